@@ -1,0 +1,779 @@
+/*
+ * oracle.c — plain, slow, single-threaded CPU ORACLE for the ABFT-protected CG
+ * hot path.  TEST INFRASTRUCTURE ONLY: only tests/, __graft_entry__.smoke() and
+ * bench.py's cpu_baseline / --impl reference legs may load it.  It shares no
+ * code, header or table generator with the CUDA path
+ * (paper_conf_cluster_pawelczakmpm17_b200/csrc/), and never calls it.
+ *
+ * Written from DESIGN.md §3-§4 (the normative code text), which restates the
+ * paper:  SED        P:207-217 (§IV)
+ *         SECDED     P:218-243 (§IV; decode rule P:230-238)
+ *         CRC32C     P:244-284 (§IV)
+ *         CSR layout P:315-327 (§V-B); element codes P:352-376 (§VI-A)
+ *         rowptr     P:377-397 (§VI-A.1); range checks P:407-416 (§VI-A.2)
+ *         vectors    P:426-451 (§VI-B); write buffering P:468-490 (§VI-C)
+ *         CG         TeaLeaf CG (ref [19]), DESIGN.md §4
+ *
+ * Every computation is the plain definition: syndromes are XORs of H-columns
+ * over a loop on every container bit, CRC32C is the bit-serial division,
+ * encoding solves the reserved bits with the inverse of the reserved-bit
+ * submatrix (Gaussian elimination over GF(2) done once per instance), SpMV is a
+ * row loop, dot products follow RED-1 literally.  Build: gcc -O2 -std=c11
+ * -ffp-contract=off -shared -fPIC -o liboracle.so oracle.c -lm
+ *
+ * Parity status: every function here is pinned by tests/test_oracle_*.py
+ * (exhaustive single/double flips, CRC32C check values of RFC 3720, survey
+ * self-check vectors, dense direct solves, closed-form eigenpairs); see
+ * DESIGN.md §10 for the pin list.  No function is "parity unpinned".
+ */
+#include <math.h>
+#include <stdint.h>
+#include <stdlib.h>
+#include <string.h>
+
+/* ------------------------------------------------------------------ enums */
+enum { S_NONE = 0, S_SED = 1, S_SECDED64 = 2, S_SECDED128 = 3, S_CRC32C = 4, N_SCHEMES = 5 };
+enum { T_ELEM = 0, T_ROWPTR = 1, T_VEC = 2, N_TARGETS = 3 };
+enum { C_DET = 0, C_COR = 1, C_UNC = 2, C_RANGE = 3 };
+enum { OUT_CLEAN = 0, OUT_CORRECTED = 1, OUT_DUE = 2 };
+enum { OK = 0, E_INVALID = -1, E_RANGE = -2, E_SHAPE = -3, E_DUE = -4, E_NOT_CONVERGED = -5 };
+
+/* counters: uint64 [N_TARGETS][N_SCHEMES][4] */
+typedef uint64_t counts_t[N_TARGETS][N_SCHEMES][4];
+
+/* ------------------------------------------------------- SECDED instances */
+/* instance ids */
+enum { I_E_SECDED = 0, I_V_SECDED64 = 1, I_R_SECDED64 = 2, I_R_SECDED128 = 3, I_V_SECDED128 = 4, N_INST = 5 };
+
+typedef struct {
+  int nbits;          /* container width */
+  int r;              /* syndrome bits */
+  int col[128];       /* H column of each container bit */
+  int nres;           /* reserved (solved) bits: check bits + overall parity */
+  int res[16];        /* container positions of reserved bits */
+  int inv[16][16];    /* inverse of the (r+1)x(nres) reserved matrix, rows = reserved bits */
+  int nforced;        /* forced-zero bits */
+  int forced[16];
+} inst_t;
+
+static inst_t INST[N_INST];
+static int inst_ready = 0;
+
+/* DESIGN.md §3.2, E-SECDED table. */
+static void build_e_secded(inst_t* I) {
+  I->nbits = 96; I->r = 7; I->nforced = 0;
+  for (int j = 0; j < 32; j++) I->col[j] = j | (0 << 5);                 /* A = val[0:32]  */
+  for (int j = 0; j < 31; j++) I->col[32 + j] = j | (1 << 5);            /* B = val[32:64] */
+  I->col[32 + 31] = 31 | (3 << 5);
+  for (int j = 0; j < 24; j++) I->col[64 + j] = j | (2 << 5);            /* C = col[0:24]  */
+  I->col[64 + 24] = 8 | (3 << 5);
+  I->col[64 + 25] = 17 | (3 << 5);
+  I->col[64 + 26] = 26 | (3 << 5);
+  I->col[64 + 27] = 27 | (3 << 5);
+  I->col[64 + 28] = 28 | (3 << 5);
+  I->col[64 + 29] = 29 | (2 << 5);
+  I->col[64 + 30] = 30 | (2 << 5);
+  I->col[64 + 31] = 31 | (1 << 5);
+  I->nres = 8;
+  for (int k = 0; k < 8; k++) I->res[k] = 88 + k;
+}
+
+/* DESIGN.md §3.2, V-SECDED64 table. */
+static void build_v_secded64(inst_t* I) {
+  I->nbits = 64; I->r = 7; I->nforced = 0;
+  for (int j = 8; j < 32; j++) I->col[j] = j;
+  for (int j = 0; j < 32; j++) I->col[32 + j] = j | (1 << 5);
+  I->col[0] = 0 | (0 << 5);
+  I->col[1] = 9 | (2 << 5);
+  I->col[2] = 18 | (2 << 5);
+  I->col[3] = 3 | (2 << 5);
+  I->col[4] = 4; I->col[5] = 5; I->col[6] = 6;
+  I->col[7] = 7 | (3 << 5);
+  I->nres = 8;
+  for (int k = 0; k < 8; k++) I->res[k] = k;
+}
+
+/* textbook extended Hamming.  cpos[k] = container bit of c_k,
+ * ppos = container bit of P, forced = forced-zero data bits. */
+static void build_textbook(inst_t* I, int nbits, int r, const int* cpos, int ppos, const int* forced, int nforced) {
+  I->nbits = nbits; I->r = r; I->nforced = nforced;
+  int is_res[128] = {0};
+  for (int k = 0; k < r; k++) { is_res[cpos[k]] = 1; I->col[cpos[k]] = 1 << k; }
+  is_res[ppos] = 1; I->col[ppos] = 0;
+  int pos = 3;
+  for (int b = 0; b < nbits; b++) {
+    if (is_res[b]) continue;
+    while ((pos & (pos - 1)) == 0) pos++;   /* skip powers of two */
+    I->col[b] = pos++;
+  }
+  I->nres = r + 1;
+  for (int k = 0; k < r; k++) I->res[k] = cpos[k];
+  I->res[r] = ppos;
+  for (int k = 0; k < nforced; k++) I->forced[k] = forced[k];
+}
+
+/* Column of bit b extended with the overall-parity row (bit r). */
+static int ext_col(const inst_t* I, int b) { return I->col[b] | (1 << I->r); }
+
+/* Invert the (r+1) x nres reserved matrix over GF(2) (square: nres = r+1). */
+static void build_inverse(inst_t* I) {
+  int n = I->nres;
+  int M[16][32];
+  for (int row = 0; row < n; row++)
+    for (int c = 0; c < n; c++) {
+      M[row][c] = (ext_col(I, I->res[c]) >> row) & 1;
+      M[row][n + c] = (row == c);
+    }
+  for (int c = 0; c < n; c++) {
+    int p = -1;
+    for (int row = c; row < n; row++) if (M[row][c]) { p = row; break; }
+    if (p < 0) abort();  /* singular: spec error */
+    if (p != c) for (int k = 0; k < 2 * n; k++) { int t = M[p][k]; M[p][k] = M[c][k]; M[c][k] = t; }
+    for (int row = 0; row < n; row++)
+      if (row != c && M[row][c]) for (int k = 0; k < 2 * n; k++) M[row][k] ^= M[c][k];
+  }
+  /* M[:, n:] = inverse: reserved value vector x = inv * syndrome_vector */
+  for (int a = 0; a < n; a++) for (int b = 0; b < n; b++) I->inv[a][b] = M[a][n + b];
+}
+
+static void init_instances(void) {
+  if (inst_ready) return;
+  build_e_secded(&INST[I_E_SECDED]);
+  build_v_secded64(&INST[I_V_SECDED64]);
+  { int c[7] = {28, 29, 30, 31, 60, 61, 62};
+    build_textbook(&INST[I_R_SECDED64], 64, 7, c, 63, NULL, 0); }
+  { int c[8] = {28, 29, 30, 31, 60, 61, 62, 63}; int f[7] = {93, 94, 95, 124, 125, 126, 127};
+    build_textbook(&INST[I_R_SECDED128], 128, 8, c, 92, f, 7); }
+  { int c[8] = {0, 1, 2, 3, 4, 64, 65, 66}; int f[1] = {68};
+    build_textbook(&INST[I_V_SECDED128], 128, 8, c, 67, f, 1); }
+  for (int i = 0; i < N_INST; i++) build_inverse(&INST[i]);
+  inst_ready = 1;
+}
+
+static int getbit(const uint32_t* w, int b) { return (w[b >> 5] >> (b & 31)) & 1; }
+static void flipbit(uint32_t* w, int b) { w[b >> 5] ^= (1u << (b & 31)); }
+static void setbit(uint32_t* w, int b, int v) { if (getbit(w, b) != v) flipbit(w, b); }
+
+/* q = parity of the container, s = XOR of H columns of set bits. */
+static void syndrome(const inst_t* I, const uint32_t* w, int* s, int* q) {
+  int ss = 0, qq = 0;
+  for (int b = 0; b < I->nbits; b++)
+    if (getbit(w, b)) { ss ^= I->col[b]; qq ^= 1; }
+  *s = ss; *q = qq;
+}
+
+/* Decode rule of DESIGN.md §3.1 / P:230-238.  Corrects w in place.  Returns
+ * OUT_* and, for OUT_CORRECTED, the flipped bit in *bit. */
+static int secded_check(const inst_t* I, uint32_t* w, int* bit) {
+  int s, q;
+  syndrome(I, w, &s, &q);
+  if (q == 0 && s == 0) return OUT_CLEAN;
+  if (q == 0) return OUT_DUE;                         /* double error */
+  int hit = -1, nhit = 0;
+  for (int b = 0; b < I->nbits; b++) if (I->col[b] == s) { hit = b; nhit++; }
+  if (nhit != 1) return OUT_DUE;                      /* not a column (R10) */
+  flipbit(w, hit);
+  if (bit) *bit = hit;
+  return OUT_CORRECTED;
+}
+
+/* Systematic encode: reserved bits := the unique solution of q = 0, s = 0. */
+static void secded_encode(const inst_t* I, uint32_t* w) {
+  for (int k = 0; k < I->nres; k++) setbit(w, I->res[k], 0);
+  int s, q;
+  syndrome(I, w, &s, &q);
+  int v = s | (q << I->r);             /* the reserved bits must cancel this */
+  for (int a = 0; a < I->nres; a++) {
+    int x = 0;
+    for (int b = 0; b < I->nres; b++) x ^= I->inv[a][b] & ((v >> b) & 1);
+    setbit(w, I->res[a], x);
+  }
+}
+
+/* ------------------------------------------------------------------ SED */
+static int parity_words(const uint32_t* w, int nbits) {
+  int p = 0;
+  for (int b = 0; b < nbits; b++) p ^= getbit(w, b);
+  return p;
+}
+
+/* -------------------------------------------------------------- CRC32C */
+/* Bit-serial CRC32C (Castagnoli, reflected 0x82F63B78, init/xorout ~0). */
+uint32_t or_crc32c(const uint8_t* msg, size_t len) {
+  uint32_t crc = 0xFFFFFFFFu;
+  for (size_t i = 0; i < len; i++) {
+    crc ^= msg[i];
+    for (int k = 0; k < 8; k++) crc = (crc >> 1) ^ (0x82F63B78u & (0u - (crc & 1u)));
+  }
+  return crc ^ 0xFFFFFFFFu;
+}
+
+/* ---------------------------------------------------- codec test hooks */
+int or_init(void) { init_instances(); return OK; }
+
+int or_inst_nbits(int inst) { init_instances(); return INST[inst].nbits; }
+int or_inst_column(int inst, int bit) { init_instances(); return INST[inst].col[bit]; }
+int or_inst_reserved(int inst, int k) { init_instances(); return k < INST[inst].nres ? INST[inst].res[k] : -1; }
+
+/* Check (and correct in place) one container; returns OUT_*; *bit = corrected bit. */
+int or_secded_check(int inst, uint32_t* words, int* bit) {
+  init_instances();
+  if (bit) *bit = -1;
+  return secded_check(&INST[inst], words, bit);
+}
+void or_secded_encode(int inst, uint32_t* words) { init_instances(); secded_encode(&INST[inst], words); }
+void or_secded_syndrome(int inst, const uint32_t* words, int* s, int* q) { init_instances(); syndrome(&INST[inst], words, s, q); }
+
+/* --------------------------------------------------- vector encodings */
+static int vec_group(int scheme) { return scheme == S_SECDED128 ? 2 : scheme == S_CRC32C ? 4 : 1; }
+static int vec_k(int scheme) {
+  switch (scheme) { case S_SED: return 1; case S_SECDED64: return 8; case S_SECDED128: return 5; case S_CRC32C: return 8; default: return 0; }
+}
+int64_t or_vec_padded_len(int64_t n, int scheme) { int64_t g = vec_group(scheme); return (n + g - 1) / g * g; }
+
+static uint64_t mask_k(int k) { return k == 0 ? ~0ull : ~((1ull << k) - 1ull); }
+
+/* DESIGN.md §3.6 round_k: + 2^(k-1), clear k LSBs; Inf/NaN truncate. */
+static uint64_t round_k(uint64_t u, int k) {
+  if (k == 0) return u;
+  if (((u >> 52) & 0x7FF) == 0x7FF) return u & mask_k(k);
+  return (u + (1ull << (k - 1))) & mask_k(k);
+}
+
+static double bits2d(uint64_t u) { double d; memcpy(&d, &u, 8); return d; }
+static uint64_t d2bits(double d) { uint64_t u; memcpy(&u, &d, 8); return u; }
+
+static void u64_to_words(const uint64_t* v, int n, uint32_t* w) {
+  for (int i = 0; i < n; i++) { w[2 * i] = (uint32_t)v[i]; w[2 * i + 1] = (uint32_t)(v[i] >> 32); }
+}
+static void words_to_u64(const uint32_t* w, int n, uint64_t* v) {
+  for (int i = 0; i < n; i++) v[i] = (uint64_t)w[2 * i] | ((uint64_t)w[2 * i + 1] << 32);
+}
+
+/* V-CRC message: 4 x (f64 with low byte zeroed) LE. */
+static uint32_t vcrc(const uint64_t* d) {
+  uint8_t m[32];
+  for (int i = 0; i < 4; i++) {
+    uint64_t u = d[i] & ~0xFFull;
+    for (int b = 0; b < 8; b++) m[8 * i + b] = (uint8_t)(u >> (8 * b));
+  }
+  return or_crc32c(m, 32);
+}
+
+/* Encode one group of G already-rounded values (reserved bits are overwritten). */
+static void vec_encode_group(uint64_t* d, int scheme) {
+  uint32_t w[4];
+  switch (scheme) {
+    case S_SED:
+      d[0] &= ~1ull;
+      u64_to_words(d, 1, w);
+      d[0] |= (uint64_t)parity_words(w, 64);
+      break;
+    case S_SECDED64:
+      u64_to_words(d, 1, w); secded_encode(&INST[I_V_SECDED64], w); words_to_u64(w, 1, d);
+      break;
+    case S_SECDED128:
+      u64_to_words(d, 2, w); secded_encode(&INST[I_V_SECDED128], w); words_to_u64(w, 2, d);
+      break;
+    case S_CRC32C: {
+      for (int i = 0; i < 4; i++) d[i] &= ~0xFFull;
+      uint32_t c = vcrc(d);
+      for (int i = 0; i < 4; i++) d[i] |= (uint64_t)((c >> (8 * i)) & 0xFF);
+      break;
+    }
+    default: break;
+  }
+}
+
+/* Check one group; corrects d in place; returns OUT_*; *word32 = index of the
+ * 32-bit word holding the corrected bit (for scrub accounting). */
+static int vec_check_group(uint64_t* d, int scheme) {
+  uint32_t w[4];
+  int out = OUT_CLEAN, bit;
+  switch (scheme) {
+    case S_SED:
+      u64_to_words(d, 1, w);
+      out = parity_words(w, 64) ? OUT_DUE : OUT_CLEAN;
+      break;
+    case S_SECDED64:
+      u64_to_words(d, 1, w); out = secded_check(&INST[I_V_SECDED64], w, &bit); words_to_u64(w, 1, d);
+      break;
+    case S_SECDED128:
+      u64_to_words(d, 2, w); out = secded_check(&INST[I_V_SECDED128], w, &bit); words_to_u64(w, 2, d);
+      break;
+    case S_CRC32C: {
+      uint32_t c = 0;
+      for (int i = 0; i < 4; i++) c |= (uint32_t)(d[i] & 0xFF) << (8 * i);
+      out = (c == vcrc(d)) ? OUT_CLEAN : OUT_DUE;
+      break;
+    }
+    default: break;
+  }
+  return out;
+}
+
+static void count_outcome(counts_t* cnt, int target, int scheme, int out) {
+  if (!cnt || out == OUT_CLEAN) return;
+  (*cnt)[target][scheme][C_DET]++;
+  if (out == OUT_CORRECTED) (*cnt)[target][scheme][C_COR]++;
+  else (*cnt)[target][scheme][C_UNC]++;
+}
+
+/* Encode a whole (padded) vector in place: round_k then ECC (a1). data holds the
+ * f64 bit patterns; entries [n, npad) are set to encoded +0.0. */
+int or_vec_encode(uint64_t* data, int64_t n, int scheme) {
+  init_instances();
+  int g = vec_group(scheme), k = vec_k(scheme);
+  int64_t npad = or_vec_padded_len(n, scheme);
+  for (int64_t i = n; i < npad; i++) data[i] = 0;
+  for (int64_t i = 0; i < npad; i++) data[i] = round_k(data[i], k);
+  for (int64_t i = 0; i < npad; i += g) vec_encode_group(data + i, scheme);
+  return OK;
+}
+
+/* Check every codeword of v (count into target VEC), write masked values to out
+ * (may be NULL); scrub = write corrections back into data.  Returns number of DUEs. */
+int64_t or_vec_check(uint64_t* data, int64_t n, int scheme, double* out, counts_t* cnt, int scrub) {
+  init_instances();
+  int g = vec_group(scheme), k = vec_k(scheme);
+  int64_t npad = or_vec_padded_len(n, scheme), dues = 0;
+  for (int64_t i = 0; i < npad; i += g) {
+    uint64_t d[4];
+    for (int j = 0; j < g; j++) d[j] = data[i + j];
+    int o = vec_check_group(d, scheme);
+    count_outcome(cnt, T_VEC, scheme, o);
+    if (o == OUT_DUE) { dues++; for (int j = 0; j < g; j++) d[j] = data[i + j]; }
+    if (o == OUT_CORRECTED && scrub) for (int j = 0; j < g; j++) data[i + j] = d[j];
+    if (out) for (int j = 0; j < g; j++) if (i + j < n) out[i + j] = bits2d(d[j] & mask_k(k));
+  }
+  return dues;
+}
+
+/* ------------------------------------------------------- rowptr codes */
+static int rp_group(int scheme) {
+  switch (scheme) { case S_SECDED64: return 2; case S_SECDED128: return 4; case S_CRC32C: return 8; default: return 1; }
+}
+static uint32_t rp_mask(int scheme) {
+  switch (scheme) { case S_NONE: return 0xFFFFFFFFu; case S_SED: return 0x7FFFFFFFu; default: return 0x0FFFFFFFu; }
+}
+int64_t or_rowptr_padded_len(int64_t nrows, int scheme) { int64_t g = rp_group(scheme); return (nrows + 1 + g - 1) / g * g; }
+
+static uint32_t rcrc(const uint32_t* e) {
+  uint8_t m[32];
+  for (int i = 0; i < 8; i++) { uint32_t u = e[i] & 0x0FFFFFFFu; for (int b = 0; b < 4; b++) m[4 * i + b] = (uint8_t)(u >> (8 * b)); }
+  return or_crc32c(m, 32);
+}
+
+static void rp_encode_group(uint32_t* e, int scheme) {
+  switch (scheme) {
+    case S_SED: e[0] &= 0x7FFFFFFFu; e[0] |= (uint32_t)parity_words(e, 31) << 31; break;
+    case S_SECDED64: secded_encode(&INST[I_R_SECDED64], e); break;
+    case S_SECDED128: secded_encode(&INST[I_R_SECDED128], e); break;
+    case S_CRC32C: {
+      for (int i = 0; i < 8; i++) e[i] &= 0x0FFFFFFFu;
+      uint32_t c = rcrc(e);
+      for (int i = 0; i < 8; i++) e[i] |= ((c >> (4 * i)) & 0xFu) << 28;
+      break;
+    }
+    default: break;
+  }
+}
+static int rp_check_group(uint32_t* e, int scheme) {
+  int bit;
+  switch (scheme) {
+    case S_SED: return parity_words(e, 32) ? OUT_DUE : OUT_CLEAN;
+    case S_SECDED64: return secded_check(&INST[I_R_SECDED64], e, &bit);
+    case S_SECDED128: return secded_check(&INST[I_R_SECDED128], e, &bit);
+    case S_CRC32C: {
+      uint32_t c = 0;
+      for (int i = 0; i < 8; i++) c |= (e[i] >> 28) << (4 * i);
+      return c == rcrc(e) ? OUT_CLEAN : OUT_DUE;
+    }
+    default: return OUT_CLEAN;
+  }
+}
+
+/* ------------------------------------------------------ element codes */
+static uint32_t col_mask(int scheme) {
+  switch (scheme) { case S_NONE: return 0xFFFFFFFFu; case S_SED: return 0x7FFFFFFFu; default: return 0x00FFFFFFu; }
+}
+
+static void el_words(uint64_t val, uint32_t col, uint32_t* w) { w[0] = (uint32_t)val; w[1] = (uint32_t)(val >> 32); w[2] = col; }
+
+/* E-CRC message of one row. */
+static uint32_t ecrc_row(const uint64_t* val, const uint32_t* col, int64_t start, int64_t end) {
+  int64_t L = end - start;
+  uint8_t* m = (uint8_t*)malloc((size_t)(12 * L));
+  for (int64_t k = 0; k < L; k++) {
+    uint64_t v = val[start + k];
+    uint32_t c = col[start + k];
+    if (k < 4) c &= 0x00FFFFFFu;
+    for (int b = 0; b < 8; b++) m[12 * k + b] = (uint8_t)(v >> (8 * b));
+    for (int b = 0; b < 4; b++) m[12 * k + 8 + b] = (uint8_t)(c >> (8 * b));
+  }
+  uint32_t crc = or_crc32c(m, (size_t)(12 * L));
+  free(m);
+  return crc;
+}
+static uint32_t ecrc_stored(const uint32_t* col, int64_t start) {
+  uint32_t c = 0;
+  for (int k = 0; k < 4; k++) c |= (col[start + k] >> 24) << (8 * k);
+  return c;
+}
+
+/* Encode a CSR matrix in place (a0): col gets ECC in its spare bits, rowptr is
+ * padded (copies of nnz) and encoded.  val is never modified.  rowptr must have
+ * or_rowptr_padded_len(nrows, rs) entries, entries [nrows+1, len) are written. */
+int or_csr_encode(const uint64_t* val, uint32_t* col, uint32_t* rowptr, int64_t nrows, int64_t ncols,
+                  int64_t nnz, int es, int rs) {
+  init_instances();
+  /* capacity checks */
+  uint64_t cmax = (es == S_NONE) ? 0xFFFFFFFFull : (es == S_SED ? 0x7FFFFFFFull : 0x00FFFFFFull);
+  uint64_t nmax = (rs == S_NONE) ? 0xFFFFFFFFull : (rs == S_SED ? 0x7FFFFFFFull : 0x0FFFFFFFull);
+  if ((uint64_t)nnz > nmax) return E_RANGE;
+  if (ncols > 0 && (uint64_t)(ncols - 1) > cmax) return E_RANGE;
+  for (int64_t e = 0; e < nnz; e++) if ((uint64_t)col[e] > cmax) return E_RANGE;
+  for (int64_t i = 0; i <= nrows; i++) if ((uint64_t)rowptr[i] > nmax) return E_RANGE;
+  if (es == S_CRC32C)
+    for (int64_t i = 0; i < nrows; i++) if (rowptr[i + 1] - rowptr[i] < 4) return E_SHAPE;
+  /* elements */
+  if (es == S_SED || es == S_SECDED64 || es == S_SECDED128) {
+    for (int64_t e = 0; e < nnz; e++) {
+      uint32_t w[3];
+      el_words(val[e], col[e], w);
+      if (es == S_SED) { w[2] &= 0x7FFFFFFFu; w[2] |= (uint32_t)parity_words(w, 95) << 31; }
+      else secded_encode(&INST[I_E_SECDED], w);
+      col[e] = w[2];
+    }
+  } else if (es == S_CRC32C) {
+    for (int64_t i = 0; i < nrows; i++) {
+      int64_t s = rowptr[i], t = rowptr[i + 1];
+      uint32_t c = ecrc_row(val, col, s, t);
+      for (int k = 0; k < 4; k++) col[s + k] = (col[s + k] & 0x00FFFFFFu) | (((c >> (8 * k)) & 0xFFu) << 24);
+    }
+  }
+  /* rowptr */
+  int64_t len = or_rowptr_padded_len(nrows, rs);
+  for (int64_t i = nrows + 1; i < len; i++) rowptr[i] = (uint32_t)nnz;
+  int g = rp_group(rs);
+  if (rs != S_NONE) for (int64_t i = 0; i < len; i += g) rp_encode_group(rowptr + i, rs);
+  return OK;
+}
+
+/* ------------------------------------------------------------- RED-1 */
+/* RB of 256, lane l sums i = l, l+32, ... with fma from +0.0,
+ * xor-butterfly 16,8,4,2,1, complete binary tree over RBs padded to 2^m. */
+static double red1_block(const double* a, const double* b, int64_t base, int64_t n) {
+  double s[32];
+  for (int l = 0; l < 32; l++) {
+    s[l] = 0.0;
+    for (int64_t i = base + l; i < base + 256 && i < n; i += 32) s[l] = fma(a[i], b[i], s[l]);
+  }
+  for (int off = 16; off >= 1; off >>= 1) {
+    double t[32];
+    for (int l = 0; l < 32; l++) t[l] = s[l] + s[l ^ off];
+    memcpy(s, t, sizeof s);
+  }
+  return s[0];
+}
+static double tree_sum(double* v, int64_t m) {   /* m = power of two */
+  while (m > 1) {
+    for (int64_t i = 0; i < m / 2; i++) v[i] = v[2 * i] + v[2 * i + 1];
+    m /= 2;
+  }
+  return v[0];
+}
+double or_dot_red1(const double* a, const double* b, int64_t n) {
+  int64_t nrb = (n + 255) / 256, m = 1;
+  while (m < nrb) m *= 2;
+  double* v = (double*)calloc((size_t)(m > 0 ? m : 1), sizeof(double));
+  for (int64_t r = 0; r < nrb; r++) v[r] = red1_block(a, b, r * 256, n);
+  double res = (n > 0) ? tree_sum(v, m) : 0.0;
+  free(v);
+  return res;
+}
+/* RB partials only (used by the multi-rank tests: per-rank subtree roots). */
+void or_red1_blocks(const double* a, const double* b, int64_t n, double* out) {
+  int64_t nrb = (n + 255) / 256;
+  for (int64_t r = 0; r < nrb; r++) out[r] = red1_block(a, b, r * 256, n);
+}
+double or_tree_sum(double* v, int64_t m) { return tree_sum(v, m); }
+
+/* ------------------------------------------------------------- SpMV */
+typedef struct {
+  int64_t nrows, ncols, nnz, row_base, col_base;
+  uint64_t* val; uint32_t* col; uint32_t* rowptr;
+  int es, rs;
+} or_csr;
+
+/* Check all elements of A (index order), counting into ELEM; fills vd/cd with
+ * decoded (masked) values and skip[] for range violations; scrubs corrections.
+ * E-CRC rows are checked in the row pass (the codeword is the row). */
+static int64_t check_elements(or_csr* A, double* vd, uint32_t* cd, uint8_t* skip, counts_t* cnt, int scrub) {
+  int64_t dues = 0;
+  uint32_t cm = col_mask(A->es);
+  for (int64_t e = 0; e < A->nnz; e++) {
+    uint32_t w[3];
+    el_words(A->val[e], A->col[e], w);
+    int o = OUT_CLEAN;
+    if (A->es == S_SED) o = parity_words(w, 96) ? OUT_DUE : OUT_CLEAN;
+    else if (A->es == S_SECDED64 || A->es == S_SECDED128) {
+      uint32_t w0[3] = {w[0], w[1], w[2]};
+      int bit;
+      o = secded_check(&INST[I_E_SECDED], w, &bit);
+      if (o == OUT_DUE) { w[0] = w0[0]; w[1] = w0[1]; w[2] = w0[2]; }
+    }
+    count_outcome(cnt, T_ELEM, A->es, o);
+    if (o == OUT_DUE) dues++;
+    if (o == OUT_CORRECTED && scrub) {
+      A->val[e] = (uint64_t)w[0] | ((uint64_t)w[1] << 32);
+      A->col[e] = w[2];
+    }
+    uint64_t v = (uint64_t)w[0] | ((uint64_t)w[1] << 32);
+    vd[e] = bits2d(v);
+    cd[e] = w[2] & cm;
+    skip[e] = 0;
+    if (A->es != S_NONE && (int64_t)cd[e] >= A->ncols) {
+      skip[e] = 1;
+      if (cnt) (*cnt)[T_ELEM][A->es][C_RANGE]++;
+      dues++;
+    }
+  }
+  return dues;
+}
+
+/* Check every rowptr group; fills rp[] with decoded masked entries. */
+static int64_t check_rowptr(or_csr* A, uint32_t* rp, counts_t* cnt, int scrub) {
+  int64_t len = or_rowptr_padded_len(A->nrows, A->rs), dues = 0;
+  int g = rp_group(A->rs);
+  uint32_t m = rp_mask(A->rs);
+  for (int64_t i = 0; i < len; i += g) {
+    uint32_t e[8];
+    for (int j = 0; j < g; j++) e[j] = A->rowptr[i + j];
+    int o = rp_check_group(e, A->rs);
+    count_outcome(cnt, T_ROWPTR, A->rs, o);
+    if (o == OUT_DUE) { dues++; for (int j = 0; j < g; j++) e[j] = A->rowptr[i + j]; }
+    if (o == OUT_CORRECTED && scrub) for (int j = 0; j < g; j++) A->rowptr[i + j] = e[j];
+    for (int j = 0; j < g; j++) rp[i + j] = e[j] & m;
+  }
+  return dues;
+}
+
+/* Protected SpMV out = A*in.  in/out are padded encoded
+ * vectors (f64 bit patterns) of logical length n_in / n_out.  The `in`
+ * codewords inside [row_base, row_base+nrows) are owned (counted, scrubbed);
+ * others are corrected silently.  dot (may be NULL) = RED-1 sum of
+ * in[row_base+i]*out[row_base+i] over masked values.  Returns number of DUE +
+ * range violations seen (the caller applies the DUE policy). */
+int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, int64_t n_out, counts_t* cnt,
+                double* dot) {
+  init_instances();
+  int64_t dues = 0;
+  int g = vec_group(vs), k = vec_k(vs);
+  double* vd = (double*)malloc(sizeof(double) * (size_t)(A->nnz + 1));
+  uint32_t* cd = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)(A->nnz + 1));
+  uint8_t* skip = (uint8_t*)malloc((size_t)(A->nnz + 1));
+  int64_t rplen = or_rowptr_padded_len(A->nrows, A->rs);
+  uint32_t* rp = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)rplen);
+  int64_t npad_in = or_vec_padded_len(n_in, vs);
+  double* xin = (double*)malloc(sizeof(double) * (size_t)npad_in);
+
+  dues += check_elements(A, vd, cd, skip, cnt, 1);
+  dues += check_rowptr(A, rp, cnt, 1);
+  /* every codeword of `in`: owned ones counted + scrubbed */
+  for (int64_t i = 0; i < npad_in; i += g) {
+    uint64_t d[4];
+    for (int j = 0; j < g; j++) d[j] = in[i + j];
+    int o = vec_check_group(d, vs);
+    int owned = (i >= A->row_base && i < A->row_base + A->nrows);
+    if (owned) { count_outcome(cnt, T_VEC, vs, o); if (o == OUT_DUE) dues++; }
+    if (o == OUT_DUE) for (int j = 0; j < g; j++) d[j] = in[i + j];
+    if (o == OUT_CORRECTED && owned) for (int j = 0; j < g; j++) in[i + j] = d[j];
+    for (int j = 0; j < g; j++) xin[i + j] = bits2d(d[j] & mask_k(k));
+  }
+  /* rows */
+  double* acc = (double*)malloc(sizeof(double) * (size_t)(A->nrows + 1));
+  for (int64_t i = 0; i < A->nrows; i++) {
+    uint32_t s = rp[i], t = rp[i + 1];
+    double a = 0.0;
+    if (!(s <= t && (int64_t)t <= A->nnz)) {
+      if (cnt && A->rs != S_NONE) (*cnt)[T_ROWPTR][A->rs][C_RANGE]++;
+      if (A->rs != S_NONE) dues++;
+      acc[i] = 0.0;
+      continue;
+    }
+    if (A->es == S_CRC32C) {           /* E-CRC: the row is the codeword */
+      int o;
+      if (t - s < 4) o = OUT_DUE;
+      else o = (ecrc_stored(A->col, s) == ecrc_row(A->val, A->col, s, t)) ? OUT_CLEAN : OUT_DUE;
+      count_outcome(cnt, T_ELEM, S_CRC32C, o);
+      if (o == OUT_DUE) dues++;
+    }
+    for (uint32_t j = s; j < t; j++) {
+      if (skip[j]) continue;
+      a = fma(vd[j], xin[A->col_base + cd[j]], a);
+    }
+    acc[i] = a;
+  }
+  /* write buffered: whole groups of `out` */
+  int64_t lo = A->row_base, hi = A->row_base + A->nrows;
+  int64_t npad_out = or_vec_padded_len(n_out, vs);
+  for (int64_t i = lo; i < hi; i += g) {
+    uint64_t d[4];
+    for (int j = 0; j < g; j++) {
+      int64_t r = i + j;
+      d[j] = (r < hi) ? round_k(d2bits(acc[r - lo]), k) : 0ull;
+    }
+    vec_encode_group(d, vs);
+    for (int j = 0; j < g; j++) if (i + j < npad_out) out[i + j] = d[j];
+  }
+  if (dot) {
+    double* a = (double*)malloc(sizeof(double) * (size_t)(A->nrows + 1));
+    double* b = (double*)malloc(sizeof(double) * (size_t)(A->nrows + 1));
+    for (int64_t i = 0; i < A->nrows; i++) {
+      a[i] = xin[lo + i];
+      b[i] = bits2d(out[lo + i] & mask_k(k));
+    }
+    *dot = or_dot_red1(a, b, A->nrows);
+    free(a); free(b);
+  }
+  free(acc); free(vd); free(cd); free(skip); free(rp); free(xin);
+  return dues;
+}
+
+/* ---------------------------------------------------------- check_all */
+int64_t or_check_csr(or_csr* A, counts_t* cnt, int scrub) {
+  init_instances();
+  double* vd = (double*)malloc(sizeof(double) * (size_t)(A->nnz + 1));
+  uint32_t* cd = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)(A->nnz + 1));
+  uint8_t* skip = (uint8_t*)malloc((size_t)(A->nnz + 1));
+  int64_t rplen = or_rowptr_padded_len(A->nrows, A->rs);
+  uint32_t* rp = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)rplen);
+  int64_t dues = check_elements(A, vd, cd, skip, cnt, scrub);
+  dues += check_rowptr(A, rp, cnt, scrub);
+  for (int64_t i = 0; i < A->nrows; i++) {
+    uint32_t s = rp[i], t = rp[i + 1];
+    if (!(s <= t && (int64_t)t <= A->nnz)) {
+      if (cnt && A->rs != S_NONE) (*cnt)[T_ROWPTR][A->rs][C_RANGE]++;
+      if (A->rs != S_NONE) dues++;
+      continue;
+    }
+    if (A->es == S_CRC32C) {
+      int o = (t - s < 4) ? OUT_DUE : (ecrc_stored(A->col, s) == ecrc_row(A->val, A->col, s, t) ? OUT_CLEAN : OUT_DUE);
+      count_outcome(cnt, T_ELEM, S_CRC32C, o);
+      if (o == OUT_DUE) dues++;
+    }
+  }
+  free(vd); free(cd); free(skip); free(rp);
+  return dues;
+}
+
+/* ---------------------------------------------------------- CG pieces */
+/* Decode a whole vector into masked doubles, counting + scrubbing (owned). */
+static int64_t vdec(uint64_t* v, int64_t n, int vs, double* out, counts_t* cnt) {
+  return or_vec_check(v, n, vs, out, cnt, 1);
+}
+/* Encode n computed doubles into v (round_k + ECC per group), padding = +0.0. */
+static void venc(uint64_t* v, const double* x, int64_t n, int vs) {
+  int g = vec_group(vs), k = vec_k(vs);
+  int64_t npad = or_vec_padded_len(n, vs);
+  for (int64_t i = 0; i < npad; i += g) {
+    uint64_t d[4];
+    for (int j = 0; j < g; j++) d[j] = (i + j < n) ? round_k(d2bits(x[i + j]), k) : 0ull;
+    vec_encode_group(d, vs);
+    for (int j = 0; j < g; j++) v[i + j] = d[j];
+  }
+}
+static void vmasked(const uint64_t* v, int64_t n, int vs, double* out) {
+  int k = vec_k(vs);
+  for (int64_t i = 0; i < n; i++) out[i] = bits2d(v[i] & mask_k(k));
+}
+
+/* calc_ur (a4): x = enc(fma(a,p,x)); r = enc(fma(-a,w,r)); returns rrn. */
+int64_t or_calc_ur(uint64_t* x, uint64_t* p, uint64_t* r, uint64_t* w, int64_t n, int vs, double alpha,
+                   counts_t* cnt, double* rrn) {
+  init_instances();
+  double* X = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* P = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* R = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* W = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  int64_t dues = vdec(x, n, vs, X, cnt) + vdec(p, n, vs, P, cnt) + vdec(r, n, vs, R, cnt) + vdec(w, n, vs, W, cnt);
+  for (int64_t i = 0; i < n; i++) {
+    X[i] = fma(alpha, P[i], X[i]);
+    R[i] = fma(-alpha, W[i], R[i]);
+  }
+  venc(x, X, n, vs);
+  venc(r, R, n, vs);
+  vmasked(r, n, vs, R);
+  *rrn = or_dot_red1(R, R, n);
+  free(X); free(P); free(R); free(W);
+  return dues;
+}
+
+/* calc_p (a5): p = enc(fma(beta, p, r)). */
+int64_t or_calc_p(uint64_t* p, uint64_t* r, int64_t n, int vs, double beta, counts_t* cnt) {
+  init_instances();
+  double* P = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* R = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  int64_t dues = vdec(r, n, vs, R, cnt) + vdec(p, n, vs, P, cnt);
+  for (int64_t i = 0; i < n; i++) P[i] = fma(beta, P[i], R[i]);
+  venc(p, P, n, vs);
+  free(P); free(R);
+  return dues;
+}
+
+/* init part 2 (a2): r = enc(b - w); p = r; returns rr0 = r.r */
+int64_t or_cg_init_r(uint64_t* b, uint64_t* w, uint64_t* r, uint64_t* p, int64_t n, int vs, counts_t* cnt, double* rr0) {
+  init_instances();
+  double* B = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* W = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  int64_t dues = vdec(b, n, vs, B, cnt) + vdec(w, n, vs, W, cnt);
+  for (int64_t i = 0; i < n; i++) B[i] = B[i] - W[i];
+  venc(r, B, n, vs);
+  int64_t npad = or_vec_padded_len(n, vs);
+  memcpy(p, r, sizeof(uint64_t) * (size_t)npad);
+  vmasked(r, n, vs, B);
+  *rr0 = or_dot_red1(B, B, n);
+  free(B); free(W);
+  return dues;
+}
+
+typedef struct { int32_t iters; int32_t status; double rr0, rrn; } or_cg_result;
+
+/* Protected CG on a single (unchunked, square) matrix, DESIGN.md §4.
+ * Vectors are padded encoded arrays of logical length n = A->nrows.
+ * due_policy: 0 abort (finish the iteration, return E_DUE), 1 continue.
+ * max_iters <= 0: only the init.  Returns status. */
+int or_cg_solve(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
+                int max_iters, int due_policy, or_cg_result* res, counts_t* cnt) {
+  init_instances();
+  int64_t n = A->nrows;
+  double rr0, rro, rrn = 0.0, pw;
+  res->iters = 0; res->status = OK; res->rr0 = 0.0; res->rrn = 0.0;
+  int64_t dues = or_spmv(A, x, n, vs, w, n, cnt, NULL);
+  dues += or_cg_init_r(b, w, r, p, n, vs, cnt, &rr0);
+  res->rr0 = rr0; res->rrn = rr0;
+  if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+  if (rr0 == 0.0) return OK;
+  rro = rr0;
+  for (int k = 1; k <= max_iters; k++) {
+    dues = or_spmv(A, p, n, vs, w, n, cnt, &pw);
+    double alpha = rro / pw;
+    dues += or_calc_ur(x, p, r, w, n, vs, alpha, cnt, &rrn);
+    res->iters = k; res->rrn = rrn;
+    int conv = sqrt(rrn) <= tol * sqrt(rr0);
+    if (!conv) {
+      double beta = rrn / rro;
+      dues += or_calc_p(p, r, n, vs, beta, cnt);
+      rro = rrn;
+    }
+    if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+    if (conv) return OK;
+  }
+  res->status = (max_iters > 0) ? E_NOT_CONVERGED : OK;
+  return res->status;
+}
+
+/* Masked-value helper for tests: clear the k reserved LSBs of each entry. */
+void or_vec_masked(const uint64_t* v, int64_t n, int vs, double* out) { vmasked(v, n, vs, out); }
+uint64_t or_round_k(uint64_t u, int k) { return round_k(u, k); }
