@@ -1,0 +1,169 @@
+/*
+ * abft.h — C ABI of libabft.so: the ABFT-protected CG hot path on B200 (sm_100a).
+ *
+ * The calls follow the paper's statement of the problem (Pawelczak et al.,
+ * CLUSTER 2017; P:a-b = /root/reference/PAPER.md lines):
+ *   protect a CSR matrix (val, col, rowptr) and dense fp64 vectors with
+ *   SED / SECDED64 / SECDED128 / CRC32C at zero storage overhead
+ *   (P:146-152); correct single flips and detect double
+ *   flips on load; let the application decide on a DUE;
+ *   run the protected SpMV and the protected CG (§V-A).
+ * The codes themselves are specified in DESIGN.md §3.
+ *
+ * Conventions
+ *  - Every large buffer is DEVICE memory allocated and owned by the caller; the
+ *    library never frees it.  Scratch (reduction partials, CG scalars) belongs
+ *    to an abft_ctx and is freed by abft_ctx_destroy.
+ *  - `stream` is a cudaStream_t passed as void* (NULL = legacy default stream).
+ *    Calls are stream-ordered and asynchronous unless documented "syncs".
+ *  - Errors are returned as abft_status codes (never exceptions);
+ *    abft_last_error() gives a thread-local message for the last non-OK return.
+ *  - Host-side metadata (sizes, schemes) is unprotected.
+ *  - Handles are not thread-safe.
+ */
+#ifndef ABFT_H_
+#define ABFT_H_
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+/* Protection schemes. */
+typedef enum { ABFT_NONE = 0, ABFT_SED = 1, ABFT_SECDED64 = 2, ABFT_SECDED128 = 3, ABFT_CRC32C = 4,
+               ABFT_SCHEME_COUNT = 5 } abft_scheme;
+/* Counter targets: CSR elements, row pointers, dense vectors. */
+typedef enum { ABFT_T_ELEM = 0, ABFT_T_ROWPTR = 1, ABFT_T_VEC = 2, ABFT_T_COUNT = 3 } abft_target;
+
+/* Per (target, scheme) fault counters.  A counters buffer is a
+ * DEVICE array abft_counts[ABFT_T_COUNT][ABFT_SCHEME_COUNT] (480 bytes). */
+typedef struct { uint64_t detected, corrected, uncorrectable, range_violations; } abft_counts;
+
+typedef enum {
+  ABFT_OK = 0,
+  ABFT_E_INVALID = -1,        /* bad argument (null pointer, size, scheme, aliasing) */
+  ABFT_E_RANGE = -2,          /* an index / nnz exceeds the scheme's capacity */
+  ABFT_E_SHAPE = -3,          /* e.g. a CRC32C row with < 4 entries */
+  ABFT_E_DUE = -4,            /* uncorrectable error seen under policy abort */
+  ABFT_E_NOT_CONVERGED = -5,  /* CG hit max_iters */
+  ABFT_E_CUDA = -6,
+  ABFT_E_NCCL = -7
+} abft_status;
+
+/* One CSR matrix (or one row-block chunk of a larger matrix, reading R7).
+ * val: f64[nnz] (never modified except by scrubbing), col: u32[nnz] (ECC in
+ * its top bits after encode), rowptr: u32[abft_rowptr_padded_len(nrows, rowptr_scheme)].
+ * Local row i writes out[row_base + i]; local column c reads in[col_base + c].
+ * stencil_n: performance hint only (row stride of a 5-point stencil, 0 = none);
+ * results never depend on it. */
+typedef struct {
+  int64_t nrows, ncols, nnz;
+  int64_t row_base, col_base;
+  double* val;
+  uint32_t* col;
+  uint32_t* rowptr;
+  int32_t elem_scheme, rowptr_scheme;
+  int64_t stencil_n;
+} abft_csr;
+
+/* A dense fp64 vector of logical length n; data has abft_vec_padded_len(n, scheme)
+ * entries (padding holds encoded +0.0). */
+typedef struct { int64_t n; double* data; int32_t scheme; } abft_vec;
+
+typedef struct abft_ctx abft_ctx;
+
+/* Create / destroy a context on `device` (owns scratch, events, graphs). */
+int abft_ctx_create(int device, abft_ctx** out);
+int abft_ctx_destroy(abft_ctx* ctx);
+
+int64_t abft_rowptr_padded_len(int64_t nrows, int32_t scheme);  /* pad with copies of nnz (R6) */
+int64_t abft_vec_padded_len(int64_t n, int32_t scheme);         /* pad with encoded +0.0 */
+
+/* a0: encode a CSR matrix in place: ECC into col's top bits and rowptr's top bits
+ * (P:361-397), validates capacities (ABFT_E_RANGE) and CRC row lengths
+ * (ABFT_E_SHAPE).  Syncs `stream` (returns the validation result). */
+int abft_csr_encode(abft_ctx* ctx, abft_csr* A, void* stream);
+
+/* a1: encode a vector in place: round_k then ECC in the k low mantissa bits
+ * (DESIGN.md §3.6).  Input: plain f64 values in data[0..n). */
+int abft_vec_encode(abft_ctx* ctx, abft_vec* v, void* stream);
+
+/* Check every codeword of v, write the masked values to out_masked (device
+ * f64[n], may be NULL), count into dcnt (device, may be NULL), scrub single
+ * flips in place. */
+int abft_vec_decode(abft_ctx* ctx, abft_vec* v, double* out_masked, abft_counts* dcnt, void* stream);
+
+/* a3: protected SpMV out = A*in over nchunks chunks.
+ * dot_out (device f64, may be NULL) receives sum_i in[row]*out[row] over the
+ * chunks' rows, RED-1 order.  in and out must not alias. */
+int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, double* dot_out,
+              abft_counts* dcnt, void* stream);
+
+typedef struct {
+  double tol;          /* stop when sqrt(r.r) <= tol*sqrt(r0.r0) (R15) */
+  int32_t max_iters;
+  int32_t due_policy;  /* 0 = abort (finish the iteration, return ABFT_E_DUE), 1 = continue */
+  int32_t poll_every;  /* iterations between host polls of the stop flag (0 = default 16) */
+} abft_cg_opts;
+
+typedef struct { int32_t iters; int32_t status; double rr0, rrn; } abft_cg_result;
+
+/* a2-a7: protected CG.  x holds x0 on entry and the solution on
+ * return; r, p, w are work vectors of the same length/scheme.  The iteration
+ * runs on the device (alpha/beta/convergence computed by the reduction
+ * kernels); the host only polls a stop flag every opts->poll_every
+ * iterations.  Syncs `stream`.  Returns res->status. */
+int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                  abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream);
+
+/* Check (and with scrub=1 correct in place) every codeword of the matrix chunks
+ * and of the nvec vectors, counting into dcnt. */
+int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs, int nvec, int scrub,
+                   abft_counts* dcnt, void* stream);
+
+/* Fault injection (not in the paper; the harness of S§3.4): XOR one stored bit
+ * at bit_offset of the device buffer dev_base.  Stream-ordered. */
+int abft_inject_bitflip(abft_ctx* ctx, void* dev_base, uint64_t bit_offset, void* stream);
+
+/* Copy the device counters to host_out[ABFT_T_COUNT*ABFT_SCHEME_COUNT].  Syncs. */
+int abft_counts_read(const abft_counts* dcnt, abft_counts* host_out, void* stream);
+int abft_counts_reset(abft_counts* dcnt, void* stream);
+
+/* Number of kernels this process launched through the library so far. */
+uint64_t abft_launch_count(void);
+
+/* Per-kernel-class device time accumulated by the CG driver when profiling is
+ * on (CUDA events on the launch stream): class 0 SpMV, 1 calc_ur, 2 calc_p,
+ * 3 reductions.  abft_profile(ctx, 1) clears and enables. */
+int abft_profile(abft_ctx* ctx, int enable);
+int abft_profile_read(abft_ctx* ctx, double* ms_out /*[4]*/, int64_t* launches_out /*[4]*/);
+
+const char* abft_last_error(void);
+
+/* ---- multi-GPU (row-block strips, reading S§8(e)) ----
+ * One process per GPU.  nccl_unique_id: 128 bytes from ncclGetUniqueId on rank 0,
+ * broadcast by the caller (torch.distributed).  The local vectors have n_halo
+ * extra entries before and after the local rows (ghost rows of the strip). */
+typedef struct abft_dist abft_dist;
+int abft_dist_init(abft_dist** out, const void* nccl_unique_id, int rank, int nranks, int device);
+int abft_dist_get_unique_id(void* out128);
+int abft_dist_destroy(abft_dist* d);
+/* Distributed protected CG: each rank passes its strip's chunks (col_base
+ * relative to the halo-extended vector) and its halo-extended vectors; halos of
+ * encoded p are exchanged with rank-1 / rank+1 before each SpMV, and the RED-1
+ * subtree roots of the two dot products are all-gathered (bit-identical to one
+ * GPU when every rank owns a power-of-two number of reduction blocks). */
+int abft_cg_solve_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b,
+                       abft_vec* x, abft_vec* r, abft_vec* p, abft_vec* w, const abft_cg_opts* opts,
+                       abft_cg_result* res, abft_counts* dcnt, void* stream);
+
+/* Host-side codec hooks (no GPU needed): run the exact __host__ __device__
+ * codec functions on the CPU for the unit tests.  inst: 0 E-SECDED, 1 V-SECDED64,
+ * 2 R-SECDED64, 3 R-SECDED128, 4 V-SECDED128.  Returns 0 clean, 1 corrected, 2 DUE. */
+int abft_codec_host_check(int inst, uint32_t* words);
+void abft_codec_host_encode(int inst, uint32_t* words);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* ABFT_H_ */

@@ -506,42 +506,6 @@ typedef struct {
   int es, rs;
 } or_csr;
 
-/* Check all elements of A (index order), counting into ELEM; fills vd/cd with
- * decoded (masked) values and skip[] for range violations; scrubs corrections.
- * E-CRC rows are checked in the row pass (the codeword is the row). */
-static int64_t check_elements(or_csr* A, double* vd, uint32_t* cd, uint8_t* skip, counts_t* cnt, int scrub) {
-  int64_t dues = 0;
-  uint32_t cm = col_mask(A->es);
-  for (int64_t e = 0; e < A->nnz; e++) {
-    uint32_t w[3];
-    el_words(A->val[e], A->col[e], w);
-    int o = OUT_CLEAN;
-    if (A->es == S_SED) o = parity_words(w, 96) ? OUT_DUE : OUT_CLEAN;
-    else if (A->es == S_SECDED64 || A->es == S_SECDED128) {
-      uint32_t w0[3] = {w[0], w[1], w[2]};
-      int bit;
-      o = secded_check(&INST[I_E_SECDED], w, &bit);
-      if (o == OUT_DUE) { w[0] = w0[0]; w[1] = w0[1]; w[2] = w0[2]; }
-    }
-    count_outcome(cnt, T_ELEM, A->es, o);
-    if (o == OUT_DUE) dues++;
-    if (o == OUT_CORRECTED && scrub) {
-      A->val[e] = (uint64_t)w[0] | ((uint64_t)w[1] << 32);
-      A->col[e] = w[2];
-    }
-    uint64_t v = (uint64_t)w[0] | ((uint64_t)w[1] << 32);
-    vd[e] = bits2d(v);
-    cd[e] = w[2] & cm;
-    skip[e] = 0;
-    if (A->es != S_NONE && (int64_t)cd[e] >= A->ncols) {
-      skip[e] = 1;
-      if (cnt) (*cnt)[T_ELEM][A->es][C_RANGE]++;
-      dues++;
-    }
-  }
-  return dues;
-}
-
 /* Check every rowptr group; fills rp[] with decoded masked entries. */
 static int64_t check_rowptr(or_csr* A, uint32_t* rp, counts_t* cnt, int scrub) {
   int64_t len = or_rowptr_padded_len(A->nrows, A->rs), dues = 0;
@@ -559,26 +523,38 @@ static int64_t check_rowptr(or_csr* A, uint32_t* rp, counts_t* cnt, int scrub) {
   return dues;
 }
 
-/* Protected SpMV out = A*in.  in/out are padded encoded
- * vectors (f64 bit patterns) of logical length n_in / n_out.  The `in`
- * codewords inside [row_base, row_base+nrows) are owned (counted, scrubbed);
- * others are corrected silently.  dot (may be NULL) = RED-1 sum of
- * in[row_base+i]*out[row_base+i] over masked values.  Returns number of DUE +
- * range violations seen (the caller applies the DUE policy). */
+/* Check one CSR element codeword (SED / E-SECDED), correcting w in place. */
+static int el_check(int es, uint32_t* w) {
+  int bit;
+  if (es == S_SED) return parity_words(w, 96) ? OUT_DUE : OUT_CLEAN;
+  if (es == S_SECDED64 || es == S_SECDED128) {
+    uint32_t w0[3] = {w[0], w[1], w[2]};
+    int o = secded_check(&INST[I_E_SECDED], w, &bit);
+    if (o == OUT_DUE) { w[0] = w0[0]; w[1] = w0[1]; w[2] = w0[2]; }
+    return o;
+  }
+  return OUT_CLEAN;
+}
+
+/* Protected SpMV out = A*in (counting per §3.8).
+ * Every rowptr group is checked once; every `in` codeword is checked once and
+ * those inside [row_base, row_base+nrows) are owned (counted, scrubbed); CSR
+ * elements are checked on each access by a row (a single flip is counted and
+ * scrubbed at its first access, a DUE at every access).  in/out are padded
+ * encoded vectors (f64 bit patterns) of logical length n_in / n_out.
+ * dot (may be NULL) = RED-1 sum of in[row_base+i]*out[row_base+i] over masked
+ * values.  Returns the number of DUEs + range violations seen. */
 int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, int64_t n_out, counts_t* cnt,
                 double* dot) {
   init_instances();
   int64_t dues = 0;
   int g = vec_group(vs), k = vec_k(vs);
-  double* vd = (double*)malloc(sizeof(double) * (size_t)(A->nnz + 1));
-  uint32_t* cd = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)(A->nnz + 1));
-  uint8_t* skip = (uint8_t*)malloc((size_t)(A->nnz + 1));
+  uint32_t cm = col_mask(A->es);
   int64_t rplen = or_rowptr_padded_len(A->nrows, A->rs);
   uint32_t* rp = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)rplen);
   int64_t npad_in = or_vec_padded_len(n_in, vs);
   double* xin = (double*)malloc(sizeof(double) * (size_t)npad_in);
 
-  dues += check_elements(A, vd, cd, skip, cnt, 1);
   dues += check_rowptr(A, rp, cnt, 1);
   /* every codeword of `in`: owned ones counted + scrubbed */
   for (int64_t i = 0; i < npad_in; i += g) {
@@ -610,8 +586,23 @@ int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, in
       if (o == OUT_DUE) dues++;
     }
     for (uint32_t j = s; j < t; j++) {
-      if (skip[j]) continue;
-      a = fma(vd[j], xin[A->col_base + cd[j]], a);
+      uint32_t w[3];
+      el_words(A->val[j], A->col[j], w);
+      int o = el_check(A->es, w);
+      count_outcome(cnt, T_ELEM, A->es, o);
+      if (o == OUT_DUE) dues++;
+      if (o == OUT_CORRECTED) {          /* scrub: later accesses see the clean codeword */
+        A->val[j] = (uint64_t)w[0] | ((uint64_t)w[1] << 32);
+        A->col[j] = w[2];
+      }
+      uint32_t c = w[2] & cm;
+      if (A->es != S_NONE && (int64_t)c >= A->ncols) {
+        if (cnt) (*cnt)[T_ELEM][A->es][C_RANGE]++;
+        dues++;
+        continue;
+      }
+      double v = bits2d((uint64_t)w[0] | ((uint64_t)w[1] << 32));
+      a = fma(v, xin[A->col_base + c], a);
     }
     acc[i] = a;
   }
@@ -637,7 +628,36 @@ int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, in
     *dot = or_dot_red1(a, b, A->nrows);
     free(a); free(b);
   }
-  free(acc); free(vd); free(cd); free(skip); free(rp); free(xin);
+  free(acc); free(rp); free(xin);
+  return dues;
+}
+
+/* Check all elements of A (index order), counting into ELEM; fills vd/cd with
+ * decoded (masked) values and skip[] for range violations; scrubs corrections.
+ * E-CRC rows are checked in the row pass (the codeword is the row). */
+static int64_t check_elements(or_csr* A, double* vd, uint32_t* cd, uint8_t* skip, counts_t* cnt, int scrub) {
+  int64_t dues = 0;
+  uint32_t cm = col_mask(A->es);
+  for (int64_t e = 0; e < A->nnz; e++) {
+    uint32_t w[3];
+    el_words(A->val[e], A->col[e], w);
+    int o = el_check(A->es, w);
+    count_outcome(cnt, T_ELEM, A->es, o);
+    if (o == OUT_DUE) dues++;
+    if (o == OUT_CORRECTED && scrub) {
+      A->val[e] = (uint64_t)w[0] | ((uint64_t)w[1] << 32);
+      A->col[e] = w[2];
+    }
+    uint64_t v = (uint64_t)w[0] | ((uint64_t)w[1] << 32);
+    vd[e] = bits2d(v);
+    cd[e] = w[2] & cm;
+    skip[e] = 0;
+    if (A->es != S_NONE && (int64_t)cd[e] >= A->ncols) {
+      skip[e] = 1;
+      if (cnt) (*cnt)[T_ELEM][A->es][C_RANGE]++;
+      dues++;
+    }
+  }
   return dues;
 }
 

@@ -1,0 +1,332 @@
+"""ctypes binding of libabft.so (include/abft.h) — argument marshalling only.
+
+Every step of the hot path runs in the library's CUDA kernels; torch is used
+for device memory, streams and process groups.  Importing this module fails
+loudly if the compiled library is missing: there is no CPU fallback.
+"""
+from __future__ import annotations
+
+import ctypes as C
+import os
+
+import torch
+
+from . import build as _build
+
+NONE, SED, SECDED64, SECDED128, CRC32C = range(5)
+SCHEMES = {"none": NONE, "sed": SED, "secded64": SECDED64, "secded128": SECDED128, "crc32c": CRC32C}
+ELEM, ROWPTR, VEC = range(3)
+OK, E_INVALID, E_RANGE, E_SHAPE, E_DUE, E_NOT_CONVERGED, E_CUDA, E_NCCL = 0, -1, -2, -3, -4, -5, -6, -7
+
+_SO = _build.SO
+if not os.path.exists(_SO):
+    raise ImportError(f"libabft.so not built ({_SO}); run __graft_entry__.build() "
+                      "or python -m paper_conf_cluster_pawelczakmpm17_b200.build")
+
+
+class CSR(C.Structure):
+    _fields_ = [("nrows", C.c_int64), ("ncols", C.c_int64), ("nnz", C.c_int64), ("row_base", C.c_int64),
+                ("col_base", C.c_int64), ("val", C.c_void_p), ("col", C.c_void_p), ("rowptr", C.c_void_p),
+                ("elem_scheme", C.c_int32), ("rowptr_scheme", C.c_int32), ("stencil_n", C.c_int64)]
+
+
+class Vec(C.Structure):
+    _fields_ = [("n", C.c_int64), ("data", C.c_void_p), ("scheme", C.c_int32)]
+
+
+class CGOpts(C.Structure):
+    _fields_ = [("tol", C.c_double), ("max_iters", C.c_int32), ("due_policy", C.c_int32), ("poll_every", C.c_int32)]
+
+
+class CGResult(C.Structure):
+    _fields_ = [("iters", C.c_int32), ("status", C.c_int32), ("rr0", C.c_double), ("rrn", C.c_double)]
+
+
+_lib = C.CDLL(_SO)
+_P = C.c_void_p
+_sig = {
+    "abft_ctx_create": (C.c_int, [C.c_int, C.POINTER(C.c_void_p)]),
+    "abft_ctx_destroy": (C.c_int, [_P]),
+    "abft_rowptr_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
+    "abft_vec_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
+    "abft_csr_encode": (C.c_int, [_P, C.POINTER(CSR), _P]),
+    "abft_vec_encode": (C.c_int, [_P, C.POINTER(Vec), _P]),
+    "abft_vec_decode": (C.c_int, [_P, C.POINTER(Vec), _P, _P, _P]),
+    "abft_spmv": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), _P, _P, _P]),
+    "abft_cg_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
+                                C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
+    "abft_check_all": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.c_int, C.c_int, _P, _P]),
+    "abft_inject_bitflip": (C.c_int, [_P, _P, C.c_uint64, _P]),
+    "abft_counts_read": (C.c_int, [_P, _P, _P]),
+    "abft_counts_reset": (C.c_int, [_P, _P]),
+    "abft_launch_count": (C.c_uint64, []),
+    "abft_profile": (C.c_int, [_P, C.c_int]),
+    "abft_profile_read": (C.c_int, [_P, _P, _P]),
+    "abft_last_error": (C.c_char_p, []),
+    "abft_dist_init": (C.c_int, [C.POINTER(C.c_void_p), _P, C.c_int, C.c_int, C.c_int]),
+    "abft_dist_get_unique_id": (C.c_int, [_P]),
+    "abft_dist_destroy": (C.c_int, [_P]),
+    "abft_cg_solve_dist": (C.c_int, [_P, _P, C.POINTER(CSR), C.c_int, C.c_int64, C.POINTER(Vec), C.POINTER(Vec),
+                                     C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts),
+                                     C.POINTER(CGResult), _P, _P]),
+    "abft_codec_host_check": (C.c_int, [C.c_int, _P]),
+    "abft_codec_host_encode": (None, [C.c_int, _P]),
+}
+for _name, (_res, _args) in _sig.items():
+    _f = getattr(_lib, _name)
+    _f.restype = _res
+    _f.argtypes = _args
+
+HEADER_SYMBOLS = sorted(_sig)
+
+
+class AbftError(RuntimeError):
+    def __init__(self, code: int, what: str):
+        super().__init__(f"{what}: status {code}: {last_error()}")
+        self.code = code
+
+
+def last_error() -> str:
+    return (_lib.abft_last_error() or b"").decode()
+
+
+def _check(code: int, what: str, allow=()) -> int:
+    if code != OK and code not in allow:
+        raise AbftError(code, what)
+    return code
+
+
+def _stream(stream) -> int | None:
+    if stream is None:
+        return torch.cuda.current_stream().cuda_stream
+    return stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
+
+
+def launch_count() -> int:
+    return int(_lib.abft_launch_count())
+
+
+def rowptr_padded_len(nrows: int, scheme: int) -> int:
+    return int(_lib.abft_rowptr_padded_len(nrows, scheme))
+
+
+def vec_padded_len(n: int, scheme: int) -> int:
+    return int(_lib.abft_vec_padded_len(n, scheme))
+
+
+def codec_host_check(inst: int, words) -> int:
+    buf = (C.c_uint32 * len(words))(*[int(w) for w in words])
+    o = _lib.abft_codec_host_check(inst, C.cast(buf, C.c_void_p))
+    words[:] = list(buf)
+    return o
+
+
+def codec_host_encode(inst: int, words) -> list:
+    buf = (C.c_uint32 * len(words))(*[int(w) for w in words])
+    _lib.abft_codec_host_encode(inst, C.cast(buf, C.c_void_p))
+    return list(buf)
+
+
+# ------------------------------------------------------------------ objects
+class Context:
+    """abft_ctx: owns reduction scratch and the device CG scalars."""
+
+    def __init__(self, device: int | None = None):
+        if not torch.cuda.is_available():
+            raise RuntimeError("the ABFT CUDA path needs a GPU (no CPU fallback)")
+        self.device = torch.cuda.current_device() if device is None else int(device)
+        h = C.c_void_p()
+        _check(_lib.abft_ctx_create(self.device, C.byref(h)), "abft_ctx_create")
+        self.h = h
+
+    def close(self):
+        if self.h:
+            _lib.abft_ctx_destroy(self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+class Vector:
+    """A protected fp64 vector: `data` is a float64 device tensor of padded length
+    whose bit patterns carry the ECC (never touch it with torch arithmetic)."""
+
+    def __init__(self, data: torch.Tensor, n: int, scheme: int):
+        assert data.dtype == torch.float64 and data.is_cuda and data.is_contiguous()
+        assert data.numel() >= vec_padded_len(n, scheme)
+        self.data, self.n, self.scheme = data, int(n), int(scheme)
+
+    @classmethod
+    def empty(cls, n: int, scheme: int, device="cuda"):
+        return cls(torch.zeros(vec_padded_len(n, scheme), dtype=torch.float64, device=device), n, scheme)
+
+    @classmethod
+    def from_values(cls, ctx: Context, values: torch.Tensor, scheme: int, stream=None):
+        v = cls.empty(values.numel(), scheme, device=values.device if values.is_cuda else "cuda")
+        v.data[:values.numel()].copy_(values.reshape(-1))
+        v.encode(ctx, stream)
+        return v
+
+    @classmethod
+    def from_words(cls, words: torch.Tensor, n: int, scheme: int):
+        """Wrap already-encoded 64-bit words (e.g. copied from the oracle)."""
+        return cls(words.view(torch.float64), n, scheme)
+
+    def cstruct(self) -> Vec:
+        return Vec(self.n, self.data.data_ptr(), self.scheme)
+
+    def encode(self, ctx: Context, stream=None):
+        v = self.cstruct()
+        _check(_lib.abft_vec_encode(ctx.h, C.byref(v), _stream(stream)), "abft_vec_encode")
+
+    def decode(self, ctx: Context, counts: "Counters | None" = None, stream=None) -> torch.Tensor:
+        out = torch.empty(max(self.n, 1), dtype=torch.float64, device=self.data.device)
+        v = self.cstruct()
+        _check(_lib.abft_vec_decode(ctx.h, C.byref(v), out.data_ptr(), counts.ptr if counts else None,
+                                    _stream(stream)), "abft_vec_decode")
+        return out[:self.n]
+
+    def words(self) -> torch.Tensor:
+        return self.data.view(torch.int64)
+
+
+class Matrix:
+    """A protected CSR matrix (one chunk): val float64 [nnz], col int32 [nnz]
+    (ECC in its top bits after encode), rowptr int32 [padded]."""
+
+    def __init__(self, val: torch.Tensor, col: torch.Tensor, rowptr: torch.Tensor, nrows: int, ncols: int,
+                 elem_scheme: int, rowptr_scheme: int, row_base: int = 0, col_base: int = 0, stencil_n: int = 0):
+        dev = val.device
+        self.nrows, self.ncols = int(nrows), int(ncols)
+        self.nnz = int(rowptr[nrows].item()) if rowptr.numel() > nrows else int(col.numel())
+        self.es, self.rs = int(elem_scheme), int(rowptr_scheme)
+        self.row_base, self.col_base, self.stencil_n = int(row_base), int(col_base), int(stencil_n)
+        self.val = val.to(dtype=torch.float64).contiguous()
+        self.col = col.to(dtype=torch.int32).contiguous()
+        rp = torch.zeros(rowptr_padded_len(self.nrows, self.rs), dtype=torch.int32, device=dev)
+        rp[:self.nrows + 1] = rowptr[:self.nrows + 1].to(device=dev, dtype=torch.int32)
+        self.rowptr = rp
+
+    def cstruct(self) -> CSR:
+        return CSR(self.nrows, self.ncols, self.nnz, self.row_base, self.col_base, self.val.data_ptr(),
+                   self.col.data_ptr(), self.rowptr.data_ptr(), self.es, self.rs, self.stencil_n)
+
+    def encode(self, ctx: Context, stream=None) -> int:
+        m = self.cstruct()
+        return _lib.abft_csr_encode(ctx.h, C.byref(m), _stream(stream))
+
+
+def _chunks(A) -> tuple:
+    mats = A if isinstance(A, (list, tuple)) else [A]
+    arr = (CSR * len(mats))(*[m.cstruct() for m in mats])
+    return arr, len(mats)
+
+
+class Counters:
+    """Device abft_counts[3][5] (uint64 x4 each)."""
+
+    def __init__(self, device="cuda"):
+        self.t = torch.zeros(3 * 5 * 4, dtype=torch.int64, device=device)
+
+    @property
+    def ptr(self) -> int:
+        return self.t.data_ptr()
+
+    def reset(self, stream=None):
+        _check(_lib.abft_counts_reset(self.ptr, _stream(stream)), "abft_counts_reset")
+
+    def read(self, stream=None):
+        import numpy as np
+        host = (C.c_uint64 * 60)()
+        _check(_lib.abft_counts_read(self.ptr, C.cast(host, C.c_void_p), _stream(stream)), "abft_counts_read")
+        return np.array(list(host), dtype=np.uint64).reshape(3, 5, 4)
+
+
+def spmv(ctx: Context, A, x: Vector, y: Vector, counts: Counters | None = None, dot: torch.Tensor | None = None,
+         stream=None):
+    arr, n = _chunks(A)
+    vx, vy = x.cstruct(), y.cstruct()
+    _check(_lib.abft_spmv(ctx.h, arr, n, C.byref(vx), C.byref(vy), dot.data_ptr() if dot is not None else None,
+                          counts.ptr if counts else None, _stream(stream)), "abft_spmv")
+
+
+def cg_solve(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vector, tol=1e-10, max_iters=10000,
+             due_policy=0, counts: Counters | None = None, poll_every=16, stream=None) -> CGResult:
+    arr, n = _chunks(A)
+    opts = CGOpts(tol, max_iters, due_policy, poll_every)
+    res = CGResult()
+    vs = [v.cstruct() for v in (b, x, r, p, w)]
+    code = _lib.abft_cg_solve(ctx.h, arr, n, *[C.byref(v) for v in vs], C.byref(opts), C.byref(res),
+                              counts.ptr if counts else None, _stream(stream))
+    _check(code, "abft_cg_solve", allow=(E_DUE, E_NOT_CONVERGED))
+    return res
+
+
+def check_all(ctx: Context, A, vecs, counts: Counters | None = None, scrub=True, stream=None):
+    if A is not None:
+        arr, n = _chunks(A)
+    else:
+        arr, n = None, 0
+    varr = (Vec * max(len(vecs), 1))(*[v.cstruct() for v in vecs])
+    _check(_lib.abft_check_all(ctx.h, arr, n, varr, len(vecs), int(scrub), counts.ptr if counts else None,
+                               _stream(stream)), "abft_check_all")
+
+
+def inject_bitflip(ctx: Context, tensor: torch.Tensor, bit_offset: int, stream=None):
+    """XOR one stored bit of a device tensor (bit offset within its storage)."""
+    nbits = tensor.numel() * tensor.element_size() * 8
+    if not 0 <= bit_offset < nbits:
+        raise ValueError("bit offset out of range")
+    _check(_lib.abft_inject_bitflip(ctx.h, tensor.data_ptr(), int(bit_offset), _stream(stream)), "abft_inject_bitflip")
+
+
+def profile(ctx: Context, enable: bool):
+    _check(_lib.abft_profile(ctx.h, int(enable)), "abft_profile")
+
+
+def profile_read(ctx: Context):
+    ms = (C.c_double * 4)()
+    n = (C.c_int64 * 4)()
+    _check(_lib.abft_profile_read(ctx.h, C.cast(ms, C.c_void_p), C.cast(n, C.c_void_p)), "abft_profile_read")
+    return list(ms), list(n)
+
+
+# ------------------------------------------------------------------ multi-GPU
+class Dist:
+    """abft_dist: an NCCL communicator for the row-block strips (one per rank)."""
+
+    def __init__(self, rank: int, nranks: int, device: int, group=None):
+        import torch.distributed as dist
+        uid = torch.zeros(128, dtype=torch.uint8)
+        if rank == 0:
+            buf = (C.c_uint8 * 128)()
+            _check(_lib.abft_dist_get_unique_id(C.cast(buf, C.c_void_p)), "abft_dist_get_unique_id")
+            uid = torch.tensor(list(buf), dtype=torch.uint8)
+        if nranks > 1:
+            obj = [uid.tolist()]
+            dist.broadcast_object_list(obj, src=0, group=group)
+            uid = torch.tensor(obj[0], dtype=torch.uint8)
+        raw = (C.c_uint8 * 128)(*uid.tolist())
+        h = C.c_void_p()
+        _check(_lib.abft_dist_init(C.byref(h), C.cast(raw, C.c_void_p), rank, nranks, device), "abft_dist_init")
+        self.h, self.rank, self.nranks = h, rank, nranks
+
+    def close(self):
+        if self.h:
+            _lib.abft_dist_destroy(self.h)
+            self.h = None
+
+    def cg_solve(self, ctx: Context, A, n_halo: int, b, x, r, p, w, tol=1e-10, max_iters=10000, due_policy=0,
+                 counts: Counters | None = None, poll_every=16, stream=None) -> CGResult:
+        arr, n = _chunks(A)
+        opts = CGOpts(tol, max_iters, due_policy, poll_every)
+        res = CGResult()
+        vs = [v.cstruct() for v in (b, x, r, p, w)]
+        code = _lib.abft_cg_solve_dist(self.h, ctx.h, arr, n, int(n_halo), *[C.byref(v) for v in vs], C.byref(opts),
+                                       C.byref(res), counts.ptr if counts else None, _stream(stream))
+        _check(code, "abft_cg_solve_dist", allow=(E_DUE, E_NOT_CONVERGED))
+        return res

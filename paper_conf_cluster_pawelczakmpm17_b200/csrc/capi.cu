@@ -1,0 +1,548 @@
+// capi.cu — the C ABI of libabft.so (include/abft.h): argument validation,
+// scratch ownership, and the device-resident CG driver.
+// Host code only; every arithmetic step runs in kernels.cu.
+#include <cuda_runtime.h>
+
+#include <atomic>
+#include <cstdarg>
+#include <cmath>
+#include <cstdio>
+#include <cstring>
+#include <string>
+#include <vector>
+
+#include <nccl.h>
+
+#include "../../include/abft.h"
+#include "internal.h"
+
+using namespace abft;
+
+static thread_local std::string g_err;
+static std::atomic<uint64_t> g_launches{0};
+
+static int fail(int code, const char* fmt, ...) __attribute__((format(printf, 2, 3)));
+static int fail(int code, const char* fmt, ...) {
+  char buf[512];
+  va_list ap;
+  va_start(ap, fmt);
+  vsnprintf(buf, sizeof buf, fmt, ap);
+  va_end(ap);
+  g_err = buf;
+  return code;
+}
+#define CUDA_TRY(x)                                                                          \
+  do {                                                                                       \
+    cudaError_t e_ = (x);                                                                    \
+    if (e_ != cudaSuccess) return fail(ABFT_E_CUDA, "%s: %s", #x, cudaGetErrorString(e_)); \
+  } while (0)
+
+static inline void count_launch(int n) { g_launches.fetch_add((uint64_t)n, std::memory_order_relaxed); }
+
+struct abft_ctx {
+  int device = 0;
+  double* partials = nullptr;
+  int64_t partials_cap = 0;
+  double* roots = nullptr;
+  uint32_t* ticket = nullptr;
+  CgState* state = nullptr;
+  int* due = nullptr;
+  uint32_t* flags = nullptr;
+  CgState* h_state = nullptr;  // pinned
+  uint32_t* h_flags = nullptr; // pinned
+  bool profile = false;
+  double prof_ms[4] = {0, 0, 0, 0};
+  int64_t prof_n[4] = {0, 0, 0, 0};
+  std::vector<cudaEvent_t> events;
+};
+
+namespace {
+
+int ensure_partials(abft_ctx* c, int64_t nrb) {
+  if (nrb <= c->partials_cap) return ABFT_OK;
+  if (c->partials) cudaFree(c->partials);
+  c->partials = nullptr;
+  int64_t cap = nrb < 1024 ? 1024 : nrb;
+  CUDA_TRY(cudaMalloc(&c->partials, sizeof(double) * cap));
+  c->partials_cap = cap;
+  return ABFT_OK;
+}
+
+bool valid_scheme(int s) { return s >= 0 && s < ABFT_SCHEME_COUNT; }
+
+int check_vec(const abft_vec* v, const char* name) {
+  if (!v || !v->data || v->n < 0 || !valid_scheme(v->scheme)) return fail(ABFT_E_INVALID, "bad vector %s", name);
+  return ABFT_OK;
+}
+
+int check_chunks(const abft_csr* A, int nchunks) {
+  if (!A || nchunks <= 0) return fail(ABFT_E_INVALID, "no matrix chunks");
+  for (int c = 0; c < nchunks; c++) {
+    const abft_csr& M = A[c];
+    if (M.nrows < 0 || M.ncols < 0 || M.nnz < 0 || !M.rowptr || (M.nnz > 0 && (!M.val || !M.col)))
+      return fail(ABFT_E_INVALID, "chunk %d: bad sizes/pointers", c);
+    if (!valid_scheme(M.elem_scheme) || !valid_scheme(M.rowptr_scheme))
+      return fail(ABFT_E_INVALID, "chunk %d: bad scheme", c);
+    if (M.row_base < 0 || M.col_base < 0) return fail(ABFT_E_INVALID, "chunk %d: negative base", c);
+  }
+  return ABFT_OK;
+}
+
+// Launch the SpMV over all chunks; partials indexed by global RB (chunks must
+// start on 256-row boundaries relative to chunk 0 when dot is requested).
+int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, bool dot,
+                DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total) {
+  const int64_t base0 = A[0].row_base;
+  const int64_t npad_in = vec_padded_len(in->n, in->scheme);
+  const int64_t npad_out = vec_padded_len(out->n, out->scheme);
+  int64_t nrb_all = 0;
+  for (int c = 0; c < nchunks; c++) {
+    const abft_csr& M = A[c];
+    const int64_t rel = M.row_base - base0;
+    if (dot && (rel % 256) != 0) return fail(ABFT_E_INVALID, "chunk %d not aligned to 256 rows", c);
+    const int64_t end_rb = (rel + M.nrows + 255) / 256;
+    if (end_rb > nrb_all) nrb_all = end_rb;
+  }
+  if (dot) {
+    int e = ensure_partials(ctx, nrb_all);
+    if (e) return e;
+  }
+  for (int c = 0; c < nchunks; c++) {
+    const abft_csr& M = A[c];
+    if (M.row_base + M.nrows > out->n) return fail(ABFT_E_INVALID, "chunk %d rows exceed out", c);
+    if (M.col_base + M.ncols > npad_in) return fail(ABFT_E_INVALID, "chunk %d cols exceed in", c);
+    SpmvArgs a{};
+    a.nrows = M.nrows;
+    a.ncols = M.ncols;
+    a.nnz = M.nnz;
+    a.row_base = M.row_base;
+    a.col_base = M.col_base;
+    a.n_in = in->n;
+    a.npad_in = npad_in;
+    a.npad_out = (M.row_base + M.nrows == out->n) ? (npad_out - M.row_base) : M.nrows;
+    a.rb_offset = (M.row_base - base0) / 256;
+    a.val = reinterpret_cast<uint64_t*>(M.val);
+    a.col = M.col;
+    a.rowptr = M.rowptr;
+    a.in = reinterpret_cast<uint64_t*>(in->data);
+    a.out = reinterpret_cast<uint64_t*>(out->data);
+    a.partials = dot ? ctx->partials : nullptr;
+    a.counts = cnt;
+    a.due = ctx->due;
+    a.state = st;
+    count_launch(launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s));
+  }
+  if (nrb_total) *nrb_total = nrb_all;
+  return ABFT_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+const char* abft_last_error(void) { return g_err.c_str(); }
+uint64_t abft_launch_count(void) { return g_launches.load(); }
+
+int64_t abft_rowptr_padded_len(int64_t nrows, int32_t scheme) { return rowptr_padded_len(nrows, scheme); }
+int64_t abft_vec_padded_len(int64_t n, int32_t scheme) { return vec_padded_len(n, scheme); }
+
+int abft_ctx_create(int device, abft_ctx** out) {
+  if (!out) return fail(ABFT_E_INVALID, "null out");
+  CUDA_TRY(cudaSetDevice(device));
+  abft_ctx* c = new abft_ctx();
+  c->device = device;
+  CUDA_TRY(cudaMalloc(&c->roots, sizeof(double) * 1024));
+  CUDA_TRY(cudaMalloc(&c->ticket, sizeof(uint32_t) * 4));
+  CUDA_TRY(cudaMemset(c->ticket, 0, sizeof(uint32_t) * 4));
+  CUDA_TRY(cudaMalloc(&c->state, sizeof(CgState)));
+  CUDA_TRY(cudaMemset(c->state, 0, sizeof(CgState)));
+  CUDA_TRY(cudaMalloc(&c->due, sizeof(int) * 4));
+  CUDA_TRY(cudaMemset(c->due, 0, sizeof(int) * 4));
+  CUDA_TRY(cudaMalloc(&c->flags, sizeof(uint32_t) * 4));
+  CUDA_TRY(cudaMallocHost(&c->h_state, sizeof(CgState)));
+  CUDA_TRY(cudaMallocHost(&c->h_flags, sizeof(uint32_t) * 4));
+  int e = ensure_partials(c, 1024);
+  if (e) return e;
+  *out = c;
+  return ABFT_OK;
+}
+
+int abft_ctx_destroy(abft_ctx* c) {
+  if (!c) return ABFT_OK;
+  cudaSetDevice(c->device);
+  cudaFree(c->partials);
+  cudaFree(c->roots);
+  cudaFree(c->ticket);
+  cudaFree(c->state);
+  cudaFree(c->due);
+  cudaFree(c->flags);
+  cudaFreeHost(c->h_state);
+  cudaFreeHost(c->h_flags);
+  for (auto e : c->events) cudaEventDestroy(e);
+  delete c;
+  return ABFT_OK;
+}
+
+int abft_csr_encode(abft_ctx* ctx, abft_csr* A, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  int e = check_chunks(A, 1);
+  if (e) return e;
+  cudaStream_t s = (cudaStream_t)stream;
+  const uint64_t cap_col = A->elem_scheme == ABFT_NONE ? 0xFFFFFFFFull
+                           : A->elem_scheme == ABFT_SED ? 0x7FFFFFFFull : 0x00FFFFFFull;
+  const uint64_t cap_nnz = A->rowptr_scheme == ABFT_NONE ? 0xFFFFFFFFull
+                           : A->rowptr_scheme == ABFT_SED ? 0x7FFFFFFFull : 0x0FFFFFFFull;
+  if (A->ncols > 0 && (uint64_t)(A->ncols - 1) > cap_col)
+    return fail(ABFT_E_RANGE, "ncols %lld exceeds the element scheme's index capacity", (long long)A->ncols);
+  if ((uint64_t)A->nnz > cap_nnz) return fail(ABFT_E_RANGE, "nnz %lld exceeds the rowptr scheme's capacity", (long long)A->nnz);
+  CUDA_TRY(cudaMemsetAsync(ctx->flags, 0, sizeof(uint32_t), s));
+  count_launch(launch_csr_encode(A, ctx->flags, s));
+  CUDA_TRY(cudaGetLastError());
+  CUDA_TRY(cudaMemcpyAsync(ctx->h_flags, ctx->flags, sizeof(uint32_t), cudaMemcpyDeviceToHost, s));
+  CUDA_TRY(cudaStreamSynchronize(s));
+  uint32_t f = ctx->h_flags[0];
+  if (f & 4u) return fail(ABFT_E_SHAPE, "CRC32C element rows need >= 4 entries");
+  if (f & 3u) return fail(ABFT_E_RANGE, "column index or rowptr entry exceeds the scheme's capacity");
+  return ABFT_OK;
+}
+
+int abft_vec_encode(abft_ctx* ctx, abft_vec* v, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  int e = check_vec(v, "v");
+  if (e) return e;
+  count_launch(launch_vec_encode(reinterpret_cast<uint64_t*>(v->data), v->n, vec_padded_len(v->n, v->scheme),
+                                 v->scheme, (cudaStream_t)stream));
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_vec_decode(abft_ctx* ctx, abft_vec* v, double* out_masked, abft_counts* dcnt, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  int e = check_vec(v, "v");
+  if (e) return e;
+  count_launch(launch_vec_check(reinterpret_cast<uint64_t*>(v->data), v->n, vec_padded_len(v->n, v->scheme),
+                                v->scheme, out_masked, reinterpret_cast<DevCounts*>(dcnt), ctx->due, 1,
+                                (cudaStream_t)stream));
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, double* dot_out,
+              abft_counts* dcnt, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  int e = check_chunks(A, nchunks);
+  if (e) return e;
+  if ((e = check_vec(in, "in")) || (e = check_vec(out, "out"))) return e;
+  if (in->data == out->data) return fail(ABFT_E_INVALID, "in and out alias");
+  if (in->scheme != out->scheme) return fail(ABFT_E_INVALID, "in/out schemes differ");
+  cudaStream_t s = (cudaStream_t)stream;
+  int64_t nrb = 0;
+  e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb);
+  if (e) return e;
+  if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_profile(abft_ctx* ctx, int enable) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  ctx->profile = enable != 0;
+  for (int i = 0; i < 4; i++) { ctx->prof_ms[i] = 0; ctx->prof_n[i] = 0; }
+  return ABFT_OK;
+}
+int abft_profile_read(abft_ctx* ctx, double* ms, int64_t* n) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  for (int i = 0; i < 4; i++) { if (ms) ms[i] = ctx->prof_ms[i]; if (n) n[i] = ctx->prof_n[i]; }
+  return ABFT_OK;
+}
+
+// --------------------------------------------------------------------- CG
+namespace {
+
+struct Prof {
+  abft_ctx* ctx;
+  cudaStream_t s;
+  std::vector<std::pair<int, int>> marks;  // (class, event index of start)
+  size_t next = 0;
+  cudaEvent_t ev(size_t i) {
+    while (ctx->events.size() <= i) {
+      cudaEvent_t e;
+      cudaEventCreate(&e);
+      ctx->events.push_back(e);
+    }
+    return ctx->events[i];
+  }
+  void begin(int cls) {
+    if (!ctx->profile) return;
+    cudaEventRecord(ev(next), s);
+    marks.push_back({cls, (int)next});
+    next += 2;
+  }
+  void end() {
+    if (!ctx->profile) return;
+    cudaEventRecord(ev(marks.back().second + 1), s);
+  }
+  void harvest() {  // after a stream sync
+    if (!ctx->profile) return;
+    for (auto& m : marks) {
+      float ms = 0;
+      if (cudaEventElapsedTime(&ms, ctx->events[m.second], ctx->events[m.second + 1]) == cudaSuccess) {
+        ctx->prof_ms[m.first] += ms;
+        ctx->prof_n[m.first] += 1;
+      }
+    }
+    marks.clear();
+    next = 0;
+  }
+};
+
+}  // namespace
+
+}  // extern "C"
+
+struct abft_dist {
+  ncclComm_t comm = nullptr;
+  int rank = 0, nranks = 1, device = 0;
+  double* sendbuf = nullptr;   // [2]
+  double* gathered = nullptr;  // [2 * nranks]
+};
+
+namespace {
+
+#define NCCL_TRY(x)                                                                        \
+  do {                                                                                     \
+    ncclResult_t r_ = (x);                                                                 \
+    if (r_ != ncclSuccess) return fail(ABFT_E_NCCL, "%s: %s", #x, ncclGetErrorString(r_)); \
+  } while (0)
+
+// Exchange the ghost rows of an extended vector (n_halo entries each side).
+int halo_exchange(abft_dist* d, uint64_t* ext, int64_t n_loc, int64_t n_halo, cudaStream_t s) {
+  if (!d || d->nranks == 1 || n_halo == 0) return ABFT_OK;
+  const size_t bytes = sizeof(uint64_t) * (size_t)n_halo;
+  NCCL_TRY(ncclGroupStart());
+  if (d->rank > 0) {
+    NCCL_TRY(ncclSend(ext + n_halo, bytes, ncclChar, d->rank - 1, d->comm, s));
+    NCCL_TRY(ncclRecv(ext, bytes, ncclChar, d->rank - 1, d->comm, s));
+  }
+  if (d->rank < d->nranks - 1) {
+    NCCL_TRY(ncclSend(ext + n_loc, bytes, ncclChar, d->rank + 1, d->comm, s));
+    NCCL_TRY(ncclRecv(ext + n_halo + n_loc, bytes, ncclChar, d->rank + 1, d->comm, s));
+  }
+  NCCL_TRY(ncclGroupEnd());
+  return ABFT_OK;
+}
+
+// Dot-product finish: single GPU -> reduce with op; multi-GPU -> subtree root +
+// DUE flag, all-gather, identical top-of-tree combine on every rank.
+int finish_dot(abft_ctx* ctx, abft_dist* d, int64_t nrb, int op, cudaStream_t s) {
+  if (!d || d->nranks == 1) {
+    count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, op, ctx->state, nullptr, ctx->due, s));
+    return ABFT_OK;
+  }
+  count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 4, nullptr, d->sendbuf, ctx->due, s));
+  NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
+  count_launch(launch_combine(d->gathered, d->nranks, op, ctx->state, ctx->due, s));
+  return ABFT_OK;
+}
+
+int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b, abft_vec* x,
+            abft_vec* r, abft_vec* p, abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt,
+            cudaStream_t s) {
+  if (!ctx || !opts || !res) return fail(ABFT_E_INVALID, "null ctx/opts/res");
+  int e = check_chunks(A, nchunks);
+  if (e) return e;
+  abft_vec* vs[5] = {b, x, r, p, w};
+  const char* names[5] = {"b", "x", "r", "p", "w"};
+  for (int i = 0; i < 5; i++) if ((e = check_vec(vs[i], names[i]))) return e;
+  const int scheme = x->scheme;
+  const int64_t n_ext = x->n;
+  for (int i = 0; i < 5; i++) {
+    if (vs[i]->scheme != scheme || vs[i]->n != n_ext) return fail(ABFT_E_INVALID, "vector %s: scheme/length differ", names[i]);
+    for (int j = 0; j < i; j++) if (vs[i]->data == vs[j]->data) return fail(ABFT_E_INVALID, "vectors alias");
+  }
+  const int64_t n = n_ext - 2 * n_halo;  // local rows
+  const int G = (int)vec_padded_len(1, scheme);
+  if (n <= 0 || n_halo < 0 || (n_halo % G) != 0) return fail(ABFT_E_SHAPE, "bad halo / local size");
+  if (n_halo > 0 && (n % G) != 0) return fail(ABFT_E_SHAPE, "local rows must be a multiple of the vector group");
+  int64_t rows = 0;
+  for (int c = 0; c < nchunks; c++) rows += A[c].nrows;
+  if (A[0].row_base != n_halo || rows != n) return fail(ABFT_E_SHAPE, "chunks must cover the local rows");
+
+  DevCounts* cnt = reinterpret_cast<DevCounts*>(dcnt);
+  const int64_t npad = vec_padded_len(n, scheme);
+  const int64_t nrb = (n + 255) / 256;
+  if ((e = ensure_partials(ctx, nrb))) return e;
+  if (nrb > (int64_t)1024 * 1024) return fail(ABFT_E_SHAPE, "more than 2^28 rows per GPU");
+  const bool multi = d && d->nranks > 1;
+
+  CgState h{};
+  h.tol = opts->tol;
+  h.max_iters = opts->max_iters;
+  h.abort_policy = opts->due_policy == 0 ? 1 : 0;
+  h.dist = multi ? 1 : 0;
+  *ctx->h_state = h;
+  CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
+  CUDA_TRY(cudaMemsetAsync(ctx->due, 0, sizeof(int), s));
+
+  VecArgs va{};
+  va.n = n;
+  va.npad = npad;
+  va.x = reinterpret_cast<uint64_t*>(x->data) + n_halo;
+  va.p = reinterpret_cast<uint64_t*>(p->data) + n_halo;
+  va.r = reinterpret_cast<uint64_t*>(r->data) + n_halo;
+  va.w = reinterpret_cast<uint64_t*>(w->data) + n_halo;
+  va.b = reinterpret_cast<uint64_t*>(b->data) + n_halo;
+  va.partials = ctx->partials;
+  va.counts = cnt;
+  va.due = ctx->due;
+  va.state = ctx->state;
+
+  Prof prof{ctx, s};
+  // init (a2): w = A x0 ; r = b - w ; p = r ; rr0
+  if ((e = halo_exchange(d, reinterpret_cast<uint64_t*>(x->data), n, n_halo, s))) return e;
+  prof.begin(0);
+  e = spmv_chunks(ctx, A, nchunks, x, w, false, cnt, nullptr, s, nullptr);
+  prof.end();
+  if (e) return e;
+  count_launch(launch_init_r(va, scheme, s));
+  if ((e = finish_dot(ctx, d, nrb, 1, s))) return e;
+  CUDA_TRY(cudaGetLastError());
+
+  const int poll = opts->poll_every > 0 ? opts->poll_every : 16;
+  int64_t launched = 0;
+  for (;;) {
+    CUDA_TRY(cudaMemcpyAsync(ctx->h_state, ctx->state, sizeof(CgState), cudaMemcpyDeviceToHost, s));
+    CUDA_TRY(cudaStreamSynchronize(s));
+    prof.harvest();
+    if (ctx->h_state->stop || launched >= opts->max_iters) break;
+    int64_t k = opts->max_iters - launched;
+    if (k > poll) k = poll;
+    for (int64_t it = 0; it < k; it++) {
+      if ((e = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e;
+      prof.begin(0);
+      e = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr);
+      prof.end();
+      if (e) return e;
+      prof.begin(3);
+      if ((e = finish_dot(ctx, d, nrb, 2, s))) return e;
+      prof.end();
+      prof.begin(1);
+      count_launch(launch_calc_ur(va, scheme, s));
+      prof.end();
+      prof.begin(3);
+      if ((e = finish_dot(ctx, d, nrb, 3, s))) return e;
+      prof.end();
+      prof.begin(2);
+      count_launch(launch_calc_p(va, scheme, s));
+      prof.end();
+      if (multi && h.abort_policy) {
+        count_launch(launch_pack_due(d->sendbuf, ctx->due, s));
+        NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
+        count_launch(launch_due_combine(d->gathered, d->nranks, ctx->state, ctx->due, s));
+      }
+    }
+    CUDA_TRY(cudaGetLastError());
+    launched += k;
+  }
+  const CgState& hs = *ctx->h_state;
+  res->iters = hs.iters;
+  res->rr0 = hs.rr0;
+  res->rrn = hs.rrn;
+  res->status = hs.stop ? hs.status : (opts->max_iters > 0 ? ABFT_E_NOT_CONVERGED : ABFT_OK);
+  if (res->status != ABFT_OK) fail(res->status, "CG finished with status %d after %d iterations", res->status, res->iters);
+  return res->status;
+}
+
+}  // namespace
+
+extern "C" {
+
+int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                  abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream) {
+  return cg_core(ctx, nullptr, A, nchunks, 0, b, x, r, p, w, opts, res, dcnt, (cudaStream_t)stream);
+}
+
+int abft_dist_get_unique_id(void* out128) {
+  if (!out128) return fail(ABFT_E_INVALID, "null out");
+  ncclUniqueId id;
+  NCCL_TRY(ncclGetUniqueId(&id));
+  memcpy(out128, &id, sizeof(id));
+  return ABFT_OK;
+}
+
+int abft_dist_init(abft_dist** out, const void* uid, int rank, int nranks, int device) {
+  if (!out || !uid || nranks < 1 || rank < 0 || rank >= nranks) return fail(ABFT_E_INVALID, "bad dist args");
+  CUDA_TRY(cudaSetDevice(device));
+  abft_dist* d = new abft_dist();
+  d->rank = rank;
+  d->nranks = nranks;
+  d->device = device;
+  ncclUniqueId id;
+  memcpy(&id, uid, sizeof(id));
+  if (nranks > 1) NCCL_TRY(ncclCommInitRank(&d->comm, nranks, id, rank));
+  CUDA_TRY(cudaMalloc(&d->sendbuf, sizeof(double) * 2));
+  CUDA_TRY(cudaMalloc(&d->gathered, sizeof(double) * 2 * nranks));
+  *out = d;
+  return ABFT_OK;
+}
+
+int abft_dist_destroy(abft_dist* d) {
+  if (!d) return ABFT_OK;
+  if (d->comm) ncclCommDestroy(d->comm);
+  cudaFree(d->sendbuf);
+  cudaFree(d->gathered);
+  delete d;
+  return ABFT_OK;
+}
+
+int abft_cg_solve_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b,
+                       abft_vec* x, abft_vec* r, abft_vec* p, abft_vec* w, const abft_cg_opts* opts,
+                       abft_cg_result* res, abft_counts* dcnt, void* stream) {
+  if (!d) return fail(ABFT_E_INVALID, "null dist");
+  return cg_core(ctx, d, A, nchunks, n_halo, b, x, r, p, w, opts, res, dcnt, (cudaStream_t)stream);
+}
+
+int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs, int nvec, int scrub,
+                   abft_counts* dcnt, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  cudaStream_t s = (cudaStream_t)stream;
+  DevCounts* cnt = reinterpret_cast<DevCounts*>(dcnt);
+  if (A && nchunks > 0) {
+    int e = check_chunks(A, nchunks);
+    if (e) return e;
+    for (int c = 0; c < nchunks; c++) count_launch(launch_check_csr(&A[c], cnt, ctx->due, scrub, s));
+  }
+  for (int i = 0; i < nvec; i++) {
+    int e = check_vec(&vecs[i], "vecs[i]");
+    if (e) return e;
+    count_launch(launch_vec_check(reinterpret_cast<uint64_t*>(vecs[i].data), vecs[i].n,
+                                  vec_padded_len(vecs[i].n, vecs[i].scheme), vecs[i].scheme, nullptr, cnt, ctx->due,
+                                  scrub, s));
+  }
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_inject_bitflip(abft_ctx* ctx, void* dev_base, uint64_t bit_offset, void* stream) {
+  if (!ctx || !dev_base) return fail(ABFT_E_INVALID, "null ctx/base");
+  count_launch(launch_inject(dev_base, bit_offset, (cudaStream_t)stream));
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_counts_read(const abft_counts* dcnt, abft_counts* host_out, void* stream) {
+  if (!dcnt || !host_out) return fail(ABFT_E_INVALID, "null counts");
+  cudaStream_t s = (cudaStream_t)stream;
+  CUDA_TRY(cudaMemcpyAsync(host_out, dcnt, sizeof(abft_counts) * ABFT_T_COUNT * ABFT_SCHEME_COUNT,
+                           cudaMemcpyDeviceToHost, s));
+  CUDA_TRY(cudaStreamSynchronize(s));
+  return ABFT_OK;
+}
+
+int abft_counts_reset(abft_counts* dcnt, void* stream) {
+  if (!dcnt) return fail(ABFT_E_INVALID, "null counts");
+  CUDA_TRY(cudaMemsetAsync(dcnt, 0, sizeof(abft_counts) * ABFT_T_COUNT * ABFT_SCHEME_COUNT, (cudaStream_t)stream));
+  return ABFT_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,68 @@
+// internal.h — host-side interface between the C ABI (capi.cu, dist.cu) and the
+// kernel translation unit (kernels.cu).  No torch types anywhere.
+#pragma once
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "../../include/abft.h"
+
+namespace abft {
+
+// Device CG scalars.  Written only by single threads of the
+// reduction kernels' last blocks and by calc_p's last block.
+struct CgState {
+  double rr0, rro, rrn, pw, alpha, beta, tol;
+  int32_t iters, max_iters, stop, status, abort_policy, converged;
+  uint32_t ticket_p;   // calc_p last-block ticket
+  int32_t dist;        // 1 = multi-GPU solve (abort decided after an all-gather)
+};
+
+struct DevCounts { unsigned long long v[3][5][4]; };
+
+// arguments of one SpMV chunk launch
+struct SpmvArgs {
+  int64_t nrows, ncols, nnz, row_base, col_base, n_in, npad_in, npad_out, rb_offset;
+  uint64_t* val;
+  uint32_t* col;
+  uint32_t* rowptr;
+  uint64_t* in;
+  uint64_t* out;
+  double* partials;  // indexed rb_offset + local RB (may be null)
+  DevCounts* counts; // may be null
+  int* due;          // DUE / range flag (never null)
+  const CgState* state;  // may be null
+};
+
+struct VecArgs {
+  int64_t n, npad;
+  uint64_t* x; uint64_t* p; uint64_t* r; uint64_t* w; uint64_t* b;
+  double* partials;
+  DevCounts* counts;
+  int* due;
+  CgState* state;
+  double* out_masked;
+};
+
+// launchers (kernels.cu); each returns the number of kernels launched
+int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, bool dot, cudaStream_t s);
+int launch_calc_ur(const VecArgs& a, int vs, cudaStream_t s);
+int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s);
+int launch_init_r(const VecArgs& a, int vs, cudaStream_t s);
+int launch_vec_encode(uint64_t* data, int64_t n, int64_t npad, int vs, cudaStream_t s);
+int launch_vec_check(uint64_t* data, int64_t n, int64_t npad, int vs, double* out_masked, DevCounts* c, int* due,
+                     int scrub, cudaStream_t s);
+// op: 0 plain dot -> *out, 1 rr0 (init), 2 pw (alpha), 3 rrn (convergence, beta),
+//     4 subtree root + DUE flag -> out[0..2) (multi-GPU all-gather payload)
+int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* ticket, int op, CgState* st,
+                  double* out, const int* due, cudaStream_t s);
+int launch_combine(const double* gathered, int P, int op, CgState* st, int* due, cudaStream_t s);
+int launch_due_combine(const double* gathered, int P, CgState* st, int* due, cudaStream_t s);
+int launch_pack_due(double* out, const int* due, cudaStream_t s);
+int launch_csr_encode(abft_csr* A, uint32_t* flags, cudaStream_t s);
+int launch_check_csr(const abft_csr* A, DevCounts* c, int* due, int scrub, cudaStream_t s);
+int launch_inject(void* base, uint64_t bit, cudaStream_t s);
+
+int64_t rowptr_padded_len(int64_t nrows, int scheme);
+int64_t vec_padded_len(int64_t n, int scheme);
+
+}  // namespace abft

@@ -1,0 +1,300 @@
+"""GPU parity: libabft.so (through the C ABI) vs the CPU oracle, element by
+element on the same seeded inputs.
+
+Bar: bit-exact for every encoded word, syndrome outcome, correction and count;
+floating point (SpMV outputs, dots, CG iterates) is also required bit-exact —
+stricter than north_star's 1e-12 per element — because both sides follow the
+same fma chain and RED-1 order (readings R14)."""
+import math
+
+import numpy as np
+import pytest
+import torch
+
+import gen
+import oracle as orc
+from tests.gpu_helpers import (col_words, gpu_matrix, gpu_vec_from_words, oracle_matrix, rowptr_words, tea,
+                               val_words, words_of)
+
+pytestmark = pytest.mark.gpu
+
+SCHEMES = ["NONE", "SED", "SECDED64", "SECDED128", "CRC32C"]
+
+
+@pytest.fixture(scope="module")
+def abft():
+    from paper_conf_cluster_pawelczakmpm17_b200 import build
+    build.build()
+    from paper_conf_cluster_pawelczakmpm17_b200 import abft as A
+    return A
+
+
+@pytest.fixture(scope="module")
+def ctx(abft):
+    return abft.Context(0)
+
+
+def _special_values(n, seed):
+    v = gen.uniform_pm1(n, seed) * 10.0 ** np.round(gen.uniform_pm1(n, seed + 1) * 30)
+    sp = [0.0, -0.0, 1.0, -1.0, math.pi, -0.1, 1e300, -1e-300, 5e-324, float("inf"), float("-inf"),
+          1.7976931348623157e308, 2.2250738585072014e-308]
+    v[:len(sp)] = sp
+    return v
+
+
+@pytest.mark.parametrize("scheme", SCHEMES)
+@pytest.mark.parametrize("n", [1, 257, 1003])
+def test_vec_encode_parity(abft, ctx, scheme, n):
+    s = getattr(orc, scheme)
+    vals = _special_values(n, 5 + n)
+    ref = orc.vec_encode(vals, s)
+    g = abft.Vector.from_values(ctx, torch.from_numpy(vals).cuda(), s)
+    torch.cuda.synchronize()
+    assert np.array_equal(words_of(g)[:len(ref)], ref)
+    # decode: masked values + zero counts
+    cnt = abft.Counters()
+    out = g.decode(ctx, cnt).cpu().numpy()
+    ref_m = orc.vec_masked(ref, n, s)
+    assert np.array_equal(out.view(np.uint64), ref_m.view(np.uint64))
+    assert cnt.read().sum() == 0
+
+
+@pytest.mark.parametrize("es", ["NONE", "SED", "SECDED64", "CRC32C"])
+@pytest.mark.parametrize("rs", SCHEMES)
+def test_csr_encode_parity(abft, ctx, es, rs):
+    n = 40
+    v, c, r = tea(n)
+    N = n * n
+    Ao, so = oracle_matrix(v, c, r, N, N, getattr(orc, es), getattr(orc, rs))
+    Ag, sg = gpu_matrix(abft, ctx, v, c, r, N, N, getattr(abft, es), getattr(abft, rs))
+    assert so == sg == 0
+    assert np.array_equal(col_words(Ag), Ao.col)
+    assert np.array_equal(rowptr_words(Ag), Ao.rowptr)
+    assert np.array_equal(val_words(Ag), Ao.val)
+
+
+def test_csr_encode_capacity_errors(abft, ctx):
+    v = np.ones(1)
+    r = np.array([0, 1], dtype=np.uint32)
+    _, st = gpu_matrix(abft, ctx, v, np.array([2**24], dtype=np.uint32), r, 1, 2**24 + 1, abft.SECDED64, abft.SECDED64)
+    assert st == abft.E_RANGE
+    _, st = gpu_matrix(abft, ctx, v, np.array([2**24 - 1], dtype=np.uint32), r, 1, 2**24, abft.SECDED64,
+                       abft.SECDED64)
+    assert st == abft.OK
+    _, st = gpu_matrix(abft, ctx, np.ones(3), np.array([0, 1, 2], dtype=np.uint32), np.array([0, 3], dtype=np.uint32),
+                       1, 3, abft.CRC32C, abft.NONE)
+    assert st == abft.E_SHAPE
+
+
+def _spmv_both(abft, ctx, n, es, rs, vs, seed=3, flips=None, kind="tea"):
+    v, c, r = tea(n, kind)
+    N = n * n
+    Ao, _ = oracle_matrix(v, c, r, N, N, es, rs)
+    Ag, _ = gpu_matrix(abft, ctx, v, c, r, N, N, es, rs)
+    x = gen.uniform_pm1(N, seed)
+    xo = orc.vec_encode(x, vs)
+    xg = gpu_vec_from_words(abft, xo, N, vs)
+    if flips:
+        flips(Ao, xo, Ag, xg)
+    out_o = np.zeros(orc.vec_padded_len(N, vs), dtype=np.uint64)
+    cnt_o = orc.new_counts()
+    d, dot_o = orc.spmv(Ao, xo, N, vs, out_o, N, cnt_o, want_dot=True)
+    yg = abft.Vector.empty(N, vs)
+    cnt_g = abft.Counters()
+    dot_g = torch.zeros(1, dtype=torch.float64, device="cuda")
+    abft.spmv(ctx, Ag, xg, yg, cnt_g, dot=dot_g)
+    torch.cuda.synchronize()
+    return dict(Ao=Ao, Ag=Ag, xo=xo, xg=xg, out_o=out_o, out_g=words_of(yg), cnt_o=cnt_o, cnt_g=cnt_g.read(),
+                dot_o=dot_o, dot_g=dot_g.item())
+
+
+@pytest.mark.parametrize("vs", SCHEMES)
+@pytest.mark.parametrize("es,rs", [("NONE", "NONE"), ("SECDED64", "SECDED64"), ("SED", "SED"),
+                                   ("SECDED64", "SECDED128"), ("CRC32C", "CRC32C"), ("SECDED64", "SED")])
+@pytest.mark.parametrize("n", [40, 64])
+def test_spmv_parity(abft, ctx, n, es, rs, vs):
+    R = _spmv_both(abft, ctx, n, getattr(orc, es), getattr(orc, rs), getattr(orc, vs))
+    assert np.array_equal(R["out_g"][:len(R["out_o"])], R["out_o"])
+    assert R["dot_g"] == R["dot_o"]
+    assert R["cnt_o"].sum() == 0 and R["cnt_g"].sum() == 0
+
+
+def _flip_u64(a, idx, bit):
+    a[idx] ^= np.uint64(1 << bit)
+
+
+def _inject_both(abft, ctx, Ao, xo, Ag, xg, rng, n_el=12, n_rp=6, n_x=9, double=False):
+    """Single (or same-word double) flips at identical storage positions on both sides."""
+    nnz = Ao.nnz
+    ops = []
+    for e in rng.choice(nnz, n_el, replace=False):
+        bits = rng.choice(96, 2 if double else 1, replace=False)
+        for b in bits:
+            ops.append(("el", int(e), int(b)))
+    G = len(Ao.rowptr)
+    for g in rng.choice(G, n_rp, replace=False):
+        for b in rng.choice(32, 2 if double else 1, replace=False):
+            ops.append(("rp", int(g), int(b)))
+    for i in rng.choice(len(xo), n_x, replace=False):
+        for b in rng.choice(64, 2 if double else 1, replace=False):
+            ops.append(("x", int(i), int(b)))
+    for kind, i, b in ops:
+        if kind == "el":
+            if b < 64:
+                Ao.val[i] ^= np.uint64(1 << b)
+                abft.inject_bitflip(ctx, Ag.val, 64 * i + b)
+            else:
+                Ao.col[i] ^= np.uint32(1 << (b - 64))
+                abft.inject_bitflip(ctx, Ag.col, 32 * i + (b - 64))
+        elif kind == "rp":
+            Ao.rowptr[i] ^= np.uint32(1 << b)
+            abft.inject_bitflip(ctx, Ag.rowptr, 32 * i + b)
+        else:
+            xo[i] ^= np.uint64(1 << b)
+            abft.inject_bitflip(ctx, xg.data, 64 * i + b)
+    return ops
+
+
+@pytest.mark.parametrize("es,rs,vs", [("SECDED64", "SECDED64", "SECDED64"), ("SED", "SED", "SED"),
+                                      ("SECDED64", "SECDED128", "SECDED128"), ("CRC32C", "CRC32C", "CRC32C")])
+@pytest.mark.parametrize("double", [False, True])
+def test_spmv_fault_parity(abft, ctx, es, rs, vs, double):
+    rng = np.random.default_rng(17 + double)
+
+    def flips(Ao, xo, Ag, xg):
+        _inject_both(abft, ctx, Ao, xo, Ag, xg, rng, double=double)
+
+    R = _spmv_both(abft, ctx, 48, getattr(orc, es), getattr(orc, rs), getattr(orc, vs), flips=flips)
+    assert np.array_equal(R["cnt_g"], R["cnt_o"]), (R["cnt_g"][R["cnt_g"] != R["cnt_o"]], R["cnt_o"])
+    assert np.array_equal(R["out_g"][:len(R["out_o"])], R["out_o"])
+    assert R["dot_g"] == R["dot_o"] or (math.isnan(R["dot_g"]) and math.isnan(R["dot_o"]))
+    # scrubbed storage identical
+    assert np.array_equal(val_words(R["Ag"]), R["Ao"].val)
+    assert np.array_equal(col_words(R["Ag"]), R["Ao"].col)
+    assert np.array_equal(rowptr_words(R["Ag"]), R["Ao"].rowptr)
+    assert np.array_equal(words_of(R["xg"])[:len(R["xo"])], R["xo"])
+    if not double and es.startswith("SECDED") and vs.startswith("SECDED"):
+        cg = R["cnt_g"]
+        assert cg[:, :, 2].sum() == 0                      # singles never DUE under SECDED
+        assert cg[:, :, 1].sum() == cg[:, :, 0].sum() > 0  # every detection corrected
+
+
+def _cg_both(abft, ctx, n, es, rs, vs, policy=1, inject=None, max_iters=5000, tol=1e-10):
+    v, c, r = tea(n)
+    N = n * n
+    Ao, _ = oracle_matrix(v, c, r, N, N, es, rs)
+    Ag, _ = gpu_matrix(abft, ctx, v, c, r, N, N, es, rs)
+    b = gen.tealeaf_rhs(n).numpy()
+    bo = orc.vec_encode(b, vs)
+    xo = bo.copy()
+    bg = gpu_vec_from_words(abft, bo, N, vs)
+    xg = gpu_vec_from_words(abft, xo, N, vs)
+    if inject:
+        inject(Ao, bo, xo, Ag, bg, xg)
+    ro, po, wo = (np.zeros_like(bo) for _ in range(3))
+    cnt_o = orc.new_counts()
+    st_o, res_o = orc.cg_solve(Ao, bo, xo, ro, po, wo, vs, tol, max_iters, policy, cnt_o)
+    rg, pg, wg = (abft.Vector.empty(N, vs) for _ in range(3))
+    cnt_g = abft.Counters()
+    res_g = abft.cg_solve(ctx, Ag, bg, xg, rg, pg, wg, tol=tol, max_iters=max_iters, due_policy=policy, counts=cnt_g,
+                          poll_every=7)
+    return dict(st_o=st_o, res_o=res_o, res_g=res_g, xo=xo, xg=words_of(xg), cnt_o=cnt_o, cnt_g=cnt_g.read(),
+                ro=ro, rg=words_of(rg), po=po, pg=words_of(pg))
+
+
+@pytest.mark.parametrize("vs", SCHEMES)
+@pytest.mark.parametrize("n", [32, 48])
+def test_cg_parity(abft, ctx, n, vs):
+    s = getattr(orc, vs)
+    es = orc.SECDED64 if s != orc.CRC32C else orc.CRC32C
+    rs = s if s != orc.NONE else orc.NONE
+    es = orc.NONE if s == orc.NONE else es
+    R = _cg_both(abft, ctx, n, es, rs, s)
+    assert R["st_o"] == orc.OK and R["res_g"].status == 0
+    assert R["res_g"].iters == R["res_o"].iters
+    assert R["res_g"].rr0 == R["res_o"].rr0 and R["res_g"].rrn == R["res_o"].rrn
+    assert np.array_equal(R["xg"][:len(R["xo"])], R["xo"])
+    assert np.array_equal(R["rg"][:len(R["ro"])], R["ro"])
+    assert np.array_equal(R["pg"][:len(R["po"])], R["po"])
+
+
+def test_cg_max_iters_and_abort(abft, ctx):
+    R = _cg_both(abft, ctx, 32, orc.SECDED64, orc.SECDED64, orc.SECDED64, max_iters=5)
+    assert R["st_o"] == orc.E_NOT_CONVERGED and R["res_g"].status == orc.E_NOT_CONVERGED
+    assert R["res_g"].iters == R["res_o"].iters == 5
+    assert np.array_equal(R["xg"][:len(R["xo"])], R["xo"])
+
+    def dbl(Ao, bo, xo, Ag, bg, xg):  # a double flip in one element -> DUE at init
+        Ao.val[100] ^= np.uint64(0b101)
+        abft.inject_bitflip(ctx, Ag.val, 64 * 100)
+        abft.inject_bitflip(ctx, Ag.val, 64 * 100 + 2)
+
+    R = _cg_both(abft, ctx, 32, orc.SECDED64, orc.SECDED64, orc.SECDED64, policy=0, inject=dbl)
+    assert R["st_o"] == orc.E_DUE and R["res_g"].status == orc.E_DUE
+    assert R["res_g"].iters == R["res_o"].iters
+    assert np.array_equal(R["cnt_g"], R["cnt_o"])
+
+
+def test_config1_fault_campaign_32(abft, ctx):
+    """Config 1: 32^2, E-SECDED on elements, SED on vectors (R-SED rowptr),
+    100 single flips over val/col/rowptr/b/x0 before init, policy continue;
+    counts, iterations and x bit-exact vs the oracle."""
+    for seed in range(1, 4):
+        rng = np.random.default_rng(seed)
+
+        def inj(Ao, bo, xo, Ag, bg, xg):
+            N = len(bo)
+            targets = rng.choice(5, 100)
+            used = set()
+            for t in targets:
+                while True:
+                    if t == 0:
+                        i, b = int(rng.integers(Ao.nnz)), int(rng.integers(64)); key = ("el", i)
+                    elif t == 1:
+                        i, b = int(rng.integers(Ao.nnz)), int(rng.integers(32)); key = ("el", i)
+                    elif t == 2:
+                        i, b = int(rng.integers(len(Ao.rowptr))), int(rng.integers(32)); key = ("rp", i)
+                    elif t == 3:
+                        i, b = int(rng.integers(N)), int(rng.integers(64)); key = ("b", i)
+                    else:
+                        i, b = int(rng.integers(N)), int(rng.integers(64)); key = ("x", i)
+                    if key not in used:
+                        used.add(key)
+                        break
+                if t == 0:
+                    Ao.val[i] ^= np.uint64(1 << b); abft.inject_bitflip(ctx, Ag.val, 64 * i + b)
+                elif t == 1:
+                    Ao.col[i] ^= np.uint32(1 << b); abft.inject_bitflip(ctx, Ag.col, 32 * i + b)
+                elif t == 2:
+                    Ao.rowptr[i] ^= np.uint32(1 << b); abft.inject_bitflip(ctx, Ag.rowptr, 32 * i + b)
+                elif t == 3:
+                    bo[i] ^= np.uint64(1 << b); abft.inject_bitflip(ctx, bg.data, 64 * i + b)
+                else:
+                    xo[i] ^= np.uint64(1 << b); abft.inject_bitflip(ctx, xg.data, 64 * i + b)
+
+        R = _cg_both(abft, ctx, 32, orc.SECDED64, orc.SED, orc.SED, policy=1, inject=inj)
+        assert np.array_equal(R["cnt_g"], R["cnt_o"]), (R["cnt_g"], R["cnt_o"])
+        assert R["res_g"].iters == R["res_o"].iters
+        assert np.array_equal(R["xg"][:len(R["xo"])], R["xo"])
+        # every element flip was corrected (E-SECDED), every vector/rowptr flip detected (SED)
+        assert R["cnt_g"][orc.ELEM, orc.SECDED64, orc.UNC] == 0
+
+
+def test_check_all_parity(abft, ctx):
+    n = 40
+    v, c, r = tea(n)
+    N = n * n
+    Ao, _ = oracle_matrix(v, c, r, N, N, orc.SECDED64, orc.SECDED64)
+    Ag, _ = gpu_matrix(abft, ctx, v, c, r, N, N, orc.SECDED64, orc.SECDED64)
+    x = gen.uniform_pm1(N, 9)
+    xo = orc.vec_encode(x, orc.SECDED64)
+    xg = gpu_vec_from_words(abft, xo, N, orc.SECDED64)
+    rng = np.random.default_rng(99)
+    _inject_both(abft, ctx, Ao, xo, Ag, xg, rng, n_el=20, n_rp=8, n_x=10)
+    cnt_o = orc.new_counts()
+    Ao.check(cnt_o)
+    orc.vec_check(xo, N, orc.SECDED64, cnt_o)
+    cnt_g = abft.Counters()
+    abft.check_all(ctx, Ag, [xg], cnt_g)
+    assert np.array_equal(cnt_g.read(), cnt_o)
+    assert np.array_equal(col_words(Ag), Ao.col) and np.array_equal(val_words(Ag), Ao.val)

@@ -1,0 +1,77 @@
+"""CPU-side checks of the CUDA library (no GPU needed):
+
+* libabft.so loads and exports every function include/abft.h declares;
+* the exact __host__ __device__ codec functions the kernels use agree with the
+  oracle bit for bit (encode) and outcome for outcome (check) on every single-
+  and double-bit flip of random codewords of every SECDED instance.
+"""
+import itertools
+import os
+import re
+
+import numpy as np
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.fixture(scope="module")
+def lib():
+    from paper_conf_cluster_pawelczakmpm17_b200 import build
+    build.build()
+    from paper_conf_cluster_pawelczakmpm17_b200 import abft
+    return abft
+
+
+def test_exports_every_header_symbol(lib):
+    hdr = open(os.path.join(ROOT, "include", "abft.h")).read()
+    hdr = re.sub(r"/\*.*?\*/", "", hdr, flags=re.S)
+    declared = set(re.findall(r"\b(abft_[a-z0-9_]+)\s*\(", hdr))
+    assert declared, "no declarations parsed"
+    import ctypes
+    so = ctypes.CDLL(lib._SO)
+    missing = [s for s in declared if not hasattr(so, s)]
+    assert not missing, missing
+    assert declared <= set(lib.HEADER_SYMBOLS)
+
+
+def _rand_words(orc, inst, rng):
+    nb = orc.inst_nbits(inst)
+    w = rng.integers(0, 2**32, size=nb // 32, dtype=np.uint64).astype(np.uint32)
+    if inst in (orc.I_R_SECDED64, orc.I_R_SECDED128):
+        w &= np.uint32(0x0FFFFFFF)
+    if inst == orc.I_V_SECDED64:
+        w[0] &= np.uint32(0xFFFFFF00)
+    if inst == orc.I_V_SECDED128:
+        w[0] &= np.uint32(0xFFFFFFE0)
+        w[2] &= np.uint32(0xFFFFFFE0)
+    if inst == orc.I_E_SECDED:
+        w[2] &= np.uint32(0x00FFFFFF)
+    return w
+
+
+@pytest.mark.parametrize("inst_name", ["I_E_SECDED", "I_V_SECDED64", "I_R_SECDED64", "I_R_SECDED128",
+                                       "I_V_SECDED128"])
+def test_host_codec_matches_oracle(lib, orc, inst_name):
+    inst = getattr(orc, inst_name)
+    nb = orc.inst_nbits(inst)
+    rng = np.random.default_rng(100 + inst)
+    for _ in range(3):
+        data = _rand_words(orc, inst, rng)
+        cw_o = orc.secded_encode(inst, data)
+        cw_g = np.array(lib.codec_host_encode(inst, list(data)), dtype=np.uint32)
+        assert np.array_equal(cw_o, cw_g), (inst_name, [hex(x) for x in cw_o], [hex(x) for x in cw_g])
+        assert lib.codec_host_check(inst, list(cw_g)) == orc.CLEAN
+        for b in range(nb):
+            w = cw_g.copy()
+            w[b // 32] ^= np.uint32(1 << (b % 32))
+            lst = list(w)
+            o = lib.codec_host_check(inst, lst)
+            assert o == orc.CORRECTED and np.array_equal(np.array(lst, dtype=np.uint32), cw_g), (inst_name, b)
+        pairs = list(itertools.combinations(range(nb), 2))
+        for idx in rng.choice(len(pairs), 300, replace=False):
+            a, b = pairs[idx]
+            w = cw_g.copy()
+            w[a // 32] ^= np.uint32(1 << (a % 32))
+            w[b // 32] ^= np.uint32(1 << (b % 32))
+            assert lib.codec_host_check(inst, list(w)) == orc.DUE
