@@ -13,7 +13,7 @@ import torch
 
 import gen
 import oracle as orc
-from tests.gpu_helpers import (col_words, gpu_matrix, gpu_vec_from_words, oracle_matrix, rowptr_words, tea,
+from gpu_helpers import (col_words, gpu_matrix, gpu_vec_from_words, oracle_matrix, rowptr_words, tea,
                                val_words, words_of)
 
 pytestmark = pytest.mark.gpu
