@@ -1,0 +1,377 @@
+"""bench.py — protected CG (BASELINE.json config 2) on B200, one JSON line.
+
+    python bench.py [--gpus N --steps K --warmup W] [--impl reference] [--grid 4096]
+
+A step is one pass of the whole hot path (rows a0-a7) over the
+4096^2 G-TEA problem: re-encode the CSR matrix (a0) and the vectors b, x0 (a1),
+then the protected CG solve to tol 1e-10 (a2-a6) with fault counters (a7).
+`value` = CG iterations per second of the protected solve (inputs resident in
+HBM); `e2e` = the same through the C ABI from pinned HOST buffers (H2D of the
+raw matrix + b and D2H of x inside every step).  The unprotected twin (scheme
+NONE everywhere, same kernels) is timed the same way for the overhead figure.
+N > 1 (torchrun): weak scaling, each rank owns a 4096-row strip of a
+4096 x 4096N grid, halos + dots over NCCL; value = it/s x N (4096^2-equivalent).
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "protected CG iters/sec and SpMV HBM GB/s vs peak; ECC overhead % vs unprotected"
+SPMV_BYTES_PER_ROW = 80    # val 40 + col 20 + rowptr 4 + p 8 + w 8
+CG_BYTES_PER_ROW = 152     # SpMV 80 + calc_ur 48 + calc_p 24
+
+
+def _peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            p = json.load(f)
+        return float(p["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons DURING the timed region."""
+    Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+         "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap,power.draw")
+
+    def __init__(self, index: int):
+        self.index, self.rows, self.proc = index, [], None
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(["nvidia-smi", "-i", str(self.index), "--query-gpu=" + self.Q,
+                                          "--format=csv,noheader,nounits", "-lms", "200"],
+                                         stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except Exception:
+            self.proc = None
+        return self
+
+    def _read(self):
+        for line in self.proc.stdout:
+            parts = [p.strip() for p in line.split(",")]
+            if len(parts) >= 7:
+                self.rows.append(parts)
+
+    def __exit__(self, *a):
+        if self.proc:
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except Exception:
+                self.proc.kill()
+
+    def summary(self):
+        if not self.rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unsampled"]}
+        sm = [float(r[0]) for r in self.rows if r[0].replace(".", "").isdigit()]
+        mx = [float(r[1]) for r in self.rows if r[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[k] for r in self.rows for k in range(4) if r[2 + k].lower() == "active"})
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(self.rows)}
+
+
+# ------------------------------------------------------------------ problem
+def build_problem(grid: int, rank: int, world: int, device):
+    """Raw (unencoded) device arrays of this rank's strip + metadata."""
+    import torch
+    import gen
+    n = grid
+    ny = grid * world
+    y0, y1 = rank * grid, (rank + 1) * grid
+    halo = n if world > 1 else 0
+    val, col, rowptr = gen.strip_csr(n, y0, y1, ny=ny, device=device, col_offset=halo)
+    b = gen.tealeaf_rhs(n, y0, y1, ny=ny, device=device)
+    N = (y1 - y0) * n
+    return dict(val=val.contiguous(), col=col.to(torch.int32).contiguous(), rowptr=rowptr.to(torch.int32).contiguous(),
+                b=b.contiguous(), N=N, n=n, halo=halo, ncols=N + 2 * halo)
+
+
+class Solver:
+    """One configuration (protected or unprotected twin) of the solve."""
+
+    def __init__(self, abft, ctx, P, es, rs, vs, dist=None):
+        import torch
+        self.abft, self.ctx, self.P, self.dist = abft, ctx, P, dist
+        self.es, self.rs, self.vs = es, rs, vs
+        N, halo = P["N"], P["halo"]
+        dev = P["val"].device
+        self.A = abft.Matrix(P["val"], P["col"].clone(), P["rowptr"], N, P["ncols"], es, rs, row_base=halo,
+                             col_base=0, stencil_n=P["n"])
+        self.col_raw = P["col"]
+        self.rp_raw = torch.zeros_like(self.A.rowptr)
+        self.rp_raw[:N + 1] = P["rowptr"]
+        n_ext = N + 2 * halo
+        self.vecs = [abft.Vector.empty(n_ext, vs, device=dev) for _ in range(5)]  # b x r p w
+        self.counts = abft.Counters(device=dev)
+        self.b_raw = P["b"]
+        self.N, self.halo = N, halo
+
+    def load_inputs(self, host=None):
+        """(Re)place the raw inputs: from device copies, or from pinned host buffers (e2e)."""
+        if host is None:
+            self.A.col.copy_(self.col_raw)
+            self.A.rowptr.copy_(self.rp_raw)
+            src_b = self.b_raw
+        else:
+            self.A.val.copy_(host["val"], non_blocking=True)
+            self.A.col.copy_(host["col"], non_blocking=True)
+            self.A.rowptr[:self.N + 1].copy_(host["rowptr"], non_blocking=True)
+            self.A.rowptr[self.N + 1:].zero_()
+            src_b = host["b"]
+        b, x = self.vecs[0], self.vecs[1]
+        h = self.halo
+        b.data[h:h + self.N].copy_(src_b, non_blocking=True)
+        x.data[h:h + self.N].copy_(src_b, non_blocking=True)
+
+    def step(self, tol, max_iters, host=None):
+        """a0 + a1 + a2..a7: returns the iteration count."""
+        self.load_inputs(host)
+        st = self.A.encode(self.ctx)
+        if st != 0:
+            raise RuntimeError(f"encode failed: {self.abft.last_error()}")
+        self.vecs[0].encode(self.ctx)
+        self.vecs[1].encode(self.ctx)
+        if self.dist is not None:
+            res = self.dist.cg_solve(self.ctx, self.A, self.halo, *self.vecs, tol=tol, max_iters=max_iters,
+                                     due_policy=1, counts=self.counts, poll_every=32)
+        else:
+            res = self.abft.cg_solve(self.ctx, self.A, *self.vecs, tol=tol, max_iters=max_iters, due_policy=1,
+                                     counts=self.counts, poll_every=32)
+        return res.iters, res.status
+
+
+def timed(solver, steps, warmup, tol, max_iters, dist_on, host=None, out_host=None, profile=False):
+    import torch
+    import torch.distributed as dist
+    abft = solver.abft
+    for _ in range(warmup):
+        solver.step(tol, max_iters, host)
+    torch.cuda.synchronize()
+    if dist_on:
+        dist.barrier()
+    if profile:
+        abft.profile(solver.ctx, True)
+    l0 = abft.launch_count()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    iters = 0
+    statuses = set()
+    e0.record()
+    for _ in range(steps):
+        it, st = solver.step(tol, max_iters, host)
+        if out_host is not None:
+            x = solver.vecs[1]
+            out_host.copy_(x.data[solver.halo:solver.halo + solver.N], non_blocking=True)
+        iters += it
+        statuses.add(st)
+    e1.record()
+    torch.cuda.synchronize()
+    launches = abft.launch_count() - l0
+    ms = e0.elapsed_time(e1)
+    prof = abft.profile_read(solver.ctx) if profile else None
+    if profile:
+        abft.profile(solver.ctx, False)
+    if dist_on:
+        t = torch.tensor([ms], dtype=torch.float64, device="cuda")
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        ms = float(t.item())
+        dist.barrier()
+    return dict(ms=ms, iters=iters, launches=launches, prof=prof, statuses=statuses)
+
+
+def read_traffic():
+    """dram bytes per SpMV launch from the committed ncu --set full summary (or None)."""
+    p = os.path.join(ROOT, "profiles", "spmv_traffic.json")
+    try:
+        with open(p) as f:
+            return json.load(f)
+    except Exception:
+        return None
+
+
+# ------------------------------------------------------------------ oracle legs
+def oracle_sample(grid_sample=512, iters=3):
+    """The CPU oracle (never tuned) on a bounded sample: `iters` protected CG
+    iterations on a grid_sample^2 G-TEA problem with the config-2 schemes,
+    single-threaded; scaled to the 4096^2 workload by row count."""
+    import numpy as np
+    import gen
+    import oracle as orc
+    n = grid_sample
+    v, c, r = gen.tealeaf_csr(n)
+    N = n * n
+    A = orc.Matrix(v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32), N, N, orc.SECDED64,
+                   orc.SECDED64)
+    A.encode()
+    b = gen.tealeaf_rhs(n).numpy()
+    B = orc.vec_encode(b, orc.SECDED64)
+    X = B.copy()
+    R, Pv, W = (np.zeros_like(B) for _ in range(3))
+    # init (untimed) then time `iters` iterations: the oracle has no per-iteration
+    # entry, so time init+k and init+0 and take the difference
+    t0 = time.perf_counter()
+    orc.cg_solve(A, B.copy(), X.copy(), R, Pv, W, orc.SECDED64, 0.0, 0, 1, None)
+    t1 = time.perf_counter()
+    orc.cg_solve(A, B.copy(), X.copy(), R, Pv, W, orc.SECDED64, 0.0, iters, 1, None)
+    t2 = time.perf_counter()
+    per_iter = ((t2 - t1) - (t1 - t0)) / iters
+    scale = (4096 * 4096) / N
+    its = 1.0 / (per_iter * scale)
+    return its, f"{iters} protected CG iterations (E-SECDED+R-SECDED64+V-SECDED64) on a {n}^2 G-TEA grid, " \
+                f"per-iteration time scaled by rows to 4096^2 ({per_iter:.3f} s/iter at {n}^2)"
+
+
+def run_reference(args):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    vals = []
+    sample = ""
+    for _ in range(args.warmup):
+        oracle_sample(args.oracle_grid, 1)
+    t0 = time.perf_counter()
+    for _ in range(args.steps):
+        v, sample = oracle_sample(args.oracle_grid, 2)
+        vals.append(v)
+    wall = time.perf_counter() - t0
+    val = statistics.median(vals)
+    line = {"impl": "reference", "metric": METRIC, "value": val, "unit": "CG it/s (4096^2, protected)",
+            "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+            "ms_per_step": 1000.0 * wall / max(args.steps, 1), "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+            "config": {"workload": "tealeaf-4096x4096-cg-full-ecc", "grid": 4096, "sample_grid": args.oracle_grid},
+            "cpu_baseline": {"value": val, "unit": "CG it/s (4096^2, protected)", "cores": 1, "kind": "oracle",
+                             "sample": sample},
+            "e2e": {"value": val, "unit": "CG it/s (4096^2, protected)", "h2d_bytes_per_step": 0,
+                    "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# ------------------------------------------------------------------ main
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=3)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--grid", type=int, default=4096)
+    ap.add_argument("--tol", type=float, default=1e-10)
+    ap.add_argument("--max-iters", type=int, default=20000)
+    ap.add_argument("--oracle-grid", type=int, default=512)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-e2e", action="store_true")
+    args = ap.parse_args()
+    if args.impl == "reference":
+        return run_reference(args)
+
+    import torch
+    import torch.distributed as dist
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    torch.cuda.set_device(local)
+    dist_on = world > 1
+    if dist_on:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    from paper_conf_cluster_pawelczakmpm17_b200 import abft
+
+    P = build_problem(args.grid, rank, world, torch.device("cuda", local))
+    ctx = abft.Context(local)
+    dobj = abft.Dist(rank, world, local) if dist_on else None
+    prot = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj)
+    with ClockSampler(local) as clk:
+        r_p = timed(prot, args.steps, args.warmup, args.tol, args.max_iters, dist_on, profile=True)
+    clocks = clk.summary()
+    del prot
+    twin = Solver(abft, ctx, P, abft.NONE, abft.NONE, abft.NONE, dobj)
+    r_u = timed(twin, args.steps, max(1, args.warmup // 2), args.tol, args.max_iters, dist_on, profile=True)
+    del twin
+
+    e2e = None
+    if not args.no_e2e:
+        prot = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj)
+        host = {k: P[k].cpu().pin_memory() for k in ("val", "col", "b")}
+        host["rowptr"] = P["rowptr"].cpu().pin_memory()
+        out_host = torch.empty(P["N"], dtype=torch.float64).pin_memory()
+        r_e = timed(prot, args.steps, 1, args.tol, args.max_iters, dist_on, host=host, out_host=out_host)
+        h2d = sum(t.numel() * t.element_size() for t in host.values())
+        e2e = {"value": world * r_e["iters"] / (r_e["ms"] / 1000.0), "unit": "CG it/s (4096^2-equivalent)",
+               "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": P["N"] * 8}
+        del prot
+
+    if rank != 0:
+        if dist_on:
+            dist.destroy_process_group()
+        return
+
+    N = P["N"]
+    its = r_p["iters"] / (r_p["ms"] / 1000.0)
+    its_u = r_u["iters"] / (r_u["ms"] / 1000.0)
+    peak, peak_src = _peaks()
+    ms_cls, n_cls = r_p["prof"]
+    spmv_ms = ms_cls[0] / max(n_cls[0], 1)
+    spmv_gbs = SPMV_BYTES_PER_ROW * N / (spmv_ms / 1000.0) / 1e9 if spmv_ms > 0 else None
+    ms_u, n_u = r_u["prof"]
+    traffic = read_traffic()
+    iter_ms_p = r_p["ms"] / max(r_p["iters"], 1)
+    iter_ms_u = r_u["ms"] / max(r_u["iters"], 1)
+    line = {
+        "metric": METRIC,
+        "value": world * its,
+        "unit": "CG it/s (4096^2-equivalent)",
+        "n_gpus": world,
+        "steps": args.steps,
+        "warmup": args.warmup,
+        "ms_per_step": r_p["ms"] / args.steps,
+        "higher_is_better": True,
+        "scaling": "weak",
+        "vs_baseline": None,
+        "dtype": "f64",
+        "data": "synthetic",
+        "config": {"workload": "tealeaf-4096x4096-cg-full-ecc", "grid": args.grid, "rows_per_gpu": N,
+                   "schemes": {"elements": "E-SECDED", "rowptr": "R-SECDED64", "vectors": "V-SECDED64"},
+                   "tol": args.tol, "iters_per_step": r_p["iters"] / args.steps,
+                   "l2": "inputs larger than L2 (2.55 GB moved per CG iteration vs 126 MB L2)",
+                   "parallelism": f"row-block strips x{world}" if world > 1 else "single GPU"},
+        "roofline": {"bound": "hbm", "kernel": "k_spmv (protected SpMV + p.w)",
+                     "achieved": spmv_gbs, "peak": peak, "unit": "GB/s",
+                     "frac": (spmv_gbs / peak) if spmv_gbs else None,
+                     "traffic": traffic.get("bytes_per_launch") if traffic else None,
+                     "bytes_per_launch_algorithmic": SPMV_BYTES_PER_ROW * N, "peak_source": peak_src,
+                     "avg_launch_ms": spmv_ms},
+        "cg_bandwidth": {"achieved_gbs": CG_BYTES_PER_ROW * N / (iter_ms_p / 1000.0) / 1e9,
+                         "frac_of_measured": CG_BYTES_PER_ROW * N / (iter_ms_p / 1000.0) / 1e9 / peak,
+                         "frac_of_8tbs": CG_BYTES_PER_ROW * N / (iter_ms_p / 1000.0) / 1e9 / 8000.0},
+        "kernel_ms": {"spmv": spmv_ms, "calc_ur": ms_cls[1] / max(n_cls[1], 1), "calc_p": ms_cls[2] / max(n_cls[2], 1),
+                      "reductions": ms_cls[3] / max(n_cls[3], 1)},
+        "unprotected": {"value": world * its_u, "iter_ms": iter_ms_u, "iters_per_step": r_u["iters"] / args.steps,
+                        "spmv_ms": ms_u[0] / max(n_u[0], 1)},
+        "overhead_pct_per_iter": 100.0 * (iter_ms_p / iter_ms_u - 1.0),
+        "clocks": clocks,
+        "gpu_launches": r_p["launches"],
+        "e2e": e2e,
+    }
+    if world == 1 and not args.no_cpu_baseline:
+        v, sample = oracle_sample(args.oracle_grid, 3)
+        line["cpu_baseline"] = {"value": v, "unit": "CG it/s (4096^2, protected)", "cores": 1, "kind": "oracle",
+                                "sample": sample}
+    print(json.dumps(line), flush=True)
+    if dist_on:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

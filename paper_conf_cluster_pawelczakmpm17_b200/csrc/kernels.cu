@@ -200,8 +200,9 @@ __device__ __forceinline__ void rowptr_pass(const SpmvArgs& a, int64_t pb, int l
     return;
   }
   constexpr int NG = 32 / G + 1;
-  const int64_t g = pb / G + lane;
-  if (lane < NG && g * G <= a.nrows) {
+  for (int gl = lane; gl < NG; gl += 32) {  // NG = 33 for G = 1: lane 0 takes the extra group
+    const int64_t g = pb / G + gl;
+    if (g * G > a.nrows) continue;
     uint32_t e[G];
     uint32_t* gp = a.rowptr + g * G;
     if (G == 1) e[0] = __ldg(gp);
@@ -230,7 +231,7 @@ __device__ __forceinline__ void rowptr_pass(const SpmvArgs& a, int64_t pb, int l
       }
     }
 #pragma unroll
-    for (int t = 0; t < G; t++) srp[lane * G + t] = e[t] & rp_keep(RS);
+    for (int t = 0; t < G; t++) srp[gl * G + t] = e[t] & rp_keep(RS);
   }
   __syncwarp();
   start = srp[lane];

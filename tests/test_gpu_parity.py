@@ -38,7 +38,7 @@ def _special_values(n, seed):
     v = gen.uniform_pm1(n, seed) * 10.0 ** np.round(gen.uniform_pm1(n, seed + 1) * 30)
     sp = [0.0, -0.0, 1.0, -1.0, math.pi, -0.1, 1e300, -1e-300, 5e-324, float("inf"), float("-inf"),
           1.7976931348623157e308, 2.2250738585072014e-308]
-    v[:len(sp)] = sp
+    v[:min(n, len(sp))] = sp[:n]
     return v
 
 
@@ -179,6 +179,16 @@ def test_spmv_fault_parity(abft, ctx, es, rs, vs, double):
         assert cg[:, :, 1].sum() == cg[:, :, 0].sum() > 0  # every detection corrected
 
 
+def words_equal_nan(a, b, scheme):
+    """Bit-exact except where both values are NaN: IEEE 754 leaves NaN sign and
+    payload unspecified, and x86 / sm_100 differ (reading R25)."""
+    keep = np.uint64(~np.uint64((1 << {0: 0, 1: 1, 2: 8, 3: 5, 4: 8}[scheme]) - 1))
+    va = (a & keep).view(np.float64)
+    vb = (b & keep).view(np.float64)
+    both_nan = np.isnan(va) & np.isnan(vb)
+    return bool(np.all((a == b) | both_nan))
+
+
 def _cg_both(abft, ctx, n, es, rs, vs, policy=1, inject=None, max_iters=5000, tol=1e-10):
     v, c, r = tea(n)
     N = n * n
@@ -275,7 +285,7 @@ def test_config1_fault_campaign_32(abft, ctx):
         R = _cg_both(abft, ctx, 32, orc.SECDED64, orc.SED, orc.SED, policy=1, inject=inj)
         assert np.array_equal(R["cnt_g"], R["cnt_o"]), (R["cnt_g"], R["cnt_o"])
         assert R["res_g"].iters == R["res_o"].iters
-        assert np.array_equal(R["xg"][:len(R["xo"])], R["xo"])
+        assert words_equal_nan(R["xg"][:len(R["xo"])], R["xo"], orc.SED)
         # every element flip was corrected (E-SECDED), every vector/rowptr flip detected (SED)
         assert R["cnt_g"][orc.ELEM, orc.SECDED64, orc.UNC] == 0
 

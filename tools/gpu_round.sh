@@ -1,0 +1,27 @@
+#!/bin/bash
+# One GPU session: tests, smoke, bench, ncu launch list + full capture of the
+# hot kernels.  Usage (under gpurun): bash tools/gpu_round.sh [tag] [what...]
+TAG=${1:-r01}; shift
+WHAT=${@:-"tests smoke bench ncu"}
+mkdir -p gpurun_out
+nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw --format=csv > gpurun_out/gpu_$TAG.txt
+python -c "import __graft_entry__ as g; g.build()" > gpurun_out/build_$TAG.log 2>&1 || { cat gpurun_out/build_$TAG.log; exit 1; }
+for w in $WHAT; do
+  case $w in
+  tests)
+    timeout 1200 python -m pytest tests -m gpu -q --tb=short --maxfail=30 > gpurun_out/tests_$TAG.log 2>&1
+    tail -30 gpurun_out/tests_$TAG.log ;;
+  smoke)
+    timeout 300 python __graft_entry__.py --smoke > gpurun_out/smoke_$TAG.log 2>&1; tail -5 gpurun_out/smoke_$TAG.log ;;
+  bench)
+    timeout 900 python bench.py > gpurun_out/bench_$TAG.json 2> gpurun_out/bench_$TAG.err; tail -3 gpurun_out/bench_$TAG.err; cat gpurun_out/bench_$TAG.json ;;
+  benchref)
+    timeout 900 python bench.py --impl reference --steps 2 --warmup 1 > gpurun_out/benchref_$TAG.json 2>&1; cat gpurun_out/benchref_$TAG.json ;;
+  ncu)
+    timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv --log-file gpurun_out/launches_$TAG.csv \
+      python bench.py --steps 1 --warmup 0 --no-e2e --no-cpu-baseline --max-iters 30 > gpurun_out/ncu_launch_bench_$TAG.json 2>&1
+    timeout 900 ncu --set full --clock-control none --import-source on -k regex:'k_spmv|k_calc_ur|k_calc_p' -s 6 -c 6 \
+      -o gpurun_out/prof_$TAG -f python bench.py --steps 1 --warmup 0 --no-e2e --no-cpu-baseline --max-iters 4 > gpurun_out/ncu_full_$TAG.log 2>&1
+    tail -3 gpurun_out/ncu_full_$TAG.log ;;
+  esac
+done
