@@ -45,16 +45,33 @@ def needs_build() -> bool:
 
 
 def build(force: bool = False, verbose: bool = False) -> str:
+    """Compile every csrc/*.cu to an object in parallel, then link libabft.so."""
     if not force and not needs_build():
         return SO
+    from concurrent.futures import ThreadPoolExecutor
     nccl = _nccl_dir()
     cus = sorted(glob.glob(os.path.join(CSRC, "*.cu")))
-    cmd = ["nvcc", *ARCH, "-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr", "-Xcompiler", "-fPIC",
-           "-shared", "-I", os.path.join(nccl, "include"), "-o", SO + ".tmp", *cus,
-           "-L", os.path.join(nccl, "lib"), "-l:libnccl.so.2", "-Xlinker", "-rpath=" + os.path.join(nccl, "lib")]
+    objdir = os.path.join(PKG, "build_obj")
+    os.makedirs(objdir, exist_ok=True)
+    flags = [*ARCH, "-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr", "-Xcompiler", "-fPIC",
+             "-I", os.path.join(nccl, "include")]
     if verbose:
-        cmd.insert(1, "-Xptxas=-v")
-        print(" ".join(cmd))
+        flags.append("-Xptxas=-v")
+
+    def compile_one(cu):
+        obj = os.path.join(objdir, os.path.basename(cu)[:-3] + ".o")
+        cmd = ["nvcc", *flags, "-c", cu, "-o", obj]
+        r = subprocess.run(cmd, capture_output=True, text=True)
+        if r.returncode != 0 or verbose:
+            sys.stderr.write(r.stdout + r.stderr)
+        if r.returncode != 0:
+            raise RuntimeError(f"nvcc failed on {cu}")
+        return obj
+
+    with ThreadPoolExecutor(max_workers=max(2, os.cpu_count() or 2)) as ex:
+        objs = list(ex.map(compile_one, cus))
+    cmd = ["nvcc", *ARCH, "-shared", "-o", SO + ".tmp", *objs, "-L", os.path.join(nccl, "lib"), "-l:libnccl.so.2",
+           "-Xlinker", "-rpath=" + os.path.join(nccl, "lib")]
     subprocess.check_call(cmd)
     os.replace(SO + ".tmp", SO)
     return SO

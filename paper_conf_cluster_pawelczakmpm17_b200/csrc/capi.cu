@@ -121,6 +121,7 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.npad_in = npad_in;
     a.npad_out = (M.row_base + M.nrows == out->n) ? (npad_out - M.row_base) : M.nrows;
     a.rb_offset = (M.row_base - base0) / 256;
+    a.stencil_n = M.stencil_n;
     a.val = reinterpret_cast<uint64_t*>(M.val);
     a.col = M.col;
     a.rowptr = M.rowptr;

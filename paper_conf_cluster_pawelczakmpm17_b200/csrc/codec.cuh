@@ -62,23 +62,39 @@ ABFT_HD uint32_t lo32(uint64_t u) { return (uint32_t)u; }
 ABFT_HD uint32_t hi32(uint64_t u) { return (uint32_t)(u >> 32); }
 ABFT_HD uint64_t mk64(uint32_t lo, uint32_t hi) { return ((uint64_t)hi << 32) | lo; }
 
-// Superset-sum (Moebius / zeta) transform of a 32-bit fold register:
-// R[i] = XOR_{j superset of i} D[j].  R[0] = parity(D), R[2^k] = parity of the
-// bits whose index has bit k set, i.e. R[1,2,4,8,16] = XOR of the indices of
-// the set bits of D.
-ABFT_HD uint32_t moebius32(uint32_t d) {
-  d ^= (d >> 1) & 0x55555555u;
-  d ^= (d >> 2) & 0x33333333u;
-  d ^= (d >> 4) & 0x0F0F0F0Fu;
-  d ^= (d >> 8) & 0x00FF00FFu;
-  d ^= (d >> 16) & 0x0000FFFFu;
+// Subset-sum (Moebius / zeta) transform of a 32-bit fold register:
+// R[i] = XOR_{j subset of i} D[j].  Then R[31] = parity(D) and, for k = 0..4,
+// R[31 - 2^k] = parity of the bits whose index has bit k CLEAR, i.e.
+// R[31] ^ R[31 - 2^k] = bit k of (XOR of the indices of the set bits of D).
+// Only left shifts: ptxas emits IMAD.SHL (FMA pipe) for them, so the 10-op
+// transform splits across the ALU and FMA pipes (measured faster on sm_100a,
+// tools/microbench/codec.cu).
+constexpr ABFT_HD uint32_t moebius32(uint32_t d) {
+  d ^= (d << 1) & 0xAAAAAAAAu;
+  d ^= (d << 2) & 0xCCCCCCCCu;
+  d ^= (d << 4) & 0xF0F0F0F0u;
+  d ^= (d << 8) & 0xFF00FF00u;
+  d ^= (d << 16) & 0xFFFF0000u;
   return d;
 }
-constexpr uint32_t MOEB_SYN_MASK = 0x00010117u;  // R bits {0,1,2,4,8,16}
-// 5-bit index syndrome from a Moebius register
+// R bits {31, 30, 29, 27, 23, 15}: all zero <=> parity 0 and index syndrome 0
+constexpr uint32_t MOEB_SYN_MASK = 0xE8808000u;
+// q and the 5-bit index syndrome from a Moebius register
+ABFT_HD int moeb_q(uint32_t r) { return (int)(r >> 31); }
 ABFT_HD int moeb_index(uint32_t r) {
-  return ((r >> 1) & 1) | (((r >> 2) & 1) << 1) | (((r >> 4) & 1) << 2) | (((r >> 8) & 1) << 3) |
-         (((r >> 16) & 1) << 4);
+  const uint32_t q = r >> 31;
+  return (int)(((r >> 30) & 1) ^ q) | (int)((((r >> 29) & 1) ^ q) << 1) | (int)((((r >> 27) & 1) ^ q) << 2) |
+         (int)((((r >> 23) & 1) ^ q) << 3) | (int)((((r >> 15) & 1) ^ q) << 4);
+}
+// inverse: the Moebius-register bits a (q, index syndrome) pair produces
+constexpr ABFT_HD uint32_t moeb_bits(int q, int idx) {
+  uint32_t r = (uint32_t)q << 31;
+  r |= (uint32_t)(q ^ (idx & 1)) << 30;
+  r |= (uint32_t)(q ^ ((idx >> 1) & 1)) << 29;
+  r |= (uint32_t)(q ^ ((idx >> 2) & 1)) << 27;
+  r |= (uint32_t)(q ^ ((idx >> 3) & 1)) << 23;
+  r |= (uint32_t)(q ^ ((idx >> 4) & 1)) << 15;
+  return r;
 }
 
 // ------------------------------------------------------ layout tables
@@ -161,9 +177,9 @@ constexpr MaskTable make_masks(const Layout& L) {
   return T;
 }
 #if defined(__CUDACC__)
-__constant__ MaskTable c_mt_r64 = make_masks(kR64);
-__constant__ MaskTable c_mt_r128 = make_masks(kR128);
-__constant__ MaskTable c_mt_v128 = make_masks(kV128);
+static __constant__ MaskTable c_mt_r64 = make_masks(kR64);
+static __constant__ MaskTable c_mt_r128 = make_masks(kR128);
+static __constant__ MaskTable c_mt_v128 = make_masks(kV128);
 #endif
 constexpr MaskTable h_mt_r64 = make_masks(kR64);
 constexpr MaskTable h_mt_r128 = make_masks(kR128);
@@ -179,11 +195,11 @@ constexpr ColMap make_colmap(const Layout& L) {
 }
 
 #if defined(__CUDACC__)
-__constant__ ColMap c_map_e96 = make_colmap(kE96);
-__constant__ ColMap c_map_v64 = make_colmap(kV64);
-__constant__ ColMap c_map_r64 = make_colmap(kR64);
-__constant__ ColMap c_map_r128 = make_colmap(kR128);
-__constant__ ColMap c_map_v128 = make_colmap(kV128);
+static __constant__ ColMap c_map_e96 = make_colmap(kE96);
+static __constant__ ColMap c_map_v64 = make_colmap(kV64);
+static __constant__ ColMap c_map_r64 = make_colmap(kR64);
+static __constant__ ColMap c_map_r128 = make_colmap(kR128);
+static __constant__ ColMap c_map_v128 = make_colmap(kV128);
 #endif
 constexpr ColMap h_map_e96 = make_colmap(kE96);
 constexpr ColMap h_map_v64 = make_colmap(kV64);
@@ -266,7 +282,7 @@ ABFT_HD uint32_t v64_bad(uint32_t a, uint32_t b) {
 ABFT_HD void v64_syndrome(uint32_t a, uint32_t b, int& s, int& q) {
   uint32_t r = moebius32(v64_fold(a, b));
   s = moeb_index(r) | ((popc32(b ^ (a & 0x80u)) & 1) << 5) | ((popc32(a & 0x8Eu) & 1) << 6);
-  q = (int)(r & 1u);
+  q = moeb_q(r);
 }
 // Slow path: correct in place; returns outcome, *word = 0/1 for the half fixed.
 ABFT_HD int v64_correct(uint64_t& u, int* word) {
@@ -277,12 +293,13 @@ ABFT_HD int v64_correct(uint64_t& u, int* word) {
   if (o == CORRECTED) u = mk64(w[0], w[1]);
   return o;
 }
-// Encoder LUT: index = ((R & 0x10117) | s5 << 3) * 0x08040200 >> 25 (a
-// bijection of the 7 syndrome bits q,s0..s5 onto 0..127; s6 of the data part
-// is always 0 because no data bit of V-SECDED64 has code bit 1).
-constexpr uint32_t V64_LUT_MUL = 0x08040200u;
-ABFT_HD uint32_t v64_lut_index(uint32_t r, uint32_t s5) {
-  return (((r & MOEB_SYN_MASK) | ((s5 & 1u) << 3)) * V64_LUT_MUL) >> 25;
+// Encoder LUT: index = ((R & MOEB_SYN_MASK) | s5) * 0x10000805 >> 25, a
+// bijection of the 7 data-syndrome bits (q, s0..s5) onto 0..127 (found by
+// search); s6 of the data part is always 0 because no data bit of V-SECDED64
+// has code bit 1.
+constexpr uint32_t V64_LUT_MUL = 0x10000805u;
+constexpr ABFT_HD uint32_t v64_lut_index(uint32_t r, uint32_t s5) {
+  return (((r & MOEB_SYN_MASK) | (s5 & 1u)) * V64_LUT_MUL) >> 25;
 }
 struct V64Lut { uint8_t r[128]; };
 constexpr V64Lut make_v64_lut() {
@@ -293,16 +310,13 @@ constexpr V64Lut make_v64_lut() {
     int s = 0, q = 0;
     for (int b = 0; b < 8; b++) if ((r >> b) & 1) { s ^= kV64.col[b]; q ^= 1; }
     if ((s >> 6) & 1) continue;
-    uint32_t R = (uint32_t)q | (uint32_t)((s & 1) << 1) | (uint32_t)(((s >> 1) & 1) << 2) |
-                 (uint32_t)(((s >> 2) & 1) << 4) | (uint32_t)(((s >> 3) & 1) << 8) | (uint32_t)(((s >> 4) & 1) << 16);
-    uint32_t idx = (((R & MOEB_SYN_MASK) | ((uint32_t)((s >> 5) & 1) << 3)) * V64_LUT_MUL) >> 25;
-    T.r[idx] = (uint8_t)r;
+    T.r[v64_lut_index(moeb_bits(q, s & 31), (uint32_t)((s >> 5) & 1))] = (uint8_t)r;
   }
   return T;
 }
 constexpr V64Lut h_v64_lut = make_v64_lut();
 #if defined(__CUDACC__)
-__constant__ V64Lut c_v64_lut = make_v64_lut();
+static __constant__ V64Lut c_v64_lut = make_v64_lut();
 #endif
 // Encode with a LUT pointer (shared-memory copy on the device: 128 B = one word
 // per bank, conflict-free for any index pattern).
@@ -412,7 +426,7 @@ ABFT_HD void e96_syndrome(uint32_t a, uint32_t b, uint32_t c, int& s, int& q) {
   uint32_t r = moebius32(e96_fold(a, b, c));
   s = moeb_index(r) | ((popc32(b ^ (c & 0x9F000000u)) & 1) << 5) |
       ((popc32((c & 0x7FFFFFFFu) ^ (b & 0x80000000u)) & 1) << 6);
-  q = (int)(r & 1u);
+  q = moeb_q(r);
 }
 ABFT_HD int e96_correct(uint64_t& v, uint32_t& c, int* word) {
   uint32_t w[3] = {lo32(v), hi32(v), c};
@@ -436,7 +450,7 @@ constexpr E96Enc make_e96_enc() {
 }
 constexpr E96Enc h_e96_enc = make_e96_enc();
 #if defined(__CUDACC__)
-__constant__ E96Enc c_e96_enc = make_e96_enc();
+static __constant__ E96Enc c_e96_enc = make_e96_enc();
 #endif
 ABFT_HD uint32_t e96_encode_col(uint64_t v, uint32_t col24) {
   uint32_t c = col24 & 0x00FFFFFFu;

@@ -22,6 +22,7 @@ struct DevCounts { unsigned long long v[3][5][4]; };
 // arguments of one SpMV chunk launch
 struct SpmvArgs {
   int64_t nrows, ncols, nnz, row_base, col_base, n_in, npad_in, npad_out, rb_offset;
+  int64_t stencil_n;  // > 0: 5-point stencil row stride (tiled fast path)
   uint64_t* val;
   uint32_t* col;
   uint32_t* rowptr;

@@ -1,0 +1,873 @@
+// kernels_impl.cuh — device helpers and kernel templates shared by the kernel
+// translation units (kernels.cu, spmv_es*.cu).
+#pragma once
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "codec.cuh"
+#include "internal.h"
+
+namespace abft {
+
+// --------------------------------------------------------------- helpers
+__host__ __device__ constexpr int vgrp(int s) { return s == SECDED128 ? 2 : s == CRC32C ? 4 : 1; }
+__host__ __device__ constexpr int rgrp(int s) { return s == SECDED64 ? 2 : s == SECDED128 ? 4 : s == CRC32C ? 8 : 1; }
+__host__ __device__ constexpr int vk(int s) { return s == SED ? 1 : s == SECDED64 ? 8 : s == SECDED128 ? 5 : s == CRC32C ? 8 : 0; }
+__host__ __device__ constexpr uint64_t vkeep(int s) { return vk(s) ? ~((1ull << vk(s)) - 1ull) : ~0ull; }
+
+static __device__ __forceinline__ double as_d(uint64_t u) { return __longlong_as_double((long long)u); }
+static __device__ __forceinline__ uint64_t as_u(double d) { return (uint64_t)__double_as_longlong(d); }
+static __device__ __forceinline__ uint64_t shfl64(uint64_t v, int src) {
+  uint32_t lo = __shfl_sync(0xffffffffu, (uint32_t)v, src);
+  uint32_t hi = __shfl_sync(0xffffffffu, (uint32_t)(v >> 32), src);
+  return mk64(lo, hi);
+}
+static __device__ __forceinline__ uint64_t ldg64(const uint64_t* p) { return (uint64_t)__ldg((const unsigned long long*)p); }
+
+static __device__ __forceinline__ void cnt_add(DevCounts* c, int t, int s, int o) {
+  if (!c) return;
+  atomicAdd(&c->v[t][s][0], 1ull);
+  atomicAdd(&c->v[t][s][o == CORRECTED ? 1 : 2], 1ull);
+}
+static __device__ __forceinline__ void cnt_range(DevCounts* c, int t, int s) {
+  if (c) atomicAdd(&c->v[t][s][3], 1ull);
+}
+// Scrub one 32-bit word; returns true iff this thread's CAS replaced it (the
+// winner counts the correction: exactly-once counting).
+static __device__ __forceinline__ bool scrub32(uint32_t* addr, uint32_t oldw, uint32_t neww) {
+  return atomicCAS((unsigned int*)addr, oldw, neww) == oldw;
+}
+
+static __device__ __forceinline__ void load_lut(uint8_t* s_lut) {
+  if (threadIdx.x < 32) reinterpret_cast<uint32_t*>(s_lut)[threadIdx.x] = reinterpret_cast<const uint32_t*>(&c_v64_lut)[threadIdx.x];
+}
+
+// Cold path of a single-codeword vector check (G = 1 schemes).
+template <int VS>
+__device__ __noinline__ uint64_t v1_fix(uint64_t w, uint64_t* addr, bool owner, DevCounts* cnt, int* due) {
+  uint64_t d = w;
+  int word = 0;
+  int o = (VS == SECDED64) ? v64_correct(d, &word) : DUE;
+  if (o == CORRECTED) {
+    if (owner) {
+      uint32_t oldw = word ? hi32(w) : lo32(w), neww = word ? hi32(d) : lo32(d);
+      if (scrub32(reinterpret_cast<uint32_t*>(addr) + word, oldw, neww)) cnt_add(cnt, T_VEC, VS, CORRECTED);
+    }
+    return d;
+  }
+  if (owner) { cnt_add(cnt, T_VEC, VS, DUE); *due = 1; }
+  return w;
+}
+// Check one G=1 codeword: returns the (corrected) stored word.
+template <int VS>
+__device__ __forceinline__ uint64_t v1_check(uint64_t w, uint64_t* addr, bool owner, DevCounts* cnt, int* due) {
+  if (VS == SED) { if (!vsed_clean(w)) return v1_fix<VS>(w, addr, owner, cnt, due); }
+  if (VS == SECDED64) { if (v64_bad(lo32(w), hi32(w))) return v1_fix<VS>(w, addr, owner, cnt, due); }
+  return w;
+}
+
+// Group check (G = 2, 4): lanes [lead, lead+G) hold the group's words; the
+// leader checks, counts and scrubs, then broadcasts the corrected words.
+// Must be called by the full warp.
+template <int VS>
+__device__ uint64_t vg_check(uint64_t my, uint64_t* group_addr, int lane, bool active, bool owner, DevCounts* cnt,
+                             int* due) {
+  constexpr int G = vgrp(VS);
+  const int lead = lane & ~(G - 1);
+  uint64_t d[G];
+#pragma unroll
+  for (int t = 0; t < G; t++) d[t] = shfl64(my, lead + t);
+  if (lane == lead && active) {
+    uint64_t o0[G];
+#pragma unroll
+    for (int t = 0; t < G; t++) o0[t] = d[t];
+    int word = 0;
+    int o = vec_check_group<VS>(d, &word);
+    if (o == CORRECTED) {
+      if (owner) {
+        uint32_t* a32 = reinterpret_cast<uint32_t*>(group_addr) + word;
+        uint64_t ow = o0[word >> 1], nw = d[word >> 1];
+        uint32_t oldw = (word & 1) ? hi32(ow) : lo32(ow), neww = (word & 1) ? hi32(nw) : lo32(nw);
+        if (scrub32(a32, oldw, neww)) cnt_add(cnt, T_VEC, VS, CORRECTED);
+      }
+    } else if (o == DUE) {
+#pragma unroll
+      for (int t = 0; t < G; t++) d[t] = o0[t];
+      if (owner) { cnt_add(cnt, T_VEC, VS, DUE); *due = 1; }
+    }
+  }
+  uint64_t res = my;
+#pragma unroll
+  for (int t = 0; t < G; t++) {
+    uint64_t v = shfl64(d[t], lead);
+    if ((lane & (G - 1)) == t) res = v;
+  }
+  return res;
+}
+
+// Encode: each lane passes its rounded value; returns its encoded word.
+template <int VS>
+__device__ __forceinline__ uint64_t v_encode(uint64_t rounded, int lane, const uint8_t* lut) {
+  constexpr int G = vgrp(VS);
+  if (G == 1) {
+    uint64_t d[1] = {rounded};
+    vec_encode_group<VS>(d, lut);
+    return d[0];
+  } else {
+    const int lead = lane & ~(G - 1);
+    uint64_t d[G > 1 ? G : 1];
+#pragma unroll
+    for (int t = 0; t < G; t++) d[t] = shfl64(rounded, lead + t);
+    if (lane == lead) vec_encode_group<VS>(d, lut);
+    uint64_t res = 0;
+#pragma unroll
+    for (int t = 0; t < G; t++) {
+      uint64_t v = shfl64(d[t], lead);
+      if ((lane & (G - 1)) == t) res = v;
+    }
+    return res;
+  }
+}
+
+// Warp-uniform vector access for one pass: load my word (if idx < npad), check
+// as owner, return the corrected stored word.
+template <int VS>
+__device__ __forceinline__ uint64_t v_load_check(uint64_t* v, int64_t idx, int64_t npad, int lane, bool owner,
+                                                 DevCounts* cnt, int* due) {
+  constexpr int G = vgrp(VS);
+  const bool in = idx < npad;
+  uint64_t w = in ? ldg64(v + idx) : 0ull;
+  if (VS == NONE) return w;
+  if (G == 1) return in ? v1_check<VS>(w, v + idx, owner, cnt, due) : w;
+  const int64_t gidx = idx & ~(int64_t)(G - 1);
+  return vg_check<VS>(w, v + gidx, lane, in, owner && in, cnt, due);
+}
+
+// Non-owner gather of in[idx] (any lane, no shuffles): returns the masked value.
+template <int VS>
+__device__ __forceinline__ double gather_in(const uint64_t* in, int64_t idx) {
+  constexpr int G = vgrp(VS);
+  if (G == 1) {
+    uint64_t w = ldg64(in + idx);
+    if (VS == SED) return as_d(w & vkeep(VS));
+    if (VS == SECDED64) {
+      if (v64_bad(lo32(w), hi32(w))) {
+        uint64_t d = w;
+        if (v64_correct(d, nullptr) == CORRECTED) w = d;
+      }
+    }
+    return as_d(w & vkeep(VS));
+  } else {
+    const int64_t g = idx & ~(int64_t)(G - 1);
+    uint64_t d[G];
+#pragma unroll
+    for (int t = 0; t < G; t++) d[t] = ldg64(in + g + t);
+    uint64_t o0 = d[idx - g];
+    int o = vec_check_group<VS>(d, nullptr);
+    uint64_t w = (o == CORRECTED) ? d[idx - g] : o0;
+    return as_d(w & vkeep(VS));
+  }
+}
+
+// ============================================================ rowptr pass
+// Decode the rowptr groups covering entries [pb, pb+32] into srp (per warp),
+// checking them (owner = the pass holding row min(gG, nrows-1)), then return
+// this lane's start/end.
+template <int RS>
+__device__ __forceinline__ void rowptr_pass(const SpmvArgs& a, int64_t pb, int lane, uint32_t* srp, uint32_t& start,
+                                            uint32_t& end) {
+  constexpr int G = rgrp(RS);
+  if (RS == NONE) {
+    const int64_t e = pb + lane;
+    start = (e <= a.nrows) ? __ldg(a.rowptr + e) : 0u;
+    end = (e + 1 <= a.nrows) ? __ldg(a.rowptr + e + 1) : 0u;
+    return;
+  }
+  constexpr int NG = 32 / G + 1;
+  for (int gl = lane; gl < NG; gl += 32) {  // NG = 33 for G = 1: lane 0 takes the extra group
+    const int64_t g = pb / G + gl;
+    if (g * G > a.nrows) continue;
+    uint32_t e[G];
+    uint32_t* gp = a.rowptr + g * G;
+    if (G == 1) e[0] = __ldg(gp);
+    else if (G == 2) { uint2 u = __ldg(reinterpret_cast<const uint2*>(gp)); e[0] = u.x; e[1 % G] = u.y; }
+    else {
+#pragma unroll
+      for (int q = 0; q < G; q += 4) {
+        uint4 u = __ldg(reinterpret_cast<const uint4*>(gp + q));
+        e[q] = u.x; e[(q + 1) % G] = u.y; e[(q + 2) % G] = u.z; e[(q + 3) % G] = u.w;
+      }
+    }
+    uint32_t o0[G];
+#pragma unroll
+    for (int t = 0; t < G; t++) o0[t] = e[t];
+    int word = 0;
+    int o = rp_check_group<RS>(e, &word);
+    if (o != CLEAN) {
+      int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
+      bool owner = own >= pb && own < pb + 32;
+      if (o == CORRECTED) {
+        if (owner && scrub32(gp + word, o0[word], e[word])) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
+      } else {
+#pragma unroll
+        for (int t = 0; t < G; t++) e[t] = o0[t];
+        if (owner) { cnt_add(a.counts, T_ROWPTR, RS, DUE); *a.due = 1; }
+      }
+    }
+#pragma unroll
+    for (int t = 0; t < G; t++) srp[gl * G + t] = e[t] & rp_keep(RS);
+  }
+  __syncwarp();
+  start = srp[lane];
+  end = srp[lane + 1];
+  __syncwarp();
+}
+
+// Cold path of an element check: correct, scrub (winner counts), or DUE.
+template <int ES>
+__device__ __noinline__ int elem_fix(uint64_t& v, uint32_t& c, uint64_t* vaddr, uint32_t* caddr, DevCounts* cnt,
+                                     int* due) {
+  uint64_t v0 = v;
+  uint32_t c0 = c;
+  int word = 0;
+  int o = (ES == SED) ? DUE : e96_correct(v, c, &word);
+  if (o == CORRECTED) {
+    bool won;
+    if (word == 2) won = scrub32(caddr, c0, c);
+    else won = scrub32(reinterpret_cast<uint32_t*>(vaddr) + word, word ? hi32(v0) : lo32(v0), word ? hi32(v) : lo32(v));
+    if (won) cnt_add(cnt, T_ELEM, ES, CORRECTED);
+  } else {
+    v = v0;
+    c = c0;
+    cnt_add(cnt, T_ELEM, ES, DUE);
+    *due = 1;
+  }
+  return o;
+}
+
+// ================================================================ SpMV (a3)
+template <int ES, int RS, int VS, bool DOT>
+__global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
+  __shared__ __align__(16) uint8_t s_lut[128];
+  __shared__ uint32_t s_rp[8][40];
+  if (VS == SECDED64) load_lut(s_lut);
+  __syncthreads();
+  if (a.state && a.state->stop) return;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  const int64_t nrb = (a.nrows + 255) >> 8;
+  if (rb >= nrb) return;
+  double dot = 0.0;
+  const uint32_t ckeep = col_keep(ES);
+  for (int k = 0; k < 8; k++) {
+    const int64_t pb = rb * 256 + k * 32;
+    if (pb >= a.nrows) break;
+    const int64_t i = pb + lane;
+    const bool valid = i < a.nrows;
+    uint32_t start, end;
+    rowptr_pass<RS>(a, pb, lane, s_rp[warp], start, end);
+    // own codeword of `in` (checked once, counted here: DESIGN.md §3.8)
+    const int64_t own = a.row_base + i;
+    const int64_t own_lim = (vgrp(VS) == 1 && !valid) ? 0 : a.npad_in;
+    const uint64_t pw_own = v_load_check<VS>(a.in, own, own_lim, lane, valid, a.counts, a.due);
+    const double p_own = as_d(pw_own & vkeep(VS));
+    double acc = 0.0;
+    if (valid) {
+      const bool ok = (start <= end) && ((int64_t)end <= a.nnz);
+      if (RS != NONE && !ok) {
+        cnt_range(a.counts, T_ROWPTR, RS);
+        *a.due = 1;
+      } else {
+        uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
+        for (uint32_t j = start; j < end; j++) {
+          uint64_t v = ldg64(a.val + j);
+          uint32_t c = __ldg(a.col + j);
+          if (ES == CRC32C) {
+            int kk = (int)(j - start);
+            crc = ecrc_update(crc, v, c, kk);
+            if (kk < 4) crc_st |= (c >> 24) << (8 * kk);
+          } else if (ES != NONE) {
+            bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
+            if (bad) elem_fix<ES>(v, c, a.val + j, a.col + j, a.counts, a.due);
+          }
+          const uint32_t cm = c & ckeep;
+          if (ES != NONE && (int64_t)cm >= a.ncols) {
+            cnt_range(a.counts, T_ELEM, ES);
+            *a.due = 1;
+            continue;
+          }
+          const int64_t idx = a.col_base + cm;
+          const double x = (idx == own) ? p_own : gather_in<VS>(a.in, idx);
+          acc = fma(as_d(v), x, acc);
+        }
+        if (ES == CRC32C) {
+          if (end - start < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
+            cnt_add(a.counts, T_ELEM, CRC32C, DUE);
+            *a.due = 1;
+          }
+        }
+      }
+    }
+    // write-buffered output (whole codewords)
+    // npad_out = local rows this chunk may write (nrows, + vector padding for the last chunk)
+    const uint64_t rounded = valid ? round_k(as_u(acc), vk(VS)) : 0ull;
+    const uint64_t enc = v_encode<VS>(rounded, lane, s_lut);
+    if (i < a.npad_out) a.out[own] = enc;
+    if (DOT && valid) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+  }
+  if (DOT) {
+#pragma unroll
+    for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
+    if (lane == 0) a.partials[a.rb_offset + rb] = dot;
+  }
+}
+
+// ====================================================== tiled stencil SpMV (a3)
+// Fast path for 5-point-stencil matrices (stencil_n = n, n % 256 == 0,
+// nrows % n == 0, G = 1 vector scheme).  A CTA owns a tile of TY grid rows x
+// 256 cells (TY reduction blocks).  It first stages the decoded `in` window —
+// the tile plus one halo row above/below and one halo cell left/right — in
+// shared memory: every codeword of the tile is checked ONCE there (owner:
+// counted + scrubbed), halo codewords are checked without counting.  This is
+// the paper's "multiple ECC element and multi-iteration aware" SpMV cache
+// in B200 form; like the paper's, the decoded copies in SMEM are
+// outside the software trust boundary.  Rows then gather their
+// neighbours from SMEM whenever col - row is one of {0, +-1, +-n}; any other
+// column (generic CSR rows, corrupted-but-in-range indices) takes the global
+// gather path, so results never depend on the stencil hint.
+constexpr int TILE_TY = 16;
+constexpr int TILE_WW = 256 + 2;
+
+template <int ES, int RS, int VS, bool DOT>
+__global__ void __launch_bounds__(256) k_spmv_tile(SpmvArgs a) {
+  extern __shared__ double s_win[];  // (TILE_TY + 2) * TILE_WW
+  __shared__ __align__(16) uint8_t s_lut[128];
+  __shared__ uint32_t s_rp[8][40];
+  if (VS == SECDED64) load_lut(s_lut);
+  const int64_t n = a.stencil_n;
+  const int64_t ny = a.nrows / n;
+  const int64_t tiles_x = n >> 8;
+  const int64_t tx0 = (blockIdx.x % tiles_x) << 8;
+  const int64_t ty0 = (int64_t)(blockIdx.x / tiles_x) * TILE_TY;
+  if (a.state && a.state->stop) return;  // uniform per block (read before any barrier use below)
+  // ---- stage the decoded window
+  const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
+  for (int sidx = threadIdx.x; sidx < (TILE_TY + 2) * TILE_WW; sidx += 256) {
+    const int wy = sidx / TILE_WW, wx = sidx - wy * TILE_WW;
+    const int64_t idx = win0 + (int64_t)wy * n + wx;
+    const int64_t gy = ty0 + wy - 1;
+    const bool owner = wy >= 1 && wy <= TILE_TY && gy < ny && wx >= 1 && wx <= 256;
+    double v = 0.0;
+    if (idx >= 0 && idx < a.npad_in) {
+      uint64_t w = ldg64(a.in + idx);
+      if (VS != NONE) w = v1_check<VS>(w, a.in + idx, owner, a.counts, a.due);
+      v = as_d(w & vkeep(VS));
+    }
+    s_win[sidx] = v;
+  }
+  __syncthreads();
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const uint32_t ckeep = col_keep(ES);
+  for (int seg = warp; seg < TILE_TY; seg += 8) {
+    const int64_t gy = ty0 + seg;
+    if (gy >= ny) break;
+    const int64_t rowseg = gy * n + tx0;        // first local row of this RB
+    double dot = 0.0;
+    for (int k = 0; k < 8; k++) {
+      const int64_t pb = rowseg + k * 32;
+      const int64_t i = pb + lane;
+      uint32_t start, end;
+      rowptr_pass<RS>(a, pb, lane, s_rp[warp], start, end);
+      const int oslot = (seg + 1) * TILE_WW + k * 32 + lane + 1;
+      const double p_own = s_win[oslot];
+      const int64_t own = a.row_base + i;
+      double acc = 0.0;
+      const bool ok = (start <= end) && ((int64_t)end <= a.nnz);
+      if (RS != NONE && !ok) {
+        cnt_range(a.counts, T_ROWPTR, RS);
+        *a.due = 1;
+      } else {
+        uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
+        const uint64_t* vp = a.val + start;
+        const uint32_t* cp = a.col + start;
+        const uint32_t len = end - start;
+        for (uint32_t j = 0; j < len; j++) {
+          uint64_t v = ldg64(vp + j);
+          uint32_t c = __ldg(cp + j);
+          if (ES == CRC32C) {
+            crc = ecrc_update(crc, v, c, (int)j);
+            if (j < 4) crc_st |= (c >> 24) << (8 * j);
+          } else if (ES != NONE) {
+            bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
+            if (bad) elem_fix<ES>(v, c, a.val + start + j, a.col + start + j, a.counts, a.due);
+          }
+          const uint32_t cm = c & ckeep;
+          if (ES != NONE && (int64_t)cm >= a.ncols) {
+            cnt_range(a.counts, T_ELEM, ES);
+            *a.due = 1;
+            continue;
+          }
+          const int64_t rel = a.col_base + (int64_t)cm - own;
+          double x;
+          if (rel == 0) x = p_own;
+          else if (rel == 1) x = s_win[oslot + 1];
+          else if (rel == -1) x = s_win[oslot - 1];
+          else if (rel == n) x = s_win[oslot + TILE_WW];
+          else if (rel == -n) x = s_win[oslot - TILE_WW];
+          else x = gather_in<VS>(a.in, own + rel);
+          acc = fma(as_d(v), x, acc);
+        }
+        if (ES == CRC32C) {
+          if (len < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
+            cnt_add(a.counts, T_ELEM, CRC32C, DUE);
+            *a.due = 1;
+          }
+        }
+      }
+      const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
+      a.out[own] = enc;
+      if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+    }
+    if (DOT) {
+#pragma unroll
+      for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
+      if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
+    }
+  }
+}
+
+// ============================================================= BLAS-1 (a4, a5, a2)
+// Full-RB fast paths (G = 1 schemes): two passes per step, so each lane has
+// 8 (calc_ur) / 4 (calc_p, init) independent 8-byte loads in flight, and all
+// addressing is pointer + immediate offset.  Lane l still visits rows
+// l, l+32, ... in ascending order (RED-1).
+template <int VS>
+__device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int lane, double alpha, const uint8_t* lut) {
+  uint64_t* X = a.x + base + lane;
+  uint64_t* P = a.p + base + lane;
+  uint64_t* R = a.r + base + lane;
+  uint64_t* W = a.w + base + lane;
+  const uint64_t keep = vkeep(VS);
+  double dot = 0.0;
+#pragma unroll 1
+  for (int k = 0; k < 256; k += 64) {
+    uint64_t x0 = ldg64(X + k), x1 = ldg64(X + k + 32), p0 = ldg64(P + k), p1 = ldg64(P + k + 32);
+    uint64_t r0 = ldg64(R + k), r1 = ldg64(R + k + 32), w0 = ldg64(W + k), w1 = ldg64(W + k + 32);
+    x0 = v1_check<VS>(x0, X + k, true, a.counts, a.due);
+    x1 = v1_check<VS>(x1, X + k + 32, true, a.counts, a.due);
+    p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
+    p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
+    r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
+    r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
+    w0 = v1_check<VS>(w0, W + k, true, a.counts, a.due);
+    w1 = v1_check<VS>(w1, W + k + 32, true, a.counts, a.due);
+    const double xn0 = fma(alpha, as_d(p0 & keep), as_d(x0 & keep));
+    const double xn1 = fma(alpha, as_d(p1 & keep), as_d(x1 & keep));
+    const double rn0 = fma(-alpha, as_d(w0 & keep), as_d(r0 & keep));
+    const double rn1 = fma(-alpha, as_d(w1 & keep), as_d(r1 & keep));
+    const uint64_t xe0 = v_encode<VS>(round_k(as_u(xn0), vk(VS)), lane, lut);
+    const uint64_t xe1 = v_encode<VS>(round_k(as_u(xn1), vk(VS)), lane, lut);
+    const uint64_t re0 = v_encode<VS>(round_k(as_u(rn0), vk(VS)), lane, lut);
+    const uint64_t re1 = v_encode<VS>(round_k(as_u(rn1), vk(VS)), lane, lut);
+    X[k] = xe0; X[k + 32] = xe1;
+    R[k] = re0; R[k + 32] = re1;
+    const double m0 = as_d(re0 & keep), m1 = as_d(re1 & keep);
+    dot = fma(m0, m0, dot);
+    dot = fma(m1, m1, dot);
+  }
+  return dot;
+}
+template <int VS>
+__device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane, double beta, const uint8_t* lut) {
+  uint64_t* P = a.p + base + lane;
+  uint64_t* R = a.r + base + lane;
+  const uint64_t keep = vkeep(VS);
+#pragma unroll 1
+  for (int k = 0; k < 256; k += 64) {
+    uint64_t r0 = ldg64(R + k), r1 = ldg64(R + k + 32), p0 = ldg64(P + k), p1 = ldg64(P + k + 32);
+    r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
+    r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
+    p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
+    p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
+    const double n0 = fma(beta, as_d(p0 & keep), as_d(r0 & keep));
+    const double n1 = fma(beta, as_d(p1 & keep), as_d(r1 & keep));
+    P[k] = v_encode<VS>(round_k(as_u(n0), vk(VS)), lane, lut);
+    P[k + 32] = v_encode<VS>(round_k(as_u(n1), vk(VS)), lane, lut);
+  }
+}
+
+
+template <int VS>
+__global__ void __launch_bounds__(256) k_calc_ur(VecArgs a) {
+  __shared__ __align__(16) uint8_t s_lut[128];
+  if (VS == SECDED64) load_lut(s_lut);
+  __syncthreads();
+  if (a.state->stop) return;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  if (rb * 256 >= a.n) return;
+  const double alpha = a.state->alpha;
+  double dot = 0.0;
+  if (vgrp(VS) == 1 && rb * 256 + 256 <= a.n) {
+    dot = ur_full<VS>(a, rb * 256, lane, alpha, s_lut);
+  } else for (int k = 0; k < 8; k++) {
+    const int64_t pb = rb * 256 + k * 32;
+    if (pb >= a.n) break;
+    const int64_t i = pb + lane;
+    const bool valid = i < a.n;
+    const int64_t lim = a.npad;
+    uint64_t xw = v_load_check<VS>(a.x, i, lim, lane, true, a.counts, a.due);
+    uint64_t pw = v_load_check<VS>(a.p, i, lim, lane, true, a.counts, a.due);
+    uint64_t rw = v_load_check<VS>(a.r, i, lim, lane, true, a.counts, a.due);
+    uint64_t ww = v_load_check<VS>(a.w, i, lim, lane, true, a.counts, a.due);
+    const uint64_t keep = vkeep(VS);
+    double X = fma(alpha, as_d(pw & keep), as_d(xw & keep));
+    double R = fma(-alpha, as_d(ww & keep), as_d(rw & keep));
+    uint64_t xe = v_encode<VS>(valid ? round_k(as_u(X), vk(VS)) : 0ull, lane, s_lut);
+    uint64_t re = v_encode<VS>(valid ? round_k(as_u(R), vk(VS)) : 0ull, lane, s_lut);
+    if (i < a.npad) { a.x[i] = xe; a.r[i] = re; }
+    if (valid) { double rm = as_d(re & keep); dot = fma(rm, rm, dot); }
+  }
+#pragma unroll
+  for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
+  if (lane == 0) a.partials[rb] = dot;
+}
+
+template <int VS>
+__global__ void __launch_bounds__(256) k_calc_p(VecArgs a) {
+  __shared__ __align__(16) uint8_t s_lut[128];
+  __shared__ bool s_last;
+  if (VS == SECDED64) load_lut(s_lut);
+  __syncthreads();
+  if (a.state->stop) return;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  const double beta = a.state->beta;
+  if (vgrp(VS) == 1 && rb * 256 + 256 <= a.n) {
+    p_full<VS>(a, rb * 256, lane, beta, s_lut);
+  } else if (rb * 256 < a.n) {
+    for (int k = 0; k < 8; k++) {
+      const int64_t pb = rb * 256 + k * 32;
+      if (pb >= a.n) break;
+      const int64_t i = pb + lane;
+      const bool valid = i < a.n;
+      const int64_t lim = a.npad;
+      uint64_t rw = v_load_check<VS>(a.r, i, lim, lane, true, a.counts, a.due);
+      uint64_t pw = v_load_check<VS>(a.p, i, lim, lane, true, a.counts, a.due);
+      const uint64_t keep = vkeep(VS);
+      double P = fma(beta, as_d(pw & keep), as_d(rw & keep));
+      uint64_t pe = v_encode<VS>(valid ? round_k(as_u(P), vk(VS)) : 0ull, lane, s_lut);
+      if (i < a.npad) a.p[i] = pe;
+    }
+  }
+  // last block finishes the iteration: DUE policy and max_iters
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    __threadfence();
+    unsigned t = atomicAdd(&a.state->ticket_p, 1u);
+    s_last = (t == gridDim.x - 1);
+  }
+  __syncthreads();
+  if (s_last && threadIdx.x == 0) {
+    __threadfence();
+    CgState* st = a.state;
+    st->ticket_p = 0;
+    volatile int* due = a.due;
+    // multi-GPU runs take the DUE decision in k_due_combine after an all-gather
+    if (!st->dist && st->abort_policy && *due) { st->stop = 1; st->status = ABFT_E_DUE; }
+    else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
+    st->rro = st->rrn;
+  }
+}
+
+// init (a2): r = enc(round(b - w)), p = r, rr0 partials
+template <int VS>
+__global__ void __launch_bounds__(256) k_init_r(VecArgs a) {
+  __shared__ __align__(16) uint8_t s_lut[128];
+  if (VS == SECDED64) load_lut(s_lut);
+  __syncthreads();
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  if (rb * 256 >= a.n) return;
+  double dot = 0.0;
+  for (int k = 0; k < 8; k++) {
+    const int64_t pb = rb * 256 + k * 32;
+    if (pb >= a.n) break;
+    const int64_t i = pb + lane;
+    const bool valid = i < a.n;
+    const int64_t lim = a.npad;
+    uint64_t bw = v_load_check<VS>(a.b, i, lim, lane, true, a.counts, a.due);
+    uint64_t ww = v_load_check<VS>(a.w, i, lim, lane, true, a.counts, a.due);
+    const uint64_t keep = vkeep(VS);
+    double R = as_d(bw & keep) - as_d(ww & keep);
+    uint64_t re = v_encode<VS>(valid ? round_k(as_u(R), vk(VS)) : 0ull, lane, s_lut);
+    if (i < a.npad) { a.r[i] = re; a.p[i] = re; }
+    if (valid) { double rm = as_d(re & keep); dot = fma(rm, rm, dot); }
+  }
+#pragma unroll
+  for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
+  if (lane == 0) a.partials[rb] = dot;
+}
+
+// ============================================================ reduction (a6)
+// Complete binary tree over the RB partials padded to a power of two: each
+// block reduces an aligned subtree of <= 1024 leaves in shared memory, the
+// last block (ticket) reduces the block roots and applies the CG scalar logic.
+static __device__ __forceinline__ double tree_smem(double* s, int m) {
+  // s[0..m) -> pairwise levels; m power of two; blockDim >= m/2
+  for (; m > 1; m >>= 1) {
+    double v = 0.0;
+    const int t = threadIdx.x;
+    if (t < m / 2) v = s[2 * t] + s[2 * t + 1];
+    __syncthreads();
+    if (t < m / 2) s[t] = v;
+    __syncthreads();
+  }
+  return s[0];
+}
+
+// CG scalar logic applied by exactly one thread.
+static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
+  if (op == 1) {  // rr0
+    st->rr0 = st->rro = st->rrn = res;
+    if (st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; }
+    else if (res == 0.0) { st->stop = 1; st->status = ABFT_OK; st->converged = 1; }
+    else if (st->max_iters <= 0) { st->stop = 1; st->status = ABFT_OK; }
+  } else if (op == 2) {  // pw -> alpha
+    st->pw = res;
+    st->alpha = st->rro / res;
+    st->iters += 1;
+  } else if (op == 3) {  // rrn -> convergence, beta
+    st->rrn = res;
+    if (sqrt(res) <= st->tol * sqrt(st->rr0)) {
+      st->stop = 1;
+      st->converged = 1;
+      st->status = (st->abort_policy && dueflag) ? ABFT_E_DUE : ABFT_OK;
+    } else {
+      st->beta = res / st->rro;
+    }
+  }
+}
+
+static __global__ void __launch_bounds__(512) k_reduce(const double* partials, int64_t nrb, int64_t leaves, double* roots,
+                                                uint32_t* ticket, int op, CgState* st, double* out, const int* due) {
+  __shared__ double s[1024];
+  __shared__ bool s_last;
+  if (st && op != 1 && st->stop) return;
+  const int64_t base = (int64_t)blockIdx.x * leaves;
+  for (int64_t t = threadIdx.x; t < leaves; t += blockDim.x) s[t] = (base + t < nrb) ? partials[base + t] : 0.0;
+  __syncthreads();
+  double root = tree_smem(s, (int)leaves);
+  if (gridDim.x == 1) {
+    s_last = true;
+  } else {
+    if (threadIdx.x == 0) {
+      roots[blockIdx.x] = root;
+      __threadfence();
+      s_last = (atomicAdd(ticket, 1u) == gridDim.x - 1);
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    const int nb = gridDim.x;
+    for (int t = threadIdx.x; t < nb; t += blockDim.x) s[t] = ((volatile double*)roots)[t];
+    __syncthreads();
+    root = tree_smem(s, nb);
+  }
+  if (threadIdx.x != 0) return;
+  if (gridDim.x > 1) *ticket = 0;
+  if (op == 0) { *out = root; return; }
+  if (op == 4) { out[0] = root; out[1] = (double)(*((volatile const int*)due)); return; }
+  apply_op(op, root, st, *((volatile const int*)due) != 0);
+}
+
+// Multi-GPU: combine the all-gathered (root, due) pairs of P ranks with the top
+// of the RED-1 tree (identical on every rank) and apply the CG scalar logic.
+static __global__ void k_combine(const double* gathered, int P, int op, CgState* st, int* due) {
+  __shared__ double s[1024];
+  if (op != 1 && st->stop) return;
+  int m = 1;
+  while (m < P) m <<= 1;
+  for (int t = threadIdx.x; t < m; t += blockDim.x) s[t] = (t < P) ? gathered[2 * t] : 0.0;
+  __syncthreads();
+  double root = tree_smem(s, m);
+  if (threadIdx.x != 0) return;
+  int any = 0;
+  for (int t = 0; t < P; t++) any |= gathered[2 * t + 1] != 0.0;
+  if (any) *due = 1;
+  apply_op(op, root, st, any != 0);
+}
+// Multi-GPU abort check after calc_p (policy abort only): gathered due flags.
+static __global__ void k_due_combine(const double* gathered, int P, CgState* st, int* due) {
+  int any = 0;
+  for (int t = 0; t < P; t++) any |= gathered[2 * t + 1] != 0.0;
+  if (any) *due = 1;
+  if (st->stop && st->status != ABFT_E_NOT_CONVERGED) return;
+  if (st->abort_policy && any) { st->stop = 1; st->status = ABFT_E_DUE; }
+}
+static __global__ void k_pack_due(double* out, const int* due) { out[1] = (double)(*((volatile const int*)due)); out[0] = 0.0; }
+
+// ========================================================== vector encode / check
+template <int VS>
+__global__ void k_vec_encode(uint64_t* d, int64_t n, int64_t npad) {
+  constexpr int G = vgrp(VS);
+  const int64_t ng = npad / G;
+  for (int64_t g = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; g < ng; g += (int64_t)gridDim.x * blockDim.x) {
+    uint64_t v[G];
+#pragma unroll
+    for (int t = 0; t < G; t++) {
+      int64_t i = g * G + t;
+      v[t] = (i < n) ? round_k(d[i], vk(VS)) : 0ull;
+    }
+#if 1
+    if (VS == SECDED64) v[0] = v64_encode_lut(v[0], c_v64_lut.r);
+    else vec_encode_group<VS>(v, nullptr);
+#endif
+#pragma unroll
+    for (int t = 0; t < G; t++) d[g * G + t] = v[t];
+  }
+}
+
+template <int VS>
+__global__ void k_vec_check(uint64_t* d, int64_t n, int64_t npad, double* out, DevCounts* cnt, int* due, int scrub) {
+  constexpr int G = vgrp(VS);
+  const int64_t ng = npad / G;
+  for (int64_t g = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; g < ng; g += (int64_t)gridDim.x * blockDim.x) {
+    uint64_t v[G], o0[G];
+#pragma unroll
+    for (int t = 0; t < G; t++) o0[t] = v[t] = d[g * G + t];
+    int word = 0;
+    int o = vec_check_group<VS>(v, &word);
+    if (o == CORRECTED) {
+      bool won = true;
+      if (scrub) {
+        uint64_t ow = o0[word >> 1], nw = v[word >> 1];
+        won = scrub32(reinterpret_cast<uint32_t*>(d + g * G) + word, (word & 1) ? hi32(ow) : lo32(ow),
+                      (word & 1) ? hi32(nw) : lo32(nw));
+      }
+      if (won) cnt_add(cnt, T_VEC, VS, CORRECTED);
+    } else if (o == DUE) {
+#pragma unroll
+      for (int t = 0; t < G; t++) v[t] = o0[t];
+      cnt_add(cnt, T_VEC, VS, DUE);
+      *due = 1;
+    }
+    if (out) {
+#pragma unroll
+      for (int t = 0; t < G; t++) if (g * G + t < n) out[g * G + t] = as_d(v[t] & vkeep(VS));
+    }
+  }
+}
+
+// ============================================================ CSR encode (a0)
+// flags[0] |= 1: col beyond capacity, |= 2: rowptr beyond capacity, |= 4: CRC row < 4 entries
+template <int ES>
+__global__ void k_encode_elems(const uint64_t* val, uint32_t* col, int64_t nnz, int64_t ncols, uint32_t* flags) {
+  for (int64_t e = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; e < nnz; e += (int64_t)gridDim.x * blockDim.x) {
+    uint32_t c = col[e];
+    if ((uint64_t)c > col_limit(ES) || (int64_t)c >= ncols) { atomicOr(flags, 1u); continue; }
+    if (ES == SED) col[e] = esed_encode_col(val[e], c);
+    else if (ES == SECDED64 || ES == SECDED128) col[e] = e96_encode_col(val[e], c);
+  }
+}
+static __global__ void k_encode_ecrc(const uint64_t* val, uint32_t* col, const uint32_t* rowptr, int64_t nrows, uint32_t* flags) {
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < nrows; i += (int64_t)gridDim.x * blockDim.x) {
+    uint32_t s = rowptr[i], t = rowptr[i + 1];
+    if (t < s + 4) { atomicOr(flags, 4u); continue; }
+    uint32_t crc = 0xFFFFFFFFu;
+    for (uint32_t j = s; j < t; j++) {
+      uint32_t c = col[j];
+      if (j < s + 4) c &= 0x00FFFFFFu;
+      crc = ecrc_update(crc, val[j], c, (int)(j - s));
+    }
+    crc ^= 0xFFFFFFFFu;
+    for (int k = 0; k < 4; k++) col[s + k] = (col[s + k] & 0x00FFFFFFu) | (((crc >> (8 * k)) & 0xFFu) << 24);
+  }
+}
+template <int RS>
+__global__ void k_encode_rowptr(uint32_t* rowptr, int64_t nrows, int64_t nnz, int64_t len, uint32_t* flags) {
+  constexpr int G = rgrp(RS);
+  for (int64_t g = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; g < len / G; g += (int64_t)gridDim.x * blockDim.x) {
+    uint32_t e[G];
+    for (int t = 0; t < G; t++) {
+      int64_t i = g * G + t;
+      e[t] = (i <= nrows) ? rowptr[i] : (uint32_t)nnz;
+      if ((uint64_t)e[t] > rp_limit(RS)) atomicOr(flags, 2u);
+    }
+    if (RS != NONE) rp_encode_group<RS>(e);
+    for (int t = 0; t < G; t++) rowptr[g * G + t] = e[t];
+  }
+}
+
+// ============================================================ check_all (a7)
+template <int ES>
+__global__ void k_check_elems(uint64_t* val, uint32_t* col, int64_t nnz, int64_t ncols, DevCounts* cnt, int* due,
+                              int scrub) {
+  for (int64_t e = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; e < nnz; e += (int64_t)gridDim.x * blockDim.x) {
+    uint64_t v = val[e], v0 = v;
+    uint32_t c = col[e], c0 = c;
+    int word = 0;
+    int o = CLEAN;
+    if (ES == SED) o = esed_clean(v, c) ? CLEAN : DUE;
+    else if (e96_bad(lo32(v), hi32(v), c)) o = e96_correct(v, c, &word);
+    if (o == CORRECTED) {
+      bool won = true;
+      if (scrub) won = (word == 2) ? scrub32(col + e, c0, c)
+                                   : scrub32(reinterpret_cast<uint32_t*>(val + e) + word, word ? hi32(v0) : lo32(v0),
+                                             word ? hi32(v) : lo32(v));
+      if (won) cnt_add(cnt, T_ELEM, ES, CORRECTED);
+    } else if (o == DUE) {
+      c = c0;
+      cnt_add(cnt, T_ELEM, ES, DUE);
+      *due = 1;
+    }
+    if ((int64_t)(c & col_keep(ES)) >= ncols) { cnt_range(cnt, T_ELEM, ES); *due = 1; }
+  }
+}
+template <int RS>
+__global__ void k_check_rowptr(uint32_t* rowptr, int64_t len, DevCounts* cnt, int* due, int scrub) {
+  constexpr int G = rgrp(RS);
+  for (int64_t g = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; g < len / G; g += (int64_t)gridDim.x * blockDim.x) {
+    uint32_t e[G], o0[G];
+    for (int t = 0; t < G; t++) o0[t] = e[t] = rowptr[g * G + t];
+    int word = 0;
+    int o = rp_check_group<RS>(e, &word);
+    if (o == CORRECTED) {
+      bool won = scrub ? scrub32(rowptr + g * G + word, o0[word], e[word]) : true;
+      if (won) cnt_add(cnt, T_ROWPTR, RS, CORRECTED);
+    } else if (o == DUE) {
+      cnt_add(cnt, T_ROWPTR, RS, DUE);
+      *due = 1;
+    }
+  }
+}
+// Row pass of check_all: range check + E-CRC rows (after the rowptr pass scrubbed).
+template <int ES, int RS>
+__global__ void k_check_rows(const uint64_t* val, const uint32_t* col, const uint32_t* rowptr, int64_t nrows,
+                             int64_t nnz, DevCounts* cnt, int* due) {
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < nrows; i += (int64_t)gridDim.x * blockDim.x) {
+    uint32_t s = rowptr[i] & rp_keep(RS), t = rowptr[i + 1] & rp_keep(RS);
+    if (!(s <= t && (int64_t)t <= nnz)) {
+      if (RS != NONE) { cnt_range(cnt, T_ROWPTR, RS); *due = 1; }
+      continue;
+    }
+    if (ES == CRC32C) {
+      bool bad = (t - s < 4);
+      if (!bad) {
+        uint32_t crc = 0xFFFFFFFFu, st = 0;
+        for (uint32_t j = s; j < t; j++) {
+          uint32_t c = col[j];
+          if (j - s < 4) st |= (c >> 24) << (8 * (j - s));
+          crc = ecrc_update(crc, val[j], c, (int)(j - s));
+        }
+        bad = (crc ^ 0xFFFFFFFFu) != st;
+      }
+      if (bad) { cnt_add(cnt, T_ELEM, CRC32C, DUE); *due = 1; }
+    }
+  }
+}
+
+static __global__ void k_inject(uint32_t* base, uint64_t bit) { atomicXor(base + (bit >> 5), 1u << (bit & 31)); }
+
+
+}  // namespace abft

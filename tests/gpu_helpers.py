@@ -17,10 +17,10 @@ def tea(n: int, kind: str = "tea"):
     return v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32)
 
 
-def gpu_matrix(abft, ctx, v, c, r, nrows, ncols, es, rs, row_base=0, col_base=0):
+def gpu_matrix(abft, ctx, v, c, r, nrows, ncols, es, rs, row_base=0, col_base=0, stencil_n=0):
     A = abft.Matrix(torch.from_numpy(v).cuda(), torch.from_numpy(c.view(np.int32)).cuda(),
                     torch.from_numpy(r.view(np.int32)).cuda(), nrows, ncols, es, rs, row_base=row_base,
-                    col_base=col_base)
+                    col_base=col_base, stencil_n=stencil_n)
     st = A.encode(ctx)
     return A, st
 
