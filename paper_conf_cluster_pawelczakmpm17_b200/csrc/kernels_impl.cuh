@@ -324,39 +324,206 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
 
 // ====================================================== tiled stencil SpMV (a3)
 // Fast path for 5-point-stencil matrices (stencil_n = n, n % 256 == 0,
-// nrows % n == 0, G = 1 vector scheme).  A CTA owns a tile of TY grid rows x
-// 256 cells (TY reduction blocks).  It first stages the decoded `in` window —
-// the tile plus one halo row above/below and one halo cell left/right — in
-// shared memory: every codeword of the tile is checked ONCE there (owner:
-// counted + scrubbed), halo codewords are checked without counting.  This is
-// the paper's "multiple ECC element and multi-iteration aware" SpMV cache
-// in B200 form; like the paper's, the decoded copies in SMEM are
-// outside the software trust boundary.  Rows then gather their
-// neighbours from SMEM whenever col - row is one of {0, +-1, +-n}; any other
-// column (generic CSR rows, corrupted-but-in-range indices) takes the global
-// gather path, so results never depend on the stencil hint.
-constexpr int TILE_TY = 16;
+// nrows % n == 0, G = 1 vector scheme).  A CTA owns a tile of TILE_TY grid
+// rows x 256 cells; warp w owns grid row w of the tile = one reduction block.
+//  1. each warp decodes its segment's 257 rowptr entries into SMEM (one check
+//     per group; owner counts) and, from them, issues TMA bulk copies
+//     (cp.async.bulk + mbarrier) of the (val, col) streams of its first two
+//     32-row passes into a double buffer — the packed element stream is
+//     contiguous per pass, so it arrives fully coalesced and without
+//     occupying registers or LSU slots;
+//  2. the CTA stages the decoded `in` window (tile + one halo row above/below
+//     + one halo cell left/right) in SMEM: every codeword of the tile is
+//     checked ONCE here (owner: counted + scrubbed), halo codewords are
+//     checked without counting.  This is the paper's "multiple ECC element and
+//     multi-iteration aware" SpMV cache in B200 form; like the
+//     paper's caches, the decoded copies in SMEM are outside the software trust
+//     boundary;
+//  3. per pass each lane checks/corrects its row's elements from SMEM, gathers
+//     neighbours from the window whenever col-row is one of {0, +-1, +-n}
+//     (anything else takes the global gather path, so results never depend on
+//     the stencil hint), encodes w, and the warp refills the buffer with pass
+//     k+2.  A pass whose element range does not fit the buffer (non-stencil
+//     rows, corrupted rowptr) reads its elements from global memory instead.
+constexpr int TILE_TY = 8;
 constexpr int TILE_WW = 256 + 2;
+constexpr int TILE_EBUF = 168;                                  // elements per pass buffer (>= 160 + align)
+constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;     // 20640
+constexpr int TILE_BUF_BYTES = TILE_EBUF * 12;                  // val 8 B + col 4 B per element
+constexpr int TILE_RP = 264;                                    // rowptr entries staged per warp
+constexpr int TILE_SMEM = TILE_WIN_BYTES + TILE_TY * (2 * TILE_BUF_BYTES + TILE_RP * 4 + 16);
+
+static __device__ __forceinline__ uint32_t smem_u32(const void* p) { return (uint32_t)__cvta_generic_to_shared(p); }
+static __device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count) : "memory");
+}
+static __device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes) : "memory");
+}
+static __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                   smem_u32(dst)),
+               "l"(src), "r"(bytes), "r"(smem_u32(bar))
+               : "memory");
+}
+static __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
+  asm volatile(
+      "{\n .reg .pred P1;\n WAIT_%=:\n mbarrier.try_wait.parity.shared::cta.b64 P1, [%0], %1;\n @!P1 bra WAIT_%=;\n}\n" ::"r"(
+          smem_u32(bar)),
+      "r"(parity)
+      : "memory");
+}
+
+// Issue the bulk copies of one pass's element range [s0, s1) into buffer buf.
+// Returns the aligned starts (e0 for val, c0 for col) or -1 if not staged.
+static __device__ __forceinline__ bool tile_issue(const SpmvArgs& a, uint32_t s0, uint32_t s1, uint8_t* buf,
+                                                  uint64_t* bar, int lane) {
+  if (!(s0 <= s1 && (int64_t)s1 <= a.nnz && s1 - s0 <= 160u)) return false;
+  if (lane == 0) {
+    const uint32_t e0 = s0 & ~1u, e1 = (s1 + 1u) & ~1u;
+    const uint32_t c0 = s0 & ~3u, c1 = (s1 + 3u) & ~3u;
+    const uint32_t vb = (e1 - e0) * 8u, cb = (c1 - c0) * 4u;
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+    mbar_expect_tx(bar, vb + cb);
+    if (vb) bulk_g2s(buf, a.val + e0, vb, bar);
+    if (cb) bulk_g2s(buf + TILE_EBUF * 8, a.col + c0, cb, bar);
+  }
+  return true;
+}
+
+// One row: check/correct its elements (from SMEM or global), gather, fma chain.
+template <int ES, int RS, int VS>
+static __device__ __forceinline__ double tile_row(const SpmvArgs& a, uint32_t start, uint32_t end, const uint64_t* sval,
+                                                 const uint32_t* scol, uint32_t sbase_v, uint32_t sbase_c, bool staged,
+                                                 const double* win, int oslot, double p_own, int64_t own) {
+  double acc = 0.0;
+  const bool ok = (start <= end) && ((int64_t)end <= a.nnz);
+  if (RS != NONE && !ok) {
+    cnt_range(a.counts, T_ROWPTR, RS);
+    *a.due = 1;
+    return 0.0;
+  }
+  const uint32_t ckeep = col_keep(ES);
+  const int64_t n = a.stencil_n;
+  uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
+  const uint32_t len = end - start;
+  for (uint32_t j = 0; j < len; j++) {
+    uint64_t v;
+    uint32_t c;
+    if (staged) {
+      v = sval[start + j - sbase_v];
+      c = scol[start + j - sbase_c];
+    } else {
+      v = ldg64(a.val + start + j);
+      c = __ldg(a.col + start + j);
+    }
+    if (ES == CRC32C) {
+      crc = ecrc_update(crc, v, c, (int)j);
+      if (j < 4) crc_st |= (c >> 24) << (8 * j);
+    } else if (ES != NONE) {
+      bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
+      if (bad) elem_fix<ES>(v, c, a.val + start + j, a.col + start + j, a.counts, a.due);
+    }
+    const uint32_t cm = c & ckeep;
+    if (ES != NONE && (int64_t)cm >= a.ncols) {
+      cnt_range(a.counts, T_ELEM, ES);
+      *a.due = 1;
+      continue;
+    }
+    const int64_t rel = a.col_base + (int64_t)cm - own;
+    double x;
+    if (rel == 0) x = p_own;
+    else if (rel == 1) x = win[oslot + 1];
+    else if (rel == -1) x = win[oslot - 1];
+    else if (rel == n) x = win[oslot + TILE_WW];
+    else if (rel == -n) x = win[oslot - TILE_WW];
+    else x = gather_in<VS>(a.in, own + rel);
+    acc = fma(as_d(v), x, acc);
+  }
+  if (ES == CRC32C) {
+    if (len < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
+      cnt_add(a.counts, T_ELEM, CRC32C, DUE);
+      *a.due = 1;
+    }
+  }
+  return acc;
+}
 
 template <int ES, int RS, int VS, bool DOT>
 __global__ void __launch_bounds__(256) k_spmv_tile(SpmvArgs a) {
-  extern __shared__ double s_win[];  // (TILE_TY + 2) * TILE_WW
+  extern __shared__ __align__(128) uint8_t s_dyn[];
   __shared__ __align__(16) uint8_t s_lut[128];
-  __shared__ uint32_t s_rp[8][40];
+  double* s_win = reinterpret_cast<double*>(s_dyn);
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  uint8_t* wbase = s_dyn + TILE_WIN_BYTES + warp * (2 * TILE_BUF_BYTES + TILE_RP * 4 + 16);
+  uint8_t* buf[2] = {wbase, wbase + TILE_BUF_BYTES};
+  uint32_t* srp = reinterpret_cast<uint32_t*>(wbase + 2 * TILE_BUF_BYTES);
+  uint64_t* bars = reinterpret_cast<uint64_t*>(wbase + 2 * TILE_BUF_BYTES + TILE_RP * 4);
   if (VS == SECDED64) load_lut(s_lut);
+  if (lane == 0) {
+    mbar_init(&bars[0], 1);
+    mbar_init(&bars[1], 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncwarp();
+  if (a.state && a.state->stop) return;  // uniform per grid
   const int64_t n = a.stencil_n;
   const int64_t ny = a.nrows / n;
   const int64_t tiles_x = n >> 8;
   const int64_t tx0 = (blockIdx.x % tiles_x) << 8;
   const int64_t ty0 = (int64_t)(blockIdx.x / tiles_x) * TILE_TY;
-  if (a.state && a.state->stop) return;  // uniform per block (read before any barrier use below)
-  // ---- stage the decoded window
+  const int64_t gy = ty0 + warp;
+  const bool has_seg = gy < ny;
+  const int64_t rowseg = gy * n + tx0;
+  // ---- 1. rowptr of the segment (entries rowseg .. rowseg+256), then the first two element copies
+  bool staged[2] = {false, false};
+  if (has_seg) {
+    constexpr int G = rgrp(RS);
+    constexpr int NG = 256 / G + 1;
+    for (int gl = lane; gl < NG; gl += 32) {
+      const int64_t g = rowseg / G + gl;
+      uint32_t e[G];
+      uint32_t* gp = a.rowptr + g * G;
+      if (G == 1) e[0] = __ldg(gp);
+      else if (G == 2) { uint2 u = __ldg(reinterpret_cast<const uint2*>(gp)); e[0] = u.x; e[1 % G] = u.y; }
+      else {
+#pragma unroll
+        for (int q = 0; q < G; q += 4) {
+          uint4 u = __ldg(reinterpret_cast<const uint4*>(gp + q));
+          e[q] = u.x; e[(q + 1) % G] = u.y; e[(q + 2) % G] = u.z; e[(q + 3) % G] = u.w;
+        }
+      }
+      if (RS != NONE) {
+        uint32_t o0[G];
+#pragma unroll
+        for (int t = 0; t < G; t++) o0[t] = e[t];
+        int word = 0;
+        int o = rp_check_group<RS>(e, &word);
+        if (o != CLEAN) {
+          const int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
+          const bool owner = own >= rowseg && own < rowseg + 256;
+          if (o == CORRECTED) {
+            if (owner && scrub32(gp + word, o0[word], e[word])) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
+          } else {
+#pragma unroll
+            for (int t = 0; t < G; t++) e[t] = o0[t];
+            if (owner) { cnt_add(a.counts, T_ROWPTR, RS, DUE); *a.due = 1; }
+          }
+        }
+      }
+#pragma unroll
+      for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[t] & rp_keep(RS);
+    }
+    __syncwarp();
+    staged[0] = tile_issue(a, srp[0], srp[32], buf[0], &bars[0], lane);
+    staged[1] = tile_issue(a, srp[32], srp[64], buf[1], &bars[1], lane);
+  }
+  // ---- 2. decoded `in` window
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
   for (int sidx = threadIdx.x; sidx < (TILE_TY + 2) * TILE_WW; sidx += 256) {
     const int wy = sidx / TILE_WW, wx = sidx - wy * TILE_WW;
     const int64_t idx = win0 + (int64_t)wy * n + wx;
-    const int64_t gy = ty0 + wy - 1;
-    const bool owner = wy >= 1 && wy <= TILE_TY && gy < ny && wx >= 1 && wx <= 256;
+    const bool owner = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny && wx >= 1 && wx <= 256;
     double v = 0.0;
     if (idx >= 0 && idx < a.npad_in) {
       uint64_t w = ldg64(a.in + idx);
@@ -366,73 +533,36 @@ __global__ void __launch_bounds__(256) k_spmv_tile(SpmvArgs a) {
     s_win[sidx] = v;
   }
   __syncthreads();
-  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  const uint32_t ckeep = col_keep(ES);
-  for (int seg = warp; seg < TILE_TY; seg += 8) {
-    const int64_t gy = ty0 + seg;
-    if (gy >= ny) break;
-    const int64_t rowseg = gy * n + tx0;        // first local row of this RB
-    double dot = 0.0;
-    for (int k = 0; k < 8; k++) {
-      const int64_t pb = rowseg + k * 32;
-      const int64_t i = pb + lane;
-      uint32_t start, end;
-      rowptr_pass<RS>(a, pb, lane, s_rp[warp], start, end);
-      const int oslot = (seg + 1) * TILE_WW + k * 32 + lane + 1;
-      const double p_own = s_win[oslot];
-      const int64_t own = a.row_base + i;
-      double acc = 0.0;
-      const bool ok = (start <= end) && ((int64_t)end <= a.nnz);
-      if (RS != NONE && !ok) {
-        cnt_range(a.counts, T_ROWPTR, RS);
-        *a.due = 1;
-      } else {
-        uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
-        const uint64_t* vp = a.val + start;
-        const uint32_t* cp = a.col + start;
-        const uint32_t len = end - start;
-        for (uint32_t j = 0; j < len; j++) {
-          uint64_t v = ldg64(vp + j);
-          uint32_t c = __ldg(cp + j);
-          if (ES == CRC32C) {
-            crc = ecrc_update(crc, v, c, (int)j);
-            if (j < 4) crc_st |= (c >> 24) << (8 * j);
-          } else if (ES != NONE) {
-            bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
-            if (bad) elem_fix<ES>(v, c, a.val + start + j, a.col + start + j, a.counts, a.due);
-          }
-          const uint32_t cm = c & ckeep;
-          if (ES != NONE && (int64_t)cm >= a.ncols) {
-            cnt_range(a.counts, T_ELEM, ES);
-            *a.due = 1;
-            continue;
-          }
-          const int64_t rel = a.col_base + (int64_t)cm - own;
-          double x;
-          if (rel == 0) x = p_own;
-          else if (rel == 1) x = s_win[oslot + 1];
-          else if (rel == -1) x = s_win[oslot - 1];
-          else if (rel == n) x = s_win[oslot + TILE_WW];
-          else if (rel == -n) x = s_win[oslot - TILE_WW];
-          else x = gather_in<VS>(a.in, own + rel);
-          acc = fma(as_d(v), x, acc);
-        }
-        if (ES == CRC32C) {
-          if (len < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
-            cnt_add(a.counts, T_ELEM, CRC32C, DUE);
-            *a.due = 1;
-          }
-        }
-      }
-      const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
-      a.out[own] = enc;
-      if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
-    }
-    if (DOT) {
+  if (!has_seg) return;
+  // ---- 3. passes
+  double dot = 0.0;
+  uint32_t phase[2] = {0u, 0u};  // completed-phase parity expected next, per buffer
 #pragma unroll
-      for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-      if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
+  for (int k = 0; k < 8; k++) {
+    const int b = k & 1;
+    const uint32_t s0 = srp[32 * k];
+    const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
+    const bool st = staged[b];
+    if (st) {
+      mbar_wait(&bars[b], phase[b]);
+      phase[b] ^= 1u;
     }
+    const uint64_t* sval = reinterpret_cast<const uint64_t*>(buf[b]);
+    const uint32_t* scol = reinterpret_cast<const uint32_t*>(buf[b] + TILE_EBUF * 8);
+    const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
+    const double p_own = s_win[oslot];
+    const int64_t own = a.row_base + rowseg + k * 32 + lane;
+    const double acc = tile_row<ES, RS, VS>(a, start, end, sval, scol, s0 & ~1u, s0 & ~3u, st, s_win, oslot, p_own, own);
+    const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
+    a.out[own] = enc;
+    if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+    __syncwarp();
+    if (k + 2 < 8) staged[b] = tile_issue(a, srp[32 * (k + 2)], srp[32 * (k + 3)], buf[b], &bars[b], lane);
+  }
+  if (DOT) {
+#pragma unroll
+    for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
+    if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
   }
 }
 
