@@ -450,13 +450,12 @@ static __device__ __forceinline__ double tile_row(const SpmvArgs& a, uint32_t st
 }
 
 template <int ES, int RS, int VS, bool DOT>
-__global__ void __launch_bounds__(256) k_spmv_tile(SpmvArgs a) {
+__global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
   extern __shared__ __align__(128) uint8_t s_dyn[];
   __shared__ __align__(16) uint8_t s_lut[128];
   double* s_win = reinterpret_cast<double*>(s_dyn);
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   uint8_t* wbase = s_dyn + TILE_WIN_BYTES + warp * (2 * TILE_BUF_BYTES + TILE_RP * 4 + 16);
-  uint8_t* buf[2] = {wbase, wbase + TILE_BUF_BYTES};
   uint32_t* srp = reinterpret_cast<uint32_t*>(wbase + 2 * TILE_BUF_BYTES);
   uint64_t* bars = reinterpret_cast<uint64_t*>(wbase + 2 * TILE_BUF_BYTES + TILE_RP * 4);
   if (VS == SECDED64) load_lut(s_lut);
@@ -476,79 +475,100 @@ __global__ void __launch_bounds__(256) k_spmv_tile(SpmvArgs a) {
   const bool has_seg = gy < ny;
   const int64_t rowseg = gy * n + tx0;
   // ---- 1. rowptr of the segment (entries rowseg .. rowseg+256), then the first two element copies
-  bool staged[2] = {false, false};
+  uint32_t stmask = 0u;  // bit b: buffer b holds the current pass (TMA issued)
   if (has_seg) {
     constexpr int G = rgrp(RS);
     constexpr int NG = 256 / G + 1;
-    for (int gl = lane; gl < NG; gl += 32) {
-      const int64_t g = rowseg / G + gl;
-      uint32_t e[G];
-      uint32_t* gp = a.rowptr + g * G;
-      if (G == 1) e[0] = __ldg(gp);
-      else if (G == 2) { uint2 u = __ldg(reinterpret_cast<const uint2*>(gp)); e[0] = u.x; e[1 % G] = u.y; }
-      else {
+    constexpr int PER = (NG + 31) / 32;
+    uint32_t e[PER][G];
 #pragma unroll
-        for (int q = 0; q < G; q += 4) {
-          uint4 u = __ldg(reinterpret_cast<const uint4*>(gp + q));
-          e[q] = u.x; e[(q + 1) % G] = u.y; e[(q + 2) % G] = u.z; e[(q + 3) % G] = u.w;
+    for (int q = 0; q < PER; q++) {  // all loads first (latency overlapped)
+      const int gl = lane + 32 * q;
+      const uint32_t* gp = a.rowptr + (rowseg / G + gl) * G;
+      if (gl < NG) {
+        if (G == 1) e[q][0] = __ldg(gp);
+        else if (G == 2) { uint2 u = __ldg(reinterpret_cast<const uint2*>(gp)); e[q][0] = u.x; e[q][1 % G] = u.y; }
+        else {
+#pragma unroll
+          for (int t = 0; t < G; t += 4) {
+            uint4 u = __ldg(reinterpret_cast<const uint4*>(gp + t));
+            e[q][t] = u.x; e[q][(t + 1) % G] = u.y; e[q][(t + 2) % G] = u.z; e[q][(t + 3) % G] = u.w;
+          }
         }
       }
+    }
+#pragma unroll
+    for (int q = 0; q < PER; q++) {
+      const int gl = lane + 32 * q;
+      if (gl >= NG) continue;
+      const int64_t g = rowseg / G + gl;
+      uint32_t* gp = a.rowptr + g * G;
       if (RS != NONE) {
         uint32_t o0[G];
 #pragma unroll
-        for (int t = 0; t < G; t++) o0[t] = e[t];
+        for (int t = 0; t < G; t++) o0[t] = e[q][t];
         int word = 0;
-        int o = rp_check_group<RS>(e, &word);
+        int o = rp_check_group<RS>(e[q], &word);
         if (o != CLEAN) {
           const int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
           const bool owner = own >= rowseg && own < rowseg + 256;
           if (o == CORRECTED) {
-            if (owner && scrub32(gp + word, o0[word], e[word])) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
+            if (owner && scrub32(gp + word, o0[word], e[q][word])) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
           } else {
 #pragma unroll
-            for (int t = 0; t < G; t++) e[t] = o0[t];
+            for (int t = 0; t < G; t++) e[q][t] = o0[t];
             if (owner) { cnt_add(a.counts, T_ROWPTR, RS, DUE); *a.due = 1; }
           }
         }
       }
 #pragma unroll
-      for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[t] & rp_keep(RS);
+      for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[q][t] & rp_keep(RS);
     }
     __syncwarp();
-    staged[0] = tile_issue(a, srp[0], srp[32], buf[0], &bars[0], lane);
-    staged[1] = tile_issue(a, srp[32], srp[64], buf[1], &bars[1], lane);
+    stmask |= tile_issue(a, srp[0], srp[32], wbase, &bars[0], lane) ? 1u : 0u;
+    stmask |= tile_issue(a, srp[32], srp[64], wbase + TILE_BUF_BYTES, &bars[1], lane) ? 2u : 0u;
   }
   // ---- 2. decoded `in` window
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
-  for (int sidx = threadIdx.x; sidx < (TILE_TY + 2) * TILE_WW; sidx += 256) {
+  constexpr int NSLOT = (TILE_TY + 2) * TILE_WW;
+  constexpr int PER_T = (NSLOT + 255) / 256;
+  uint64_t wv[PER_T];
+#pragma unroll
+  for (int q = 0; q < PER_T; q++) {  // all loads first (latency overlapped)
+    const int sidx = threadIdx.x + 256 * q;
+    const int wy = sidx / TILE_WW, wx = sidx - wy * TILE_WW;
+    const int64_t idx = win0 + (int64_t)wy * n + wx;
+    wv[q] = (sidx < NSLOT && idx >= 0 && idx < a.npad_in) ? ldg64(a.in + idx) : 0ull;
+  }
+#pragma unroll
+  for (int q = 0; q < PER_T; q++) {
+    const int sidx = threadIdx.x + 256 * q;
+    if (sidx >= NSLOT) continue;
     const int wy = sidx / TILE_WW, wx = sidx - wy * TILE_WW;
     const int64_t idx = win0 + (int64_t)wy * n + wx;
     const bool owner = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny && wx >= 1 && wx <= 256;
-    double v = 0.0;
-    if (idx >= 0 && idx < a.npad_in) {
-      uint64_t w = ldg64(a.in + idx);
-      if (VS != NONE) w = v1_check<VS>(w, a.in + idx, owner, a.counts, a.due);
-      v = as_d(w & vkeep(VS));
-    }
-    s_win[sidx] = v;
+    uint64_t w = wv[q];
+    if (VS != NONE && idx >= 0 && idx < a.npad_in) w = v1_check<VS>(w, a.in + idx, owner, a.counts, a.due);
+    s_win[sidx] = as_d(w & vkeep(VS));
   }
   __syncthreads();
   if (!has_seg) return;
   // ---- 3. passes
   double dot = 0.0;
-  uint32_t phase[2] = {0u, 0u};  // completed-phase parity expected next, per buffer
-#pragma unroll
+  uint32_t phmask = 0u;  // bit b: completed-phase parity expected next for buffer b
+#pragma unroll 1
   for (int k = 0; k < 8; k++) {
     const int b = k & 1;
     const uint32_t s0 = srp[32 * k];
     const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
-    const bool st = staged[b];
+    const bool st = (stmask >> b) & 1u;
     if (st) {
-      mbar_wait(&bars[b], phase[b]);
-      phase[b] ^= 1u;
+      mbar_wait(&bars[b], (phmask >> b) & 1u);
+      phmask ^= 1u << b;
     }
-    const uint64_t* sval = reinterpret_cast<const uint64_t*>(buf[b]);
-    const uint32_t* scol = reinterpret_cast<const uint32_t*>(buf[b] + TILE_EBUF * 8);
+    uint8_t* bb = wbase + b * TILE_BUF_BYTES;
+    const uint64_t* sval = reinterpret_cast<const uint64_t*>(bb);
+    const uint32_t* scol = reinterpret_cast<const uint32_t*>(bb + TILE_EBUF * 8);
     const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
     const double p_own = s_win[oslot];
     const int64_t own = a.row_base + rowseg + k * 32 + lane;
@@ -557,7 +577,10 @@ __global__ void __launch_bounds__(256) k_spmv_tile(SpmvArgs a) {
     a.out[own] = enc;
     if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
     __syncwarp();
-    if (k + 2 < 8) staged[b] = tile_issue(a, srp[32 * (k + 2)], srp[32 * (k + 3)], buf[b], &bars[b], lane);
+    if (k + 2 < 8) {
+      const bool ok = tile_issue(a, srp[32 * (k + 2)], srp[32 * (k + 3)], bb, &bars[b], lane);
+      stmask = (stmask & ~(1u << b)) | ((ok ? 1u : 0u) << b);
+    }
   }
   if (DOT) {
 #pragma unroll

@@ -23,5 +23,9 @@ for w in $WHAT; do
     timeout 900 ncu --set full --clock-control none --import-source on -k regex:'k_spmv|k_calc_ur|k_calc_p' -s 6 -c 6 \
       -o gpurun_out/prof_$TAG -f python bench.py --steps 1 --warmup 0 --no-e2e --no-cpu-baseline --max-iters 4 > gpurun_out/ncu_full_$TAG.log 2>&1
     tail -3 gpurun_out/ncu_full_$TAG.log ;;
+  ncuspmv)
+    timeout 900 ncu --set full --clock-control none --import-source on -k regex:'k_spmv' -s 2 -c 4 \
+      -o gpurun_out/prof_$TAG -f python bench.py --steps 1 --warmup 0 --no-e2e --no-cpu-baseline --max-iters 3 > gpurun_out/ncu_full_$TAG.log 2>&1
+    tail -3 gpurun_out/ncu_full_$TAG.log ;;
   esac
 done
