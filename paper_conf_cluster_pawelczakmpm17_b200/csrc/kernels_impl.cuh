@@ -391,9 +391,10 @@ static __device__ __forceinline__ bool tile_issue(const SpmvArgs& a, uint32_t s0
   return true;
 }
 
-// One row: check/correct its elements (from SMEM or global), gather, fma chain.
+// One row, general case: check/correct its elements (from SMEM or global),
+// gather, fma chain.  Also the cold path of the 5-entry fast path below.
 template <int ES, int RS, int VS>
-static __device__ __forceinline__ double tile_row(const SpmvArgs& a, uint32_t start, uint32_t end, const uint64_t* sval,
+static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start, uint32_t end, const uint64_t* sval,
                                                  const uint32_t* scol, uint32_t sbase_v, uint32_t sbase_c, bool staged,
                                                  const double* win, int oslot, double p_own, int64_t own) {
   double acc = 0.0;
@@ -445,6 +446,50 @@ static __device__ __forceinline__ double tile_row(const SpmvArgs& a, uint32_t st
       cnt_add(a.counts, T_ELEM, CRC32C, DUE);
       *a.due = 1;
     }
+  }
+  return acc;
+}
+
+// 5-entry stencil rows (the TeaLeaf layout, reading R16): straight-line code,
+// one uniform branch for "any element needs correction / any index is not
+// the canonical stencil neighbour or in range" -> tile_row (identical
+// semantics, so counts and results do not depend on which path ran).
+template <int ES, int RS, int VS>
+static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, uint32_t start, uint32_t end,
+                                                   const uint64_t* sval, const uint32_t* scol, uint32_t sbase_v,
+                                                   uint32_t sbase_c, bool staged, const double* win, int oslot,
+                                                   double p_own, int64_t own) {
+  if (ES == CRC32C || !staged || end - start != 5u || start > end || (int64_t)end > a.nnz)
+    return tile_row<ES, RS, VS>(a, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
+  const int n32 = (int)a.stencil_n;
+  const int own_col = (int)(own - a.col_base);
+  const uint32_t ckeep = col_keep(ES);
+  uint64_t v[5];
+  uint32_t c[5];
+#pragma unroll
+  for (int t = 0; t < 5; t++) {
+    v[t] = sval[start + t - sbase_v];
+    c[t] = scol[start + t - sbase_c];
+  }
+  uint32_t bad = 0;
+  int sd[5];
+  const int canon[5] = {-n32, -1, 0, 1, n32};
+  const int canon_sd[5] = {-TILE_WW, -1, 0, 1, TILE_WW};
+#pragma unroll
+  for (int t = 0; t < 5; t++) {
+    if (ES == SED) bad |= esed_clean(v[t], c[t]) ? 0u : 1u;
+    else if (ES != NONE) bad |= e96_bad(lo32(v[t]), hi32(v[t]), c[t]);
+    const uint32_t cm = c[t] & ckeep;
+    const int d = (int)cm - own_col;
+    sd[t] = (d == 0) ? 0 : canon_sd[t];
+    if (!((d == 0 || d == canon[t]) && (int64_t)cm < a.ncols)) bad |= 2u;
+  }
+  if (bad) return tile_row<ES, RS, VS>(a, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
+  double acc = 0.0;
+#pragma unroll
+  for (int t = 0; t < 5; t++) {
+    const double x = (sd[t] == 0) ? p_own : win[oslot + sd[t]];
+    acc = fma(as_d(v[t]), x, acc);
   }
   return acc;
 }
@@ -572,7 +617,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
     const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
     const double p_own = s_win[oslot];
     const int64_t own = a.row_base + rowseg + k * 32 + lane;
-    const double acc = tile_row<ES, RS, VS>(a, start, end, sval, scol, s0 & ~1u, s0 & ~3u, st, s_win, oslot, p_own, own);
+    const double acc = tile_row5<ES, RS, VS>(a, start, end, sval, scol, s0 & ~1u, s0 & ~3u, st, s_win, oslot, p_own, own);
     const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
     a.out[own] = enc;
     if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
