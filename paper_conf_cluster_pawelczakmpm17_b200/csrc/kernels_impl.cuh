@@ -455,12 +455,12 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
 // the canonical stencil neighbour or in range" -> tile_row (identical
 // semantics, so counts and results do not depend on which path ran).
 template <int ES, int RS, int VS>
-static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, uint32_t start, uint32_t end,
+static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const SpmvArgs& sa, uint32_t start, uint32_t end,
                                                    const uint64_t* sval, const uint32_t* scol, uint32_t sbase_v,
                                                    uint32_t sbase_c, bool staged, const double* win, int oslot,
                                                    double p_own, int64_t own) {
   if (ES == CRC32C || !staged || end - start != 5u || start > end || (int64_t)end > a.nnz)
-    return tile_row<ES, RS, VS>(a, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
   const int n32 = (int)a.stencil_n;
   const int own_col = (int)(own - a.col_base);
   const uint32_t ckeep = col_keep(ES);
@@ -484,7 +484,7 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, uint32_t s
     sd[t] = (d == 0) ? 0 : canon_sd[t];
     if (!((d == 0 || d == canon[t]) && (int64_t)cm < a.ncols)) bad |= 2u;
   }
-  if (bad) return tile_row<ES, RS, VS>(a, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
+  if (bad) return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
   double acc = 0.0;
 #pragma unroll
   for (int t = 0; t < 5; t++) {
@@ -498,6 +498,10 @@ template <int ES, int RS, int VS, bool DOT>
 __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
   extern __shared__ __align__(128) uint8_t s_dyn[];
   __shared__ __align__(16) uint8_t s_lut[128];
+  // the cold row path takes the arguments by reference: give it a SMEM copy so
+  // the kernel parameters are never spilled to local memory
+  __shared__ SpmvArgs s_args;
+  if (threadIdx.x == 0) s_args = a;
   double* s_win = reinterpret_cast<double*>(s_dyn);
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   uint8_t* wbase = s_dyn + TILE_WIN_BYTES + warp * (2 * TILE_BUF_BYTES + TILE_RP * 4 + 16);
@@ -575,26 +579,40 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
   }
   // ---- 2. decoded `in` window
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
-  constexpr int NSLOT = (TILE_TY + 2) * TILE_WW;
-  constexpr int PER_T = (NSLOT + 255) / 256;
-  uint64_t wv[PER_T];
+  constexpr int WPER = (TILE_WW + 31) / 32;                      // 9 slots per lane per window row
+  for (int wy = warp; wy < TILE_TY + 2; wy += 8) {
+    const int64_t rbase = win0 + (int64_t)wy * n;                 // in-index of (wy, 0)
+    const bool row_in = rbase >= 0 && rbase + TILE_WW <= a.npad_in;  // uniform: no per-slot bounds
+    const bool row_own = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny;
+    const uint64_t* src = a.in + rbase;
+    double* dst = s_win + wy * TILE_WW;
+    uint64_t wv[WPER];
 #pragma unroll
-  for (int q = 0; q < PER_T; q++) {  // all loads first (latency overlapped)
-    const int sidx = threadIdx.x + 256 * q;
-    const int wy = sidx / TILE_WW, wx = sidx - wy * TILE_WW;
-    const int64_t idx = win0 + (int64_t)wy * n + wx;
-    wv[q] = (sidx < NSLOT && idx >= 0 && idx < a.npad_in) ? ldg64(a.in + idx) : 0ull;
-  }
+    for (int q = 0; q < WPER; q++) {
+      const int wx = lane + 32 * q;
+      const int64_t idx = rbase + wx;
+      const bool ok = wx < TILE_WW && (row_in || (idx >= 0 && idx < a.npad_in));
+      wv[q] = ok ? ldg64(src + wx) : 0ull;
+    }
+    uint32_t badm = 0;
 #pragma unroll
-  for (int q = 0; q < PER_T; q++) {
-    const int sidx = threadIdx.x + 256 * q;
-    if (sidx >= NSLOT) continue;
-    const int wy = sidx / TILE_WW, wx = sidx - wy * TILE_WW;
-    const int64_t idx = win0 + (int64_t)wy * n + wx;
-    const bool owner = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny && wx >= 1 && wx <= 256;
-    uint64_t w = wv[q];
-    if (VS != NONE && idx >= 0 && idx < a.npad_in) w = v1_check<VS>(w, a.in + idx, owner, a.counts, a.due);
-    s_win[sidx] = as_d(w & vkeep(VS));
+    for (int q = 0; q < WPER; q++) {
+      const int wx = lane + 32 * q;
+      if (VS == SED) badm |= (vsed_clean(wv[q]) ? 0u : 1u) << q;
+      if (VS == SECDED64) badm |= (v64_bad(lo32(wv[q]), hi32(wv[q])) ? 1u : 0u) << q;
+      if (wx < TILE_WW) dst[wx] = as_d(wv[q] & vkeep(VS));
+    }
+    if (VS != NONE && badm) {  // cold: reload, correct (owner counts + scrubs), overwrite
+      for (int q = 0; q < WPER; q++) {
+        if (!((badm >> q) & 1u)) continue;
+        const int wx = lane + 32 * q;
+        const int64_t idx = rbase + wx;
+        if (wx >= TILE_WW || idx < 0 || idx >= a.npad_in) continue;
+        const bool owner = row_own && wx >= 1 && wx <= 256;
+        const uint64_t w = v1_check<VS>(ldg64(src + wx), a.in + idx, owner, a.counts, a.due);
+        dst[wx] = as_d(w & vkeep(VS));
+      }
+    }
   }
   __syncthreads();
   if (!has_seg) return;
@@ -617,7 +635,8 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
     const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
     const double p_own = s_win[oslot];
     const int64_t own = a.row_base + rowseg + k * 32 + lane;
-    const double acc = tile_row5<ES, RS, VS>(a, start, end, sval, scol, s0 & ~1u, s0 & ~3u, st, s_win, oslot, p_own, own);
+    const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s0 & ~1u, s0 & ~3u, st, s_win, oslot,
+                                             p_own, own);
     const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
     a.out[own] = enc;
     if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
