@@ -79,6 +79,9 @@ constexpr ABFT_HD uint32_t moebius32(uint32_t d) {
 }
 // R bits {31, 30, 29, 27, 23, 15}: all zero <=> parity 0 and index syndrome 0
 constexpr uint32_t MOEB_SYN_MASK = 0xE8808000u;
+// "any syndrome or parity bit set" over OR-accumulated Moebius registers and
+// code-row popcounts of several codewords
+ABFT_HD bool syn_bad(uint32_t acc_r, uint32_t acc_p) { return ((acc_r & MOEB_SYN_MASK) | (acc_p & 1u)) != 0u; }
 // q and the 5-bit index syndrome from a Moebius register
 ABFT_HD int moeb_q(uint32_t r) { return (int)(r >> 31); }
 ABFT_HD int moeb_index(uint32_t r) {
@@ -274,6 +277,10 @@ ABFT_HD uint32_t v64_fold(uint32_t a, uint32_t b) {
   return (a & ~0x6u) ^ b ^ (t & 0x00040200u);
 }
 // Returns nonzero iff the codeword is NOT clean (fast path).
+ABFT_HD void v64_acc(uint32_t a, uint32_t b, uint32_t& acc_r, uint32_t& acc_p) {
+  acc_r |= moebius32(v64_fold(a, b));
+  acc_p |= (uint32_t)(popc32(b ^ (a & 0x80u)) | popc32(a & 0x8Eu));
+}
 ABFT_HD uint32_t v64_bad(uint32_t a, uint32_t b) {
   uint32_t r = moebius32(v64_fold(a, b));
   uint32_t s56 = (uint32_t)(popc32(b ^ (a & 0x80u)) | popc32(a & 0x8Eu)) & 1u;
@@ -414,13 +421,22 @@ ABFT_HD uint64_t col_limit(int s) { return s == NONE ? 0xFFFFFFFFull : s == SED 
 // ---- E-SECDED (folded).  Fold register: A ^ B ^ C with C24, C25 moved to fold
 // positions 8 and 17 (PRMT copies col's top byte into bytes 1 and 2).
 ABFT_HD uint32_t e96_fold(uint32_t a, uint32_t b, uint32_t c) {
-  uint32_t t = byte_perm(c, 0u, 0x4334u);           // [0, c.b3, c.b3, 0]
-  return a ^ b ^ (c & ~0x03000000u) ^ (t & 0x00020100u);
+  // t = [0, c.b3, c.b3, c.b3]; XOR-ing t & 0x03020100 removes C24/C25 from
+  // fold positions 24/25 and inserts them at 8/17 (PRMT + 2 LOP3).
+  uint32_t t = byte_perm(c, 0u, 0x3334u);
+  return (a ^ b ^ c) ^ (t & 0x03020100u);
 }
+// Accumulating fast check (OR the Moebius registers and the code-row popcounts
+// of several codewords, test once with syn_bad): one branch per row / step.
+ABFT_HD void e96_acc(uint32_t a, uint32_t b, uint32_t c, uint32_t& acc_r, uint32_t& acc_p) {
+  acc_r |= moebius32(e96_fold(a, b, c));
+  acc_p |= (uint32_t)(popc32(b ^ (c & 0x9F000000u)) | popc32((b & 0x80000000u) | (c & 0x7FFFFFFFu)));
+}
+
 ABFT_HD uint32_t e96_bad(uint32_t a, uint32_t b, uint32_t c) {
-  uint32_t r = moebius32(e96_fold(a, b, c));
-  uint32_t s56 = (uint32_t)(popc32(b ^ (c & 0x9F000000u)) | popc32((c & 0x7FFFFFFFu) ^ (b & 0x80000000u))) & 1u;
-  return (r & MOEB_SYN_MASK) | s56;
+  uint32_t r = 0, p = 0;
+  e96_acc(a, b, c, r, p);
+  return syn_bad(r, p) ? 1u : 0u;
 }
 ABFT_HD void e96_syndrome(uint32_t a, uint32_t b, uint32_t c, int& s, int& q) {
   uint32_t r = moebius32(e96_fold(a, b, c));

@@ -471,18 +471,25 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
     v[t] = sval[start + t - sbase_v];
     c[t] = scol[start + t - sbase_c];
   }
-  uint32_t bad = 0;
+  uint32_t acc_r = 0, acc_p = 0, bad = 0;
   int sd[5];
   const int canon[5] = {-n32, -1, 0, 1, n32};
   const int canon_sd[5] = {-TILE_WW, -1, 0, 1, TILE_WW};
+  const uint32_t ncols32 = (uint32_t)a.ncols;
+  uint32_t cmax = 0;
 #pragma unroll
   for (int t = 0; t < 5; t++) {
-    if (ES == SED) bad |= esed_clean(v[t], c[t]) ? 0u : 1u;
-    else if (ES != NONE) bad |= e96_bad(lo32(v[t]), hi32(v[t]), c[t]);
+    if (ES == SED) acc_p |= (uint32_t)(popc64(v[t]) + popc32(c[t]));
+    else if (ES != NONE) e96_acc(lo32(v[t]), hi32(v[t]), c[t], acc_r, acc_p);
     const uint32_t cm = c[t] & ckeep;
+    cmax = max(cmax, cm);
     const int d = (int)cm - own_col;
     sd[t] = (d == 0) ? 0 : canon_sd[t];
-    if (!((d == 0 || d == canon[t]) && (int64_t)cm < a.ncols)) bad |= 2u;
+    bad |= (d == 0 || d == canon[t]) ? 0u : 1u;
+  }
+  if (ES != NONE) {
+    if (syn_bad(acc_r, acc_p)) bad = 1u;
+    if (a.ncols > 0xFFFFFFFFll ? false : cmax >= ncols32) bad = 1u;
   }
   if (bad) return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
   double acc = 0.0;
