@@ -50,7 +50,8 @@ struct abft_ctx {
   uint32_t* flags = nullptr;
   CgState* h_state = nullptr;  // pinned
   uint32_t* h_flags = nullptr; // pinned
-  bool profile = false;
+  int profile = 0;        // bitmask of kernel classes to time: 1 SpMV, 2 calc_ur, 4 calc_p, 8 reductions
+  bool use_graphs = true; // capture poll_every iterations into a CUDA graph (single GPU)
   double prof_ms[4] = {0, 0, 0, 0};
   int64_t prof_n[4] = {0, 0, 0, 0};
   std::vector<cudaEvent_t> events;
@@ -247,7 +248,7 @@ int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_
 
 int abft_profile(abft_ctx* ctx, int enable) {
   if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
-  ctx->profile = enable != 0;
+  ctx->profile = enable;
   for (int i = 0; i < 4; i++) { ctx->prof_ms[i] = 0; ctx->prof_n[i] = 0; }
   return ABFT_OK;
 }
@@ -273,17 +274,20 @@ struct Prof {
     }
     return ctx->events[i];
   }
+  bool on = false;
   void begin(int cls) {
-    if (!ctx->profile) return;
+    on = (ctx->profile >> cls) & 1;
+    if (!on) return;
     cudaEventRecord(ev(next), s);
     marks.push_back({cls, (int)next});
     next += 2;
   }
   void end() {
-    if (!ctx->profile) return;
+    if (!on) return;
     cudaEventRecord(ev(marks.back().second + 1), s);
+    on = false;
   }
-  void harvest() {  // after a stream sync
+  void harvest(bool keep = false) {  // after a stream sync; keep = marks belong to a graph
     if (!ctx->profile) return;
     for (auto& m : marks) {
       float ms = 0;
@@ -292,8 +296,10 @@ struct Prof {
         ctx->prof_n[m.first] += 1;
       }
     }
-    marks.clear();
-    next = 0;
+    if (!keep) {
+      marks.clear();
+      next = 0;
+    }
   }
 };
 
@@ -410,28 +416,23 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   CUDA_TRY(cudaGetLastError());
 
   const int poll = opts->poll_every > 0 ? opts->poll_every : 16;
-  int64_t launched = 0;
-  for (;;) {
-    CUDA_TRY(cudaMemcpyAsync(ctx->h_state, ctx->state, sizeof(CgState), cudaMemcpyDeviceToHost, s));
-    CUDA_TRY(cudaStreamSynchronize(s));
-    prof.harvest();
-    if (ctx->h_state->stop || launched >= opts->max_iters) break;
-    int64_t k = opts->max_iters - launched;
-    if (k > poll) k = poll;
+  // k iterations of (a3)..(a5) + the DUE/convergence logic, all device-side
+  auto issue = [&](int64_t k) -> int {
     for (int64_t it = 0; it < k; it++) {
-      if ((e = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e;
+      int e2;
+      if ((e2 = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e2;
       prof.begin(0);
-      e = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr);
+      e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr);
       prof.end();
-      if (e) return e;
+      if (e2) return e2;
       prof.begin(3);
-      if ((e = finish_dot(ctx, d, nrb, 2, s))) return e;
+      if ((e2 = finish_dot(ctx, d, nrb, 2, s))) return e2;
       prof.end();
       prof.begin(1);
       count_launch(launch_calc_ur(va, scheme, s));
       prof.end();
       prof.begin(3);
-      if ((e = finish_dot(ctx, d, nrb, 3, s))) return e;
+      if ((e2 = finish_dot(ctx, d, nrb, 3, s))) return e2;
       prof.end();
       prof.begin(2);
       count_launch(launch_calc_p(va, scheme, s));
@@ -443,8 +444,56 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       }
     }
     CUDA_TRY(cudaGetLastError());
+    return ABFT_OK;
+  };
+  // CUDA graph of `poll` iterations (single GPU): one launch per poll, no
+  // per-kernel CPU launch cost; kernels read alpha/beta/stop from device state.
+  cudaGraphExec_t gexec = nullptr;
+  std::vector<std::pair<int, int>> gmarks;
+  uint64_t glaunches = 0;
+  const bool graphs = ctx->use_graphs && !multi;
+  bool last_graph = false;
+  int64_t launched = 0;
+  for (;;) {
+    CUDA_TRY(cudaMemcpyAsync(ctx->h_state, ctx->state, sizeof(CgState), cudaMemcpyDeviceToHost, s));
+    CUDA_TRY(cudaStreamSynchronize(s));
+    if (last_graph) {  // the graph's event nodes were re-recorded by this replay
+      prof.marks = gmarks;
+      prof.harvest(true);
+      prof.marks.clear();
+    } else {
+      prof.harvest();
+    }
+    last_graph = false;
+    if (ctx->h_state->stop || launched >= opts->max_iters) break;
+    int64_t k = opts->max_iters - launched;
+    if (k > poll) k = poll;
+    if (graphs && k == poll) {
+      if (!gexec) {
+        prof.harvest();  // start the graph's marks from a clean list
+        const uint64_t l0 = g_launches.load();
+        cudaGraph_t graph = nullptr;
+        CUDA_TRY(cudaStreamBeginCapture(s, cudaStreamCaptureModeThreadLocal));
+        e = issue(k);
+        cudaError_t ce = cudaStreamEndCapture(s, &graph);
+        if (e) return e;
+        if (ce != cudaSuccess) return fail(ABFT_E_CUDA, "graph capture: %s", cudaGetErrorString(ce));
+        CUDA_TRY(cudaGraphInstantiate(&gexec, graph, 0));
+        cudaGraphDestroy(graph);
+        glaunches = g_launches.load() - l0;
+        g_launches.fetch_sub(glaunches);  // counted per replay below
+        gmarks = prof.marks;
+      }
+      prof.marks.clear();
+      CUDA_TRY(cudaGraphLaunch(gexec, s));
+      count_launch((int)glaunches);
+      last_graph = true;
+    } else {
+      if ((e = issue(k))) return e;
+    }
     launched += k;
   }
+  if (gexec) cudaGraphExecDestroy(gexec);
   const CgState& hs = *ctx->h_state;
   res->iters = hs.iters;
   res->rr0 = hs.rr0;

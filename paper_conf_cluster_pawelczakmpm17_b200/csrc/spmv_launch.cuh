@@ -13,8 +13,9 @@ template <int ES, int RS, int VS, bool DOT>
 static void spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   const size_t smem = TILE_SMEM;
   static bool attr = false;
-  if (!attr) {
-    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, DOT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (!attr) {  // both variants at once: never inside a later CUDA-graph capture
+    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     attr = true;
   }
   const int64_t ny = a.nrows / a.stencil_n;
