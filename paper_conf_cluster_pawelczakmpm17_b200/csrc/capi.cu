@@ -52,6 +52,7 @@ struct abft_ctx {
   uint32_t* h_flags = nullptr; // pinned
   int profile = 0;        // bitmask of kernel classes to time: 1 SpMV, 2 calc_ur, 4 calc_p, 8 reductions
   bool use_graphs = true; // capture poll_every iterations into a CUDA graph (single GPU)
+  cudaStream_t cap_stream = nullptr;
   double prof_ms[4] = {0, 0, 0, 0};
   int64_t prof_n[4] = {0, 0, 0, 0};
   std::vector<cudaEvent_t> events;
@@ -181,6 +182,7 @@ int abft_ctx_destroy(abft_ctx* c) {
   cudaFreeHost(c->h_state);
   cudaFreeHost(c->h_flags);
   for (auto e : c->events) cudaEventDestroy(e);
+  if (c->cap_stream) cudaStreamDestroy(c->cap_stream);
   delete c;
   return ABFT_OK;
 }
@@ -417,7 +419,8 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
 
   const int poll = opts->poll_every > 0 ? opts->poll_every : 16;
   // k iterations of (a3)..(a5) + the DUE/convergence logic, all device-side
-  auto issue = [&](int64_t k) -> int {
+  auto issue = [&](int64_t k, cudaStream_t s) -> int {
+    prof.s = s;
     for (int64_t it = 0; it < k; it++) {
       int e2;
       if ((e2 = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e2;
@@ -472,10 +475,14 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       if (!gexec) {
         prof.harvest();  // start the graph's marks from a clean list
         const uint64_t l0 = g_launches.load();
+        // capture on the context's private stream (the caller's may be the
+        // legacy default stream, which cannot be captured); replay on `s`
+        if (!ctx->cap_stream) CUDA_TRY(cudaStreamCreateWithFlags(&ctx->cap_stream, cudaStreamNonBlocking));
         cudaGraph_t graph = nullptr;
-        CUDA_TRY(cudaStreamBeginCapture(s, cudaStreamCaptureModeThreadLocal));
-        e = issue(k);
-        cudaError_t ce = cudaStreamEndCapture(s, &graph);
+        CUDA_TRY(cudaStreamBeginCapture(ctx->cap_stream, cudaStreamCaptureModeThreadLocal));
+        e = issue(k, ctx->cap_stream);
+        cudaError_t ce = cudaStreamEndCapture(ctx->cap_stream, &graph);
+        prof.s = s;
         if (e) return e;
         if (ce != cudaSuccess) return fail(ABFT_E_CUDA, "graph capture: %s", cudaGetErrorString(ce));
         CUDA_TRY(cudaGraphInstantiate(&gexec, graph, 0));
@@ -489,7 +496,7 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       count_launch((int)glaunches);
       last_graph = true;
     } else {
-      if ((e = issue(k))) return e;
+      if ((e = issue(k, s))) return e;
     }
     launched += k;
   }
