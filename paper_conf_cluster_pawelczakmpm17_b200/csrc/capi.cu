@@ -280,13 +280,13 @@ struct Prof {
   void begin(int cls) {
     on = (ctx->profile >> cls) & 1;
     if (!on) return;
-    cudaEventRecord(ev(next), s);
+    cudaEventRecordWithFlags(ev(next), s, cudaEventRecordExternal);  // observable when captured in a graph
     marks.push_back({cls, (int)next});
     next += 2;
   }
   void end() {
     if (!on) return;
-    cudaEventRecord(ev(marks.back().second + 1), s);
+    cudaEventRecordWithFlags(ev(marks.back().second + 1), s, cudaEventRecordExternal);
     on = false;
   }
   void harvest(bool keep = false) {  // after a stream sync; keep = marks belong to a graph
@@ -296,6 +296,8 @@ struct Prof {
       if (cudaEventElapsedTime(&ms, ctx->events[m.second], ctx->events[m.second + 1]) == cudaSuccess) {
         ctx->prof_ms[m.first] += ms;
         ctx->prof_n[m.first] += 1;
+      } else {
+        (void)cudaGetLastError();  // a failed timing query must not poison later calls
       }
     }
     if (!keep) {
