@@ -280,13 +280,13 @@ struct Prof {
   void begin(int cls) {
     on = (ctx->profile >> cls) & 1;
     if (!on) return;
-    cudaEventRecordWithFlags(ev(next), s, cudaEventRecordExternal);  // observable when captured in a graph
+    cudaEventRecord(ev(next), s);
     marks.push_back({cls, (int)next});
     next += 2;
   }
   void end() {
     if (!on) return;
-    cudaEventRecordWithFlags(ev(marks.back().second + 1), s, cudaEventRecordExternal);
+    cudaEventRecord(ev(marks.back().second + 1), s);
     on = false;
   }
   void harvest(bool keep = false) {  // after a stream sync; keep = marks belong to a graph
@@ -456,7 +456,9 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   cudaGraphExec_t gexec = nullptr;
   std::vector<std::pair<int, int>> gmarks;
   uint64_t glaunches = 0;
-  const bool graphs = ctx->use_graphs && !multi;
+  // (profiling brackets kernels with events, which are not timeable inside a
+  // graph replay: profiled solves launch kernels directly)
+  const bool graphs = ctx->use_graphs && !multi && ctx->profile == 0;
   bool last_graph = false;
   int64_t launched = 0;
   for (;;) {
