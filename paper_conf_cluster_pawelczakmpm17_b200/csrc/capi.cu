@@ -346,7 +346,7 @@ int halo_exchange(abft_dist* d, uint64_t* ext, int64_t n_loc, int64_t n_halo, cu
 // Dot-product finish: single GPU -> reduce with op; multi-GPU -> subtree root +
 // DUE flag, all-gather, identical top-of-tree combine on every rank.
 int finish_dot(abft_ctx* ctx, abft_dist* d, int64_t nrb, int op, cudaStream_t s) {
-  if (!d || d->nranks == 1) {
+  if (!d) {
     count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, op, ctx->state, nullptr, ctx->due, s));
     return ABFT_OK;
   }
@@ -384,7 +384,9 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   const int64_t nrb = (n + 255) / 256;
   if ((e = ensure_partials(ctx, nrb))) return e;
   if (nrb > (int64_t)1024 * 1024) return fail(ABFT_E_SHAPE, "more than 2^28 rows per GPU");
-  const bool multi = d && d->nranks > 1;
+  // the dist path runs whenever a communicator is given (also with 1 rank, so the
+  // all-gather / top-of-tree combine code is exercised on a single GPU)
+  const bool multi = d != nullptr;
 
   CgState h{};
   h.tol = opts->tol;
@@ -540,7 +542,7 @@ int abft_dist_init(abft_dist** out, const void* uid, int rank, int nranks, int d
   d->device = device;
   ncclUniqueId id;
   memcpy(&id, uid, sizeof(id));
-  if (nranks > 1) NCCL_TRY(ncclCommInitRank(&d->comm, nranks, id, rank));
+  NCCL_TRY(ncclCommInitRank(&d->comm, nranks, id, rank));
   CUDA_TRY(cudaMalloc(&d->sendbuf, sizeof(double) * 2));
   CUDA_TRY(cudaMalloc(&d->gathered, sizeof(double) * 2 * nranks));
   *out = d;

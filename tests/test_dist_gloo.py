@@ -1,0 +1,150 @@
+"""Multi-rank host logic on CPU (torch.distributed gloo, world size 2 and 4).
+
+Each rank owns a strip of grid rows of the G-TEA problem with one ghost grid
+row above/below its local vectors.  Per CG iteration the ranks
+exchange the encoded boundary rows of p (ECC travels with the data), run the
+oracle SpMV / calc_ur / calc_p on their strip, and all-gather one RED-1
+subtree root per dot product, combining them with the top of the tree.  This is
+the algorithm `abft_cg_solve_dist` runs over NCCL; here it is checked against
+the single-process oracle CG: identical iteration count, bit-identical x and r,
+and fault counters that sum to the single-process counts (owner rule).
+"""
+import os
+
+import numpy as np
+import pytest
+import torch
+import torch.distributed as dist
+import torch.multiprocessing as mp
+
+import gen
+import oracle as orc
+
+N_GRID = 32
+
+
+def _single(scheme, flips):
+    n = N_GRID
+    N = n * n
+    v, c, r = gen.tealeaf_csr(n)
+    es = rs = orc.SECDED64
+    A = orc.Matrix(v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32), N, N, es, rs)
+    A.encode()
+    b = gen.tealeaf_rhs(n).numpy()
+    B = orc.vec_encode(b, scheme)
+    X = B.copy()
+    for (i, bit) in flips:
+        X[i] ^= np.uint64(1 << bit)
+    R, P, W = (np.zeros_like(B) for _ in range(3))
+    cnt = orc.new_counts()
+    st, res = orc.cg_solve(A, B, X, R, P, W, scheme, 1e-10, 500, 1, cnt)
+    return res.iters, X[:N], R[:N], cnt
+
+
+def _worker(rank, world, port, scheme, flips, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        n = N_GRID
+        rows = n // world
+        y0, y1 = rank * rows, (rank + 1) * rows
+        N = rows * n
+        h = n
+        v, c, r = gen.strip_csr(n, y0, y1, ny=n, col_offset=h)
+        es = rs = orc.SECDED64
+        A = orc.Matrix(v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32), N, N + 2 * h, es, rs,
+                       row_base=h, col_base=0)
+        A.encode()
+        b = gen.tealeaf_rhs(n, y0, y1, ny=n).numpy()
+        ext = N + 2 * h
+
+        def vec(vals=None):
+            out = np.zeros(ext, dtype=np.uint64)
+            if vals is not None:
+                out[h:h + N] = orc.vec_encode(vals, scheme)[:N]
+            return out
+
+        B, X = vec(b), vec(b)
+        for (i, bit) in flips:  # global index -> owner rank's local slot
+            if y0 * n <= i < y1 * n:
+                X[h + i - y0 * n] ^= np.uint64(1 << bit)
+        R, Pv, W = vec(), vec(), vec()
+        cnt = orc.new_counts()
+
+        def halo(a):
+            t = torch.from_numpy(a.view(np.int64))
+            reqs = []
+            if rank > 0:
+                reqs.append(dist.isend(t[h:2 * h].clone(), rank - 1))
+                top = torch.empty(h, dtype=torch.int64)
+                reqs.append(dist.irecv(top, rank - 1))
+            if rank < world - 1:
+                reqs.append(dist.isend(t[N:N + h].clone(), rank + 1))
+                bot = torch.empty(h, dtype=torch.int64)
+                reqs.append(dist.irecv(bot, rank + 1))
+            for rq in reqs:
+                rq.wait()
+            if rank > 0:
+                a[0:h] = top.numpy().view(np.uint64)
+            if rank < world - 1:
+                a[h + N:] = bot.numpy().view(np.uint64)
+
+        def combine(root):
+            g = [torch.zeros(1, dtype=torch.float64) for _ in range(world)]
+            dist.all_gather(g, torch.tensor([root], dtype=torch.float64))
+            return orc.tree_sum(np.array([x.item() for x in g]))
+
+        loc = slice(h, h + N)
+        halo(X)
+        orc.spmv(A, X, ext, scheme, W, ext, cnt)
+        _, rr0_loc = orc.cg_init_r(B[loc], W[loc], R[loc], Pv[loc], N, scheme, cnt)
+        rr0 = rro = combine(rr0_loc)
+        iters = 0
+        for k in range(1, 501):
+            halo(Pv)
+            _, pw_loc = orc.spmv(A, Pv, ext, scheme, W, ext, cnt, want_dot=True)
+            pw = combine(pw_loc)
+            alpha = rro / pw
+            xl, pl, rl, wl = X[loc].copy(), Pv[loc].copy(), R[loc].copy(), W[loc].copy()
+            _, rrn_loc = orc.calc_ur(xl, pl, rl, wl, N, scheme, alpha, cnt)
+            X[loc], Pv[loc], R[loc], W[loc] = xl, pl, rl, wl
+            rrn = combine(rrn_loc)
+            iters = k
+            if np.sqrt(rrn) <= 1e-10 * np.sqrt(rr0):
+                break
+            beta = rrn / rro
+            pl, rl = Pv[loc].copy(), R[loc].copy()
+            orc.calc_p(pl, rl, N, scheme, beta, cnt)
+            Pv[loc], R[loc] = pl, rl
+            rro = rrn
+        q.put((rank, iters, X[loc].copy(), R[loc].copy(), cnt))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("world", [2, 4])
+@pytest.mark.parametrize("scheme_name", ["SECDED64", "SED"])
+def test_distributed_cg_matches_single_process(world, scheme_name):
+    scheme = getattr(orc, scheme_name)
+    orc.build()
+    flips = [(5, 7), (300, 40), (700, 63), (1000, 2)]   # single flips in x0 on several ranks
+    it1, x1, r1, cnt1 = _single(scheme, flips)
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = 29500 + world * 7 + scheme
+    procs = [ctx.Process(target=_worker, args=(rk, world, port, scheme, flips, q)) for rk in range(world)]
+    for p in procs:
+        p.start()
+    out = [q.get(timeout=300) for _ in range(world)]
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    out.sort(key=lambda t: t[0])
+    assert all(o[1] == it1 for o in out), ([o[1] for o in out], it1)
+    xg = np.concatenate([o[2] for o in out])
+    rg = np.concatenate([o[3] for o in out])
+    assert np.array_equal(xg, x1)
+    assert np.array_equal(rg, r1)
+    cnt = sum(o[4] for o in out)
+    assert np.array_equal(cnt, cnt1), (cnt, cnt1)
