@@ -67,7 +67,8 @@ def run(grid, rates, seeds, kinds, out_path, check_spmv=True):
     col = col.to(torch.int32)
     rowptr = rowptr.to(torch.int32)
     nnz = 5 * N
-    A = abft.Matrix(val, col.clone(), rowptr, N, N, S, S, stencil_n=n if n % 256 == 0 else 0)
+    val0 = val.clone()   # pristine values: DUE'd (unscrubbed) flips must not leak into the next trial
+    A = abft.Matrix(val.clone(), col.clone(), rowptr, N, N, S, S, stencil_n=n if n % 256 == 0 else 0)
     rp_len = A.rowptr.numel()
     vec_vals = [gen.tealeaf_rhs(n, device=dev)] + [torch.from_numpy(gen.uniform_pm1(N, 100 + j)).to(dev)
                                                   for j in range(4)]
@@ -84,6 +85,7 @@ def run(grid, rates, seeds, kinds, out_path, check_spmv=True):
         for rate in rates:
             for seed in range(1, seeds + 1):
                 t0 = time.time()
+                A.val.copy_(val0)
                 A.col.copy_(col)
                 A.rowptr.zero_()
                 A.rowptr[:N + 1].copy_(rowptr)
