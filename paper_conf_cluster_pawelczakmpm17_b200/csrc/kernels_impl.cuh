@@ -396,9 +396,13 @@ static __device__ __forceinline__ bool tile_issue(const SpmvArgs& a, uint32_t s0
 template <int ES, int RS, int VS>
 static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start, uint32_t end, const uint64_t* sval,
                                                  const uint32_t* scol, uint32_t sbase_v, uint32_t sbase_c, bool staged,
-                                                 const double* win, int oslot, double p_own, int64_t own) {
+                                                 const double* win, int oslot, double p_own, int64_t own, uint32_t s0,
+                                                 uint32_t s1) {
   double acc = 0.0;
   const bool ok = (start <= end) && ((int64_t)end <= a.nnz);
+  // a corrupted (DUE) rowptr entry can put this row outside the staged pass
+  // range: read it from global memory then
+  staged = staged && start >= s0 && end <= s1;
   if (RS != NONE && !ok) {
     cnt_range(a.counts, T_ROWPTR, RS);
     *a.due = 1;
@@ -458,9 +462,9 @@ template <int ES, int RS, int VS>
 static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const SpmvArgs& sa, uint32_t start, uint32_t end,
                                                    const uint64_t* sval, const uint32_t* scol, uint32_t sbase_v,
                                                    uint32_t sbase_c, bool staged, const double* win, int oslot,
-                                                   double p_own, int64_t own) {
-  if (ES == CRC32C || !staged || end - start != 5u || start > end || (int64_t)end > a.nnz)
-    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
+                                                   double p_own, int64_t own, uint32_t s0, uint32_t s1) {
+  if (ES == CRC32C || !staged || end - start != 5u || start > end || start < s0 || end > s1)
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own, s0, s1);
   const int n32 = (int)a.stencil_n;
   const int own_col = (int)(own - a.col_base);
   const uint32_t ckeep = col_keep(ES);
@@ -491,7 +495,8 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
     if (syn_bad(acc_r, acc_p)) bad = 1u;
     if (a.ncols > 0xFFFFFFFFll ? false : cmax >= ncols32) bad = 1u;
   }
-  if (bad) return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own);
+  if (bad)
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own, s0, s1);
   double acc = 0.0;
 #pragma unroll
   for (int t = 0; t < 5; t++) {
@@ -642,8 +647,9 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
     const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
     const double p_own = s_win[oslot];
     const int64_t own = a.row_base + rowseg + k * 32 + lane;
+    const uint32_t s1 = srp[32 * k + 32];
     const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s0 & ~1u, s0 & ~3u, st, s_win, oslot,
-                                             p_own, own);
+                                             p_own, own, s0, s1);
     const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
     a.out[own] = enc;
     if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);

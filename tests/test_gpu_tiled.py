@@ -128,3 +128,35 @@ def test_tiled_cg_parity(abft, ctx):
     assert res_g.rrn == res_o.rrn
     assert np.array_equal(words_of(xg)[:N], xo)
     assert np.array_equal(cnt_g.read(), cnt_o)
+
+
+@pytest.mark.parametrize("seed", [1, 2, 3])
+def test_tiled_spmv_rowptr_due_parity(abft, ctx, seed):
+    """Same-word double flips in rowptr entries (DUE, used as masked stored bits
+    under policy continue): rows may point anywhere in [0, nnz] or outside it;
+    the tiled kernel must fall back to global reads and match the oracle."""
+    n = 256
+    N = n * n
+    S = orc.SECDED64
+    rng = np.random.default_rng(100 + seed)
+    v, c, r = gen.tealeaf_csr(n)
+    v, c, r = v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32)
+    Ao, _ = oracle_matrix(v, c, r, N, N, S, S)
+    Ag, _ = gpu_matrix(abft, ctx, v, c, r, N, N, S, S, stencil_n=n)
+    for g in rng.choice(N // 2, 6, replace=False):
+        i = 2 * int(g) + int(rng.integers(2))
+        for b in rng.choice(28, 2, replace=False):   # value bits: the decoded entry really moves
+            Ao.rowptr[i] ^= np.uint32(1 << int(b))
+            abft.inject_bitflip(ctx, Ag.rowptr, 32 * i + int(b))
+    x = gen.uniform_pm1(N, 5)
+    xo = orc.vec_encode(x, S)
+    xg = gpu_vec_from_words(abft, xo, N, S)
+    out_o = np.zeros(N, dtype=np.uint64)
+    cnt_o = orc.new_counts()
+    orc.spmv(Ao, xo, N, S, out_o, N, cnt_o)
+    yg = abft.Vector.empty(N, S)
+    cnt_g = abft.Counters()
+    abft.spmv(ctx, Ag, xg, yg, cnt_g)
+    torch.cuda.synchronize()
+    assert np.array_equal(cnt_g.read(), cnt_o)
+    assert np.array_equal(words_of(yg)[:N], out_o)
