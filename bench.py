@@ -85,19 +85,29 @@ class ClockSampler:
 
 
 # ------------------------------------------------------------------ problem
-def build_problem(grid: int, rank: int, world: int, device):
-    """Raw (unencoded) device arrays of this rank's strip + metadata."""
+def build_problem(grid: int, rank: int, world: int, device, chunk_rows=None):
+    """Raw (unencoded) device arrays of this rank's rows, as row-block chunks
+    whose column windows fit the 24-bit element index (reading R7)."""
     import torch
     import gen
     n = grid
     ny = grid * world
-    y0, y1 = rank * grid, (rank + 1) * grid
+    y0r, y1r = rank * grid, (rank + 1) * grid
     halo = n if world > 1 else 0
-    val, col, rowptr = gen.strip_csr(n, y0, y1, ny=ny, device=device, col_offset=halo)
-    b = gen.tealeaf_rhs(n, y0, y1, ny=ny, device=device)
-    N = (y1 - y0) * n
-    return dict(val=val.contiguous(), col=col.to(torch.int32).contiguous(), rowptr=rowptr.to(torch.int32).contiguous(),
-                b=b.contiguous(), N=N, n=n, halo=halo, ncols=N + 2 * halo)
+    chunks = []
+    for (c0, c1, cb) in gen.chunk_plan(n, y1r - y0r, chunk_rows=chunk_rows):
+        # local grid rows [c0, c1) of this rank's strip; vector index = halo + local row index
+        gy0, gy1 = y0r + c0, y0r + c1
+        row_base = halo + c0 * n
+        col_base = max(0, row_base - n) if world > 1 or c0 > 0 else 0
+        val, col, rowptr = gen.strip_csr(n, gy0, gy1, ny=ny, device=device, col_offset=row_base - col_base)
+        ncols = min(halo + (y1r - y0r) * n + halo, row_base + (c1 - c0) * n + n) - col_base
+        chunks.append(dict(val=val.contiguous(), col=col.to(torch.int32).contiguous(),
+                           rowptr=rowptr.to(torch.int32).contiguous(), row_base=row_base, col_base=col_base,
+                           nrows=(c1 - c0) * n, ncols=ncols))
+    b = gen.tealeaf_rhs(n, y0r, y1r, ny=ny, device=device)
+    N = (y1r - y0r) * n
+    return dict(chunks=chunks, b=b.contiguous(), N=N, n=n, halo=halo)
 
 
 class Solver:
@@ -108,12 +118,15 @@ class Solver:
         self.abft, self.ctx, self.P, self.dist = abft, ctx, P, dist
         self.es, self.rs, self.vs = es, rs, vs
         N, halo = P["N"], P["halo"]
-        dev = P["val"].device
-        self.A = abft.Matrix(P["val"], P["col"].clone(), P["rowptr"], N, P["ncols"], es, rs, row_base=halo,
-                             col_base=0, stencil_n=P["n"])
-        self.col_raw = P["col"]
-        self.rp_raw = torch.zeros_like(self.A.rowptr)
-        self.rp_raw[:N + 1] = P["rowptr"]
+        dev = P["b"].device
+        self.A, self.raw = [], []
+        for ch in P["chunks"]:
+            M = abft.Matrix(ch["val"], ch["col"].clone(), ch["rowptr"], ch["nrows"], ch["ncols"], es, rs,
+                            row_base=ch["row_base"], col_base=ch["col_base"], stencil_n=P["n"])
+            rp_raw = torch.zeros_like(M.rowptr)
+            rp_raw[:ch["nrows"] + 1] = ch["rowptr"]
+            self.A.append(M)
+            self.raw.append((ch["col"], rp_raw))
         n_ext = N + 2 * halo
         self.vecs = [abft.Vector.empty(n_ext, vs, device=dev) for _ in range(5)]  # b x r p w
         self.counts = abft.Counters(device=dev)
@@ -122,16 +135,17 @@ class Solver:
 
     def load_inputs(self, host=None):
         """(Re)place the raw inputs: from device copies, or from pinned host buffers (e2e)."""
-        if host is None:
-            self.A.col.copy_(self.col_raw)
-            self.A.rowptr.copy_(self.rp_raw)
-            src_b = self.b_raw
-        else:
-            self.A.val.copy_(host["val"], non_blocking=True)
-            self.A.col.copy_(host["col"], non_blocking=True)
-            self.A.rowptr[:self.N + 1].copy_(host["rowptr"], non_blocking=True)
-            self.A.rowptr[self.N + 1:].zero_()
-            src_b = host["b"]
+        for i, (M, (col_raw, rp_raw)) in enumerate(zip(self.A, self.raw)):
+            if host is None:
+                M.col.copy_(col_raw)
+                M.rowptr.copy_(rp_raw)
+            else:
+                hv, hc, hr = host["chunks"][i]
+                M.val.copy_(hv, non_blocking=True)
+                M.col.copy_(hc, non_blocking=True)
+                M.rowptr[:M.nrows + 1].copy_(hr, non_blocking=True)
+                M.rowptr[M.nrows + 1:].zero_()
+        src_b = self.b_raw if host is None else host["b"]
         b, x = self.vecs[0], self.vecs[1]
         h = self.halo
         b.data[h:h + self.N].copy_(src_b, non_blocking=True)
@@ -140,9 +154,10 @@ class Solver:
     def step(self, tol, max_iters, host=None):
         """a0 + a1 + a2..a7: returns the iteration count."""
         self.load_inputs(host)
-        st = self.A.encode(self.ctx)
-        if st != 0:
-            raise RuntimeError(f"encode failed: {self.abft.last_error()}")
+        for M in self.A:
+            st = M.encode(self.ctx)
+            if st != 0:
+                raise RuntimeError(f"encode failed: {self.abft.last_error()}")
         self.vecs[0].encode(self.ctx)
         self.vecs[1].encode(self.ctx)
         if self.dist is not None:
@@ -152,6 +167,13 @@ class Solver:
             res = self.abft.cg_solve(self.ctx, self.A, *self.vecs, tol=tol, max_iters=max_iters, due_policy=1,
                                      counts=self.counts, poll_every=32)
         return res.iters, res.status
+
+
+def host_inputs(P):
+    """Pinned host copies of the raw inputs (the e2e leg's H2D source)."""
+    chunks = [(c["val"].cpu().pin_memory(), c["col"].cpu().pin_memory(), c["rowptr"].cpu().pin_memory())
+              for c in P["chunks"]]
+    return {"chunks": chunks, "b": P["b"].cpu().pin_memory()}
 
 
 def timed(solver, steps, warmup, tol, max_iters, dist_on, host=None, out_host=None, profile=0):
@@ -271,6 +293,7 @@ def main():
     ap.add_argument("--tol", type=float, default=1e-10)
     ap.add_argument("--max-iters", type=int, default=20000)
     ap.add_argument("--oracle-grid", type=int, default=512)
+    ap.add_argument("--chunk-rows", type=int, default=None, help="grid rows per row-block chunk (default: fit 2^24 cols)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     args = ap.parse_args()
@@ -288,7 +311,7 @@ def main():
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     from paper_conf_cluster_pawelczakmpm17_b200 import abft
 
-    P = build_problem(args.grid, rank, world, torch.device("cuda", local))
+    P = build_problem(args.grid, rank, world, torch.device("cuda", local), args.chunk_rows)
     ctx = abft.Context(local)
     dobj = abft.Dist(rank, world, local) if dist_on else None
     prot = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj)
@@ -309,12 +332,12 @@ def main():
     e2e = None
     if not args.no_e2e:
         prot = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj)
-        host = {k: P[k].cpu().pin_memory() for k in ("val", "col", "b")}
-        host["rowptr"] = P["rowptr"].cpu().pin_memory()
+        host = host_inputs(P)
         out_host = torch.empty(P["N"], dtype=torch.float64).pin_memory()
         r_e = timed(prot, args.steps, 1, args.tol, args.max_iters, dist_on, host=host, out_host=out_host)
-        h2d = sum(t.numel() * t.element_size() for t in host.values())
-        e2e = {"value": world * r_e["iters"] / (r_e["ms"] / 1000.0), "unit": "CG it/s (4096^2-equivalent)",
+        h2d = sum(t.numel() * t.element_size() for c in host["chunks"] for t in c) + host["b"].numel() * 8
+        e2e = {"value": world * r_e["iters"] / (r_e["ms"] / 1000.0) * P["N"] / float(4096 * 4096),
+               "unit": "CG it/s (4096^2-equivalent)",
                "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": P["N"] * 8}
         del prot
 
@@ -324,8 +347,9 @@ def main():
         return
 
     N = P["N"]
-    its = r_p["iters"] / (r_p["ms"] / 1000.0)
-    its_u = r_u["iters"] / (r_u["ms"] / 1000.0)
+    eq = N / float(4096 * 4096)   # 4096^2-equivalent: scale by rows per GPU
+    its = r_p["iters"] / (r_p["ms"] / 1000.0) * eq
+    its_u = r_u["iters"] / (r_u["ms"] / 1000.0) * eq
     peak, peak_src = _peaks()
     ms_t, n_t = r_ps["prof"]         # roofline pass: SpMV launches only
     spmv_ms = ms_t[0] / max(n_t[0], 1)
@@ -348,7 +372,8 @@ def main():
         "vs_baseline": None,
         "dtype": "f64",
         "data": "synthetic",
-        "config": {"workload": "tealeaf-4096x4096-cg-full-ecc", "grid": args.grid, "rows_per_gpu": N,
+        "config": {"workload": f"tealeaf-{args.grid}x{args.grid}-cg-full-ecc", "grid": args.grid, "rows_per_gpu": N,
+                   "chunks": len(P["chunks"]),
                    "schemes": {"elements": "E-SECDED", "rowptr": "R-SECDED64", "vectors": "V-SECDED64"},
                    "tol": args.tol, "iters_per_step": r_p["iters"] / args.steps,
                    "l2": "inputs larger than L2 (2.55 GB moved per CG iteration vs 126 MB L2)",

@@ -164,3 +164,34 @@ def fault_positions(seed: int, count: int, nbits_total: int) -> np.ndarray:
     modulo mapping of splitmix64 outputs (bias < 2^-40 for the sizes used)."""
     r = splitmix64(np.arange(count, dtype=np.uint64), seed)
     return (r % np.uint64(nbits_total)).astype(np.int64)
+
+
+def chunk_plan(n: int, ny: int | None = None, max_cols: int = 1 << 24, chunk_rows: int | None = None):
+    """Row-block chunks (reading R7 / S§8(c) O11) of an n x ny grid so that each
+    chunk's column window [(y0-1)*n, (y1+1)*n) fits the 24-bit element index and
+    its nnz fits 28-bit rowptr entries.  Returns [(y0, y1, col_base)]."""
+    ny = n if ny is None else ny
+
+    def plan(rows):
+        out = []
+        for y0 in range(0, ny, rows):
+            y1 = min(ny, y0 + rows)
+            out.append((y0, y1, max(0, (y0 - 1) * n)))
+        return out
+
+    def fits(pl):
+        return all((min(ny, y1 + 1) * n - cb) <= max_cols and 5 * (y1 - y0) * n <= (1 << 28) - 1
+                   for (y0, y1, cb) in pl)
+
+    if chunk_rows is not None:
+        return plan(chunk_rows)
+    rows = ny
+    while not fits(plan(rows)):
+        rows //= 2
+    return plan(rows)
+
+
+def chunk_csr(n: int, y0: int, y1: int, col_base: int, ny: int | None = None, device="cpu", kind: str = "tea"):
+    """CSR of grid rows [y0, y1) with column indices relative to col_base
+    (global index - col_base), for a chunk that reads the global vector."""
+    return strip_csr(n, y0, y1, ny=ny, kind=kind, device=device, col_offset=y0 * n - col_base)

@@ -56,6 +56,7 @@ struct abft_ctx {
   double prof_ms[4] = {0, 0, 0, 0};
   int64_t prof_n[4] = {0, 0, 0, 0};
   std::vector<cudaEvent_t> events;
+  RedState* red = nullptr;   // fused-reduction counters/roots (zero between reductions)
 };
 
 namespace {
@@ -93,7 +94,7 @@ int check_chunks(const abft_csr* A, int nchunks) {
 // Launch the SpMV over all chunks; partials indexed by global RB (chunks must
 // start on 256-row boundaries relative to chunk 0 when dot is requested).
 int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, bool dot,
-                DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total) {
+                DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total, RedArgs red = RedArgs{}) {
   const int64_t base0 = A[0].row_base;
   const int64_t npad_in = vec_padded_len(in->n, in->scheme);
   const int64_t npad_out = vec_padded_len(out->n, out->scheme);
@@ -133,6 +134,8 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.counts = cnt;
     a.due = ctx->due;
     a.state = st;
+    a.red = red;
+    if (a.red.rs) a.red.nrb = nrb_all;
     count_launch(launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s));
   }
   if (nrb_total) *nrb_total = nrb_all;
@@ -162,6 +165,8 @@ int abft_ctx_create(int device, abft_ctx** out) {
   CUDA_TRY(cudaMalloc(&c->due, sizeof(int) * 4));
   CUDA_TRY(cudaMemset(c->due, 0, sizeof(int) * 4));
   CUDA_TRY(cudaMalloc(&c->flags, sizeof(uint32_t) * 4));
+  CUDA_TRY(cudaMalloc(&c->red, sizeof(RedState)));
+  CUDA_TRY(cudaMemset(c->red, 0, sizeof(RedState)));
   CUDA_TRY(cudaMallocHost(&c->h_state, sizeof(CgState)));
   CUDA_TRY(cudaMallocHost(&c->h_flags, sizeof(uint32_t) * 4));
   int e = ensure_partials(c, 1024);
@@ -179,6 +184,7 @@ int abft_ctx_destroy(abft_ctx* c) {
   cudaFree(c->state);
   cudaFree(c->due);
   cudaFree(c->flags);
+  cudaFree(c->red);
   cudaFreeHost(c->h_state);
   cudaFreeHost(c->h_flags);
   for (auto e : c->events) cudaEventDestroy(e);
@@ -241,9 +247,11 @@ int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_
   if (in->scheme != out->scheme) return fail(ABFT_E_INVALID, "in/out schemes differ");
   cudaStream_t s = (cudaStream_t)stream;
   int64_t nrb = 0;
-  e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb);
+  RedArgs red{};
+  if (dot_out) { red.rs = ctx->red; red.op = 0; red.out = dot_out; red.due = ctx->due; }
+  e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb,
+                  red);
   if (e) return e;
-  if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
   CUDA_TRY(cudaGetLastError());
   return ABFT_OK;
 }
@@ -343,14 +351,21 @@ int halo_exchange(abft_dist* d, uint64_t* ext, int64_t n_loc, int64_t n_halo, cu
   return ABFT_OK;
 }
 
-// Dot-product finish: single GPU -> reduce with op; multi-GPU -> subtree root +
-// DUE flag, all-gather, identical top-of-tree combine on every rank.
-int finish_dot(abft_ctx* ctx, abft_dist* d, int64_t nrb, int op, cudaStream_t s) {
-  if (!d) {
-    count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, op, ctx->state, nullptr, ctx->due, s));
-    return ABFT_OK;
-  }
-  count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 4, nullptr, d->sendbuf, ctx->due, s));
+// Fused dot-product finish: single GPU -> the producer kernel's
+// last warp applies `op`; multi-GPU -> it writes (subtree root, DUE flag) to
+// sendbuf, then all-gather + identical top-of-tree combine on every rank.
+RedArgs red_for(abft_ctx* ctx, abft_dist* d, int64_t nrb, int op) {
+  RedArgs r{};
+  r.rs = ctx->red;
+  r.nrb = nrb;
+  r.due = ctx->due;
+  r.st = ctx->state;
+  if (d) { r.op = 4; r.out = d->sendbuf; }
+  else r.op = op;
+  return r;
+}
+int finish_dot(abft_ctx* ctx, abft_dist* d, int op, cudaStream_t s) {
+  if (!d) return ABFT_OK;
   NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
   count_launch(launch_combine(d->gathered, d->nranks, op, ctx->state, ctx->due, s));
   return ABFT_OK;
@@ -409,6 +424,7 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   va.counts = cnt;
   va.due = ctx->due;
   va.state = ctx->state;
+  va.red = red_for(ctx, d, nrb, 1);
 
   Prof prof{ctx, s};
   // init (a2): w = A x0 ; r = b - w ; p = r ; rr0
@@ -418,7 +434,7 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   prof.end();
   if (e) return e;
   count_launch(launch_init_r(va, scheme, s));
-  if ((e = finish_dot(ctx, d, nrb, 1, s))) return e;
+  if ((e = finish_dot(ctx, d, 1, s))) return e;
   CUDA_TRY(cudaGetLastError());
 
   const int poll = opts->poll_every > 0 ? opts->poll_every : 16;
@@ -429,18 +445,24 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       int e2;
       if ((e2 = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e2;
       prof.begin(0);
-      e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr);
+      e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2));
       prof.end();
       if (e2) return e2;
-      prof.begin(3);
-      if ((e2 = finish_dot(ctx, d, nrb, 2, s))) return e2;
-      prof.end();
+      if (d) {
+        prof.begin(3);
+        if ((e2 = finish_dot(ctx, d, 2, s))) return e2;
+        prof.end();
+      }
       prof.begin(1);
-      count_launch(launch_calc_ur(va, scheme, s));
+      VecArgs vu = va;
+      vu.red = red_for(ctx, d, nrb, 3);
+      count_launch(launch_calc_ur(vu, scheme, s));
       prof.end();
-      prof.begin(3);
-      if ((e2 = finish_dot(ctx, d, nrb, 3, s))) return e2;
-      prof.end();
+      if (d) {
+        prof.begin(3);
+        if ((e2 = finish_dot(ctx, d, 3, s))) return e2;
+        prof.end();
+      }
       prof.begin(2);
       count_launch(launch_calc_p(va, scheme, s));
       prof.end();

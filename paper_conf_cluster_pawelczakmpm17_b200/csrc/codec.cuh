@@ -541,6 +541,36 @@ ABFT_HD void rp_encode_group(uint32_t* e) {
   }
 }
 
+// OR-accumulable fast check of a rowptr group: bit 0 of the result is set
+// iff the group is not clean (parity rows' popcounts OR-ed).
+template <int RS>
+ABFT_HD uint32_t rp_acc(const uint32_t* e) {
+  if (RS == SED) return (uint32_t)popc32(e[0]);
+  if (RS == SECDED64 || RS == SECDED128) {
+    constexpr int NW = (RS == SECDED64) ? 2 : 4;
+    constexpr int R = (RS == SECDED64) ? 7 : 8;
+    const MaskTable& M = (RS == SECDED64) ? ABFT_MT(r64) : ABFT_MT(r128);
+    uint32_t q = 0;
+#pragma unroll
+    for (int i = 0; i < NW; i++) q ^= e[i];
+    uint32_t acc = (uint32_t)popc32(q);
+#pragma unroll
+    for (int k = 0; k < R; k++) {
+      uint32_t t = 0;
+#pragma unroll
+      for (int i = 0; i < NW; i++) t ^= e[i] & M.m[k][i];
+      acc |= (uint32_t)popc32(t);
+    }
+    return acc;
+  }
+  if (RS == CRC32C) {
+    uint32_t st = 0;
+    for (int i = 0; i < 8; i++) st |= (e[i] >> 28) << (4 * i);
+    return st == rcrc_compute(e) ? 0u : 1u;
+  }
+  return 0u;
+}
+
 // Fast-path check of a rowptr group; corrects in place.
 template <int RS>
 ABFT_HD int rp_check_group(uint32_t* e, int* word) {

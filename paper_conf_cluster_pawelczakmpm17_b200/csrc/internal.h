@@ -19,6 +19,25 @@ struct CgState {
 
 struct DevCounts { unsigned long long v[3][5][4]; };
 
+// Fused RED-1 reduction state (ctx scratch, zero between reductions): the warp
+// that writes the last partial of a 1024-leaf group reduces the group, the
+// warp that completes the last group reduces the group roots and applies the
+// CG scalar logic (op) — no separate reduction kernel.
+struct RedState {
+  unsigned int group_ctr[1024];
+  unsigned int top_ctr;
+  unsigned int pad[3];
+  double roots[1024];
+};
+struct RedArgs {
+  RedState* rs;     // null: no fused finish (partials only)
+  int64_t nrb;      // total reduction blocks of the vector (all chunks)
+  int op;           // 0 dot -> out[0], 1 rr0, 2 pw, 3 rrn, 4 root+due -> out[0..2)
+  double* out;
+  CgState* st;
+  const int* due;
+};
+
 // arguments of one SpMV chunk launch
 struct SpmvArgs {
   int64_t nrows, ncols, nnz, row_base, col_base, n_in, npad_in, npad_out, rb_offset;
@@ -32,6 +51,7 @@ struct SpmvArgs {
   DevCounts* counts; // may be null
   int* due;          // DUE / range flag (never null)
   const CgState* state;  // may be null
+  RedArgs red;
 };
 
 struct VecArgs {
@@ -42,6 +62,7 @@ struct VecArgs {
   int* due;
   CgState* state;
   double* out_masked;
+  RedArgs red;
 };
 
 // launchers (kernels.cu); each returns the number of kernels launched

@@ -42,6 +42,9 @@ static __device__ __forceinline__ void load_lut(uint8_t* s_lut) {
   if (threadIdx.x < 32) reinterpret_cast<uint32_t*>(s_lut)[threadIdx.x] = reinterpret_cast<const uint32_t*>(&c_v64_lut)[threadIdx.x];
 }
 
+struct RedArgs;
+static __device__ void red_push(double* partials, int64_t rb, double val, const RedArgs& r, int lane);
+
 // Cold path of a single-codeword vector check (G = 1 schemes).
 template <int VS>
 __device__ __noinline__ uint64_t v1_fix(uint64_t w, uint64_t* addr, bool owner, DevCounts* cnt, int* due) {
@@ -318,7 +321,8 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
   if (DOT) {
 #pragma unroll
     for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-    if (lane == 0) a.partials[a.rb_offset + rb] = dot;
+    if (a.red.rs) red_push(a.partials, a.rb_offset + rb, dot, a.red, lane);
+    else if (lane == 0) a.partials[a.rb_offset + rb] = dot;
   }
 }
 
@@ -558,13 +562,17 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
         }
       }
     }
+    uint32_t acc = 0;
 #pragma unroll
-    for (int q = 0; q < PER; q++) {
-      const int gl = lane + 32 * q;
-      if (gl >= NG) continue;
-      const int64_t g = rowseg / G + gl;
-      uint32_t* gp = a.rowptr + g * G;
-      if (RS != NONE) {
+    for (int q = 0; q < PER; q++)
+      if (RS != NONE && lane + 32 * q < NG) acc |= rp_acc<RS>(e[q]);
+    if (RS != NONE && (acc & 1u)) {  // cold: locate, correct, count (owner), per group
+#pragma unroll
+      for (int q = 0; q < PER; q++) {
+        const int gl = lane + 32 * q;
+        if (gl >= NG) continue;
+        const int64_t g = rowseg / G + gl;
+        uint32_t* gp = a.rowptr + g * G;
         uint32_t o0[G];
 #pragma unroll
         for (int t = 0; t < G; t++) o0[t] = e[q][t];
@@ -582,6 +590,11 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
           }
         }
       }
+    }
+#pragma unroll
+    for (int q = 0; q < PER; q++) {
+      const int gl = lane + 32 * q;
+      if (gl >= NG) continue;
 #pragma unroll
       for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[q][t] & rp_keep(RS);
     }
@@ -662,7 +675,8 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
   if (DOT) {
 #pragma unroll
     for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-    if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
+    if (a.red.rs) red_push(a.partials, a.rb_offset + (rowseg >> 8), dot, a.red, lane);
+    else if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
   }
 }
 
@@ -760,7 +774,8 @@ __global__ void __launch_bounds__(256) k_calc_ur(VecArgs a) {
   }
 #pragma unroll
   for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-  if (lane == 0) a.partials[rb] = dot;
+  if (a.red.rs) red_push(a.partials, rb, dot, a.red, lane);
+  else if (lane == 0) a.partials[rb] = dot;
 }
 
 template <int VS>
@@ -836,7 +851,8 @@ __global__ void __launch_bounds__(256) k_init_r(VecArgs a) {
   }
 #pragma unroll
   for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-  if (lane == 0) a.partials[rb] = dot;
+  if (a.red.rs) red_push(a.partials, rb, dot, a.red, lane);
+  else if (lane == 0) a.partials[rb] = dot;
 }
 
 // ============================================================ reduction (a6)
@@ -877,6 +893,71 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
       st->beta = res / st->rro;
     }
   }
+}
+
+// ---- fused RED-1 finish: called by a whole warp after it
+// produced the partial of reduction block rb.
+static __device__ __forceinline__ int64_t p2ceil(int64_t v) {
+  int64_t p = 1;
+  while (p < v) p <<= 1;
+  return p;
+}
+// Pairwise tree of m = 2^j values held by lanes 0..m-1 (m <= 32): butterfly
+// over offsets 1..m/2 combines adjacent subtrees first; lane 0 gets the root.
+static __device__ __forceinline__ double warp_tree(double v, int m) {
+  for (int off = 1; off < m; off <<= 1) v = v + __shfl_xor_sync(0xffffffffu, v, off);
+  return v;
+}
+// Tree over L = 2^j leaves src[0..L) (src[i] for i >= valid read as 0) by one warp.
+static __device__ double warp_subtree(const double* src, int64_t L, int64_t valid, int lane) {
+  if (L <= 32) {
+    double v = (lane < L && lane < valid) ? __ldcg(src + lane) : 0.0;
+    return warp_tree(v, (int)L);
+  }
+  const int per = (int)(L / 32);  // leaves per lane, power of two <= 32
+  double t[32];
+  for (int i = 0; i < per; i++) {
+    const int64_t j = (int64_t)lane * per + i;
+    t[i] = (j < valid) ? __ldcg(src + j) : 0.0;
+  }
+  for (int m = per; m > 1; m >>= 1)
+    for (int i = 0; i < m / 2; i++) t[i] = t[2 * i] + t[2 * i + 1];
+  return warp_tree(t[0], 32);
+}
+static __device__ void red_push(double* partials, int64_t rb, double val, const RedArgs& r, int lane) {
+  const int64_t P2 = p2ceil(r.nrb);
+  const int64_t L = P2 < 1024 ? P2 : 1024;
+  const int64_t g = rb / L;
+  const int64_t ngr = (r.nrb + L - 1) / L;   // groups holding real partials
+  unsigned last = 0;
+  if (lane == 0) {
+    partials[rb] = val;
+    __threadfence();
+    const int64_t expect = (r.nrb - g * L) < L ? (r.nrb - g * L) : L;
+    last = (atomicAdd(&r.rs->group_ctr[g], 1u) == (unsigned)expect - 1u);
+  }
+  last = __shfl_sync(0xffffffffu, last, 0);
+  if (!last) return;
+  __threadfence();
+  const double root = warp_subtree(partials + g * L, L, r.nrb - g * L, lane);
+  unsigned top = 0;
+  if (lane == 0) {
+    r.rs->group_ctr[g] = 0;
+    r.rs->roots[g] = root;
+    __threadfence();
+    top = (atomicAdd(&r.rs->top_ctr, 1u) == (unsigned)ngr - 1u);
+  }
+  top = __shfl_sync(0xffffffffu, top, 0);
+  if (!top) return;
+  __threadfence();
+  const int64_t ng = P2 / L;
+  const double res = warp_subtree(r.rs->roots, ng, ngr, lane);
+  if (lane != 0) return;
+  r.rs->top_ctr = 0;
+  const int dueflag = *((volatile const int*)r.due);
+  if (r.op == 0) r.out[0] = res;
+  else if (r.op == 4) { r.out[0] = res; r.out[1] = (double)dueflag; }
+  else apply_op(r.op, res, r.st, dueflag != 0);
 }
 
 static __global__ void __launch_bounds__(512) k_reduce(const double* partials, int64_t nrb, int64_t leaves, double* roots,
