@@ -685,6 +685,28 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
 // 8 (calc_ur) / 4 (calc_p, init) independent 8-byte loads in flight, and all
 // addressing is pointer + immediate offset.  Lane l still visits rows
 // l, l+32, ... in ascending order (RED-1).
+// OR-accumulated fast check of up to 8 G=1 codewords (zero words are clean in
+// every scheme): true iff any of them needs the per-word cold path.
+template <int VS>
+__device__ __forceinline__ bool vacc_bad(uint64_t w0, uint64_t w1, uint64_t w2, uint64_t w3, uint64_t w4, uint64_t w5,
+                                         uint64_t w6, uint64_t w7) {
+  if (VS == SED) return ((popc64(w0) | popc64(w1) | popc64(w2) | popc64(w3) | popc64(w4) | popc64(w5) |
+                          popc64(w6) | popc64(w7)) & 1) != 0;
+  if (VS == SECDED64) {
+    uint32_t r = 0, p = 0;
+    v64_acc(lo32(w0), hi32(w0), r, p);
+    v64_acc(lo32(w1), hi32(w1), r, p);
+    v64_acc(lo32(w2), hi32(w2), r, p);
+    v64_acc(lo32(w3), hi32(w3), r, p);
+    v64_acc(lo32(w4), hi32(w4), r, p);
+    v64_acc(lo32(w5), hi32(w5), r, p);
+    v64_acc(lo32(w6), hi32(w6), r, p);
+    v64_acc(lo32(w7), hi32(w7), r, p);
+    return syn_bad(r, p);
+  }
+  return false;
+}
+
 template <int VS>
 __device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int lane, double alpha, const uint8_t* lut) {
   uint64_t* X = a.x + base + lane;
@@ -697,14 +719,16 @@ __device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int la
   for (int k = 0; k < 256; k += 64) {
     uint64_t x0 = ldg64(X + k), x1 = ldg64(X + k + 32), p0 = ldg64(P + k), p1 = ldg64(P + k + 32);
     uint64_t r0 = ldg64(R + k), r1 = ldg64(R + k + 32), w0 = ldg64(W + k), w1 = ldg64(W + k + 32);
-    x0 = v1_check<VS>(x0, X + k, true, a.counts, a.due);
-    x1 = v1_check<VS>(x1, X + k + 32, true, a.counts, a.due);
-    p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
-    p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
-    r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
-    r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
-    w0 = v1_check<VS>(w0, W + k, true, a.counts, a.due);
-    w1 = v1_check<VS>(w1, W + k + 32, true, a.counts, a.due);
+    if (vacc_bad<VS>(x0, x1, p0, p1, r0, r1, w0, w1)) {  // cold: locate per word
+      x0 = v1_check<VS>(x0, X + k, true, a.counts, a.due);
+      x1 = v1_check<VS>(x1, X + k + 32, true, a.counts, a.due);
+      p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
+      p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
+      r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
+      r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
+      w0 = v1_check<VS>(w0, W + k, true, a.counts, a.due);
+      w1 = v1_check<VS>(w1, W + k + 32, true, a.counts, a.due);
+    }
     const double xn0 = fma(alpha, as_d(p0 & keep), as_d(x0 & keep));
     const double xn1 = fma(alpha, as_d(p1 & keep), as_d(x1 & keep));
     const double rn0 = fma(-alpha, as_d(w0 & keep), as_d(r0 & keep));
@@ -729,10 +753,12 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
 #pragma unroll 1
   for (int k = 0; k < 256; k += 64) {
     uint64_t r0 = ldg64(R + k), r1 = ldg64(R + k + 32), p0 = ldg64(P + k), p1 = ldg64(P + k + 32);
-    r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
-    r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
-    p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
-    p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
+    if (vacc_bad<VS>(r0, r1, p0, p1, 0ull, 0ull, 0ull, 0ull)) {  // cold: locate per word
+      r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
+      r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
+      p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
+      p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
+    }
     const double n0 = fma(beta, as_d(p0 & keep), as_d(r0 & keep));
     const double n1 = fma(beta, as_d(p1 & keep), as_d(r1 & keep));
     P[k] = v_encode<VS>(round_k(as_u(n0), vk(VS)), lane, lut);
