@@ -247,11 +247,9 @@ int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_
   if (in->scheme != out->scheme) return fail(ABFT_E_INVALID, "in/out schemes differ");
   cudaStream_t s = (cudaStream_t)stream;
   int64_t nrb = 0;
-  RedArgs red{};
-  if (dot_out) { red.rs = ctx->red; red.op = 0; red.out = dot_out; red.due = ctx->due; }
-  e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb,
-                  red);
+  e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb);
   if (e) return e;
+  if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
   CUDA_TRY(cudaGetLastError());
   return ABFT_OK;
 }
@@ -354,18 +352,21 @@ int halo_exchange(abft_dist* d, uint64_t* ext, int64_t n_loc, int64_t n_halo, cu
 // Fused dot-product finish: single GPU -> the producer kernel's
 // last warp applies `op`; multi-GPU -> it writes (subtree root, DUE flag) to
 // sendbuf, then all-gather + identical top-of-tree combine on every rank.
-RedArgs red_for(abft_ctx* ctx, abft_dist* d, int64_t nrb, int op) {
-  RedArgs r{};
-  r.rs = ctx->red;
-  r.nrb = nrb;
-  r.due = ctx->due;
-  r.st = ctx->state;
-  if (d) { r.op = 4; r.out = d->sendbuf; }
-  else r.op = op;
-  return r;
+RedArgs red_for(abft_ctx*, abft_dist*, int64_t, int) {
+  // Fused last-warp reductions (RedState) measured slower than a separate
+  // reduction kernel: the per-warp __threadfence before the group counter
+  // stalls every producer warp on its own outstanding stores (r14: SpMV
+  // 0.295 -> 0.327 ms).  Kept disabled; partials are reduced by k_reduce.
+  return RedArgs{};
 }
-int finish_dot(abft_ctx* ctx, abft_dist* d, int op, cudaStream_t s) {
-  if (!d) return ABFT_OK;
+// Dot-product finish: single GPU -> k_reduce applies `op`; multi-GPU -> subtree
+// root + DUE flag, all-gather, identical top-of-tree combine on every rank.
+int finish_dot(abft_ctx* ctx, abft_dist* d, int64_t nrb, int op, cudaStream_t s) {
+  if (!d) {
+    count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, op, ctx->state, nullptr, ctx->due, s));
+    return ABFT_OK;
+  }
+  count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 4, nullptr, d->sendbuf, ctx->due, s));
   NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
   count_launch(launch_combine(d->gathered, d->nranks, op, ctx->state, ctx->due, s));
   return ABFT_OK;
@@ -434,7 +435,7 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   prof.end();
   if (e) return e;
   count_launch(launch_init_r(va, scheme, s));
-  if ((e = finish_dot(ctx, d, 1, s))) return e;
+  if ((e = finish_dot(ctx, d, nrb, 1, s))) return e;
   CUDA_TRY(cudaGetLastError());
 
   const int poll = opts->poll_every > 0 ? opts->poll_every : 16;
@@ -448,21 +449,17 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2));
       prof.end();
       if (e2) return e2;
-      if (d) {
-        prof.begin(3);
-        if ((e2 = finish_dot(ctx, d, 2, s))) return e2;
-        prof.end();
-      }
+      prof.begin(3);
+      if ((e2 = finish_dot(ctx, d, nrb, 2, s))) return e2;
+      prof.end();
       prof.begin(1);
       VecArgs vu = va;
       vu.red = red_for(ctx, d, nrb, 3);
       count_launch(launch_calc_ur(vu, scheme, s));
       prof.end();
-      if (d) {
-        prof.begin(3);
-        if ((e2 = finish_dot(ctx, d, 3, s))) return e2;
-        prof.end();
-      }
+      prof.begin(3);
+      if ((e2 = finish_dot(ctx, d, nrb, 3, s))) return e2;
+      prof.end();
       prof.begin(2);
       count_launch(launch_calc_p(va, scheme, s));
       prof.end();

@@ -124,7 +124,7 @@ int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* 
   while (p2 < nrb) p2 <<= 1;
   int64_t leaves = p2 < 1024 ? p2 : 1024;
   int blocks = (int)(p2 / leaves);
-  k_reduce<<<blocks, 512, 0, s>>>(partials, nrb, leaves, roots, ticket, op, st, out, due);
+  k_reduce<<<blocks, 256, 0, s>>>(partials, nrb, leaves, roots, ticket, op, st, out, due);
   return 1;
 }
 

@@ -986,30 +986,38 @@ static __device__ void red_push(double* partials, int64_t rb, double val, const 
   else apply_op(r.op, res, r.st, dueflag != 0);
 }
 
-static __global__ void __launch_bounds__(512) k_reduce(const double* partials, int64_t nrb, int64_t leaves, double* roots,
+static __global__ void __launch_bounds__(256) k_reduce(const double* partials, int64_t nrb, int64_t leaves, double* roots,
                                                 uint32_t* ticket, int op, CgState* st, double* out, const int* due) {
-  __shared__ double s[1024];
+  // Block b reduces leaves [b*L, b*L+L): warp w the aligned sub-range of L/8
+  // leaves (warp trees keep the pairwise order), then warp 0 combines the 8
+  // warp roots; the last block (ticket) combines the block roots.
+  __shared__ double s_w[8];
   __shared__ bool s_last;
   if (st && op != 1 && st->stop) return;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t base = (int64_t)blockIdx.x * leaves;
-  for (int64_t t = threadIdx.x; t < leaves; t += blockDim.x) s[t] = (base + t < nrb) ? partials[base + t] : 0.0;
+  const int nw = leaves >= 8 ? 8 : 1;
+  const int64_t per = leaves / nw;
+  if (warp < nw) {
+    const double r = warp_subtree(partials + base + warp * per, per, nrb - base - warp * per, lane);
+    if (lane == 0) s_w[warp] = r;
+  }
   __syncthreads();
-  double root = tree_smem(s, (int)leaves);
-  if (gridDim.x == 1) {
-    s_last = true;
-  } else {
+  double root = 0.0;
+  if (warp == 0) {
+    const double v = (lane < nw) ? s_w[lane] : 0.0;
+    root = warp_tree(v, nw);
+  }
+  if (gridDim.x > 1) {
     if (threadIdx.x == 0) {
       roots[blockIdx.x] = root;
       __threadfence();
       s_last = (atomicAdd(ticket, 1u) == gridDim.x - 1);
     }
     __syncthreads();
-    if (!s_last) return;
+    if (!s_last || warp != 0) return;
     __threadfence();
-    const int nb = gridDim.x;
-    for (int t = threadIdx.x; t < nb; t += blockDim.x) s[t] = ((volatile double*)roots)[t];
-    __syncthreads();
-    root = tree_smem(s, nb);
+    root = warp_subtree(roots, gridDim.x, gridDim.x, lane);
   }
   if (threadIdx.x != 0) return;
   if (gridDim.x > 1) *ticket = 0;
