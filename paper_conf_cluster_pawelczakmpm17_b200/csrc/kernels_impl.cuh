@@ -395,6 +395,42 @@ static __device__ __forceinline__ bool tile_issue(const SpmvArgs& a, uint32_t s0
   return true;
 }
 
+// Register-staged alternative to the TMA bulk copy (TILE_TMA = false): the
+// warp loads the pass's packed (val, col) range with 16-byte coalesced loads
+// (<= 4 per lane), writes it to the pass buffer one pass later.  Fewer issue
+// slots than the elected-lane cp.async.bulk sequence.
+constexpr bool TILE_TMA = false;
+struct PassRegs { uint4 q[4]; };
+static __device__ __forceinline__ bool pass_ok(uint32_t s0, uint32_t s1, int64_t nnz) {
+  return s0 <= s1 && (int64_t)s1 <= nnz && s1 - s0 <= 160u;
+}
+static __device__ __forceinline__ void pass_load(const SpmvArgs& a, uint32_t s0, uint32_t s1, int lane, PassRegs& R) {
+  const uint32_t e0 = s0 & ~1u, e1 = (s1 + 1u) & ~1u;
+  const uint32_t c0 = s0 & ~3u, c1 = (s1 + 3u) & ~3u;
+  const int nv = (int)((e1 - e0) >> 1), nc = (int)((c1 - c0) >> 2);
+  const uint4* vsrc = reinterpret_cast<const uint4*>(a.val + e0);
+  const uint4* csrc = reinterpret_cast<const uint4*>(a.col + c0);
+#pragma unroll
+  for (int q = 0; q < 4; q++) {
+    const int j = lane + 32 * q;
+    if (j < nv) R.q[q] = __ldg(vsrc + j);
+    else if (j - nv < nc) R.q[q] = __ldg(csrc + (j - nv));
+  }
+}
+static __device__ __forceinline__ void pass_store(uint32_t s0, uint32_t s1, int lane, const PassRegs& R, uint8_t* buf) {
+  const uint32_t e0 = s0 & ~1u, e1 = (s1 + 1u) & ~1u;
+  const uint32_t c0 = s0 & ~3u, c1 = (s1 + 3u) & ~3u;
+  const int nv = (int)((e1 - e0) >> 1), nc = (int)((c1 - c0) >> 2);
+  uint4* vdst = reinterpret_cast<uint4*>(buf);
+  uint4* cdst = reinterpret_cast<uint4*>(buf + TILE_EBUF * 8);
+#pragma unroll
+  for (int q = 0; q < 4; q++) {
+    const int j = lane + 32 * q;
+    if (j < nv) vdst[j] = R.q[q];
+    else if (j - nv < nc) cdst[j - nv] = R.q[q];
+  }
+}
+
 // One row, general case: check/correct its elements (from SMEM or global),
 // gather, fma chain.  Also the cold path of the 5-entry fast path below.
 template <int ES, int RS, int VS>
@@ -479,34 +515,33 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
     v[t] = sval[start + t - sbase_v];
     c[t] = scol[start + t - sbase_c];
   }
-  uint32_t acc_r = 0, acc_p = 0, bad = 0;
-  int sd[5];
-  const int canon[5] = {-n32, -1, 0, 1, n32};
-  const int canon_sd[5] = {-TILE_WW, -1, 0, 1, TILE_WW};
-  const uint32_t ncols32 = (uint32_t)a.ncols;
-  uint32_t cmax = 0;
+  uint32_t acc_r = 0, acc_p = 0;
 #pragma unroll
   for (int t = 0; t < 5; t++) {
     if (ES == SED) acc_p |= (uint32_t)(popc64(v[t]) + popc32(c[t]));
     else if (ES != NONE) e96_acc(lo32(v[t]), hi32(v[t]), c[t], acc_r, acc_p);
-    const uint32_t cm = c[t] & ckeep;
-    cmax = max(cmax, cm);
-    const int d = (int)cm - own_col;
-    sd[t] = (d == 0) ? 0 : canon_sd[t];
-    bad |= (d == 0 || d == canon[t]) ? 0u : 1u;
   }
-  if (ES != NONE) {
-    if (syn_bad(acc_r, acc_p)) bad = 1u;
-    if (a.ncols > 0xFFFFFFFFll ? false : cmax >= ncols32) bad = 1u;
-  }
-  if (bad)
-    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own, s0, s1);
-  double acc = 0.0;
+  // canonical stencil neighbours [i-n, i-1, i, i+1, i+n] or the row itself (R16)
+  int d[5];
+  uint32_t cmax = 0;
 #pragma unroll
   for (int t = 0; t < 5; t++) {
-    const double x = (sd[t] == 0) ? p_own : win[oslot + sd[t]];
-    acc = fma(as_d(v[t]), x, acc);
+    const uint32_t cm = c[t] & ckeep;
+    cmax = max(cmax, cm);
+    d[t] = (int)cm - own_col;
   }
+  const bool canon = (d[0] == 0 || d[0] == -n32) && ((unsigned)(d[1] + 1) <= 1u) && d[2] == 0 &&
+                     ((unsigned)d[3] <= 1u) && (d[4] == 0 || d[4] == n32);
+  const bool in_range = (ES == NONE) || cmax < (uint32_t)a.ncols;
+  if ((ES != NONE && syn_bad(acc_r, acc_p)) || !canon || !in_range)
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own, s0, s1);
+  // slot offsets: d itself for +-1 / 0, +-window width for +-n
+  const int o0 = d[0] ? -TILE_WW : 0, o4 = d[4] ? TILE_WW : 0;
+  double acc = fma(as_d(v[0]), win[oslot + o0], 0.0);
+  acc = fma(as_d(v[1]), win[oslot + d[1]], acc);
+  acc = fma(as_d(v[2]), p_own, acc);
+  acc = fma(as_d(v[3]), win[oslot + d[3]], acc);
+  acc = fma(as_d(v[4]), win[oslot + o4], acc);
   return acc;
 }
 
@@ -541,6 +576,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
   const int64_t rowseg = gy * n + tx0;
   // ---- 1. rowptr of the segment (entries rowseg .. rowseg+256), then the first two element copies
   uint32_t stmask = 0u;  // bit b: buffer b holds the current pass (TMA issued)
+  PassRegs pre;          // register-staged next pass (TILE_TMA = false)
   if (has_seg) {
     constexpr int G = rgrp(RS);
     constexpr int NG = 256 / G + 1;
@@ -599,8 +635,17 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
       for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[q][t] & rp_keep(RS);
     }
     __syncwarp();
-    stmask |= tile_issue(a, srp[0], srp[32], wbase, &bars[0], lane) ? 1u : 0u;
-    stmask |= tile_issue(a, srp[32], srp[64], wbase + TILE_BUF_BYTES, &bars[1], lane) ? 2u : 0u;
+    if (TILE_TMA) {
+      stmask |= tile_issue(a, srp[0], srp[32], wbase, &bars[0], lane) ? 1u : 0u;
+      stmask |= tile_issue(a, srp[32], srp[64], wbase + TILE_BUF_BYTES, &bars[1], lane) ? 2u : 0u;
+    } else {
+      if (pass_ok(srp[0], srp[32], a.nnz)) {       // pass 0 -> buffer 0 now, pass 1 in flight
+        pass_load(a, srp[0], srp[32], lane, pre);
+        pass_store(srp[0], srp[32], lane, pre, wbase);
+        stmask |= 1u;
+      }
+      if (pass_ok(srp[32], srp[64], a.nnz)) pass_load(a, srp[32], srp[64], lane, pre);
+    }
   }
   // ---- 2. decoded `in` window
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
@@ -650,7 +695,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
     const uint32_t s0 = srp[32 * k];
     const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
     const bool st = (stmask >> b) & 1u;
-    if (st) {
+    if (TILE_TMA && st) {
       mbar_wait(&bars[b], (phmask >> b) & 1u);
       phmask ^= 1u << b;
     }
@@ -667,9 +712,21 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
     a.out[own] = enc;
     if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
     __syncwarp();
-    if (k + 2 < 8) {
-      const bool ok = tile_issue(a, srp[32 * (k + 2)], srp[32 * (k + 3)], bb, &bars[b], lane);
-      stmask = (stmask & ~(1u << b)) | ((ok ? 1u : 0u) << b);
+    if (TILE_TMA) {
+      if (k + 2 < 8) {
+        const bool ok = tile_issue(a, srp[32 * (k + 2)], srp[32 * (k + 3)], bb, &bars[b], lane);
+        stmask = (stmask & ~(1u << b)) | ((ok ? 1u : 0u) << b);
+      }
+    } else if (k + 1 < 8) {
+      // pass k+1: registers -> the other buffer (pass k-1 is done with it); then prefetch pass k+2
+      const uint32_t t0 = srp[32 * (k + 1)], t1 = srp[32 * (k + 2)];
+      const int nb = b ^ 1;
+      const bool ok = pass_ok(t0, t1, a.nnz);
+      if (ok) pass_store(t0, t1, lane, pre, wbase + nb * TILE_BUF_BYTES);
+      stmask = (stmask & ~(1u << nb)) | ((ok ? 1u : 0u) << nb);
+      __syncwarp();
+      if (k + 2 < 8 && pass_ok(srp[32 * (k + 2)], srp[32 * (k + 3)], a.nnz))
+        pass_load(a, srp[32 * (k + 2)], srp[32 * (k + 3)], lane, pre);
     }
   }
   if (DOT) {
@@ -768,7 +825,7 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
 
 
 template <int VS>
-__global__ void __launch_bounds__(256) k_calc_ur(VecArgs a) {
+__global__ void __launch_bounds__(256, 4) k_calc_ur(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
   if (VS == SECDED64) load_lut(s_lut);
   __syncthreads();
@@ -805,7 +862,7 @@ __global__ void __launch_bounds__(256) k_calc_ur(VecArgs a) {
 }
 
 template <int VS>
-__global__ void __launch_bounds__(256) k_calc_p(VecArgs a) {
+__global__ void __launch_bounds__(256, 6) k_calc_p(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
   __shared__ bool s_last;
   if (VS == SECDED64) load_lut(s_lut);
