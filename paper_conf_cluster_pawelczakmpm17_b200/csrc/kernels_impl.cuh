@@ -399,7 +399,7 @@ static __device__ __forceinline__ bool tile_issue(const SpmvArgs& a, uint32_t s0
 // warp loads the pass's packed (val, col) range with 16-byte coalesced loads
 // (<= 4 per lane), writes it to the pass buffer one pass later.  Fewer issue
 // slots than the elected-lane cp.async.bulk sequence.
-constexpr bool TILE_TMA = false;
+constexpr bool TILE_TMA = true;
 struct PassRegs { uint4 q[4]; };
 static __device__ __forceinline__ bool pass_ok(uint32_t s0, uint32_t s1, int64_t nnz) {
   return s0 <= s1 && (int64_t)s1 <= nnz && s1 - s0 <= 160u;
