@@ -565,7 +565,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
   }
   __syncwarp();
-  if (a.state && a.state->stop) return;  // uniform per grid
+  const int stop_v = a.state ? a.state->stop : 0;  // checked after the prologue loads are in flight
   const int64_t n = a.stencil_n;
   const int64_t ny = a.nrows / n;
   const int64_t tiles_x = n >> 8;
@@ -598,6 +598,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
         }
       }
     }
+    if (stop_v) return;
     uint32_t acc = 0;
 #pragma unroll
     for (int q = 0; q < PER; q++)
@@ -647,6 +648,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
       if (pass_ok(srp[32], srp[64], a.nnz)) pass_load(a, srp[32], srp[64], lane, pre);
     }
   }
+  if (stop_v) return;  // uniform per grid
   // ---- 2. decoded `in` window
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
   constexpr int WPER = (TILE_WW + 31) / 32;                      // 9 slots per lane per window row
@@ -765,17 +767,40 @@ __device__ __forceinline__ bool vacc_bad(uint64_t w0, uint64_t w1, uint64_t w2, 
 }
 
 template <int VS>
-__device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int lane, double alpha, const uint8_t* lut) {
+struct UrStep { uint64_t x0, x1, p0, p1, r0, r1, w0, w1; };
+template <int VS>
+__device__ __forceinline__ void ur_load(const uint64_t* X, const uint64_t* P, const uint64_t* R, const uint64_t* W, int k,
+                                        UrStep<VS>& s) {
+  s.x0 = ldg64(X + k); s.x1 = ldg64(X + k + 32); s.p0 = ldg64(P + k); s.p1 = ldg64(P + k + 32);
+  s.r0 = ldg64(R + k); s.r1 = ldg64(R + k + 32); s.w0 = ldg64(W + k); s.w1 = ldg64(W + k + 32);
+}
+template <int VS>
+__device__ __forceinline__ void ur_step(const VecArgs& a, uint64_t* X, uint64_t* P, uint64_t* R, uint64_t* W, int k,
+                                        const UrStep<VS>& s, double alpha, int lane, const uint8_t* lut, double& dot);
+// Full RB of calc_ur; step 0's loads were issued by the caller before the
+// kernel's barrier / stop check so their latency overlaps the state loads.
+template <int VS>
+__device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int lane, double alpha, const uint8_t* lut,
+                                          UrStep<VS> s) {
   uint64_t* X = a.x + base + lane;
   uint64_t* P = a.p + base + lane;
   uint64_t* R = a.r + base + lane;
   uint64_t* W = a.w + base + lane;
-  const uint64_t keep = vkeep(VS);
   double dot = 0.0;
+  ur_step<VS>(a, X, P, R, W, 0, s, alpha, lane, lut, dot);
 #pragma unroll 1
-  for (int k = 0; k < 256; k += 64) {
-    uint64_t x0 = ldg64(X + k), x1 = ldg64(X + k + 32), p0 = ldg64(P + k), p1 = ldg64(P + k + 32);
-    uint64_t r0 = ldg64(R + k), r1 = ldg64(R + k + 32), w0 = ldg64(W + k), w1 = ldg64(W + k + 32);
+  for (int k = 64; k < 256; k += 64) {
+    ur_load<VS>(X, P, R, W, k, s);
+    ur_step<VS>(a, X, P, R, W, k, s, alpha, lane, lut, dot);
+  }
+  return dot;
+}
+template <int VS>
+__device__ __forceinline__ void ur_step(const VecArgs& a, uint64_t* X, uint64_t* P, uint64_t* R, uint64_t* W, int k,
+                                        const UrStep<VS>& s, double alpha, int lane, const uint8_t* lut, double& dot) {
+  const uint64_t keep = vkeep(VS);
+  {
+    uint64_t x0 = s.x0, x1 = s.x1, p0 = s.p0, p1 = s.p1, r0 = s.r0, r1 = s.r1, w0 = s.w0, w1 = s.w1;
     if (vacc_bad<VS>(x0, x1, p0, p1, r0, r1, w0, w1)) {  // cold: locate per word
       x0 = v1_check<VS>(x0, X + k, true, a.counts, a.due);
       x1 = v1_check<VS>(x1, X + k + 32, true, a.counts, a.due);
@@ -800,43 +825,54 @@ __device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int la
     dot = fma(m0, m0, dot);
     dot = fma(m1, m1, dot);
   }
-  return dot;
 }
 template <int VS>
-__device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane, double beta, const uint8_t* lut) {
+__device__ __forceinline__ void p_step(const VecArgs& a, uint64_t* P, uint64_t* R, int k, uint64_t r0, uint64_t r1,
+                                       uint64_t p0, uint64_t p1, double beta, int lane, const uint8_t* lut) {
+  const uint64_t keep = vkeep(VS);
+  if (vacc_bad<VS>(r0, r1, p0, p1, 0ull, 0ull, 0ull, 0ull)) {  // cold: locate per word
+    r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
+    r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
+    p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
+    p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
+  }
+  const double n0 = fma(beta, as_d(p0 & keep), as_d(r0 & keep));
+  const double n1 = fma(beta, as_d(p1 & keep), as_d(r1 & keep));
+  P[k] = v_encode<VS>(round_k(as_u(n0), vk(VS)), lane, lut);
+  P[k + 32] = v_encode<VS>(round_k(as_u(n1), vk(VS)), lane, lut);
+}
+// Full RB of calc_p; step 0's words were loaded by the caller ahead of the
+// barrier / stop check.
+template <int VS>
+__device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane, double beta, const uint8_t* lut,
+                                       uint64_t r0, uint64_t r1, uint64_t p0, uint64_t p1) {
   uint64_t* P = a.p + base + lane;
   uint64_t* R = a.r + base + lane;
-  const uint64_t keep = vkeep(VS);
+  p_step<VS>(a, P, R, 0, r0, r1, p0, p1, beta, lane, lut);
 #pragma unroll 1
-  for (int k = 0; k < 256; k += 64) {
-    uint64_t r0 = ldg64(R + k), r1 = ldg64(R + k + 32), p0 = ldg64(P + k), p1 = ldg64(P + k + 32);
-    if (vacc_bad<VS>(r0, r1, p0, p1, 0ull, 0ull, 0ull, 0ull)) {  // cold: locate per word
-      r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
-      r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
-      p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
-      p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
-    }
-    const double n0 = fma(beta, as_d(p0 & keep), as_d(r0 & keep));
-    const double n1 = fma(beta, as_d(p1 & keep), as_d(r1 & keep));
-    P[k] = v_encode<VS>(round_k(as_u(n0), vk(VS)), lane, lut);
-    P[k + 32] = v_encode<VS>(round_k(as_u(n1), vk(VS)), lane, lut);
-  }
+  for (int k = 64; k < 256; k += 64)
+    p_step<VS>(a, P, R, k, ldg64(R + k), ldg64(R + k + 32), ldg64(P + k), ldg64(P + k + 32), beta, lane, lut);
 }
 
 
 template <int VS>
 __global__ void __launch_bounds__(256, 4) k_calc_ur(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
-  if (VS == SECDED64) load_lut(s_lut);
-  __syncthreads();
-  if (a.state->stop) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
-  if (rb * 256 >= a.n) return;
+  const bool full = vgrp(VS) == 1 && rb * 256 + 256 <= a.n;
+  UrStep<VS> s0{};
+  if (full)  // issue step 0 first: its latency overlaps the state loads and the barrier
+    ur_load<VS>(a.x + rb * 256 + lane, a.p + rb * 256 + lane, a.r + rb * 256 + lane, a.w + rb * 256 + lane, 0, s0);
+  const int stop = a.state->stop;
   const double alpha = a.state->alpha;
+  if (VS == SECDED64) load_lut(s_lut);
+  __syncthreads();
+  if (stop) return;
+  if (rb * 256 >= a.n) return;
   double dot = 0.0;
-  if (vgrp(VS) == 1 && rb * 256 + 256 <= a.n) {
-    dot = ur_full<VS>(a, rb * 256, lane, alpha, s_lut);
+  if (full) {
+    dot = ur_full<VS>(a, rb * 256, lane, alpha, s_lut, s0);
   } else for (int k = 0; k < 8; k++) {
     const int64_t pb = rb * 256 + k * 32;
     if (pb >= a.n) break;
@@ -865,14 +901,22 @@ template <int VS>
 __global__ void __launch_bounds__(256, 6) k_calc_p(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
   __shared__ bool s_last;
-  if (VS == SECDED64) load_lut(s_lut);
-  __syncthreads();
-  if (a.state->stop) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  const bool full = vgrp(VS) == 1 && rb * 256 + 256 <= a.n;
+  uint64_t r0 = 0, r1 = 0, p0 = 0, p1 = 0;
+  if (full) {  // issue step 0 first: its latency overlaps the state loads and the barrier
+    const uint64_t* R = a.r + rb * 256 + lane;
+    const uint64_t* P = a.p + rb * 256 + lane;
+    r0 = ldg64(R); r1 = ldg64(R + 32); p0 = ldg64(P); p1 = ldg64(P + 32);
+  }
+  const int stop = a.state->stop;
   const double beta = a.state->beta;
-  if (vgrp(VS) == 1 && rb * 256 + 256 <= a.n) {
-    p_full<VS>(a, rb * 256, lane, beta, s_lut);
+  if (VS == SECDED64) load_lut(s_lut);
+  __syncthreads();
+  if (stop) return;
+  if (full) {
+    p_full<VS>(a, rb * 256, lane, beta, s_lut, r0, r1, p0, p1);
   } else if (rb * 256 < a.n) {
     for (int k = 0; k < 8; k++) {
       const int64_t pb = rb * 256 + k * 32;

@@ -27,5 +27,10 @@ for w in $WHAT; do
     timeout 900 ncu --set full --clock-control none --import-source on -k regex:'k_spmv' -s 2 -c 4 \
       -o gpurun_out/prof_$TAG -f python bench.py --steps 1 --warmup 0 --no-e2e --no-cpu-baseline --max-iters 3 > gpurun_out/ncu_full_$TAG.log 2>&1
     tail -3 gpurun_out/ncu_full_$TAG.log ;;
+  sweep)
+    timeout 1500 python tools/sweep.py --out gpurun_out/sweep_$TAG.json > gpurun_out/sweep_$TAG.log 2>&1; tail -4 gpurun_out/sweep_$TAG.log ;;
+  big)
+    timeout 1200 python bench.py --grid 16384 --steps 2 --warmup 3 --max-iters 3000 --no-cpu-baseline > gpurun_out/bench16k_$TAG.json 2> gpurun_out/bench16k_$TAG.err
+    tail -3 gpurun_out/bench16k_$TAG.err; cat gpurun_out/bench16k_$TAG.json ;;
   esac
 done
