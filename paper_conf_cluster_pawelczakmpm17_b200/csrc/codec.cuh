@@ -58,6 +58,21 @@ ABFT_HD uint32_t byte_perm(uint32_t x, uint32_t y, uint32_t s) {
   return r;
 #endif
 }
+// LOP3 with an explicit truth table (a = 0xF0, b = 0xCC, c = 0xAA): ptxas does
+// not always merge a mask-and-combine into one LOP3 on its own.
+template <uint32_t LUT>
+ABFT_HD uint32_t lop3(uint32_t a, uint32_t b, uint32_t c) {
+#if defined(__CUDA_ARCH__)
+  uint32_t r;
+  asm("lop3.b32 %0, %1, %2, %3, %4;" : "=r"(r) : "r"(a), "r"(b), "r"(c), "n"(LUT));
+  return r;
+#else
+  uint32_t r = 0;
+  for (int i = 0; i < 8; i++)
+    if ((LUT >> i) & 1u) r |= ((i & 4) ? a : ~a) & ((i & 2) ? b : ~b) & ((i & 1) ? c : ~c);
+  return r;
+#endif
+}
 ABFT_HD uint32_t lo32(uint64_t u) { return (uint32_t)u; }
 ABFT_HD uint32_t hi32(uint64_t u) { return (uint32_t)(u >> 32); }
 ABFT_HD uint64_t mk64(uint32_t lo, uint32_t hi) { return ((uint64_t)hi << 32) | lo; }
@@ -274,7 +289,7 @@ ABFT_HD uint64_t vsed_encode(uint64_t rounded) {
 // positions 9 and 18 (one PRMT copies byte 0 into bytes 1 and 2).
 ABFT_HD uint32_t v64_fold(uint32_t a, uint32_t b) {
   uint32_t t = byte_perm(a, 0u, 0x4004u);           // [0, a.b0, a.b0, 0]
-  return (a & ~0x6u) ^ b ^ (t & 0x00040200u);
+  return lop3<0x78>(lop3<0x6C>(a, b, ~0x6u), t, 0x00040200u);   // (a & ~6) ^ b ^ (t & mask)
 }
 // Returns nonzero iff the codeword is NOT clean (fast path).
 ABFT_HD void v64_acc(uint32_t a, uint32_t b, uint32_t& acc_r, uint32_t& acc_p) {
@@ -424,13 +439,14 @@ ABFT_HD uint32_t e96_fold(uint32_t a, uint32_t b, uint32_t c) {
   // t = [0, c.b3, c.b3, c.b3]; XOR-ing t & 0x03020100 removes C24/C25 from
   // fold positions 24/25 and inserts them at 8/17 (PRMT + 2 LOP3).
   uint32_t t = byte_perm(c, 0u, 0x3334u);
-  return (a ^ b ^ c) ^ (t & 0x03020100u);
+  return lop3<0x78>(lop3<0x96>(a, b, c), t, 0x03020100u);   // (a ^ b ^ c) ^ (t & mask)
 }
 // Accumulating fast check (OR the Moebius registers and the code-row popcounts
 // of several codewords, test once with syn_bad): one branch per row / step.
+// Code rows: s5 = parity(b ^ (c & 0x9F000000)), s6 = parity(b[31] | c[0:31]).
 ABFT_HD void e96_acc(uint32_t a, uint32_t b, uint32_t c, uint32_t& acc_r, uint32_t& acc_p) {
   acc_r |= moebius32(e96_fold(a, b, c));
-  acc_p |= (uint32_t)(popc32(b ^ (c & 0x9F000000u)) | popc32((b & 0x80000000u) | (c & 0x7FFFFFFFu)));
+  acc_p |= (uint32_t)(popc32(lop3<0x78>(b, c, 0x9F000000u)) | popc32(lop3<0xE4>(b, c, 0x80000000u)));
 }
 
 ABFT_HD uint32_t e96_bad(uint32_t a, uint32_t b, uint32_t c) {
@@ -549,7 +565,7 @@ ABFT_HD uint32_t rp_acc(const uint32_t* e) {
   if (RS == SECDED64 || RS == SECDED128) {
     constexpr int NW = (RS == SECDED64) ? 2 : 4;
     constexpr int R = (RS == SECDED64) ? 7 : 8;
-    const MaskTable& M = (RS == SECDED64) ? ABFT_MT(r64) : ABFT_MT(r128);
+    constexpr MaskTable M = (RS == SECDED64) ? h_mt_r64 : h_mt_r128;   // masks as immediates
     uint32_t q = 0;
 #pragma unroll
     for (int i = 0; i < NW; i++) q ^= e[i];

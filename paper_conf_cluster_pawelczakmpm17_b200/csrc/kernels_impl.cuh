@@ -1,6 +1,7 @@
 // kernels_impl.cuh — device helpers and kernel templates shared by the kernel
 // translation units (kernels.cu, spmv_es*.cu).
 #pragma once
+#include <cuda.h>
 #include <cuda_runtime.h>
 #include <stdint.h>
 
@@ -328,14 +329,19 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
 
 // ====================================================== tiled stencil SpMV (a3)
 // Fast path for 5-point-stencil matrices (stencil_n = n, n % 256 == 0,
-// nrows % n == 0, G = 1 vector scheme).  A CTA owns a tile of TILE_TY grid
-// rows x 256 cells; warp w owns grid row w of the tile = one reduction block.
+// nrows % n == 0, nnz == 5 nrows, G = 1 vector scheme).  A CTA owns a tile of
+// TILE_TY grid rows x 256 cells; warp w owns grid row w of the tile = one
+// reduction block, processed as 8 passes of 32 rows.
+//  0. thread 0 is the CTA's TMA producer: the (val, col) element streams of one
+//     pass of all TILE_TY warps form a 2-D box [TILE_TY grid rows][160
+//     elements] of the matrix viewed as [ny][5n] (tensor maps built on the
+//     host), so ONE pair of cp.async.bulk.tensor copies per pass feeds the
+//     whole CTA through a TILE_NST-stage full/empty mbarrier ring.  The box
+//     position assumes the stencil layout rowptr[i] = 5i; every row compares
+//     its decoded rowptr with that assumption and reads global memory instead
+//     whenever it disagrees, so results never depend on the guess;
 //  1. each warp decodes its segment's 257 rowptr entries into SMEM (one check
-//     per group; owner counts) and, from them, issues TMA bulk copies
-//     (cp.async.bulk + mbarrier) of the (val, col) streams of its first two
-//     32-row passes into a double buffer — the packed element stream is
-//     contiguous per pass, so it arrives fully coalesced and without
-//     occupying registers or LSU slots;
+//     per group; owner counts);
 //  2. the CTA stages the decoded `in` window (tile + one halo row above/below
 //     + one halo cell left/right) in SMEM: every codeword of the tile is
 //     checked ONCE here (owner: counted + scrubbed), halo codewords are
@@ -343,19 +349,24 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
 //     multi-iteration aware" SpMV cache in B200 form; like the
 //     paper's caches, the decoded copies in SMEM are outside the software trust
 //     boundary;
-//  3. per pass each lane checks/corrects its row's elements from SMEM, gathers
-//     neighbours from the window whenever col-row is one of {0, +-1, +-n}
-//     (anything else takes the global gather path, so results never depend on
-//     the stencil hint), encodes w, and the warp refills the buffer with pass
-//     k+2.  A pass whose element range does not fit the buffer (non-stencil
-//     rows, corrupted rowptr) reads its elements from global memory instead.
+//  3. per pass each lane checks/corrects its row's elements from the stage,
+//     gathers neighbours from the window whenever col-row is one of {0, +-1,
+//     +-n} (anything else takes the global gather path, so results never
+//     depend on the stencil hint), encodes w, and releases the stage.
+struct TileMaps { CUtensorMap val, col; };
+
 constexpr int TILE_TY = 8;
 constexpr int TILE_WW = 256 + 2;
-constexpr int TILE_EBUF = 168;                                  // elements per pass buffer (>= 160 + align)
-constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;     // 20640
-constexpr int TILE_BUF_BYTES = TILE_EBUF * 12;                  // val 8 B + col 4 B per element
-constexpr int TILE_RP = 264;                                    // rowptr entries staged per warp
-constexpr int TILE_SMEM = TILE_WIN_BYTES + TILE_TY * (2 * TILE_BUF_BYTES + TILE_RP * 4 + 16);
+constexpr int TILE_PE = 160;                                   // elements per warp per pass (32 rows x 5)
+constexpr int TILE_NST = 3;                                    // pipeline stages
+constexpr int TILE_STAGE_VAL = TILE_TY * TILE_PE * 8;          // 10240
+constexpr int TILE_STAGE = TILE_STAGE_VAL + TILE_TY * TILE_PE * 4;   // + 5120
+constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 20640
+constexpr int TILE_RP = 264;                                   // rowptr entries staged per warp
+constexpr int TILE_OFF_WIN = TILE_NST * TILE_STAGE;            // stages first (128-B aligned)
+constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
+constexpr int TILE_OFF_BAR = TILE_OFF_RP + TILE_TY * TILE_RP * 4;
+constexpr int TILE_SMEM = TILE_OFF_BAR + 2 * TILE_NST * 8 + 128;   // + alignment slack
 
 static __device__ __forceinline__ uint32_t smem_u32(const void* p) { return (uint32_t)__cvta_generic_to_shared(p); }
 static __device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
@@ -364,11 +375,8 @@ static __device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) 
 static __device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
   asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes) : "memory");
 }
-static __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
-  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
-                   smem_u32(dst)),
-               "l"(src), "r"(bytes), "r"(smem_u32(bar))
-               : "memory");
+static __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
 static __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
   asm volatile(
@@ -377,71 +385,33 @@ static __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity)
       "r"(parity)
       : "memory");
 }
-
-// Issue the bulk copies of one pass's element range [s0, s1) into buffer buf.
-// Returns the aligned starts (e0 for val, c0 for col) or -1 if not staged.
-static __device__ __forceinline__ bool tile_issue(const SpmvArgs& a, uint32_t s0, uint32_t s1, uint8_t* buf,
-                                                  uint64_t* bar, int lane) {
-  if (!(s0 <= s1 && (int64_t)s1 <= a.nnz && s1 - s0 <= 160u)) return false;
-  if (lane == 0) {
-    const uint32_t e0 = s0 & ~1u, e1 = (s1 + 1u) & ~1u;
-    const uint32_t c0 = s0 & ~3u, c1 = (s1 + 3u) & ~3u;
-    const uint32_t vb = (e1 - e0) * 8u, cb = (c1 - c0) * 4u;
-    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
-    mbar_expect_tx(bar, vb + cb);
-    if (vb) bulk_g2s(buf, a.val + e0, vb, bar);
-    if (cb) bulk_g2s(buf + TILE_EBUF * 8, a.col + c0, cb, bar);
-  }
-  return true;
+static __device__ __forceinline__ void tma_2d(void* dst, const CUtensorMap* map, int x, int y, uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.tensor.2d.shared::cluster.global.tile.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], [%4];" ::"r"(
+          smem_u32(dst)),
+      "l"(reinterpret_cast<uint64_t>(map)), "r"(x), "r"(y), "r"(smem_u32(bar))
+      : "memory");
+}
+// Producer: the element boxes of pass k of the tile (tx0, ty0) into stage buffer `stage`.
+static __device__ __forceinline__ void tile_produce(const TileMaps& tm, uint8_t* stage, uint64_t* full, int64_t tx0,
+                                                    int64_t ty0, int k) {
+  mbar_expect_tx(full, TILE_STAGE);
+  const int x = (int)(5 * (tx0 + 32 * k)), y = (int)ty0;
+  tma_2d(stage, &tm.val, x, y, full);
+  tma_2d(stage + TILE_STAGE_VAL, &tm.col, x, y, full);
 }
 
-// Register-staged alternative to the TMA bulk copy (TILE_TMA = false): the
-// warp loads the pass's packed (val, col) range with 16-byte coalesced loads
-// (<= 4 per lane), writes it to the pass buffer one pass later.  Fewer issue
-// slots than the elected-lane cp.async.bulk sequence.
-constexpr bool TILE_TMA = true;
-struct PassRegs { uint4 q[4]; };
-static __device__ __forceinline__ bool pass_ok(uint32_t s0, uint32_t s1, int64_t nnz) {
-  return s0 <= s1 && (int64_t)s1 <= nnz && s1 - s0 <= 160u;
-}
-static __device__ __forceinline__ void pass_load(const SpmvArgs& a, uint32_t s0, uint32_t s1, int lane, PassRegs& R) {
-  const uint32_t e0 = s0 & ~1u, e1 = (s1 + 1u) & ~1u;
-  const uint32_t c0 = s0 & ~3u, c1 = (s1 + 3u) & ~3u;
-  const int nv = (int)((e1 - e0) >> 1), nc = (int)((c1 - c0) >> 2);
-  const uint4* vsrc = reinterpret_cast<const uint4*>(a.val + e0);
-  const uint4* csrc = reinterpret_cast<const uint4*>(a.col + c0);
-#pragma unroll
-  for (int q = 0; q < 4; q++) {
-    const int j = lane + 32 * q;
-    if (j < nv) R.q[q] = __ldg(vsrc + j);
-    else if (j - nv < nc) R.q[q] = __ldg(csrc + (j - nv));
-  }
-}
-static __device__ __forceinline__ void pass_store(uint32_t s0, uint32_t s1, int lane, const PassRegs& R, uint8_t* buf) {
-  const uint32_t e0 = s0 & ~1u, e1 = (s1 + 1u) & ~1u;
-  const uint32_t c0 = s0 & ~3u, c1 = (s1 + 3u) & ~3u;
-  const int nv = (int)((e1 - e0) >> 1), nc = (int)((c1 - c0) >> 2);
-  uint4* vdst = reinterpret_cast<uint4*>(buf);
-  uint4* cdst = reinterpret_cast<uint4*>(buf + TILE_EBUF * 8);
-#pragma unroll
-  for (int q = 0; q < 4; q++) {
-    const int j = lane + 32 * q;
-    if (j < nv) vdst[j] = R.q[q];
-    else if (j - nv < nc) cdst[j - nv] = R.q[q];
-  }
-}
-
-// One row, general case: check/correct its elements (from SMEM or global),
-// gather, fma chain.  Also the cold path of the 5-entry fast path below.
+// One row, general case: check/correct its elements (from the stage or
+// global), gather, fma chain.  Also the cold path of the 5-entry fast path
+// below.  sval/scol hold elements [s0, s1) of the chunk (if staged).
 template <int ES, int RS, int VS>
 static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start, uint32_t end, const uint64_t* sval,
-                                                 const uint32_t* scol, uint32_t sbase_v, uint32_t sbase_c, bool staged,
-                                                 const double* win, int oslot, double p_own, int64_t own, uint32_t s0,
-                                                 uint32_t s1) {
+                                                 const uint32_t* scol, bool staged, const double* win, int oslot,
+                                                 double p_own, int64_t own, uint32_t s0, uint32_t s1) {
   double acc = 0.0;
   const bool ok = (start <= end) && ((int64_t)end <= a.nnz);
-  // a corrupted (DUE) rowptr entry can put this row outside the staged pass
-  // range: read it from global memory then
+  // a corrupted (DUE) rowptr entry can put this row outside the staged range:
+  // read it from global memory then
   staged = staged && start >= s0 && end <= s1;
   if (RS != NONE && !ok) {
     cnt_range(a.counts, T_ROWPTR, RS);
@@ -456,8 +426,8 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
     uint64_t v;
     uint32_t c;
     if (staged) {
-      v = sval[start + j - sbase_v];
-      c = scol[start + j - sbase_c];
+      v = sval[start + j - s0];
+      c = scol[start + j - s0];
     } else {
       v = ldg64(a.val + start + j);
       c = __ldg(a.col + start + j);
@@ -494,17 +464,18 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
   return acc;
 }
 
-// 5-entry stencil rows (the TeaLeaf layout, reading R16): straight-line code,
-// one uniform branch for "any element needs correction / any index is not
-// the canonical stencil neighbour or in range" -> tile_row (identical
-// semantics, so counts and results do not depend on which path ran).
+// 5-entry stencil rows (the TeaLeaf layout, reading R16) at the assumed
+// position start = s0 + 5 lane: straight-line code, one uniform branch for
+// "any element needs correction / any index is not the canonical stencil
+// neighbour or in range / rowptr disagrees" -> tile_row (identical semantics,
+// so counts and results do not depend on which path ran).
 template <int ES, int RS, int VS>
 static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const SpmvArgs& sa, uint32_t start, uint32_t end,
-                                                   const uint64_t* sval, const uint32_t* scol, uint32_t sbase_v,
-                                                   uint32_t sbase_c, bool staged, const double* win, int oslot,
-                                                   double p_own, int64_t own, uint32_t s0, uint32_t s1) {
-  if (ES == CRC32C || !staged || end - start != 5u || start > end || start < s0 || end > s1)
-    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own, s0, s1);
+                                                   const uint64_t* sval, const uint32_t* scol, const double* win,
+                                                   int oslot, double p_own, int64_t own, uint32_t s0, int lane) {
+  const uint32_t s1 = s0 + TILE_PE;
+  if (ES == CRC32C || start != s0 + 5u * (uint32_t)lane || end != start + 5u)
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1);
   const int n32 = (int)a.stencil_n;
   const int own_col = (int)(own - a.col_base);
   const uint32_t ckeep = col_keep(ES);
@@ -512,8 +483,8 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
   uint32_t c[5];
 #pragma unroll
   for (int t = 0; t < 5; t++) {
-    v[t] = sval[start + t - sbase_v];
-    c[t] = scol[start + t - sbase_c];
+    v[t] = sval[5 * lane + t];
+    c[t] = scol[5 * lane + t];
   }
   uint32_t acc_r = 0, acc_p = 0;
 #pragma unroll
@@ -534,7 +505,7 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
                      ((unsigned)d[3] <= 1u) && (d[4] == 0 || d[4] == n32);
   const bool in_range = (ES == NONE) || cmax < (uint32_t)a.ncols;
   if ((ES != NONE && syn_bad(acc_r, acc_p)) || !canon || !in_range)
-    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, sbase_v, sbase_c, staged, win, oslot, p_own, own, s0, s1);
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1);
   // slot offsets: d itself for +-1 / 0, +-window width for +-n
   const int o0 = d[0] ? -TILE_WW : 0, o4 = d[4] ? TILE_WW : 0;
   double acc = fma(as_d(v[0]), win[oslot + o0], 0.0);
@@ -546,37 +517,41 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
 }
 
 template <int ES, int RS, int VS, bool DOT>
-__global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
-  extern __shared__ __align__(128) uint8_t s_dyn[];
+__global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __grid_constant__ TileMaps tm) {
+  extern __shared__ uint8_t s_raw[];
   __shared__ __align__(16) uint8_t s_lut[128];
   // the cold row path takes the arguments by reference: give it a SMEM copy so
   // the kernel parameters are never spilled to local memory
   __shared__ SpmvArgs s_args;
-  if (threadIdx.x == 0) s_args = a;
-  double* s_win = reinterpret_cast<double*>(s_dyn);
+  uint8_t* s_dyn = s_raw + ((128u - (smem_u32(s_raw) & 127u)) & 127u);
+  double* s_win = reinterpret_cast<double*>(s_dyn + TILE_OFF_WIN);
+  uint64_t* full = reinterpret_cast<uint64_t*>(s_dyn + TILE_OFF_BAR);
+  uint64_t* empty = full + TILE_NST;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  uint8_t* wbase = s_dyn + TILE_WIN_BYTES + warp * (2 * TILE_BUF_BYTES + TILE_RP * 4 + 16);
-  uint32_t* srp = reinterpret_cast<uint32_t*>(wbase + 2 * TILE_BUF_BYTES);
-  uint64_t* bars = reinterpret_cast<uint64_t*>(wbase + 2 * TILE_BUF_BYTES + TILE_RP * 4);
-  if (VS == SECDED64) load_lut(s_lut);
-  if (lane == 0) {
-    mbar_init(&bars[0], 1);
-    mbar_init(&bars[1], 1);
-    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-  }
-  __syncwarp();
-  const int stop_v = a.state ? a.state->stop : 0;  // checked after the prologue loads are in flight
+  uint32_t* srp = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_RP) + warp * TILE_RP;
   const int64_t n = a.stencil_n;
   const int64_t ny = a.nrows / n;
   const int64_t tiles_x = n >> 8;
   const int64_t tx0 = (blockIdx.x % tiles_x) << 8;
   const int64_t ty0 = (int64_t)(blockIdx.x / tiles_x) * TILE_TY;
+  // ---- 0. producer: barriers, then the first TILE_NST passes in flight
+  if (threadIdx.x == 0) {
+    s_args = a;
+#pragma unroll
+    for (int s = 0; s < TILE_NST; s++) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], TILE_TY);
+    }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+#pragma unroll
+    for (int k = 0; k < TILE_NST; k++) tile_produce(tm, s_dyn + k * TILE_STAGE, &full[k], tx0, ty0, k);
+  }
+  if (VS == SECDED64) load_lut(s_lut);
+  const int stop_v = a.state ? a.state->stop : 0;  // checked after the prologue loads are in flight
   const int64_t gy = ty0 + warp;
   const bool has_seg = gy < ny;
   const int64_t rowseg = gy * n + tx0;
-  // ---- 1. rowptr of the segment (entries rowseg .. rowseg+256), then the first two element copies
-  uint32_t stmask = 0u;  // bit b: buffer b holds the current pass (TMA issued)
-  PassRegs pre;          // register-staged next pass (TILE_TMA = false)
+  // ---- 1. rowptr of the segment (entries rowseg .. rowseg+256)
   if (has_seg) {
     constexpr int G = rgrp(RS);
     constexpr int NG = 256 / G + 1;
@@ -598,57 +573,54 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
         }
       }
     }
-    if (stop_v) return;
-    uint32_t acc = 0;
+    if (!stop_v) {
+      uint32_t acc = 0;
 #pragma unroll
-    for (int q = 0; q < PER; q++)
-      if (RS != NONE && lane + 32 * q < NG) acc |= rp_acc<RS>(e[q]);
-    if (RS != NONE && (acc & 1u)) {  // cold: locate, correct, count (owner), per group
+      for (int q = 0; q < PER; q++)
+        if (RS != NONE && lane + 32 * q < NG) acc |= rp_acc<RS>(e[q]);
+      if (RS != NONE && (acc & 1u)) {  // cold: locate, correct, count (owner), per group
+#pragma unroll
+        for (int q = 0; q < PER; q++) {
+          const int gl = lane + 32 * q;
+          if (gl >= NG) continue;
+          const int64_t g = rowseg / G + gl;
+          uint32_t* gp = a.rowptr + g * G;
+          uint32_t o0[G];
+#pragma unroll
+          for (int t = 0; t < G; t++) o0[t] = e[q][t];
+          int word = 0;
+          int o = rp_check_group<RS>(e[q], &word);
+          if (o != CLEAN) {
+            const int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
+            const bool owner = own >= rowseg && own < rowseg + 256;
+            if (o == CORRECTED) {
+              uint32_t ow = 0, nw = 0;   // select, not index: keeps e[][] out of local memory
+#pragma unroll
+              for (int t = 0; t < G; t++)
+                if (t == word) { ow = o0[t]; nw = e[q][t]; }
+              if (owner && scrub32(gp + word, ow, nw)) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
+            } else {
+#pragma unroll
+              for (int t = 0; t < G; t++) e[q][t] = o0[t];
+              if (owner) { cnt_add(a.counts, T_ROWPTR, RS, DUE); *a.due = 1; }
+            }
+          }
+        }
+      }
 #pragma unroll
       for (int q = 0; q < PER; q++) {
         const int gl = lane + 32 * q;
         if (gl >= NG) continue;
-        const int64_t g = rowseg / G + gl;
-        uint32_t* gp = a.rowptr + g * G;
-        uint32_t o0[G];
 #pragma unroll
-        for (int t = 0; t < G; t++) o0[t] = e[q][t];
-        int word = 0;
-        int o = rp_check_group<RS>(e[q], &word);
-        if (o != CLEAN) {
-          const int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
-          const bool owner = own >= rowseg && own < rowseg + 256;
-          if (o == CORRECTED) {
-            if (owner && scrub32(gp + word, o0[word], e[q][word])) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
-          } else {
-#pragma unroll
-            for (int t = 0; t < G; t++) e[q][t] = o0[t];
-            if (owner) { cnt_add(a.counts, T_ROWPTR, RS, DUE); *a.due = 1; }
-          }
-        }
+        for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[q][t] & rp_keep(RS);
       }
-    }
-#pragma unroll
-    for (int q = 0; q < PER; q++) {
-      const int gl = lane + 32 * q;
-      if (gl >= NG) continue;
-#pragma unroll
-      for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[q][t] & rp_keep(RS);
-    }
-    __syncwarp();
-    if (TILE_TMA) {
-      stmask |= tile_issue(a, srp[0], srp[32], wbase, &bars[0], lane) ? 1u : 0u;
-      stmask |= tile_issue(a, srp[32], srp[64], wbase + TILE_BUF_BYTES, &bars[1], lane) ? 2u : 0u;
-    } else {
-      if (pass_ok(srp[0], srp[32], a.nnz)) {       // pass 0 -> buffer 0 now, pass 1 in flight
-        pass_load(a, srp[0], srp[32], lane, pre);
-        pass_store(srp[0], srp[32], lane, pre, wbase);
-        stmask |= 1u;
-      }
-      if (pass_ok(srp[32], srp[64], a.nnz)) pass_load(a, srp[32], srp[64], lane, pre);
     }
   }
-  if (stop_v) return;  // uniform per grid
+  if (stop_v) {  // uniform per grid: drain the producer's copies before the CTA exits
+    if (threadIdx.x == 0)
+      for (int s = 0; s < TILE_NST; s++) mbar_wait(&full[s], 0u);
+    return;
+  }
   // ---- 2. decoded `in` window
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
   constexpr int WPER = (TILE_WW + 31) / 32;                      // 9 slots per lane per window row
@@ -687,51 +659,36 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(SpmvArgs a) {
     }
   }
   __syncthreads();
-  if (!has_seg) return;
-  // ---- 3. passes
+  // ---- 3. passes (every warp takes part in the stage protocol)
   double dot = 0.0;
-  uint32_t phmask = 0u;  // bit b: completed-phase parity expected next for buffer b
-#pragma unroll 1
+  const uint32_t seg_e = (uint32_t)(5 * rowseg);   // assumed element start of the segment
+#pragma unroll
   for (int k = 0; k < 8; k++) {
-    const int b = k & 1;
-    const uint32_t s0 = srp[32 * k];
-    const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
-    const bool st = (stmask >> b) & 1u;
-    if (TILE_TMA && st) {
-      mbar_wait(&bars[b], (phmask >> b) & 1u);
-      phmask ^= 1u << b;
+    const int st = k % TILE_NST;
+    const uint32_t ph = (uint32_t)((k / TILE_NST) & 1);
+    uint8_t* stage = s_dyn + st * TILE_STAGE;
+    mbar_wait(&full[st], ph);
+    if (has_seg) {
+      const uint64_t* sval = reinterpret_cast<const uint64_t*>(stage) + warp * TILE_PE;
+      const uint32_t* scol = reinterpret_cast<const uint32_t*>(stage + TILE_STAGE_VAL) + warp * TILE_PE;
+      const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
+      const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
+      const double p_own = s_win[oslot];
+      const int64_t own = a.row_base + rowseg + k * 32 + lane;
+      const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s_win, oslot, p_own, own,
+                                               seg_e + 160u * k, lane);
+      const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
+      a.out[own] = enc;
+      if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
     }
-    uint8_t* bb = wbase + b * TILE_BUF_BYTES;
-    const uint64_t* sval = reinterpret_cast<const uint64_t*>(bb);
-    const uint32_t* scol = reinterpret_cast<const uint32_t*>(bb + TILE_EBUF * 8);
-    const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
-    const double p_own = s_win[oslot];
-    const int64_t own = a.row_base + rowseg + k * 32 + lane;
-    const uint32_t s1 = srp[32 * k + 32];
-    const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s0 & ~1u, s0 & ~3u, st, s_win, oslot,
-                                             p_own, own, s0, s1);
-    const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
-    a.out[own] = enc;
-    if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
     __syncwarp();
-    if (TILE_TMA) {
-      if (k + 2 < 8) {
-        const bool ok = tile_issue(a, srp[32 * (k + 2)], srp[32 * (k + 3)], bb, &bars[b], lane);
-        stmask = (stmask & ~(1u << b)) | ((ok ? 1u : 0u) << b);
-      }
-    } else if (k + 1 < 8) {
-      // pass k+1: registers -> the other buffer (pass k-1 is done with it); then prefetch pass k+2
-      const uint32_t t0 = srp[32 * (k + 1)], t1 = srp[32 * (k + 2)];
-      const int nb = b ^ 1;
-      const bool ok = pass_ok(t0, t1, a.nnz);
-      if (ok) pass_store(t0, t1, lane, pre, wbase + nb * TILE_BUF_BYTES);
-      stmask = (stmask & ~(1u << nb)) | ((ok ? 1u : 0u) << nb);
-      __syncwarp();
-      if (k + 2 < 8 && pass_ok(srp[32 * (k + 2)], srp[32 * (k + 3)], a.nnz))
-        pass_load(a, srp[32 * (k + 2)], srp[32 * (k + 3)], lane, pre);
+    if (lane == 0) mbar_arrive(&empty[st]);
+    if (k + TILE_NST < 8 && threadIdx.x == 0) {  // refill the stage once every warp released it
+      mbar_wait(&empty[st], ph);
+      tile_produce(tm, stage, &full[st], tx0, ty0, k + TILE_NST);
     }
   }
-  if (DOT) {
+  if (DOT && has_seg) {
 #pragma unroll
     for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
     if (a.red.rs) red_push(a.partials, a.rb_offset + (rowseg >> 8), dot, a.red, lane);

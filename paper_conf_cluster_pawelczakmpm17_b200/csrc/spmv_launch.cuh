@@ -1,33 +1,74 @@
 // spmv_launch.cuh — host-side SpMV launch templates (tiled stencil fast path or
 // generic CSR kernel), instantiated per element scheme in spmv_es_*.cu.
 #pragma once
+#include <cudaTypedefs.h>
+
 #include "kernels_impl.cuh"
 
 namespace abft {
 namespace {
+// Tiled path preconditions (host metadata; the kernel still checks every row's
+// decoded rowptr against the assumed stencil layout).
 static bool tile_ok(const SpmvArgs& a, int vs) {
   const int64_t n = a.stencil_n;
-  return n > 0 && (n % 256) == 0 && (a.nrows % n) == 0 && vgrp(vs) == 1 && a.npad_out >= a.nrows;
+  return n > 0 && (n % 256) == 0 && (a.nrows % n) == 0 && vgrp(vs) == 1 && a.npad_out >= a.nrows &&
+         a.nnz == 5 * a.nrows && a.nnz < (int64_t(1) << 32) && (a.nrows / n) < (int64_t(1) << 31) &&
+         (reinterpret_cast<uintptr_t>(a.val) & 15u) == 0 && (reinterpret_cast<uintptr_t>(a.col) & 15u) == 0;
+}
+// The driver's tensor-map encoder, resolved once through the runtime (no -lcuda).
+static PFN_cuTensorMapEncodeTiled_v12000 tmap_encoder() {
+  static PFN_cuTensorMapEncodeTiled_v12000 fn = nullptr;
+  static bool tried = false;
+  if (!tried) {
+    tried = true;
+    void* p = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &p, cudaEnableDefault, &q) == cudaSuccess &&
+        q == cudaDriverEntryPointSuccess)
+      fn = reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(p);
+  }
+  return fn;
+}
+// The chunk's element arrays viewed as [ny grid rows][5n elements]; box = one
+// pass of all TILE_TY warps of a tile: [TILE_TY][TILE_PE].
+static bool tile_maps(const SpmvArgs& a, TileMaps* m) {
+  auto enc = tmap_encoder();
+  if (!enc) return false;
+  const int64_t n = a.stencil_n, ny = a.nrows / n;
+  cuuint64_t dims[2] = {(cuuint64_t)(5 * n), (cuuint64_t)ny};
+  cuuint32_t box[2] = {(cuuint32_t)TILE_PE, (cuuint32_t)TILE_TY};
+  cuuint32_t estr[2] = {1, 1};
+  cuuint64_t sv[1] = {(cuuint64_t)(5 * n * 8)}, sc[1] = {(cuuint64_t)(5 * n * 4)};
+  CUresult r1 = enc(&m->val, CU_TENSOR_MAP_DATA_TYPE_UINT64, 2, a.val, dims, sv, box, estr,
+                    CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  CUresult r2 = enc(&m->col, CU_TENSOR_MAP_DATA_TYPE_UINT32, 2, a.col, dims, sc, box, estr,
+                    CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                    CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  return r1 == CUDA_SUCCESS && r2 == CUDA_SUCCESS;
 }
 template <int ES, int RS, int VS, bool DOT>
-static void spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
+static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
+  TileMaps tm;
+  if (!tile_maps(a, &tm)) return false;
   const size_t smem = TILE_SMEM;
   static bool attr = false;
   if (!attr) {  // both variants at once: never inside a later CUDA-graph capture
     cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, true>, cudaFuncAttributePreferredSharedMemoryCarveout, 100);
+    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, false>, cudaFuncAttributePreferredSharedMemoryCarveout, 100);
     attr = true;
   }
   const int64_t ny = a.nrows / a.stencil_n;
   const int64_t blocks = (a.stencil_n / 256) * ((ny + TILE_TY - 1) / TILE_TY);
-  k_spmv_tile<ES, RS, VS, DOT><<<(unsigned)blocks, 256, smem, s>>>(a);
+  k_spmv_tile<ES, RS, VS, DOT><<<(unsigned)blocks, 256, smem, s>>>(a, tm);
+  return true;
 }
 template <int ES, int RS, int VS>
 static void spmv3(const SpmvArgs& a, bool dot, cudaStream_t s) {
   if (vgrp(VS) == 1 && tile_ok(a, VS)) {
-    if (dot) spmv_tile_launch<ES, RS, VS, true>(a, s);
-    else spmv_tile_launch<ES, RS, VS, false>(a, s);
-    return;
+    if (dot ? spmv_tile_launch<ES, RS, VS, true>(a, s) : spmv_tile_launch<ES, RS, VS, false>(a, s)) return;
   }
   const int64_t nrb = (a.nrows + 255) / 256;
   const int blocks = (int)((nrb + 7) / 8);
