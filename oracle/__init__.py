@@ -65,6 +65,8 @@ def lib():
         L.or_tree_sum.argtypes = [dp, C.c_int64]
         L.or_spmv.restype = C.c_int64
         L.or_spmv.argtypes = [C.c_void_p, u64p, C.c_int64, C.c_int, u64p, C.c_int64, C.c_void_p, dp]
+        L.or_spmv_mode.restype = C.c_int64
+        L.or_spmv_mode.argtypes = [C.c_void_p, u64p, C.c_int64, C.c_int, u64p, C.c_int64, C.c_void_p, dp, C.c_int]
         L.or_check_csr.restype = C.c_int64
         L.or_check_csr.argtypes = [C.c_void_p, C.c_void_p, C.c_int]
         L.or_calc_ur.restype = C.c_int64
@@ -75,6 +77,8 @@ def lib():
         L.or_cg_init_r.argtypes = [u64p, u64p, u64p, u64p, C.c_int64, C.c_int, C.c_void_p, dp]
         L.or_cg_solve.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
                                   C.c_int, C.c_void_p, C.c_void_p]
+        L.or_cg_solve_ex.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
+                                     C.c_int, C.c_void_p, C.c_void_p, C.c_int]
         L.or_vec_masked.argtypes = [u64p, C.c_int64, C.c_int, dp]
         L.or_round_k.restype = C.c_uint64
         L.or_round_k.argtypes = [C.c_uint64, C.c_int]
@@ -227,16 +231,22 @@ class Matrix:
                    _p(self.col, C.c_uint32), _p(self.rowptr, C.c_uint32), self.es, self.rs)
 
     def check(self, counts=None, scrub=True) -> int:
+        """scrub: False count only, True count + scrub, 2 detection only."""
         s = self.cstruct()
         return lib().or_check_csr(C.byref(s), counts.ctypes.data if counts is not None else None, int(scrub))
 
 
+# matrix check modes of one SpMV access (DESIGN.md §3.9, P:398-425)
+MODE_CORRECT, MODE_DETECT, MODE_RANGE = 0, 1, 2
+
+
 def spmv(A: Matrix, x: np.ndarray, n_in: int, scheme: int, out: np.ndarray, n_out: int, counts=None,
-         want_dot=False):
+         want_dot=False, mode=MODE_CORRECT):
     s = A.cstruct()
     dot = C.c_double(0.0)
-    d = lib().or_spmv(C.byref(s), _p(x, C.c_uint64), n_in, scheme, _p(out, C.c_uint64), n_out,
-                      counts.ctypes.data if counts is not None else None, C.byref(dot) if want_dot else None)
+    d = lib().or_spmv_mode(C.byref(s), _p(x, C.c_uint64), n_in, scheme, _p(out, C.c_uint64), n_out,
+                           counts.ctypes.data if counts is not None else None, C.byref(dot) if want_dot else None,
+                           int(mode))
     return (d, dot.value) if want_dot else d
 
 
@@ -259,11 +269,14 @@ def cg_init_r(b, w, r, p, n, scheme, counts=None):
     return d, rr0.value
 
 
-def cg_solve(A: Matrix, b, x, r, p, w, scheme, tol=1e-10, max_iters=10000, due_policy=1, counts=None):
-    """Protected CG on encoded uint64 vectors (x: in x0, out x)."""
+def cg_solve(A: Matrix, b, x, r, p, w, scheme, tol=1e-10, max_iters=10000, due_policy=1, counts=None,
+             check_interval=1):
+    """Protected CG on encoded uint64 vectors (x: in x0, out x).
+    check_interval N > 1: the matrix is checked (detection only) on every N-th
+    access and range-checked otherwise, plus a final check."""
     s = A.cstruct()
     res = CGResult()
-    st = lib().or_cg_solve(C.byref(s), _p(b, C.c_uint64), _p(x, C.c_uint64), _p(r, C.c_uint64), _p(p, C.c_uint64),
-                           _p(w, C.c_uint64), scheme, tol, max_iters, due_policy, C.byref(res),
-                           counts.ctypes.data if counts is not None else None)
+    st = lib().or_cg_solve_ex(C.byref(s), _p(b, C.c_uint64), _p(x, C.c_uint64), _p(r, C.c_uint64),
+                              _p(p, C.c_uint64), _p(w, C.c_uint64), scheme, tol, max_iters, due_policy, C.byref(res),
+                              counts.ctypes.data if counts is not None else None, int(check_interval))
     return st, res

@@ -13,6 +13,8 @@
  *         rowptr     P:377-397 (§VI-A.1); range checks P:407-416 (§VI-A.2)
  *         vectors    P:426-451 (§VI-B); write buffering P:468-490 (§VI-C)
  *         CG         TeaLeaf CG (ref [19]), DESIGN.md §4
+ *         interval   "less frequent correctness checking" P:398-425 (§VI-A.2),
+ *                    DESIGN.md §3.9 (reading R27)
  *
  * Every computation is the plain definition: syndromes are XORs of H-columns
  * over a loop on every container bit, CRC32C is the bit-serial division,
@@ -506,15 +508,23 @@ typedef struct {
   int es, rs;
 } or_csr;
 
+/* Matrix check modes: every access checked and
+ * corrected (N = 1); an interval access checked for detection only (a found
+ * error may have been used by the unchecked accesses before it, so it is a
+ * DUE: "we lose the ability to correct any errors"); an unchecked
+ * access, range checks only. */
+enum { M_CORRECT = 0, M_DETECT = 1, M_RANGE = 2 };
+
 /* Check every rowptr group; fills rp[] with decoded masked entries. */
-static int64_t check_rowptr(or_csr* A, uint32_t* rp, counts_t* cnt, int scrub) {
+static int64_t check_rowptr(or_csr* A, uint32_t* rp, counts_t* cnt, int scrub, int mode) {
   int64_t len = or_rowptr_padded_len(A->nrows, A->rs), dues = 0;
   int g = rp_group(A->rs);
   uint32_t m = rp_mask(A->rs);
   for (int64_t i = 0; i < len; i += g) {
     uint32_t e[8];
     for (int j = 0; j < g; j++) e[j] = A->rowptr[i + j];
-    int o = rp_check_group(e, A->rs);
+    int o = (mode == M_RANGE) ? OUT_CLEAN : rp_check_group(e, A->rs);
+    if (o == OUT_CORRECTED && mode == M_DETECT) o = OUT_DUE;
     count_outcome(cnt, T_ROWPTR, A->rs, o);
     if (o == OUT_DUE) { dues++; for (int j = 0; j < g; j++) e[j] = A->rowptr[i + j]; }
     if (o == OUT_CORRECTED && scrub) for (int j = 0; j < g; j++) A->rowptr[i + j] = e[j];
@@ -544,8 +554,8 @@ static int el_check(int es, uint32_t* w) {
  * encoded vectors (f64 bit patterns) of logical length n_in / n_out.
  * dot (may be NULL) = RED-1 sum of in[row_base+i]*out[row_base+i] over masked
  * values.  Returns the number of DUEs + range violations seen. */
-int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, int64_t n_out, counts_t* cnt,
-                double* dot) {
+int64_t or_spmv_mode(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, int64_t n_out, counts_t* cnt,
+                     double* dot, int mode) {
   init_instances();
   int64_t dues = 0;
   int g = vec_group(vs), k = vec_k(vs);
@@ -555,7 +565,7 @@ int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, in
   int64_t npad_in = or_vec_padded_len(n_in, vs);
   double* xin = (double*)malloc(sizeof(double) * (size_t)npad_in);
 
-  dues += check_rowptr(A, rp, cnt, 1);
+  dues += check_rowptr(A, rp, cnt, 1, mode);
   /* every codeword of `in`: owned ones counted + scrubbed */
   for (int64_t i = 0; i < npad_in; i += g) {
     uint64_t d[4];
@@ -578,7 +588,7 @@ int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, in
       acc[i] = 0.0;
       continue;
     }
-    if (A->es == S_CRC32C) {           /* E-CRC: the row is the codeword */
+    if (A->es == S_CRC32C && mode != M_RANGE) {   /* E-CRC: the row is the codeword */
       int o;
       if (t - s < 4) o = OUT_DUE;
       else o = (ecrc_stored(A->col, s) == ecrc_row(A->val, A->col, s, t)) ? OUT_CLEAN : OUT_DUE;
@@ -588,7 +598,11 @@ int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, in
     for (uint32_t j = s; j < t; j++) {
       uint32_t w[3];
       el_words(A->val[j], A->col[j], w);
-      int o = el_check(A->es, w);
+      int o = (mode == M_RANGE) ? OUT_CLEAN : el_check(A->es, w);
+      if (o == OUT_CORRECTED && mode == M_DETECT) {   /* detection only: stored bits, no scrub */
+        o = OUT_DUE;
+        el_words(A->val[j], A->col[j], w);
+      }
       count_outcome(cnt, T_ELEM, A->es, o);
       if (o == OUT_DUE) dues++;
       if (o == OUT_CORRECTED) {          /* scrub: later accesses see the clean codeword */
@@ -631,17 +645,23 @@ int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, in
   free(acc); free(rp); free(xin);
   return dues;
 }
+int64_t or_spmv(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* out, int64_t n_out, counts_t* cnt,
+                double* dot) {
+  return or_spmv_mode(A, in, n_in, vs, out, n_out, cnt, dot, M_CORRECT);
+}
 
 /* Check all elements of A (index order), counting into ELEM; fills vd/cd with
  * decoded (masked) values and skip[] for range violations; scrubs corrections.
  * E-CRC rows are checked in the row pass (the codeword is the row). */
-static int64_t check_elements(or_csr* A, double* vd, uint32_t* cd, uint8_t* skip, counts_t* cnt, int scrub) {
+static int64_t check_elements(or_csr* A, double* vd, uint32_t* cd, uint8_t* skip, counts_t* cnt, int scrub,
+                              int mode) {
   int64_t dues = 0;
   uint32_t cm = col_mask(A->es);
   for (int64_t e = 0; e < A->nnz; e++) {
     uint32_t w[3];
     el_words(A->val[e], A->col[e], w);
     int o = el_check(A->es, w);
+    if (o == OUT_CORRECTED && mode == M_DETECT) { o = OUT_DUE; el_words(A->val[e], A->col[e], w); }
     count_outcome(cnt, T_ELEM, A->es, o);
     if (o == OUT_DUE) dues++;
     if (o == OUT_CORRECTED && scrub) {
@@ -662,15 +682,19 @@ static int64_t check_elements(or_csr* A, double* vd, uint32_t* cd, uint8_t* skip
 }
 
 /* ---------------------------------------------------------- check_all */
+/* scrub: 0 count only, 1 count + scrub single flips, 2 detection only (every
+ * failing codeword is a DUE: the end-of-solve check of interval mode) */
 int64_t or_check_csr(or_csr* A, counts_t* cnt, int scrub) {
   init_instances();
+  int mode = (scrub == 2) ? M_DETECT : M_CORRECT;
+  if (scrub == 2) scrub = 0;
   double* vd = (double*)malloc(sizeof(double) * (size_t)(A->nnz + 1));
   uint32_t* cd = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)(A->nnz + 1));
   uint8_t* skip = (uint8_t*)malloc((size_t)(A->nnz + 1));
   int64_t rplen = or_rowptr_padded_len(A->nrows, A->rs);
   uint32_t* rp = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)rplen);
-  int64_t dues = check_elements(A, vd, cd, skip, cnt, scrub);
-  dues += check_rowptr(A, rp, cnt, scrub);
+  int64_t dues = check_elements(A, vd, cd, skip, cnt, scrub, mode);
+  dues += check_rowptr(A, rp, cnt, scrub, mode);
   for (int64_t i = 0; i < A->nrows; i++) {
     uint32_t s = rp[i], t = rp[i + 1];
     if (!(s <= t && (int64_t)t <= A->nnz)) {
@@ -764,20 +788,27 @@ typedef struct { int32_t iters; int32_t status; double rr0, rrn; } or_cg_result;
  * Vectors are padded encoded arrays of logical length n = A->nrows.
  * due_policy: 0 abort (finish the iteration, return E_DUE), 1 continue.
  * max_iters <= 0: only the init.  Returns status. */
-int or_cg_solve(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
-                int max_iters, int due_policy, or_cg_result* res, counts_t* cnt) {
-  init_instances();
+/* Matrix access a (init SpMV = 0, iteration k's SpMV = k) under check
+ * interval N: N <= 1 every access checked + corrected; otherwise
+ * access a is checked (detection only) iff a % N == 0, else range-checked. */
+static int access_mode(int64_t a, int interval) {
+  if (interval <= 1) return M_CORRECT;
+  return (a % interval == 0) ? M_DETECT : M_RANGE;
+}
+
+static int cg_run(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
+                  int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval) {
   int64_t n = A->nrows;
   double rr0, rro, rrn = 0.0, pw;
   res->iters = 0; res->status = OK; res->rr0 = 0.0; res->rrn = 0.0;
-  int64_t dues = or_spmv(A, x, n, vs, w, n, cnt, NULL);
+  int64_t dues = or_spmv_mode(A, x, n, vs, w, n, cnt, NULL, access_mode(0, interval));
   dues += or_cg_init_r(b, w, r, p, n, vs, cnt, &rr0);
   res->rr0 = rr0; res->rrn = rr0;
   if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
   if (rr0 == 0.0) return OK;
   rro = rr0;
   for (int k = 1; k <= max_iters; k++) {
-    dues = or_spmv(A, p, n, vs, w, n, cnt, &pw);
+    dues = or_spmv_mode(A, p, n, vs, w, n, cnt, &pw, access_mode(k, interval));
     double alpha = rro / pw;
     dues += or_calc_ur(x, p, r, w, n, vs, alpha, cnt, &rrn);
     res->iters = k; res->rrn = rrn;
@@ -792,6 +823,26 @@ int or_cg_solve(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, u
   }
   res->status = (max_iters > 0) ? E_NOT_CONVERGED : OK;
   return res->status;
+}
+
+/* interval > 1: after the solve, if its last matrix access (= res->iters) was
+ * not a checked one, an extra detection-only integrity check of the whole
+ * matrix "just in case N does not divide the number of iterations performed"
+ * (P:418-421); a DUE found there turns OK / NOT_CONVERGED into E_DUE under
+ * policy abort. */
+int or_cg_solve_ex(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
+                   int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval) {
+  init_instances();
+  int st = cg_run(A, b, x, r, p, w, vs, tol, max_iters, due_policy, res, cnt, interval);
+  if (interval > 1 && res->iters % interval != 0) {
+    int64_t dues = or_check_csr(A, cnt, 2);
+    if (dues && due_policy == 0 && st != E_DUE) { res->status = E_DUE; st = E_DUE; }
+  }
+  return st;
+}
+int or_cg_solve(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
+                int max_iters, int due_policy, or_cg_result* res, counts_t* cnt) {
+  return or_cg_solve_ex(A, b, x, r, p, w, vs, tol, max_iters, due_policy, res, cnt, 1);
 }
 
 /* Masked-value helper for tests: clear the k reserved LSBs of each entry. */
