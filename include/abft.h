@@ -99,11 +99,29 @@ int abft_vec_decode(abft_ctx* ctx, abft_vec* v, double* out_masked, abft_counts*
 int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, double* dot_out,
               abft_counts* dcnt, void* stream);
 
+/* Matrix check mode of one SpMV access ("less frequent correctness checking",
+ * P:398-425): */
+typedef enum {
+  ABFT_CHECK_CORRECT = 0,  /* check every element / rowptr group, correct + scrub single flips (default) */
+  ABFT_CHECK_DETECT = 1,   /* check, detection only: any failing codeword is a DUE, never scrubbed */
+  ABFT_CHECK_RANGE = 2     /* no ECC check: stored bits masked + range checks only */
+} abft_check_mode;
+/* abft_spmv with an explicit matrix check mode (vectors are always checked). */
+int abft_spmv_ex(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, double* dot_out,
+                 abft_counts* dcnt, int32_t check_mode, void* stream);
+
 typedef struct {
   double tol;          /* stop when sqrt(r.r) <= tol*sqrt(r0.r0) (R15) */
   int32_t max_iters;
   int32_t due_policy;  /* 0 = abort (finish the iteration, return ABFT_E_DUE), 1 = continue */
   int32_t poll_every;  /* iterations between host polls of the stop flag (0 = default 16) */
+  /* check_interval N: 0/1 = check + correct the
+   * matrix on every access; N > 1 = matrix access a (init SpMV = 0, iteration
+   * k's SpMV = k) is checked for detection only iff a % N == 0 and only
+   * range-checked otherwise, plus a detection-only check of the whole matrix
+   * after the solve when N does not divide the iteration count (a DUE found
+   * there returns ABFT_E_DUE under policy abort).  Vectors: every access. */
+  int32_t check_interval;
 } abft_cg_opts;
 
 typedef struct { int32_t iters; int32_t status; double rr0, rrn; } abft_cg_result;
@@ -116,8 +134,9 @@ typedef struct { int32_t iters; int32_t status; double rr0, rrn; } abft_cg_resul
 int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
                   abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream);
 
-/* Check (and with scrub=1 correct in place) every codeword of the matrix chunks
- * and of the nvec vectors, counting into dcnt. */
+/* Check every codeword of the matrix chunks and of the nvec vectors, counting
+ * into dcnt.  scrub: 0 count only, 1 count and correct single flips in place,
+ * 2 detection only (every failing codeword is a DUE, nothing is written). */
 int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs, int nvec, int scrub,
                    abft_counts* dcnt, void* stream);
 

@@ -334,7 +334,8 @@ int or_vec_encode(uint64_t* data, int64_t n, int scheme) {
 }
 
 /* Check every codeword of v (count into target VEC), write masked values to out
- * (may be NULL); scrub = write corrections back into data.  Returns number of DUEs. */
+ * (may be NULL); scrub = write corrections back into data (2: detection only, every
+ * failing codeword is a DUE).  Returns number of DUEs. */
 int64_t or_vec_check(uint64_t* data, int64_t n, int scheme, double* out, counts_t* cnt, int scrub) {
   init_instances();
   int g = vec_group(scheme), k = vec_k(scheme);
@@ -343,6 +344,7 @@ int64_t or_vec_check(uint64_t* data, int64_t n, int scheme, double* out, counts_
     uint64_t d[4];
     for (int j = 0; j < g; j++) d[j] = data[i + j];
     int o = vec_check_group(d, scheme);
+    if (o == OUT_CORRECTED && scrub == 2) o = OUT_DUE;   /* detection only */
     count_outcome(cnt, T_VEC, scheme, o);
     if (o == OUT_DUE) { dues++; for (int j = 0; j < g; j++) d[j] = data[i + j]; }
     if (o == OUT_CORRECTED && scrub) for (int j = 0; j < g; j++) data[i + j] = d[j];

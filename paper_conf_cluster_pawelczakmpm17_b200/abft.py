@@ -35,7 +35,8 @@ class Vec(C.Structure):
 
 
 class CGOpts(C.Structure):
-    _fields_ = [("tol", C.c_double), ("max_iters", C.c_int32), ("due_policy", C.c_int32), ("poll_every", C.c_int32)]
+    _fields_ = [("tol", C.c_double), ("max_iters", C.c_int32), ("due_policy", C.c_int32), ("poll_every", C.c_int32),
+                ("check_interval", C.c_int32)]
 
 
 class CGResult(C.Structure):
@@ -53,6 +54,7 @@ _sig = {
     "abft_vec_encode": (C.c_int, [_P, C.POINTER(Vec), _P]),
     "abft_vec_decode": (C.c_int, [_P, C.POINTER(Vec), _P, _P, _P]),
     "abft_spmv": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), _P, _P, _P]),
+    "abft_spmv_ex": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), _P, _P, C.c_int32, _P]),
     "abft_cg_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                 C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
     "abft_check_all": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.c_int, C.c_int, _P, _P]),
@@ -246,18 +248,23 @@ class Counters:
         return np.array(list(host), dtype=np.uint64).reshape(3, 5, 4)
 
 
+# matrix check modes of one SpMV access (abft_check_mode)
+CHECK_CORRECT, CHECK_DETECT, CHECK_RANGE = 0, 1, 2
+
+
 def spmv(ctx: Context, A, x: Vector, y: Vector, counts: Counters | None = None, dot: torch.Tensor | None = None,
-         stream=None):
+         stream=None, mode: int = CHECK_CORRECT):
     arr, n = _chunks(A)
     vx, vy = x.cstruct(), y.cstruct()
-    _check(_lib.abft_spmv(ctx.h, arr, n, C.byref(vx), C.byref(vy), dot.data_ptr() if dot is not None else None,
-                          counts.ptr if counts else None, _stream(stream)), "abft_spmv")
+    _check(_lib.abft_spmv_ex(ctx.h, arr, n, C.byref(vx), C.byref(vy), dot.data_ptr() if dot is not None else None,
+                             counts.ptr if counts else None, int(mode), _stream(stream)), "abft_spmv_ex")
 
 
 def cg_solve(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vector, tol=1e-10, max_iters=10000,
-             due_policy=0, counts: Counters | None = None, poll_every=16, stream=None) -> CGResult:
+             due_policy=0, counts: Counters | None = None, poll_every=16, stream=None,
+             check_interval=1) -> CGResult:
     arr, n = _chunks(A)
-    opts = CGOpts(tol, max_iters, due_policy, poll_every)
+    opts = CGOpts(tol, max_iters, due_policy, poll_every, check_interval)
     res = CGResult()
     vs = [v.cstruct() for v in (b, x, r, p, w)]
     code = _lib.abft_cg_solve(ctx.h, arr, n, *[C.byref(v) for v in vs], C.byref(opts), C.byref(res),
@@ -321,9 +328,9 @@ class Dist:
             self.h = None
 
     def cg_solve(self, ctx: Context, A, n_halo: int, b, x, r, p, w, tol=1e-10, max_iters=10000, due_policy=0,
-                 counts: Counters | None = None, poll_every=16, stream=None) -> CGResult:
+                 counts: Counters | None = None, poll_every=16, stream=None, check_interval=1) -> CGResult:
         arr, n = _chunks(A)
-        opts = CGOpts(tol, max_iters, due_policy, poll_every)
+        opts = CGOpts(tol, max_iters, due_policy, poll_every, check_interval)
         res = CGResult()
         vs = [v.cstruct() for v in (b, x, r, p, w)]
         code = _lib.abft_cg_solve_dist(self.h, ctx.h, arr, n, int(n_halo), *[C.byref(v) for v in vs], C.byref(opts),

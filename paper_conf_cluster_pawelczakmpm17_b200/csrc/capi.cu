@@ -94,7 +94,8 @@ int check_chunks(const abft_csr* A, int nchunks) {
 // Launch the SpMV over all chunks; partials indexed by global RB (chunks must
 // start on 256-row boundaries relative to chunk 0 when dot is requested).
 int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, bool dot,
-                DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total, RedArgs red = RedArgs{}) {
+                DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total, RedArgs red = RedArgs{},
+                int check_mode = MODE_CORRECT, int check_interval = 0) {
   const int64_t base0 = A[0].row_base;
   const int64_t npad_in = vec_padded_len(in->n, in->scheme);
   const int64_t npad_out = vec_padded_len(out->n, out->scheme);
@@ -136,6 +137,8 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.state = st;
     a.red = red;
     if (a.red.rs) a.red.nrb = nrb_all;
+    a.check_mode = check_mode;
+    a.check_interval = check_interval;
     count_launch(launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s));
   }
   if (nrb_total) *nrb_total = nrb_all;
@@ -239,7 +242,13 @@ int abft_vec_decode(abft_ctx* ctx, abft_vec* v, double* out_masked, abft_counts*
 
 int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, double* dot_out,
               abft_counts* dcnt, void* stream) {
+  return abft_spmv_ex(ctx, A, nchunks, in, out, dot_out, dcnt, ABFT_CHECK_CORRECT, stream);
+}
+
+int abft_spmv_ex(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, double* dot_out,
+                 abft_counts* dcnt, int32_t check_mode, void* stream) {
   if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  if (check_mode < ABFT_CHECK_CORRECT || check_mode > ABFT_CHECK_RANGE) return fail(ABFT_E_INVALID, "bad check mode");
   int e = check_chunks(A, nchunks);
   if (e) return e;
   if ((e = check_vec(in, "in")) || (e = check_vec(out, "out"))) return e;
@@ -247,7 +256,8 @@ int abft_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_
   if (in->scheme != out->scheme) return fail(ABFT_E_INVALID, "in/out schemes differ");
   cudaStream_t s = (cudaStream_t)stream;
   int64_t nrb = 0;
-  e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb);
+  e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb,
+                  RedArgs{}, check_mode);
   if (e) return e;
   if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
   CUDA_TRY(cudaGetLastError());
@@ -399,6 +409,8 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   const int64_t npad = vec_padded_len(n, scheme);
   const int64_t nrb = (n + 255) / 256;
   if ((e = ensure_partials(ctx, nrb))) return e;
+  if (opts->check_interval < 0) return fail(ABFT_E_INVALID, "negative check interval");
+  const int interval = opts->check_interval > 1 ? opts->check_interval : 0;
   if (nrb > (int64_t)1024 * 1024) return fail(ABFT_E_SHAPE, "more than 2^28 rows per GPU");
   // the dist path runs whenever a communicator is given (also with 1 rank, so the
   // all-gather / top-of-tree combine code is exercised on a single GPU)
@@ -431,7 +443,7 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   // init (a2): w = A x0 ; r = b - w ; p = r ; rr0
   if ((e = halo_exchange(d, reinterpret_cast<uint64_t*>(x->data), n, n_halo, s))) return e;
   prof.begin(0);
-  e = spmv_chunks(ctx, A, nchunks, x, w, false, cnt, nullptr, s, nullptr);
+  e = spmv_chunks(ctx, A, nchunks, x, w, false, cnt, nullptr, s, nullptr, RedArgs{}, MODE_CORRECT, interval);
   prof.end();
   if (e) return e;
   count_launch(launch_init_r(va, scheme, s));
@@ -446,7 +458,8 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       int e2;
       if ((e2 = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e2;
       prof.begin(0);
-      e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2));
+      e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2),
+                       MODE_CORRECT, interval);
       prof.end();
       if (e2) return e2;
       prof.begin(3);
@@ -531,6 +544,26 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   res->rr0 = hs.rr0;
   res->rrn = hs.rrn;
   res->status = hs.stop ? hs.status : (opts->max_iters > 0 ? ABFT_E_NOT_CONVERGED : ABFT_OK);
+  // interval mode: detection-only integrity check of the whole matrix when the
+  // last access (= iteration count) was not a checked one
+  if (interval && hs.iters % interval != 0) {
+    CUDA_TRY(cudaMemsetAsync(ctx->due, 0, sizeof(int), s));
+    for (int c = 0; c < nchunks; c++) count_launch(launch_check_csr(&A[c], cnt, ctx->due, 2, s));
+    int any = 0;
+    if (multi) {
+      count_launch(launch_pack_due(d->sendbuf, ctx->due, s));
+      NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
+      std::vector<double> g(2 * (size_t)d->nranks);
+      CUDA_TRY(cudaMemcpyAsync(g.data(), d->gathered, sizeof(double) * g.size(), cudaMemcpyDeviceToHost, s));
+      CUDA_TRY(cudaStreamSynchronize(s));
+      for (int rk = 0; rk < d->nranks; rk++) any |= g[2 * rk + 1] != 0.0;
+    } else {
+      CUDA_TRY(cudaMemcpyAsync(ctx->h_flags, ctx->due, sizeof(int), cudaMemcpyDeviceToHost, s));
+      CUDA_TRY(cudaStreamSynchronize(s));
+      any = ctx->h_flags[0] != 0;
+    }
+    if (any && h.abort_policy && res->status != ABFT_E_DUE) res->status = ABFT_E_DUE;
+  }
   if (res->status != ABFT_OK) fail(res->status, "CG finished with status %d after %d iterations", res->status, res->iters);
   return res->status;
 }

@@ -52,7 +52,12 @@ struct SpmvArgs {
   int* due;          // DUE / range flag (never null)
   const CgState* state;  // may be null
   RedArgs red;
+  // matrix check mode of this access: MODE_CORRECT / DETECT /
+  // RANGE; with check_interval > 1 the kernel derives it from the device
+  // iteration counter instead (access k = state->iters + 1, init = 0)
+  int32_t check_mode, check_interval;
 };
+enum { MODE_CORRECT = 0, MODE_DETECT = 1, MODE_RANGE = 2 };
 
 struct VecArgs {
   int64_t n, npad;

@@ -43,6 +43,15 @@ static __device__ __forceinline__ void load_lut(uint8_t* s_lut) {
   if (threadIdx.x < 32) reinterpret_cast<uint32_t*>(s_lut)[threadIdx.x] = reinterpret_cast<const uint32_t*>(&c_v64_lut)[threadIdx.x];
 }
 
+// Matrix check mode of this SpMV access.
+static __device__ __forceinline__ int spmv_mode(const SpmvArgs& a) {
+  if (a.check_interval > 1) {
+    const int64_t acc = a.state ? (int64_t)a.state->iters + 1 : 0;   // init = access 0
+    return (acc % a.check_interval) ? MODE_RANGE : MODE_DETECT;
+  }
+  return a.check_mode;
+}
+
 struct RedArgs;
 static __device__ void red_push(double* partials, int64_t rb, double val, const RedArgs& r, int lane);
 
@@ -179,7 +188,7 @@ __device__ __forceinline__ double gather_in(const uint64_t* in, int64_t idx) {
 // this lane's start/end.
 template <int RS>
 __device__ __forceinline__ void rowptr_pass(const SpmvArgs& a, int64_t pb, int lane, uint32_t* srp, uint32_t& start,
-                                            uint32_t& end) {
+                                            uint32_t& end, int mode) {
   constexpr int G = rgrp(RS);
   if (RS == NONE) {
     const int64_t e = pb + lane;
@@ -206,7 +215,8 @@ __device__ __forceinline__ void rowptr_pass(const SpmvArgs& a, int64_t pb, int l
 #pragma unroll
     for (int t = 0; t < G; t++) o0[t] = e[t];
     int word = 0;
-    int o = rp_check_group<RS>(e, &word);
+    int o = (mode == MODE_RANGE) ? CLEAN : rp_check_group<RS>(e, &word);
+    if (o == CORRECTED && mode == MODE_DETECT) o = DUE;   // interval mode: detection only
     if (o != CLEAN) {
       int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
       bool owner = own >= pb && own < pb + 32;
@@ -230,11 +240,12 @@ __device__ __forceinline__ void rowptr_pass(const SpmvArgs& a, int64_t pb, int l
 // Cold path of an element check: correct, scrub (winner counts), or DUE.
 template <int ES>
 __device__ __noinline__ int elem_fix(uint64_t& v, uint32_t& c, uint64_t* vaddr, uint32_t* caddr, DevCounts* cnt,
-                                     int* due) {
+                                     int* due, int mode) {
   uint64_t v0 = v;
   uint32_t c0 = c;
   int word = 0;
   int o = (ES == SED) ? DUE : e96_correct(v, c, &word);
+  if (o == CORRECTED && mode == MODE_DETECT) o = DUE;   // interval mode: detection only
   if (o == CORRECTED) {
     bool won;
     if (word == 2) won = scrub32(caddr, c0, c);
@@ -263,13 +274,14 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
   if (rb >= nrb) return;
   double dot = 0.0;
   const uint32_t ckeep = col_keep(ES);
+  const int mode = spmv_mode(a);
   for (int k = 0; k < 8; k++) {
     const int64_t pb = rb * 256 + k * 32;
     if (pb >= a.nrows) break;
     const int64_t i = pb + lane;
     const bool valid = i < a.nrows;
     uint32_t start, end;
-    rowptr_pass<RS>(a, pb, lane, s_rp[warp], start, end);
+    rowptr_pass<RS>(a, pb, lane, s_rp[warp], start, end, mode);
     // own codeword of `in` (checked once, counted here: DESIGN.md §3.8)
     const int64_t own = a.row_base + i;
     const int64_t own_lim = (vgrp(VS) == 1 && !valid) ? 0 : a.npad_in;
@@ -288,11 +300,11 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
           uint32_t c = __ldg(a.col + j);
           if (ES == CRC32C) {
             int kk = (int)(j - start);
-            crc = ecrc_update(crc, v, c, kk);
+            if (mode != MODE_RANGE) crc = ecrc_update(crc, v, c, kk);
             if (kk < 4) crc_st |= (c >> 24) << (8 * kk);
-          } else if (ES != NONE) {
+          } else if (ES != NONE && mode != MODE_RANGE) {
             bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
-            if (bad) elem_fix<ES>(v, c, a.val + j, a.col + j, a.counts, a.due);
+            if (bad) elem_fix<ES>(v, c, a.val + j, a.col + j, a.counts, a.due, mode);
           }
           const uint32_t cm = c & ckeep;
           if (ES != NONE && (int64_t)cm >= a.ncols) {
@@ -304,7 +316,7 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
           const double x = (idx == own) ? p_own : gather_in<VS>(a.in, idx);
           acc = fma(as_d(v), x, acc);
         }
-        if (ES == CRC32C) {
+        if (ES == CRC32C && mode != MODE_RANGE) {
           if (end - start < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
             cnt_add(a.counts, T_ELEM, CRC32C, DUE);
             *a.due = 1;
@@ -407,7 +419,7 @@ static __device__ __forceinline__ void tile_produce(const TileMaps& tm, uint8_t*
 template <int ES, int RS, int VS>
 static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start, uint32_t end, const uint64_t* sval,
                                                  const uint32_t* scol, bool staged, const double* win, int oslot,
-                                                 double p_own, int64_t own, uint32_t s0, uint32_t s1) {
+                                                 double p_own, int64_t own, uint32_t s0, uint32_t s1, int mode) {
   double acc = 0.0;
   const bool ok = (start <= end) && ((int64_t)end <= a.nnz);
   // a corrupted (DUE) rowptr entry can put this row outside the staged range:
@@ -433,11 +445,11 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
       c = __ldg(a.col + start + j);
     }
     if (ES == CRC32C) {
-      crc = ecrc_update(crc, v, c, (int)j);
+      if (mode != MODE_RANGE) crc = ecrc_update(crc, v, c, (int)j);
       if (j < 4) crc_st |= (c >> 24) << (8 * j);
-    } else if (ES != NONE) {
+    } else if (ES != NONE && mode != MODE_RANGE) {
       bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
-      if (bad) elem_fix<ES>(v, c, a.val + start + j, a.col + start + j, a.counts, a.due);
+      if (bad) elem_fix<ES>(v, c, a.val + start + j, a.col + start + j, a.counts, a.due, mode);
     }
     const uint32_t cm = c & ckeep;
     if (ES != NONE && (int64_t)cm >= a.ncols) {
@@ -455,7 +467,7 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
     else x = gather_in<VS>(a.in, own + rel);
     acc = fma(as_d(v), x, acc);
   }
-  if (ES == CRC32C) {
+  if (ES == CRC32C && mode != MODE_RANGE) {
     if (len < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
       cnt_add(a.counts, T_ELEM, CRC32C, DUE);
       *a.due = 1;
@@ -472,10 +484,11 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
 template <int ES, int RS, int VS>
 static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const SpmvArgs& sa, uint32_t start, uint32_t end,
                                                    const uint64_t* sval, const uint32_t* scol, const double* win,
-                                                   int oslot, double p_own, int64_t own, uint32_t s0, int lane) {
+                                                   int oslot, double p_own, int64_t own, uint32_t s0, int lane,
+                                                   int mode) {
   const uint32_t s1 = s0 + TILE_PE;
-  if (ES == CRC32C || start != s0 + 5u * (uint32_t)lane || end != start + 5u)
-    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1);
+  if ((ES == CRC32C && mode != MODE_RANGE) || start != s0 + 5u * (uint32_t)lane || end != start + 5u)
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1, mode);
   const int n32 = (int)a.stencil_n;
   const int own_col = (int)(own - a.col_base);
   const uint32_t ckeep = col_keep(ES);
@@ -487,10 +500,12 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
     c[t] = scol[5 * lane + t];
   }
   uint32_t acc_r = 0, acc_p = 0;
+  if (mode != MODE_RANGE) {   // uniform: interval mode's unchecked accesses skip the codec
 #pragma unroll
-  for (int t = 0; t < 5; t++) {
-    if (ES == SED) acc_p |= (uint32_t)(popc64(v[t]) + popc32(c[t]));
-    else if (ES != NONE) e96_acc(lo32(v[t]), hi32(v[t]), c[t], acc_r, acc_p);
+    for (int t = 0; t < 5; t++) {
+      if (ES == SED) acc_p |= (uint32_t)(popc64(v[t]) + popc32(c[t]));
+      else if (ES == SECDED64 || ES == SECDED128) e96_acc(lo32(v[t]), hi32(v[t]), c[t], acc_r, acc_p);
+    }
   }
   // canonical stencil neighbours [i-n, i-1, i, i+1, i+n] or the row itself (R16)
   int d[5];
@@ -505,7 +520,7 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
                      ((unsigned)d[3] <= 1u) && (d[4] == 0 || d[4] == n32);
   const bool in_range = (ES == NONE) || cmax < (uint32_t)a.ncols;
   if ((ES != NONE && syn_bad(acc_r, acc_p)) || !canon || !in_range)
-    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1);
+    return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1, mode);
   // slot offsets: d itself for +-1 / 0, +-window width for +-n
   const int o0 = d[0] ? -TILE_WW : 0, o4 = d[4] ? TILE_WW : 0;
   double acc = fma(as_d(v[0]), win[oslot + o0], 0.0);
@@ -548,6 +563,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   }
   if (VS == SECDED64) load_lut(s_lut);
   const int stop_v = a.state ? a.state->stop : 0;  // checked after the prologue loads are in flight
+  const int mode = spmv_mode(a);
   const int64_t gy = ty0 + warp;
   const bool has_seg = gy < ny;
   const int64_t rowseg = gy * n + tx0;
@@ -575,9 +591,11 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
     }
     if (!stop_v) {
       uint32_t acc = 0;
+      if (mode != MODE_RANGE) {
 #pragma unroll
-      for (int q = 0; q < PER; q++)
-        if (RS != NONE && lane + 32 * q < NG) acc |= rp_acc<RS>(e[q]);
+        for (int q = 0; q < PER; q++)
+          if (RS != NONE && lane + 32 * q < NG) acc |= rp_acc<RS>(e[q]);
+      }
       if (RS != NONE && (acc & 1u)) {  // cold: locate, correct, count (owner), per group
 #pragma unroll
         for (int q = 0; q < PER; q++) {
@@ -590,6 +608,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
           for (int t = 0; t < G; t++) o0[t] = e[q][t];
           int word = 0;
           int o = rp_check_group<RS>(e[q], &word);
+          if (o == CORRECTED && mode == MODE_DETECT) o = DUE;   // interval mode: detection only
           if (o != CLEAN) {
             const int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
             const bool owner = own >= rowseg && own < rowseg + 256;
@@ -676,7 +695,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       const double p_own = s_win[oslot];
       const int64_t own = a.row_base + rowseg + k * 32 + lane;
       const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s_win, oslot, p_own, own,
-                                               seg_e + 160u * k, lane);
+                                               seg_e + 160u * k, lane, mode);
       const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
       a.out[own] = enc;
       if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
@@ -1141,6 +1160,7 @@ __global__ void k_vec_check(uint64_t* d, int64_t n, int64_t npad, double* out, D
     for (int t = 0; t < G; t++) o0[t] = v[t] = d[g * G + t];
     int word = 0;
     int o = vec_check_group<VS>(v, &word);
+    if (o == CORRECTED && scrub == 2) o = DUE;   // detection only
     if (o == CORRECTED) {
       bool won = true;
       if (scrub) {
@@ -1213,6 +1233,7 @@ __global__ void k_check_elems(uint64_t* val, uint32_t* col, int64_t nnz, int64_t
     int o = CLEAN;
     if (ES == SED) o = esed_clean(v, c) ? CLEAN : DUE;
     else if (e96_bad(lo32(v), hi32(v), c)) o = e96_correct(v, c, &word);
+    if (o == CORRECTED && scrub == 2) o = DUE;   // detection only (interval mode's final check)
     if (o == CORRECTED) {
       bool won = true;
       if (scrub) won = (word == 2) ? scrub32(col + e, c0, c)
@@ -1235,6 +1256,7 @@ __global__ void k_check_rowptr(uint32_t* rowptr, int64_t len, DevCounts* cnt, in
     for (int t = 0; t < G; t++) o0[t] = e[t] = rowptr[g * G + t];
     int word = 0;
     int o = rp_check_group<RS>(e, &word);
+    if (o == CORRECTED && scrub == 2) o = DUE;   // detection only (interval mode's final check)
     if (o == CORRECTED) {
       bool won = scrub ? scrub32(rowptr + g * G + word, o0[word], e[word]) : true;
       if (won) cnt_add(cnt, T_ROWPTR, RS, CORRECTED);
