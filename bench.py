@@ -113,9 +113,10 @@ def build_problem(grid: int, rank: int, world: int, device, chunk_rows=None):
 class Solver:
     """One configuration (protected or unprotected twin) of the solve."""
 
-    def __init__(self, abft, ctx, P, es, rs, vs, dist=None):
+    def __init__(self, abft, ctx, P, es, rs, vs, dist=None, check_interval=1):
         import torch
         self.abft, self.ctx, self.P, self.dist = abft, ctx, P, dist
+        self.check_interval = check_interval
         self.es, self.rs, self.vs = es, rs, vs
         N, halo = P["N"], P["halo"]
         dev = P["b"].device
@@ -162,10 +163,11 @@ class Solver:
         self.vecs[1].encode(self.ctx)
         if self.dist is not None:
             res = self.dist.cg_solve(self.ctx, self.A, self.halo, *self.vecs, tol=tol, max_iters=max_iters,
-                                     due_policy=1, counts=self.counts, poll_every=32)
+                                     due_policy=1, counts=self.counts, poll_every=32,
+                                     check_interval=self.check_interval)
         else:
             res = self.abft.cg_solve(self.ctx, self.A, *self.vecs, tol=tol, max_iters=max_iters, due_policy=1,
-                                     counts=self.counts, poll_every=32)
+                                     counts=self.counts, poll_every=32, check_interval=self.check_interval)
         return res.iters, res.status
 
 

@@ -10,6 +10,11 @@ window of protected CG iterations (tol 0) after one warm-up solve; reported
 per-iteration time and overhead vs the unprotected twin.  SECDED128 on CSR
 elements maps to E-SECDED (reading R3).  SECDED128/CRC32C vectors (groups of
 2/4 doubles) run the generic kernels (the tiled SpMV fast path is G = 1 only).
+
+--intervals 1,2,4,...: additionally the check-interval sweep of the paper's
+Figs 6-8: the whole CSR matrix (elements + row pointers) protected
+with SED / SECDED64 / CRC32C, vectors unprotected, matrix checked (detection
+only) every N-th access and range-checked otherwise.
 """
 from __future__ import annotations
 
@@ -28,6 +33,8 @@ def main():
     ap.add_argument("--iters", type=int, default=200)
     ap.add_argument("--reps", type=int, default=2)
     ap.add_argument("--out", default=os.path.join(ROOT, "gpurun_out", "sweep.json"))
+    ap.add_argument("--intervals", default="", help="comma-separated check intervals (matrix-only configs)")
+    ap.add_argument("--no-schemes", action="store_true", help="skip the per-scheme sweep")
     a = ap.parse_args()
     import torch
     import bench
@@ -36,17 +43,22 @@ def main():
     P = bench.build_problem(a.grid, 0, 1, torch.device("cuda", 0))
     ctx = abft.Context(0)
     names = ["NONE", "SED", "SECDED64", "SECDED128", "CRC32C"]
-    configs = []
-    for s in names:
-        configs.append(("all", s, (s, s, s)))
-    for s in names[1:]:
-        configs.append(("elements", s, (s, "NONE", "NONE")))
-        configs.append(("rowptr", s, ("NONE", s, "NONE")))
-        configs.append(("vectors", s, ("NONE", "NONE", s)))
+    configs = [("all", "NONE", ("NONE", "NONE", "NONE"), 1)]
+    if not a.no_schemes:
+        for s in names[1:]:
+            configs.append(("all", s, (s, s, s), 1))
+        for s in names[1:]:
+            configs.append(("elements", s, (s, "NONE", "NONE"), 1))
+            configs.append(("rowptr", s, ("NONE", s, "NONE"), 1))
+            configs.append(("vectors", s, ("NONE", "NONE", s), 1))
+    for N in [int(t) for t in a.intervals.split(",") if t]:
+        for s in ("SED", "SECDED64", "CRC32C"):
+            configs.append(("matrix", s, (s, s, "NONE"), N))
     rows = []
     base = None
-    for (what, s, (es, rs, vs)) in configs:
-        sol = bench.Solver(abft, ctx, P, getattr(abft, es), getattr(abft, rs), getattr(abft, vs))
+    for (what, s, (es, rs, vs), interval) in configs:
+        sol = bench.Solver(abft, ctx, P, getattr(abft, es), getattr(abft, rs), getattr(abft, vs),
+                           check_interval=interval)
         sol.step(0.0, 5)   # warm-up (graph capture, attributes)
         best = None
         for _ in range(a.reps):
@@ -60,7 +72,8 @@ def main():
             best = ms if best is None else min(best, ms)
         if what == "all" and s == "NONE":
             base = best
-        row = {"structures": what, "scheme": s, "elem": es, "rowptr": rs, "vectors": vs, "iter_ms": best,
+        row = {"structures": what, "scheme": s, "elem": es, "rowptr": rs, "vectors": vs, "check_interval": interval,
+               "iter_ms": best,
                "overhead_pct": None if base is None else 100.0 * (best / base - 1.0),
                "cg_gbs": 152.0 * P["N"] / (best / 1000.0) / 1e9}
         rows.append(row)
