@@ -134,6 +134,17 @@ typedef struct { int32_t iters; int32_t status; double rr0, rrn; } abft_cg_resul
 int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
                   abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream);
 
+/* a4 / a5 as single calls (the CG driver fuses them into its device-side loop):
+ * calc_ur  x = enc(fma(alpha, p, x)); r = enc(fma(-alpha, w, r)); rrn_out = r.r (RED-1)
+ * calc_p   p = enc(fma(beta, p, r))
+ * (TeaLeaf CG).  Every operand codeword is checked on
+ * load and single flips corrected (counted into dcnt, may be NULL); x, r, p, w
+ * must have equal length and scheme and must not alias.  rrn_out: device f64
+ * (may be NULL). */
+int abft_calc_ur(abft_ctx* ctx, abft_vec* x, abft_vec* p, abft_vec* r, abft_vec* w, double alpha, double* rrn_out,
+                 abft_counts* dcnt, void* stream);
+int abft_calc_p(abft_ctx* ctx, abft_vec* p, abft_vec* r, double beta, abft_counts* dcnt, void* stream);
+
 /* Check every codeword of the matrix chunks and of the nvec vectors, counting
  * into dcnt.  scrub: 0 count only, 1 count and correct single flips in place,
  * 2 detection only (every failing codeword is a DUE, nothing is written). */

@@ -58,6 +58,9 @@ _sig = {
     "abft_cg_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                 C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
     "abft_check_all": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.c_int, C.c_int, _P, _P]),
+    "abft_calc_ur": (C.c_int, [_P, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.c_double, _P, _P,
+                               _P]),
+    "abft_calc_p": (C.c_int, [_P, C.POINTER(Vec), C.POINTER(Vec), C.c_double, _P, _P]),
     "abft_inject_bitflip": (C.c_int, [_P, _P, C.c_uint64, _P]),
     "abft_counts_read": (C.c_int, [_P, _P, _P]),
     "abft_counts_reset": (C.c_int, [_P, _P]),
@@ -271,6 +274,22 @@ def cg_solve(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vec
                               counts.ptr if counts else None, _stream(stream))
     _check(code, "abft_cg_solve", allow=(E_DUE, E_NOT_CONVERGED))
     return res
+
+
+def calc_ur(ctx: Context, x: Vector, p: Vector, r: Vector, w: Vector, alpha: float,
+            rrn: torch.Tensor | None = None, counts: Counters | None = None, stream=None):
+    """a4: x = enc(fma(alpha, p, x)); r = enc(fma(-alpha, w, r)); rrn[0] = r.r (RED-1)."""
+    vs = [v.cstruct() for v in (x, p, r, w)]
+    _check(_lib.abft_calc_ur(ctx.h, *[C.byref(v) for v in vs], float(alpha),
+                             rrn.data_ptr() if rrn is not None else None, counts.ptr if counts else None,
+                             _stream(stream)), "abft_calc_ur")
+
+
+def calc_p(ctx: Context, p: Vector, r: Vector, beta: float, counts: Counters | None = None, stream=None):
+    """a5: p = enc(fma(beta, p, r))."""
+    vp, vr = p.cstruct(), r.cstruct()
+    _check(_lib.abft_calc_p(ctx.h, C.byref(vp), C.byref(vr), float(beta), counts.ptr if counts else None,
+                            _stream(stream)), "abft_calc_p")
 
 
 def check_all(ctx: Context, A, vecs, counts: Counters | None = None, scrub=True, stream=None):

@@ -57,6 +57,7 @@ struct abft_ctx {
   int64_t prof_n[4] = {0, 0, 0, 0};
   std::vector<cudaEvent_t> events;
   RedState* red = nullptr;   // fused-reduction counters/roots (zero between reductions)
+  CrcTables* crc = nullptr;  // CRC32C lookup tables (device)
 };
 
 namespace {
@@ -139,6 +140,7 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     if (a.red.rs) a.red.nrb = nrb_all;
     a.check_mode = check_mode;
     a.check_interval = check_interval;
+    a.crc = ctx->crc;
     count_launch(launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s));
   }
   if (nrb_total) *nrb_total = nrb_all;
@@ -172,6 +174,12 @@ int abft_ctx_create(int device, abft_ctx** out) {
   CUDA_TRY(cudaMemset(c->red, 0, sizeof(RedState)));
   CUDA_TRY(cudaMallocHost(&c->h_state, sizeof(CgState)));
   CUDA_TRY(cudaMallocHost(&c->h_flags, sizeof(uint32_t) * 4));
+  {
+    std::vector<CrcTables> h(1);
+    build_crc_tables(h.data());
+    CUDA_TRY(cudaMalloc(&c->crc, sizeof(CrcTables)));
+    CUDA_TRY(cudaMemcpy(c->crc, h.data(), sizeof(CrcTables), cudaMemcpyHostToDevice));
+  }
   int e = ensure_partials(c, 1024);
   if (e) return e;
   *out = c;
@@ -188,6 +196,7 @@ int abft_ctx_destroy(abft_ctx* c) {
   cudaFree(c->due);
   cudaFree(c->flags);
   cudaFree(c->red);
+  cudaFree(c->crc);
   cudaFreeHost(c->h_state);
   cudaFreeHost(c->h_flags);
   for (auto e : c->events) cudaEventDestroy(e);
@@ -438,6 +447,7 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   va.due = ctx->due;
   va.state = ctx->state;
   va.red = red_for(ctx, d, nrb, 1);
+  va.crc = ctx->crc;
 
   Prof prof{ctx, s};
   // init (a2): w = A x0 ; r = b - w ; p = r ; rr0
@@ -634,6 +644,70 @@ int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs
                                   vec_padded_len(vecs[i].n, vecs[i].scheme), vecs[i].scheme, nullptr, cnt, ctx->due,
                                   scrub, s));
   }
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+// a4 / a5 as single calls: a scratch CG state carries alpha / beta (never stops)
+static int blas1_setup(abft_ctx* ctx, abft_vec* const* v, int nv, double alpha, double beta, VecArgs& va,
+                       cudaStream_t s) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  const char* names[4] = {"x", "p", "r", "w"};
+  for (int i = 0; i < nv; i++) {
+    int e = check_vec(v[i], names[i]);
+    if (e) return e;
+    if (v[i]->scheme != v[0]->scheme || v[i]->n != v[0]->n) return fail(ABFT_E_INVALID, "vectors differ");
+    for (int j = 0; j < i; j++) if (v[i]->data == v[j]->data) return fail(ABFT_E_INVALID, "vectors alias");
+  }
+  const int64_t n = v[0]->n, nrb = (n + 255) / 256;
+  int e = ensure_partials(ctx, nrb);
+  if (e) return e;
+  CgState h{};
+  h.alpha = alpha;
+  h.beta = beta;
+  h.max_iters = 0x7FFFFFFF;
+  *ctx->h_state = h;
+  CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
+  va = VecArgs{};
+  va.n = n;
+  va.npad = vec_padded_len(n, v[0]->scheme);
+  va.partials = ctx->partials;
+  va.due = ctx->due;
+  va.state = ctx->state;
+  va.crc = ctx->crc;
+  return ABFT_OK;
+}
+
+int abft_calc_ur(abft_ctx* ctx, abft_vec* x, abft_vec* p, abft_vec* r, abft_vec* w, double alpha, double* rrn_out,
+                 abft_counts* dcnt, void* stream) {
+  cudaStream_t s = (cudaStream_t)stream;
+  abft_vec* v[4] = {x, p, r, w};
+  VecArgs va;
+  int e = blas1_setup(ctx, v, 4, alpha, 0.0, va, s);
+  if (e) return e;
+  va.x = reinterpret_cast<uint64_t*>(x->data);
+  va.p = reinterpret_cast<uint64_t*>(p->data);
+  va.r = reinterpret_cast<uint64_t*>(r->data);
+  va.w = reinterpret_cast<uint64_t*>(w->data);
+  va.counts = reinterpret_cast<DevCounts*>(dcnt);
+  count_launch(launch_calc_ur(va, x->scheme, s));
+  if (rrn_out)
+    count_launch(launch_reduce(ctx->partials, (x->n + 255) / 256, ctx->roots, ctx->ticket, 0, nullptr, rrn_out,
+                               ctx->due, s));
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_calc_p(abft_ctx* ctx, abft_vec* p, abft_vec* r, double beta, abft_counts* dcnt, void* stream) {
+  cudaStream_t s = (cudaStream_t)stream;
+  abft_vec* v[2] = {p, r};
+  VecArgs va;
+  int e = blas1_setup(ctx, v, 2, 0.0, beta, va, s);
+  if (e) return e;
+  va.p = reinterpret_cast<uint64_t*>(p->data);
+  va.r = reinterpret_cast<uint64_t*>(r->data);
+  va.counts = reinterpret_cast<DevCounts*>(dcnt);
+  count_launch(launch_calc_p(va, p->scheme, s));
   CUDA_TRY(cudaGetLastError());
   return ABFT_OK;
 }

@@ -366,6 +366,22 @@ ABFT_HD void v128_encode(uint64_t* d) {   // d[0..1] already rounded (low 5 bits
   d[0] = mk64(w[0], w[1]);
   d[1] = mk64(w[2], w[3]);
 }
+// Fast "not clean?" test of a pair (bit 0 of the result set <=> q or some
+// syndrome bit is 1): OR of the 9 row popcounts, masks as immediates.
+ABFT_HD uint32_t v128_acc(uint64_t d0, uint64_t d1) {
+  constexpr MaskTable M = h_mt_v128;
+  const uint32_t w[4] = {lo32(d0), hi32(d0), lo32(d1), hi32(d1)};
+  uint32_t acc = (uint32_t)popc32(w[0] ^ w[1] ^ w[2] ^ w[3]);
+#pragma unroll
+  for (int k = 0; k < 8; k++) {
+    uint32_t t = 0;
+#pragma unroll
+    for (int i = 0; i < 4; i++)
+      if (M.m[k][i]) t ^= w[i] & M.m[k][i];
+    acc |= (uint32_t)popc32(t);
+  }
+  return acc;
+}
 ABFT_HD int v128_check(uint64_t* d, int* word) {
   uint32_t w[4] = {lo32(d[0]), hi32(d[0]), lo32(d[1]), hi32(d[1])};
   int s, q;

@@ -19,6 +19,14 @@ struct CgState {
 
 struct DevCounts { unsigned long long v[3][5][4]; };
 
+// CRC32C lookup tables (reflected 0x82F63B78), built once per
+// context on the host and copied to shared memory by the kernels that use them.
+struct CrcTables {
+  uint32_t slice[4][256];     // slicing-by-4: slice[k][b] = CRC register of byte b followed by k zero bytes
+  uint32_t vpos[4][7][256];   // V-CRC: linear CRC part of byte b at message byte 8t + j + 1 of the 32-byte quad
+};
+void build_crc_tables(CrcTables* host_out);
+
 // Fused RED-1 reduction state (ctx scratch, zero between reductions): the warp
 // that writes the last partial of a 1024-leaf group reduces the group, the
 // warp that completes the last group reduces the group roots and applies the
@@ -56,6 +64,7 @@ struct SpmvArgs {
   // RANGE; with check_interval > 1 the kernel derives it from the device
   // iteration counter instead (access k = state->iters + 1, init = 0)
   int32_t check_mode, check_interval;
+  const CrcTables* crc;   // device tables (CRC32C schemes only)
 };
 enum { MODE_CORRECT = 0, MODE_DETECT = 1, MODE_RANGE = 2 };
 
@@ -68,6 +77,7 @@ struct VecArgs {
   CgState* state;
   double* out_masked;
   RedArgs red;
+  const CrcTables* crc;   // device tables (CRC32C schemes only)
 };
 
 // launchers (kernels.cu); each returns the number of kernels launched

@@ -58,6 +58,29 @@ static inline int grid_for(int64_t n, int threads, int max_blocks = 148 * 16) {
 
 static inline int blocks_rb(int64_t n) { return (int)(((n + 255) / 256 + 7) / 8); }
 
+// CRC32C tables: reflected polynomial 0x82F63B78, bytes LSB first.
+void build_crc_tables(CrcTables* T) {
+  for (uint32_t b = 0; b < 256; b++) {
+    uint32_t c = b;
+    for (int k = 0; k < 8; k++) c = (c >> 1) ^ (0x82F63B78u & (0u - (c & 1u)));
+    T->slice[0][b] = c;
+  }
+  for (int k = 1; k < 4; k++)
+    for (uint32_t b = 0; b < 256; b++) {
+      const uint32_t c = T->slice[k - 1][b];
+      T->slice[k][b] = (c >> 8) ^ T->slice[0][c & 0xFFu];
+    }
+  // linear part of byte b at position p of a 32-byte message: register T0[b]
+  // after that byte (init 0), then 31 - p zero bytes
+  for (int t = 0; t < 4; t++)
+    for (int j = 1; j < 8; j++)
+      for (uint32_t b = 0; b < 256; b++) {
+        uint32_t c = T->slice[0][b];
+        for (int z = 0; z < 31 - (8 * t + j); z++) c = (c >> 8) ^ T->slice[0][c & 0xFFu];
+        T->vpos[t][j - 1][b] = c;
+      }
+}
+
 int launch_calc_ur(const VecArgs& a, int vs, cudaStream_t s) {
   if (a.n <= 0) return 0;
   int nb = blocks_rb(a.n);
@@ -66,7 +89,7 @@ int launch_calc_ur(const VecArgs& a, int vs, cudaStream_t s) {
     case SED: k_calc_ur<SED><<<nb, 256, 0, s>>>(a); break;
     case SECDED64: k_calc_ur<SECDED64><<<nb, 256, 0, s>>>(a); break;
     case SECDED128: k_calc_ur<SECDED128><<<nb, 256, 0, s>>>(a); break;
-    default: k_calc_ur<CRC32C><<<nb, 256, 0, s>>>(a); break;
+    default: k_calc_ur<CRC32C><<<nb, 256, vec_dyn_smem<CRC32C>(), s>>>(a); break;
   }
   return 1;
 }
@@ -78,7 +101,7 @@ int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s) {
     case SED: k_calc_p<SED><<<nb, 256, 0, s>>>(a); break;
     case SECDED64: k_calc_p<SECDED64><<<nb, 256, 0, s>>>(a); break;
     case SECDED128: k_calc_p<SECDED128><<<nb, 256, 0, s>>>(a); break;
-    default: k_calc_p<CRC32C><<<nb, 256, 0, s>>>(a); break;
+    default: k_calc_p<CRC32C><<<nb, 256, vec_dyn_smem<CRC32C>(), s>>>(a); break;
   }
   return 1;
 }

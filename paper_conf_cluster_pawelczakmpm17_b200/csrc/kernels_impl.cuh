@@ -43,6 +43,107 @@ static __device__ __forceinline__ void load_lut(uint8_t* s_lut) {
   if (threadIdx.x < 32) reinterpret_cast<uint32_t*>(s_lut)[threadIdx.x] = reinterpret_cast<const uint32_t*>(&c_v64_lut)[threadIdx.x];
 }
 
+// ====================================== CRC32C tables in shared memory (§3.5)
+// Table-driven CRC32C: the plain bit-serial division costs 8 shift/XOR steps per
+// byte; slicing-by-4 does a 32-bit word with 4 SMEM lookups.
+constexpr uint32_t VCRC_ZERO = 0x8A9136AAu;   // CRC32C of 32 zero bytes (RFC 3720 check value, PIN-4)
+constexpr int CRC_SLICE_WORDS = 4 * 256;
+constexpr int CRC_VPOS_WORDS = 4 * 7 * 256;
+static __device__ __forceinline__ void smem_fill(uint32_t* dst, const uint32_t* src, int nwords) {
+  for (int i = 4 * (int)threadIdx.x; i < nwords; i += 4 * (int)blockDim.x)
+    *reinterpret_cast<uint4*>(dst + i) = __ldg(reinterpret_cast<const uint4*>(src + i));
+}
+// one little-endian 32-bit message word through the reflected CRC register
+static __device__ __forceinline__ uint32_t crc_word(uint32_t c, uint32_t w, const uint32_t* T) {
+  c ^= w;
+  return T[768 + (c & 0xFFu)] ^ T[512 + ((c >> 8) & 0xFFu)] ^ T[256 + ((c >> 16) & 0xFFu)] ^ T[c >> 24];
+}
+// R-CRC octet: bit 0 set <=> stored nibbles != CRC of the masked entries
+static __device__ __forceinline__ uint32_t rcrc_acc_tab(const uint32_t* e, const uint32_t* T) {
+  uint32_t c = 0xFFFFFFFFu, st = 0;
+#pragma unroll
+  for (int i = 0; i < 8; i++) {
+    c = crc_word(c, e[i] & 0x0FFFFFFFu, T);
+    st |= (e[i] >> 28) << (4 * i);
+  }
+  return (c ^ 0xFFFFFFFFu) != st ? 1u : 0u;
+}
+
+// ================================== lane-split group vector codecs (G = 2, 4)
+// In every warp-wide vector access lane l holds index base + l, so the 2 / 4
+// words of an aligned group sit in adjacent lanes.
+static __device__ __forceinline__ uint64_t shfl_xor64(uint64_t v, int m) {
+  const uint32_t lo = __shfl_xor_sync(0xffffffffu, (uint32_t)v, m);
+  const uint32_t hi = __shfl_xor_sync(0xffffffffu, (uint32_t)(v >> 32), m);
+  return mk64(lo, hi);
+}
+// V-SECDED128 "pair gather": lanes 2m, 2m+1 hold the halves of group A in w0
+// (pass k) and of group B in w1 (pass k+32); after one exchange the even lane
+// holds A and the odd lane B whole (d0 = first double, d1 = second), so each
+// lane runs the textbook code with immediate masks.
+static __device__ __forceinline__ void pair_gather(uint64_t w0, uint64_t w1, int lane, uint64_t& d0, uint64_t& d1) {
+  const bool odd = lane & 1;
+  const uint64_t r = shfl_xor64(odd ? w0 : w1, 1);
+  d0 = odd ? r : w0;
+  d1 = odd ? w1 : r;
+}
+static __device__ __forceinline__ void pair_scatter(uint64_t d0, uint64_t d1, int lane, uint64_t& w0, uint64_t& w1) {
+  const bool odd = lane & 1;
+  const uint64_t r = shfl_xor64(odd ? d0 : d1, 1);
+  w0 = odd ? r : d0;
+  w1 = odd ? d1 : r;
+}
+// V-CRC (G = 4): CRC32C is affine in the message, crc(m) = L(m) ^ crc(0^32), so
+// each lane adds the linear part of its double's 7 message bytes (position
+// tables vp = vpos[lane & 3]) and the group XORs 4 partials.
+static __device__ __forceinline__ uint32_t vcrc_lin(uint64_t w, const uint32_t* vp) {
+  const uint32_t lo = lo32(w), hi = hi32(w);
+  return vp[(lo >> 8) & 0xFFu] ^ vp[256 + ((lo >> 16) & 0xFFu)] ^ vp[512 + (lo >> 24)] ^ vp[768 + (hi & 0xFFu)] ^
+         vp[1024 + ((hi >> 8) & 0xFFu)] ^ vp[1280 + ((hi >> 16) & 0xFFu)] ^ vp[1536 + (hi >> 24)];
+}
+static __device__ __forceinline__ uint32_t xor4(uint32_t p) {
+  p ^= __shfl_xor_sync(0xffffffffu, p, 1);
+  return p ^ __shfl_xor_sync(0xffffffffu, p, 2);
+}
+static __device__ __forceinline__ const uint32_t* vcrc_tab(const uint8_t* cs, int lane) {
+  return reinterpret_cast<const uint32_t*>(cs) + (lane & 3) * 7 * 256;
+}
+static __device__ __forceinline__ bool vcrc_bad_lane(uint64_t w, const uint32_t* vp, int lane) {
+  return xor4(vcrc_lin(w, vp) ^ ((lo32(w) & 0xFFu) << (8 * (lane & 3)))) != VCRC_ZERO;
+}
+static __device__ __forceinline__ uint64_t vcrc_encode_lane(uint64_t rounded, const uint32_t* vp, int lane) {
+  const uint64_t d = rounded & ~0xFFull;
+  const uint32_t crc = xor4(vcrc_lin(d, vp)) ^ VCRC_ZERO;
+  return d | ((crc >> (8 * (lane & 3))) & 0xFFu);
+}
+// Whole warp, G > 1 schemes: does any group holding w0 (pass k) or w1 (pass
+// k+32) fail its check?  cs: V-CRC position tables in SMEM (CRC32C).
+template <int VS>
+__device__ __forceinline__ bool gbad2(uint64_t w0, uint64_t w1, int lane, const uint8_t* cs) {
+  if (VS == SECDED128) {
+    uint64_t d0, d1;
+    pair_gather(w0, w1, lane, d0, d1);
+    return (v128_acc(d0, d1) & 1u) != 0u;
+  }
+  const uint32_t* vp = vcrc_tab(cs, lane);
+  return vcrc_bad_lane(w0, vp, lane) | vcrc_bad_lane(w1, vp, lane);
+}
+// Whole warp, G > 1 schemes: encode the rounded values r0 (pass k), r1 (pass k+32).
+template <int VS>
+__device__ __forceinline__ void genc2(uint64_t r0, uint64_t r1, int lane, const uint8_t* cs, uint64_t& e0,
+                                      uint64_t& e1) {
+  if (VS == SECDED128) {
+    uint64_t d[2];
+    pair_gather(r0, r1, lane, d[0], d[1]);
+    v128_encode(d);
+    pair_scatter(d[0], d[1], lane, e0, e1);
+  } else {
+    const uint32_t* vp = vcrc_tab(cs, lane);
+    e0 = vcrc_encode_lane(r0, vp, lane);
+    e1 = vcrc_encode_lane(r1, vp, lane);
+  }
+}
+
 // Matrix check mode of this SpMV access.
 static __device__ __forceinline__ int spmv_mode(const SpmvArgs& a) {
   if (a.check_interval > 1) {
@@ -378,7 +479,13 @@ constexpr int TILE_RP = 264;                                   // rowptr entries
 constexpr int TILE_OFF_WIN = TILE_NST * TILE_STAGE;            // stages first (128-B aligned)
 constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
 constexpr int TILE_OFF_BAR = TILE_OFF_RP + TILE_TY * TILE_RP * 4;
-constexpr int TILE_SMEM = TILE_OFF_BAR + 2 * TILE_NST * 8 + 128;   // + alignment slack
+constexpr int TILE_OFF_CRC = TILE_OFF_BAR + 64;                // CRC32C tables (only for CRC schemes)
+constexpr int TILE_SMEM = TILE_OFF_CRC + 128;                   // + alignment slack
+// dynamic SMEM of one tile kernel: + slicing tables (E-CRC / R-CRC), + V-CRC position tables
+template <int ES, int RS, int VS>
+constexpr int tile_smem() {
+  return TILE_SMEM + ((ES == CRC32C || RS == CRC32C) ? 4 * CRC_SLICE_WORDS : 0) + (VS == CRC32C ? 4 * CRC_VPOS_WORDS : 0);
+}
 
 static __device__ __forceinline__ uint32_t smem_u32(const void* p) { return (uint32_t)__cvta_generic_to_shared(p); }
 static __device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
@@ -485,9 +592,9 @@ template <int ES, int RS, int VS>
 static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const SpmvArgs& sa, uint32_t start, uint32_t end,
                                                    const uint64_t* sval, const uint32_t* scol, const double* win,
                                                    int oslot, double p_own, int64_t own, uint32_t s0, int lane,
-                                                   int mode) {
+                                                   int mode, const uint32_t* crc_slice) {
   const uint32_t s1 = s0 + TILE_PE;
-  if ((ES == CRC32C && mode != MODE_RANGE) || start != s0 + 5u * (uint32_t)lane || end != start + 5u)
+  if (start != s0 + 5u * (uint32_t)lane || end != start + 5u)
     return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1, mode);
   const int n32 = (int)a.stencil_n;
   const int own_col = (int)(own - a.col_base);
@@ -501,6 +608,17 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
   }
   uint32_t acc_r = 0, acc_p = 0;
   if (mode != MODE_RANGE) {   // uniform: interval mode's unchecked accesses skip the codec
+    if (ES == CRC32C) {       // E-CRC over the row, slicing-by-4 tables
+      uint32_t crc = 0xFFFFFFFFu, st = 0;
+#pragma unroll
+      for (int t = 0; t < 5; t++) {
+        crc = crc_word(crc, lo32(v[t]), crc_slice);
+        crc = crc_word(crc, hi32(v[t]), crc_slice);
+        crc = crc_word(crc, t < 4 ? (c[t] & 0x00FFFFFFu) : c[t], crc_slice);
+        if (t < 4) st |= (c[t] >> 24) << (8 * t);
+      }
+      acc_p = ((crc ^ 0xFFFFFFFFu) != st) ? 1u : 0u;
+    }
 #pragma unroll
     for (int t = 0; t < 5; t++) {
       if (ES == SED) acc_p |= (uint32_t)(popc64(v[t]) + popc32(c[t]));
@@ -544,6 +662,9 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   uint64_t* empty = full + TILE_NST;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   uint32_t* srp = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_RP) + warp * TILE_RP;
+  constexpr bool SLICE = (ES == CRC32C || RS == CRC32C);
+  uint32_t* s_slice = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_CRC);
+  uint8_t* s_vpos = s_dyn + TILE_OFF_CRC + (SLICE ? 4 * CRC_SLICE_WORDS : 0);
   const int64_t n = a.stencil_n;
   const int64_t ny = a.nrows / n;
   const int64_t tiles_x = n >> 8;
@@ -562,6 +683,10 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
     for (int k = 0; k < TILE_NST; k++) tile_produce(tm, s_dyn + k * TILE_STAGE, &full[k], tx0, ty0, k);
   }
   if (VS == SECDED64) load_lut(s_lut);
+  if (SLICE) smem_fill(s_slice, &a.crc->slice[0][0], CRC_SLICE_WORDS);
+  if (VS == CRC32C) smem_fill(reinterpret_cast<uint32_t*>(s_vpos), &a.crc->vpos[0][0][0], CRC_VPOS_WORDS);
+  if (SLICE || VS == CRC32C) __syncthreads();
+  const uint8_t* cs = (VS == CRC32C) ? s_vpos : s_lut;   // vector codec tables
   const int stop_v = a.state ? a.state->stop : 0;  // checked after the prologue loads are in flight
   const int mode = spmv_mode(a);
   const int64_t gy = ty0 + warp;
@@ -594,7 +719,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       if (mode != MODE_RANGE) {
 #pragma unroll
         for (int q = 0; q < PER; q++)
-          if (RS != NONE && lane + 32 * q < NG) acc |= rp_acc<RS>(e[q]);
+          if (RS != NONE && lane + 32 * q < NG) acc |= (RS == CRC32C) ? rcrc_acc_tab(e[q], s_slice) : rp_acc<RS>(e[q]);
       }
       if (RS != NONE && (acc & 1u)) {  // cold: locate, correct, count (owner), per group
 #pragma unroll
@@ -643,6 +768,49 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   // ---- 2. decoded `in` window
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
   constexpr int WPER = (TILE_WW + 31) / 32;                      // 9 slots per lane per window row
+  constexpr int VG = vgrp(VS);
+  if (VG > 1) {  // G = 2 / 4: load aligned groups (win0 = -1 mod 256), lane-split fast check
+    for (int wy = warp; wy < TILE_TY + 2; wy += 8) {
+      const int64_t a0 = win0 + (int64_t)wy * n - (VG - 1);      // in-index of lane 0's word, aligned to G
+      const bool row_own = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny;
+      double* dst = s_win + wy * TILE_WW;
+      uint64_t wv[WPER];
+      bool ok[WPER];
+#pragma unroll
+      for (int q = 0; q < WPER; q++) {
+        const int64_t idx = a0 + 32 * q + lane;
+        ok[q] = idx >= 0 && idx < a.npad_in;   // identical across a group (npad_in is a multiple of G)
+        wv[q] = ok[q] ? ldg64(a.in + idx) : 0ull;
+      }
+      bool bad = false;
+      if (VS == SECDED128) {   // zero groups are clean
+#pragma unroll
+        for (int q = 0; q + 1 < WPER; q += 2) bad |= gbad2<VS>(wv[q], wv[q + 1], lane, cs);
+        bad |= gbad2<VS>(wv[WPER - 1], 0ull, lane, cs);
+      } else {
+        const uint32_t* vp = vcrc_tab(cs, lane);
+#pragma unroll
+        for (int q = 0; q < WPER; q++) {
+          const bool b = vcrc_bad_lane(wv[q], vp, lane);   // every lane: shuffles inside
+          bad |= ok[q] & b;
+        }
+      }
+      if (__any_sync(0xffffffffu, bad)) {   // cold: locate / correct per group (owner counts + scrubs)
+#pragma unroll 1
+        for (int q = 0; q < WPER; q++) {
+          const int slot = 32 * q + lane - (VG - 1);
+          const bool owner = row_own && slot >= 1 && slot <= 256;   // groups never straddle the tile edge
+          wv[q] = vg_check<VS>(wv[q], a.in + (a0 + 32 * q + (lane & ~(VG - 1))), lane, ok[q], owner && ok[q],
+                               a.counts, a.due);
+        }
+      }
+#pragma unroll
+      for (int q = 0; q < WPER; q++) {
+        const int slot = 32 * q + lane - (VG - 1);
+        if (slot >= 0 && slot < TILE_WW) dst[slot] = as_d(wv[q] & vkeep(VS));
+      }
+    }
+  } else
   for (int wy = warp; wy < TILE_TY + 2; wy += 8) {
     const int64_t rbase = win0 + (int64_t)wy * n;                 // in-index of (wy, 0)
     const bool row_in = rbase >= 0 && rbase + TILE_WW <= a.npad_in;  // uniform: no per-slot bounds
@@ -680,6 +848,8 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   __syncthreads();
   // ---- 3. passes (every warp takes part in the stage protocol)
   double dot = 0.0;
+  uint64_t acc_prev = 0;   // SECDED128: rounded result of the even pass awaiting its pair
+  double p_prev = 0.0;
   const uint32_t seg_e = (uint32_t)(5 * rowseg);   // assumed element start of the segment
 #pragma unroll
   for (int k = 0; k < 8; k++) {
@@ -695,10 +865,28 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       const double p_own = s_win[oslot];
       const int64_t own = a.row_base + rowseg + k * 32 + lane;
       const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s_win, oslot, p_own, own,
-                                               seg_e + 160u * k, lane, mode);
-      const uint64_t enc = v_encode<VS>(round_k(as_u(acc), vk(VS)), lane, s_lut);
-      a.out[own] = enc;
-      if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+                                               seg_e + 160u * k, lane, mode, s_slice);
+      const uint64_t rounded = round_k(as_u(acc), vk(VS));
+      if (VS == SECDED128) {   // encode pass pairs (k-1, k): pair gather
+        if ((k & 1) == 0) {
+          acc_prev = rounded;
+          p_prev = p_own;
+        } else {
+          uint64_t e0, e1;
+          genc2<VS>(acc_prev, rounded, lane, cs, e0, e1);
+          a.out[own - 32] = e0;
+          a.out[own] = e1;
+          if (DOT) {
+            dot = fma(p_prev, as_d(e0 & vkeep(VS)), dot);
+            dot = fma(p_own, as_d(e1 & vkeep(VS)), dot);
+          }
+        }
+      } else {
+        const uint64_t enc = (VS == CRC32C) ? vcrc_encode_lane(rounded, vcrc_tab(cs, lane), lane)
+                                            : v_encode<VS>(rounded, lane, s_lut);
+        a.out[own] = enc;
+        if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+      }
     }
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[st]);
@@ -716,10 +904,12 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
 }
 
 // ============================================================= BLAS-1 (a4, a5, a2)
-// Full-RB fast paths (G = 1 schemes): two passes per step, so each lane has
-// 8 (calc_ur) / 4 (calc_p, init) independent 8-byte loads in flight, and all
-// addressing is pointer + immediate offset.  Lane l still visits rows
-// l, l+32, ... in ascending order (RED-1).
+// Full-RB fast paths: two passes per step, so each lane has 8 (calc_ur) / 4
+// (calc_p) independent 8-byte loads in flight, and all addressing is pointer +
+// immediate offset.  Lane l still visits rows l, l+32, ... in ascending order
+// (RED-1).  G = 1 schemes check each word in its lane; G = 2 / 4 schemes use
+// the lane-split group codecs (pair gather / V-CRC partials), the pass pair
+// (k, k+32) being exactly what the SECDED128 pair gather needs.
 // OR-accumulated fast check of up to 8 G=1 codewords (zero words are clean in
 // every scheme): true iff any of them needs the per-word cold path.
 template <int VS>
@@ -741,6 +931,33 @@ __device__ __forceinline__ bool vacc_bad(uint64_t w0, uint64_t w1, uint64_t w2, 
   }
   return false;
 }
+// Check the words w0 (this lane's row of pass k at addr) and w1 (pass k+32):
+// fast test, then (warp-uniform cold branch) locate / correct / count per group.
+template <int VS>
+__device__ __forceinline__ void vcheck2(uint64_t& w0, uint64_t& w1, uint64_t* addr, const VecArgs& a, int lane,
+                                        const uint8_t* cs, bool any_bad) {
+  constexpr int G = vgrp(VS);
+  if (G == 1) {
+    if (any_bad) {
+      w0 = v1_check<VS>(w0, addr, true, a.counts, a.due);
+      w1 = v1_check<VS>(w1, addr + 32, true, a.counts, a.due);
+    }
+  } else if (__any_sync(0xffffffffu, any_bad)) {
+    w0 = vg_check<VS>(w0, addr - (lane & (G - 1)), lane, true, true, a.counts, a.due);
+    w1 = vg_check<VS>(w1, addr + 32 - (lane & (G - 1)), lane, true, true, a.counts, a.due);
+  }
+}
+// Encode two rounded values (rows of pass k and k+32).
+template <int VS>
+__device__ __forceinline__ void venc2(uint64_t r0, uint64_t r1, int lane, const uint8_t* cs, uint64_t& e0,
+                                      uint64_t& e1) {
+  if (vgrp(VS) == 1) {
+    e0 = v_encode<VS>(r0, lane, cs);
+    e1 = v_encode<VS>(r1, lane, cs);
+  } else {
+    genc2<VS>(r0, r1, lane, cs, e0, e1);
+  }
+}
 
 template <int VS>
 struct UrStep { uint64_t x0, x1, p0, p1, r0, r1, w0, w1; };
@@ -752,103 +969,129 @@ __device__ __forceinline__ void ur_load(const uint64_t* X, const uint64_t* P, co
 }
 template <int VS>
 __device__ __forceinline__ void ur_step(const VecArgs& a, uint64_t* X, uint64_t* P, uint64_t* R, uint64_t* W, int k,
-                                        const UrStep<VS>& s, double alpha, int lane, const uint8_t* lut, double& dot);
+                                        const UrStep<VS>& s, double alpha, int lane, const uint8_t* cs, double& dot);
 // Full RB of calc_ur; step 0's loads were issued by the caller before the
 // kernel's barrier / stop check so their latency overlaps the state loads.
 template <int VS>
-__device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int lane, double alpha, const uint8_t* lut,
+__device__ __forceinline__ double ur_full(const VecArgs& a, int64_t base, int lane, double alpha, const uint8_t* cs,
                                           UrStep<VS> s) {
   uint64_t* X = a.x + base + lane;
   uint64_t* P = a.p + base + lane;
   uint64_t* R = a.r + base + lane;
   uint64_t* W = a.w + base + lane;
   double dot = 0.0;
-  ur_step<VS>(a, X, P, R, W, 0, s, alpha, lane, lut, dot);
+  ur_step<VS>(a, X, P, R, W, 0, s, alpha, lane, cs, dot);
 #pragma unroll 1
   for (int k = 64; k < 256; k += 64) {
     ur_load<VS>(X, P, R, W, k, s);
-    ur_step<VS>(a, X, P, R, W, k, s, alpha, lane, lut, dot);
+    ur_step<VS>(a, X, P, R, W, k, s, alpha, lane, cs, dot);
   }
   return dot;
 }
 template <int VS>
 __device__ __forceinline__ void ur_step(const VecArgs& a, uint64_t* X, uint64_t* P, uint64_t* R, uint64_t* W, int k,
-                                        const UrStep<VS>& s, double alpha, int lane, const uint8_t* lut, double& dot) {
+                                        const UrStep<VS>& s, double alpha, int lane, const uint8_t* cs, double& dot) {
   const uint64_t keep = vkeep(VS);
-  {
-    uint64_t x0 = s.x0, x1 = s.x1, p0 = s.p0, p1 = s.p1, r0 = s.r0, r1 = s.r1, w0 = s.w0, w1 = s.w1;
+  uint64_t x0 = s.x0, x1 = s.x1, p0 = s.p0, p1 = s.p1, r0 = s.r0, r1 = s.r1, w0 = s.w0, w1 = s.w1;
+  if (vgrp(VS) == 1) {
     if (vacc_bad<VS>(x0, x1, p0, p1, r0, r1, w0, w1)) {  // cold: locate per word
-      x0 = v1_check<VS>(x0, X + k, true, a.counts, a.due);
-      x1 = v1_check<VS>(x1, X + k + 32, true, a.counts, a.due);
-      p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
-      p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
-      r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
-      r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
-      w0 = v1_check<VS>(w0, W + k, true, a.counts, a.due);
-      w1 = v1_check<VS>(w1, W + k + 32, true, a.counts, a.due);
+      vcheck2<VS>(x0, x1, X + k, a, lane, cs, true);
+      vcheck2<VS>(p0, p1, P + k, a, lane, cs, true);
+      vcheck2<VS>(r0, r1, R + k, a, lane, cs, true);
+      vcheck2<VS>(w0, w1, W + k, a, lane, cs, true);
     }
-    const double xn0 = fma(alpha, as_d(p0 & keep), as_d(x0 & keep));
-    const double xn1 = fma(alpha, as_d(p1 & keep), as_d(x1 & keep));
-    const double rn0 = fma(-alpha, as_d(w0 & keep), as_d(r0 & keep));
-    const double rn1 = fma(-alpha, as_d(w1 & keep), as_d(r1 & keep));
-    const uint64_t xe0 = v_encode<VS>(round_k(as_u(xn0), vk(VS)), lane, lut);
-    const uint64_t xe1 = v_encode<VS>(round_k(as_u(xn1), vk(VS)), lane, lut);
-    const uint64_t re0 = v_encode<VS>(round_k(as_u(rn0), vk(VS)), lane, lut);
-    const uint64_t re1 = v_encode<VS>(round_k(as_u(rn1), vk(VS)), lane, lut);
-    X[k] = xe0; X[k + 32] = xe1;
-    R[k] = re0; R[k + 32] = re1;
-    const double m0 = as_d(re0 & keep), m1 = as_d(re1 & keep);
-    dot = fma(m0, m0, dot);
-    dot = fma(m1, m1, dot);
+  } else {
+    const bool bad = gbad2<VS>(x0, x1, lane, cs) | gbad2<VS>(p0, p1, lane, cs) | gbad2<VS>(r0, r1, lane, cs) |
+                     gbad2<VS>(w0, w1, lane, cs);
+    if (__any_sync(0xffffffffu, bad)) {  // cold, warp-uniform: locate per group
+      vcheck2<VS>(x0, x1, X + k, a, lane, cs, true);
+      vcheck2<VS>(p0, p1, P + k, a, lane, cs, true);
+      vcheck2<VS>(r0, r1, R + k, a, lane, cs, true);
+      vcheck2<VS>(w0, w1, W + k, a, lane, cs, true);
+    }
   }
+  const double xn0 = fma(alpha, as_d(p0 & keep), as_d(x0 & keep));
+  const double xn1 = fma(alpha, as_d(p1 & keep), as_d(x1 & keep));
+  const double rn0 = fma(-alpha, as_d(w0 & keep), as_d(r0 & keep));
+  const double rn1 = fma(-alpha, as_d(w1 & keep), as_d(r1 & keep));
+  uint64_t xe0, xe1, re0, re1;
+  venc2<VS>(round_k(as_u(xn0), vk(VS)), round_k(as_u(xn1), vk(VS)), lane, cs, xe0, xe1);
+  venc2<VS>(round_k(as_u(rn0), vk(VS)), round_k(as_u(rn1), vk(VS)), lane, cs, re0, re1);
+  X[k] = xe0; X[k + 32] = xe1;
+  R[k] = re0; R[k + 32] = re1;
+  const double m0 = as_d(re0 & keep), m1 = as_d(re1 & keep);
+  dot = fma(m0, m0, dot);
+  dot = fma(m1, m1, dot);
 }
 template <int VS>
 __device__ __forceinline__ void p_step(const VecArgs& a, uint64_t* P, uint64_t* R, int k, uint64_t r0, uint64_t r1,
-                                       uint64_t p0, uint64_t p1, double beta, int lane, const uint8_t* lut) {
+                                       uint64_t p0, uint64_t p1, double beta, int lane, const uint8_t* cs) {
   const uint64_t keep = vkeep(VS);
-  if (vacc_bad<VS>(r0, r1, p0, p1, 0ull, 0ull, 0ull, 0ull)) {  // cold: locate per word
-    r0 = v1_check<VS>(r0, R + k, true, a.counts, a.due);
-    r1 = v1_check<VS>(r1, R + k + 32, true, a.counts, a.due);
-    p0 = v1_check<VS>(p0, P + k, true, a.counts, a.due);
-    p1 = v1_check<VS>(p1, P + k + 32, true, a.counts, a.due);
+  if (vgrp(VS) == 1) {
+    if (vacc_bad<VS>(r0, r1, p0, p1, 0ull, 0ull, 0ull, 0ull)) {  // cold: locate per word
+      vcheck2<VS>(r0, r1, R + k, a, lane, cs, true);
+      vcheck2<VS>(p0, p1, P + k, a, lane, cs, true);
+    }
+  } else {
+    const bool bad = gbad2<VS>(r0, r1, lane, cs) | gbad2<VS>(p0, p1, lane, cs);
+    if (__any_sync(0xffffffffu, bad)) {
+      vcheck2<VS>(r0, r1, R + k, a, lane, cs, true);
+      vcheck2<VS>(p0, p1, P + k, a, lane, cs, true);
+    }
   }
   const double n0 = fma(beta, as_d(p0 & keep), as_d(r0 & keep));
   const double n1 = fma(beta, as_d(p1 & keep), as_d(r1 & keep));
-  P[k] = v_encode<VS>(round_k(as_u(n0), vk(VS)), lane, lut);
-  P[k + 32] = v_encode<VS>(round_k(as_u(n1), vk(VS)), lane, lut);
+  uint64_t e0, e1;
+  venc2<VS>(round_k(as_u(n0), vk(VS)), round_k(as_u(n1), vk(VS)), lane, cs, e0, e1);
+  P[k] = e0;
+  P[k + 32] = e1;
 }
 // Full RB of calc_p; step 0's words were loaded by the caller ahead of the
 // barrier / stop check.
 template <int VS>
-__device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane, double beta, const uint8_t* lut,
+__device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane, double beta, const uint8_t* cs,
                                        uint64_t r0, uint64_t r1, uint64_t p0, uint64_t p1) {
   uint64_t* P = a.p + base + lane;
   uint64_t* R = a.r + base + lane;
-  p_step<VS>(a, P, R, 0, r0, r1, p0, p1, beta, lane, lut);
+  p_step<VS>(a, P, R, 0, r0, r1, p0, p1, beta, lane, cs);
 #pragma unroll 1
   for (int k = 64; k < 256; k += 64)
-    p_step<VS>(a, P, R, k, ldg64(R + k), ldg64(R + k + 32), ldg64(P + k), ldg64(P + k + 32), beta, lane, lut);
+    p_step<VS>(a, P, R, k, ldg64(R + k), ldg64(R + k + 32), ldg64(P + k), ldg64(P + k + 32), beta, lane, cs);
 }
 
+// Codec tables of the BLAS-1 / SpMV kernels in shared memory: the V-SECDED64
+// encoder LUT (128 B) or the V-CRC position tables (28 KB, dynamic).
+template <int VS>
+constexpr size_t vec_dyn_smem() { return VS == CRC32C ? sizeof(uint32_t) * CRC_VPOS_WORDS : 0; }
+template <int VS>
+__device__ __forceinline__ const uint8_t* vec_codec_smem(uint8_t* s_lut, uint8_t* s_dyn, const CrcTables* crc) {
+  if (VS == SECDED64) { load_lut(s_lut); return s_lut; }
+  if (VS == CRC32C) {
+    smem_fill(reinterpret_cast<uint32_t*>(s_dyn), &crc->vpos[0][0][0], CRC_VPOS_WORDS);
+    return s_dyn;
+  }
+  return s_lut;
+}
 
 template <int VS>
-__global__ void __launch_bounds__(256, 4) k_calc_ur(VecArgs a) {
+__global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 3 : 4) k_calc_ur(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
+  extern __shared__ __align__(16) uint8_t s_dyn_v[];
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
-  const bool full = vgrp(VS) == 1 && rb * 256 + 256 <= a.n;
+  const bool full = rb * 256 + 256 <= a.n;
   UrStep<VS> s0{};
   if (full)  // issue step 0 first: its latency overlaps the state loads and the barrier
     ur_load<VS>(a.x + rb * 256 + lane, a.p + rb * 256 + lane, a.r + rb * 256 + lane, a.w + rb * 256 + lane, 0, s0);
   const int stop = a.state->stop;
   const double alpha = a.state->alpha;
-  if (VS == SECDED64) load_lut(s_lut);
+  const uint8_t* cs = vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
   __syncthreads();
   if (stop) return;
   if (rb * 256 >= a.n) return;
   double dot = 0.0;
   if (full) {
-    dot = ur_full<VS>(a, rb * 256, lane, alpha, s_lut, s0);
+    dot = ur_full<VS>(a, rb * 256, lane, alpha, cs, s0);
   } else for (int k = 0; k < 8; k++) {
     const int64_t pb = rb * 256 + k * 32;
     if (pb >= a.n) break;
@@ -874,12 +1117,13 @@ __global__ void __launch_bounds__(256, 4) k_calc_ur(VecArgs a) {
 }
 
 template <int VS>
-__global__ void __launch_bounds__(256, 6) k_calc_p(VecArgs a) {
+__global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : 6) k_calc_p(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
+  extern __shared__ __align__(16) uint8_t s_dyn_v[];
   __shared__ bool s_last;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
-  const bool full = vgrp(VS) == 1 && rb * 256 + 256 <= a.n;
+  const bool full = rb * 256 + 256 <= a.n;
   uint64_t r0 = 0, r1 = 0, p0 = 0, p1 = 0;
   if (full) {  // issue step 0 first: its latency overlaps the state loads and the barrier
     const uint64_t* R = a.r + rb * 256 + lane;
@@ -888,11 +1132,11 @@ __global__ void __launch_bounds__(256, 6) k_calc_p(VecArgs a) {
   }
   const int stop = a.state->stop;
   const double beta = a.state->beta;
-  if (VS == SECDED64) load_lut(s_lut);
+  const uint8_t* cs = vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
   __syncthreads();
   if (stop) return;
   if (full) {
-    p_full<VS>(a, rb * 256, lane, beta, s_lut, r0, r1, p0, p1);
+    p_full<VS>(a, rb * 256, lane, beta, cs, r0, r1, p0, p1);
   } else if (rb * 256 < a.n) {
     for (int k = 0; k < 8; k++) {
       const int64_t pb = rb * 256 + k * 32;

@@ -11,7 +11,7 @@ namespace {
 // decoded rowptr against the assumed stencil layout).
 static bool tile_ok(const SpmvArgs& a, int vs) {
   const int64_t n = a.stencil_n;
-  return n > 0 && (n % 256) == 0 && (a.nrows % n) == 0 && vgrp(vs) == 1 && a.npad_out >= a.nrows &&
+  return n > 0 && (n % 256) == 0 && (a.nrows % n) == 0 && a.npad_out >= a.nrows &&
          a.nnz == 5 * a.nrows && a.nnz < (int64_t(1) << 32) && (a.nrows / n) < (int64_t(1) << 31) &&
          (reinterpret_cast<uintptr_t>(a.val) & 15u) == 0 && (reinterpret_cast<uintptr_t>(a.col) & 15u) == 0;
 }
@@ -51,7 +51,7 @@ template <int ES, int RS, int VS, bool DOT>
 static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   TileMaps tm;
   if (!tile_maps(a, &tm)) return false;
-  const size_t smem = TILE_SMEM;
+  const size_t smem = tile_smem<ES, RS, VS>();
   static bool attr = false;
   if (!attr) {  // both variants at once: never inside a later CUDA-graph capture
     cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -67,7 +67,7 @@ static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
 }
 template <int ES, int RS, int VS>
 static void spmv3(const SpmvArgs& a, bool dot, cudaStream_t s) {
-  if (vgrp(VS) == 1 && tile_ok(a, VS)) {
+  if (tile_ok(a, VS)) {
     if (dot ? spmv_tile_launch<ES, RS, VS, true>(a, s) : spmv_tile_launch<ES, RS, VS, false>(a, s)) return;
   }
   const int64_t nrb = (a.nrows + 255) / 256;

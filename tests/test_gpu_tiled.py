@@ -51,15 +51,25 @@ def _flip(abft, ctx, Ao, Ag, xo, xg, rng, n_el, n_rp, xs):
         abft.inject_bitflip(ctx, Ag.rowptr, 32 * int(g) + b)
 
 
-@pytest.mark.parametrize("vs", ["NONE", "SED", "SECDED64"])
+def _schemes(S):
+    """Element / rowptr schemes paired with vector scheme S in the tiled tests:
+    CRC32C everywhere for CRC32C (table-driven E-CRC / R-CRC / V-CRC), R-SECDED128
+    with V-SECDED128, E-SECDED + R-SECDED64 otherwise."""
+    if S == orc.NONE:
+        return orc.NONE, orc.NONE
+    if S == orc.CRC32C:
+        return orc.CRC32C, orc.CRC32C
+    return orc.SECDED64, (orc.SECDED128 if S == orc.SECDED128 else orc.SECDED64)
+
+
+@pytest.mark.parametrize("vs", ["NONE", "SED", "SECDED64", "SECDED128", "CRC32C"])
 @pytest.mark.parametrize("splits", [(), (40,), (16, 100)])
 @pytest.mark.parametrize("faults", [False, True])
 def test_tiled_spmv_parity(abft, ctx, vs, splits, faults):
     n = 256
     N = n * n
     S = getattr(orc, vs)
-    es = orc.SECDED64 if S != orc.NONE else orc.NONE
-    rs = orc.SECDED64 if S != orc.NONE else orc.NONE
+    es, rs = _schemes(S)
     rng = np.random.default_rng(7 + len(splits) + 10 * faults)
     x = gen.uniform_pm1(N, 11)
     xo = orc.vec_encode(x, S)
@@ -105,14 +115,16 @@ def test_tiled_spmv_parity(abft, ctx, vs, splits, faults):
         assert dot_g.item() == orc.dot_red1(masked_x, masked_y)
 
 
-def test_tiled_cg_parity(abft, ctx):
+@pytest.mark.parametrize("vs", ["SECDED64", "SECDED128", "CRC32C"])
+def test_tiled_cg_parity(abft, ctx, vs):
     n = 256
     N = n * n
-    S = orc.SECDED64
+    S = getattr(orc, vs)
+    es, rs = _schemes(S)
     v, c, r = gen.tealeaf_csr(n)
     v, c, r = v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32)
-    Ao, _ = oracle_matrix(v, c, r, N, N, S, S)
-    Ag, _ = gpu_matrix(abft, ctx, v, c, r, N, N, S, S, stencil_n=n)
+    Ao, _ = oracle_matrix(v, c, r, N, N, es, rs)
+    Ag, _ = gpu_matrix(abft, ctx, v, c, r, N, N, es, rs, stencil_n=n)
     b = gen.tealeaf_rhs(n).numpy()
     bo = orc.vec_encode(b, S)
     xo = bo.copy()
