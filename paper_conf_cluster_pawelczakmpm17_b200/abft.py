@@ -18,7 +18,7 @@ SCHEMES = {"none": NONE, "sed": SED, "secded64": SECDED64, "secded128": SECDED12
 ELEM, ROWPTR, VEC = range(3)
 OK, E_INVALID, E_RANGE, E_SHAPE, E_DUE, E_NOT_CONVERGED, E_CUDA, E_NCCL = 0, -1, -2, -3, -4, -5, -6, -7
 
-_SO = _build.SO
+_SO = os.environ.get("ABFT_SO", _build.SO)   # override: kernel-variant timing tools only
 if not os.path.exists(_SO):
     raise ImportError(f"libabft.so not built ({_SO}); run __graft_entry__.build() "
                       "or python -m paper_conf_cluster_pawelczakmpm17_b200.build")

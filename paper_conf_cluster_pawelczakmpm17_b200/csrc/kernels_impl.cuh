@@ -851,7 +851,11 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   uint64_t acc_prev = 0;   // SECDED128: rounded result of the even pass awaiting its pair
   double p_prev = 0.0;
   const uint32_t seg_e = (uint32_t)(5 * rowseg);   // assumed element start of the segment
-#pragma unroll
+#ifndef ABFT_TILE_UNROLL
+#define ABFT_TILE_UNROLL 1
+#endif
+  constexpr int kPassUnroll = ABFT_TILE_UNROLL;
+#pragma unroll kPassUnroll
   for (int k = 0; k < 8; k++) {
     const int st = k % TILE_NST;
     const uint32_t ph = (uint32_t)((k / TILE_NST) & 1);

@@ -1,0 +1,62 @@
+"""Time the hot kernels alone on the 4096^2 G-TEA problem (CUDA events, inputs
+resident): protected (E-SECDED / R-SECDED64 / V-SECDED64) and unprotected
+SpMV, calc_ur, calc_p.  For comparing kernel variants quickly:
+
+    ABFT_SO=path/to/libabft_variant.so python tools/spmv_time.py [--grid 4096] [--reps 50]
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--grid", type=int, default=4096)
+    ap.add_argument("--reps", type=int, default=50)
+    ap.add_argument("--schemes", default="2,0")
+    a = ap.parse_args()
+    import torch
+    import bench
+    from paper_conf_cluster_pawelczakmpm17_b200 import abft
+    torch.cuda.set_device(0)
+    P = bench.build_problem(a.grid, 0, 1, torch.device("cuda", 0))
+    ctx = abft.Context(0)
+    out = {"so": os.environ.get("ABFT_SO", "default")}
+    for s in [int(t) for t in a.schemes.split(",")]:
+        sol = bench.Solver(abft, ctx, P, s, s, s)
+        sol.step(0.0, 1)
+        b, x, r, p, w = sol.vecs
+        cnt = sol.counts
+        dot = torch.zeros(1, dtype=torch.float64, device="cuda")
+
+        def t(fn):
+            for _ in range(3):
+                fn()
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            torch.cuda.synchronize()
+            e0.record()
+            for _ in range(a.reps):
+                fn()
+            e1.record()
+            torch.cuda.synchronize()
+            return e0.elapsed_time(e1) / a.reps
+        res = {
+            "spmv_ms": t(lambda: abft.spmv(ctx, sol.A, p, w, cnt, dot=dot)),
+            "calc_ur_ms": t(lambda: abft.calc_ur(ctx, x, p, r, w, 1e-30, rrn=dot, counts=cnt)),
+            "calc_p_ms": t(lambda: abft.calc_p(ctx, p, r, 1e-30, counts=cnt)),
+        }
+        res["spmv_gbs"] = 80.0 * P["N"] / (res["spmv_ms"] * 1e-3) / 1e9
+        res["counts"] = int(cnt.read().sum())
+        out[f"scheme{s}"] = res
+        del sol
+    print(json.dumps(out))
+
+
+if __name__ == "__main__":
+    main()

@@ -72,10 +72,17 @@ def main():
             best = ms if best is None else min(best, ms)
         if what == "all" and s == "NONE":
             base = best
+        # per-kernel-class breakdown: one extra profiled (non-graph) step
+        abft.profile(ctx, 15)
+        it2, _ = sol.step(0.0, a.iters)
+        torch.cuda.synchronize()
+        ms_cls, n_cls = abft.profile_read(ctx)
+        abft.profile(ctx, 0)
+        kms = {k: (ms_cls[i] / n_cls[i] if n_cls[i] else None) for i, k in enumerate(["spmv", "calc_ur", "calc_p", "reductions"])}
         row = {"structures": what, "scheme": s, "elem": es, "rowptr": rs, "vectors": vs, "check_interval": interval,
                "iter_ms": best,
                "overhead_pct": None if base is None else 100.0 * (best / base - 1.0),
-               "cg_gbs": 152.0 * P["N"] / (best / 1000.0) / 1e9}
+               "cg_gbs": 152.0 * P["N"] / (best / 1000.0) / 1e9, "kernel_ms": kms}
         rows.append(row)
         print(json.dumps(row), flush=True)
         del sol
