@@ -29,6 +29,9 @@ sys.path.insert(0, ROOT)
 METRIC = "protected CG iters/sec and SpMV HBM GB/s vs peak; ECC overhead % vs unprotected"
 SPMV_BYTES_PER_ROW = 80    # val 40 + col 20 + rowptr 4 + p 8 + w 8
 CG_BYTES_PER_ROW = 152     # SpMV 80 + calc_ur 48 + calc_p 24
+# fused calc_p: the SpMV reads p_{k-1} and r and writes p_k
+FUSED_SPMV_BYTES_PER_ROW = 96   # val 40 + col 20 + rowptr 4 + p_{k-1} 8 + r 8 + p_k 8 + w 8
+FUSED_CG_BYTES_PER_ROW = 144    # fused SpMV 96 + calc_ur 48
 
 
 def _peaks():
@@ -298,6 +301,8 @@ def main():
     ap.add_argument("--chunk-rows", type=int, default=None, help="grid rows per row-block chunk (default: fit 2^24 cols)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--fuse", action="store_true", help="main line on the fused calc_p path (DESIGN.md §6.1)")
+    ap.add_argument("--no-fused-extra", action="store_true", help="skip the fused-calc_p side measurement")
     args = ap.parse_args()
     if args.impl == "reference":
         return run_reference(args)
@@ -315,6 +320,11 @@ def main():
 
     P = build_problem(args.grid, rank, world, torch.device("cuda", local), args.chunk_rows)
     ctx = abft.Context(local)
+    # fused calc_p (opt-in) runs on the single-GPU tiled path (the dist path exchanges p halos unfused)
+    fused = args.fuse and not dist_on
+    ctx.set_fused_cg(fused)
+    spmv_bpr = FUSED_SPMV_BYTES_PER_ROW if fused else SPMV_BYTES_PER_ROW
+    cg_bpr = FUSED_CG_BYTES_PER_ROW if fused else CG_BYTES_PER_ROW
     dobj = abft.Dist(rank, world, local) if dist_on else None
     prot = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj)
     with ClockSampler(local) as clk:
@@ -330,6 +340,29 @@ def main():
     r_u = timed(twin, args.steps, max(1, args.warmup // 2), args.tol, args.max_iters, dist_on)
     r_uk = timed(twin, 1, 0, args.tol, args.max_iters, dist_on, profile=15)
     del twin
+
+    # side measurement: the other calc_p arrangement (fused <-> unfused), protected and unprotected
+    alt = None
+    if not dist_on and not args.no_fused_extra:
+        ctx.set_fused_cg(not fused)
+        a_p = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj)
+        r_ap = timed(a_p, args.steps, 1, args.tol, args.max_iters, dist_on)
+        r_apk = timed(a_p, 1, 0, args.tol, args.max_iters, dist_on, profile=15)
+        del a_p
+        a_u = Solver(abft, ctx, P, abft.NONE, abft.NONE, abft.NONE, dobj)
+        r_au = timed(a_u, args.steps, 1, args.tol, args.max_iters, dist_on)
+        del a_u
+        ctx.set_fused_cg(fused)
+        eq_ = P["N"] / float(4096 * 4096)
+        ip, iu = r_ap["ms"] / max(r_ap["iters"], 1), r_au["ms"] / max(r_au["iters"], 1)
+        ms_a, n_a = r_apk["prof"]
+        alt = {"fused_calc_p": not fused,
+               "value": r_ap["iters"] / (r_ap["ms"] / 1000.0) * eq_,
+               "unprotected_value": r_au["iters"] / (r_au["ms"] / 1000.0) * eq_,
+               "overhead_pct_per_iter": 100.0 * (ip / iu - 1.0),
+               "bytes_per_row_per_iter": CG_BYTES_PER_ROW if fused else FUSED_CG_BYTES_PER_ROW,
+               "kernel_ms": {"spmv": ms_a[0] / max(n_a[0], 1), "calc_ur": ms_a[1] / max(n_a[1], 1),
+                             "calc_p": ms_a[2] / max(n_a[2], 1), "reductions": ms_a[3] / max(n_a[3], 1)}}
 
     e2e = None
     if not args.no_e2e:
@@ -355,7 +388,7 @@ def main():
     peak, peak_src = _peaks()
     ms_t, n_t = r_ps["prof"]         # roofline pass: SpMV launches only
     spmv_ms = ms_t[0] / max(n_t[0], 1)
-    spmv_gbs = SPMV_BYTES_PER_ROW * N / (spmv_ms / 1000.0) / 1e9 if spmv_ms > 0 else None
+    spmv_gbs = spmv_bpr * N / (spmv_ms / 1000.0) / 1e9 if spmv_ms > 0 else None
     ms_cls, n_cls = r_pk["prof"]     # separate profiled step: all kernel classes
     ms_u, n_u = r_uk["prof"]
     traffic = read_traffic()
@@ -379,16 +412,20 @@ def main():
                    "schemes": {"elements": "E-SECDED", "rowptr": "R-SECDED64", "vectors": "V-SECDED64"},
                    "tol": args.tol, "iters_per_step": r_p["iters"] / args.steps,
                    "l2": "inputs larger than L2 (2.55 GB moved per CG iteration vs 126 MB L2)",
-                   "parallelism": f"row-block strips x{world}" if world > 1 else "single GPU"},
-        "roofline": {"bound": "hbm", "kernel": "k_spmv (protected SpMV + p.w)",
+                   "parallelism": f"row-block strips x{world}" if world > 1 else "single GPU",
+                   "fused_calc_p": fused, "bytes_per_row_per_iter": cg_bpr},
+        "roofline": {"bound": "hbm",
+                     "kernel": "k_spmv_tile (fused calc_p + protected SpMV + p.w)" if fused
+                     else "k_spmv_tile (protected SpMV + p.w)",
                      "achieved": spmv_gbs, "peak": peak, "unit": "GB/s",
                      "frac": (spmv_gbs / peak) if spmv_gbs else None,
                      "traffic": traffic.get("bytes_per_launch") if traffic else None,
-                     "bytes_per_launch_algorithmic": SPMV_BYTES_PER_ROW * N, "peak_source": peak_src,
+                     "bytes_per_launch_algorithmic": spmv_bpr * N, "peak_source": peak_src,
                      "avg_launch_ms": spmv_ms},
-        "cg_bandwidth": {"achieved_gbs": CG_BYTES_PER_ROW * N / (iter_ms_p / 1000.0) / 1e9,
-                         "frac_of_measured": CG_BYTES_PER_ROW * N / (iter_ms_p / 1000.0) / 1e9 / peak,
-                         "frac_of_8tbs": CG_BYTES_PER_ROW * N / (iter_ms_p / 1000.0) / 1e9 / 8000.0},
+        "cg_bandwidth": {"achieved_gbs": cg_bpr * N / (iter_ms_p / 1000.0) / 1e9,
+                         "frac_of_measured": cg_bpr * N / (iter_ms_p / 1000.0) / 1e9 / peak,
+                         "frac_of_8tbs": cg_bpr * N / (iter_ms_p / 1000.0) / 1e9 / 8000.0,
+                         "bytes_per_row_per_iter": cg_bpr},
         "kernel_ms": {"spmv": ms_cls[0] / max(n_cls[0], 1), "calc_ur": ms_cls[1] / max(n_cls[1], 1),
                       "calc_p": ms_cls[2] / max(n_cls[2], 1), "reductions": ms_cls[3] / max(n_cls[3], 1),
                       "note": "one extra untimed step with every kernel class bracketed by events"},
@@ -396,6 +433,7 @@ def main():
                         "spmv_ms": ms_u[0] / max(n_u[0], 1), "calc_ur_ms": ms_u[1] / max(n_u[1], 1),
                         "calc_p_ms": ms_u[2] / max(n_u[2], 1), "reductions_ms": ms_u[3] / max(n_u[3], 1)},
         "overhead_pct_per_iter": 100.0 * (iter_ms_p / iter_ms_u - 1.0),
+        "alt_calc_p_arrangement": alt,
         "clocks": clocks,
         "gpu_launches": r_p["launches"],
         "e2e": e2e,

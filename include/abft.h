@@ -75,6 +75,14 @@ typedef struct abft_ctx abft_ctx;
 /* Create / destroy a context on `device` (owns scratch, events, graphs). */
 int abft_ctx_create(int device, abft_ctx** out);
 int abft_ctx_destroy(abft_ctx* ctx);
+/* Fused calc_p (opt-in, default off): when every chunk is on the tiled
+ * stencil path, the vector scheme has group size 1 (NONE / SED / SECDED64) and
+ * the solve is single-GPU, abft_cg_solve computes calc_p of iteration k
+ * (p = enc(fma(beta, p, r))) inside the SpMV of iteration k+1:
+ * bit-identical iterates, counters and statuses, 8 fewer bytes per row per
+ * iteration.  The context then owns a second p buffer (padded length of p).
+ * enable = 0 runs the unfused sequence. */
+int abft_ctx_set_fused_cg(abft_ctx* ctx, int enable);
 
 int64_t abft_rowptr_padded_len(int64_t nrows, int32_t scheme);  /* pad with copies of nnz (R6) */
 int64_t abft_vec_padded_len(int64_t n, int32_t scheme);         /* pad with encoded +0.0 */
@@ -144,6 +152,17 @@ int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, ab
 int abft_calc_ur(abft_ctx* ctx, abft_vec* x, abft_vec* p, abft_vec* r, abft_vec* w, double alpha, double* rrn_out,
                  abft_counts* dcnt, void* stream);
 int abft_calc_p(abft_ctx* ctx, abft_vec* p, abft_vec* r, double beta, abft_counts* dcnt, void* stream);
+
+/* a5 + a3 fused: p_out = enc(fma(beta, p_prev, r)) (calc_p,
+ * P:294-314) and out = A*p_out (+ dot_out = p_out.out, RED-1) in ONE tiled
+ * kernel — the same words and counters as abft_calc_p(p_prev, r, beta)
+ * followed by abft_spmv(p_prev, out), except that p_prev itself is left as
+ * it was (single flips scrubbed) and the new p goes to p_out.  Requires the
+ * tiled stencil path (stencil_n) for every chunk and a group-size-1 vector
+ * scheme (NONE / SED / SECDED64), else ABFT_E_SHAPE.  p_prev, r, p_out, out:
+ * equal length and scheme, pairwise distinct. */
+int abft_calc_p_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* p_prev, abft_vec* r, double beta,
+                     abft_vec* p_out, abft_vec* out, double* dot_out, abft_counts* dcnt, void* stream);
 
 /* Check every codeword of the matrix chunks and of the nvec vectors, counting
  * into dcnt.  scrub: 0 count only, 1 count and correct single flips in place,

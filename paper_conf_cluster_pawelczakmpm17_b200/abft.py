@@ -48,6 +48,7 @@ _P = C.c_void_p
 _sig = {
     "abft_ctx_create": (C.c_int, [C.c_int, C.POINTER(C.c_void_p)]),
     "abft_ctx_destroy": (C.c_int, [_P]),
+    "abft_ctx_set_fused_cg": (C.c_int, [_P, C.c_int]),
     "abft_rowptr_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
     "abft_vec_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
     "abft_csr_encode": (C.c_int, [_P, C.POINTER(CSR), _P]),
@@ -61,6 +62,8 @@ _sig = {
     "abft_calc_ur": (C.c_int, [_P, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.c_double, _P, _P,
                                _P]),
     "abft_calc_p": (C.c_int, [_P, C.POINTER(Vec), C.POINTER(Vec), C.c_double, _P, _P]),
+    "abft_calc_p_spmv": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.c_double,
+                                   C.POINTER(Vec), C.POINTER(Vec), _P, _P, _P]),
     "abft_inject_bitflip": (C.c_int, [_P, _P, C.c_uint64, _P]),
     "abft_counts_read": (C.c_int, [_P, _P, _P]),
     "abft_counts_reset": (C.c_int, [_P, _P]),
@@ -143,6 +146,10 @@ class Context:
         h = C.c_void_p()
         _check(_lib.abft_ctx_create(self.device, C.byref(h)), "abft_ctx_create")
         self.h = h
+
+    def set_fused_cg(self, enable: bool):
+        """Fused calc_p in the CG's SpMV (abft_ctx_set_fused_cg; default off)."""
+        _check(_lib.abft_ctx_set_fused_cg(self.h, 1 if enable else 0), "abft_ctx_set_fused_cg")
 
     def close(self):
         if self.h:
@@ -290,6 +297,16 @@ def calc_p(ctx: Context, p: Vector, r: Vector, beta: float, counts: Counters | N
     vp, vr = p.cstruct(), r.cstruct()
     _check(_lib.abft_calc_p(ctx.h, C.byref(vp), C.byref(vr), float(beta), counts.ptr if counts else None,
                             _stream(stream)), "abft_calc_p")
+
+
+def calc_p_spmv(ctx: Context, A, p_prev: Vector, r: Vector, beta: float, p_out: Vector, y: Vector,
+                counts: Counters | None = None, dot: torch.Tensor | None = None, stream=None):
+    """a5 + a3 in one kernel: p_out = enc(fma(beta, p_prev, r)); y = A p_out (+ dot = p_out.y)."""
+    arr, n = _chunks(A)
+    vs = [v.cstruct() for v in (p_prev, r, p_out, y)]
+    _check(_lib.abft_calc_p_spmv(ctx.h, arr, n, C.byref(vs[0]), C.byref(vs[1]), float(beta), C.byref(vs[2]),
+                                 C.byref(vs[3]), dot.data_ptr() if dot is not None else None,
+                                 counts.ptr if counts else None, _stream(stream)), "abft_calc_p_spmv")
 
 
 def check_all(ctx: Context, A, vecs, counts: Counters | None = None, scrub=True, stream=None):

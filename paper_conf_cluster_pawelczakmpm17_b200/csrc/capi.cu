@@ -58,6 +58,9 @@ struct abft_ctx {
   std::vector<cudaEvent_t> events;
   RedState* red = nullptr;   // fused-reduction counters/roots (zero between reductions)
   CrcTables* crc = nullptr;  // CRC32C lookup tables (device)
+  bool fuse_p = false;       // fused calc_p in the CG's SpMV when eligible (opt-in)
+  uint64_t* p_alt = nullptr; // second p buffer of the fused CG
+  int64_t p_alt_len = 0;
 };
 
 namespace {
@@ -94,9 +97,13 @@ int check_chunks(const abft_csr* A, int nchunks) {
 
 // Launch the SpMV over all chunks; partials indexed by global RB (chunks must
 // start on 256-row boundaries relative to chunk 0 when dot is requested).
+// fused calc_p (CG driver): p_cur != null => in = p_{k-1}, r_f = r;
+// probe = true only builds the arguments and reports whether every chunk can
+// take the fused tiled kernel (nothing is launched).
 int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, bool dot,
                 DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total, RedArgs red = RedArgs{},
-                int check_mode = MODE_CORRECT, int check_interval = 0) {
+                int check_mode = MODE_CORRECT, int check_interval = 0, uint64_t* p_cur = nullptr,
+                uint64_t* r_f = nullptr, bool probe = false) {
   const int64_t base0 = A[0].row_base;
   const int64_t npad_in = vec_padded_len(in->n, in->scheme);
   const int64_t npad_out = vec_padded_len(out->n, out->scheme);
@@ -108,7 +115,7 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     const int64_t end_rb = (rel + M.nrows + 255) / 256;
     if (end_rb > nrb_all) nrb_all = end_rb;
   }
-  if (dot) {
+  if (dot && !probe) {
     int e = ensure_partials(ctx, nrb_all);
     if (e) return e;
   }
@@ -141,7 +148,15 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.check_mode = check_mode;
     a.check_interval = check_interval;
     a.crc = ctx->crc;
-    count_launch(launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s));
+    a.p_cur = p_cur;
+    a.r_f = r_f;
+    if (probe) {
+      if (!spmv_fusable(a, in->scheme)) return ABFT_E_SHAPE;
+      continue;
+    }
+    const int l = launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s);
+    if (l < 0) return fail(ABFT_E_CUDA, "chunk %d: fused calc_p SpMV could not be launched", c);
+    count_launch(l);
   }
   if (nrb_total) *nrb_total = nrb_all;
   return ABFT_OK;
@@ -186,6 +201,12 @@ int abft_ctx_create(int device, abft_ctx** out) {
   return ABFT_OK;
 }
 
+int abft_ctx_set_fused_cg(abft_ctx* c, int enable) {
+  if (!c) return fail(ABFT_E_INVALID, "null ctx");
+  c->fuse_p = enable != 0;
+  return ABFT_OK;
+}
+
 int abft_ctx_destroy(abft_ctx* c) {
   if (!c) return ABFT_OK;
   cudaSetDevice(c->device);
@@ -195,6 +216,7 @@ int abft_ctx_destroy(abft_ctx* c) {
   cudaFree(c->state);
   cudaFree(c->due);
   cudaFree(c->flags);
+  cudaFree(c->p_alt);
   cudaFree(c->red);
   cudaFree(c->crc);
   cudaFreeHost(c->h_state);
@@ -425,11 +447,30 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   // all-gather / top-of-tree combine code is exercised on a single GPU)
   const bool multi = d != nullptr;
 
+  // fused calc_p: single GPU, every chunk on the tiled path,
+  // G = 1 vector scheme; p is double-buffered with ctx->p_alt
+  const int64_t npad_ext = vec_padded_len(n_ext, scheme);
+  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0;
+  if (fused) {
+    abft_vec ptmp = *p;
+    fused = spmv_chunks(ctx, A, nchunks, &ptmp, w, true, cnt, nullptr, s, nullptr, RedArgs{}, MODE_CORRECT, 0,
+                        reinterpret_cast<uint64_t*>(p->data), reinterpret_cast<uint64_t*>(r->data), true) == ABFT_OK;
+  }
+  if (fused && ctx->p_alt_len < npad_ext) {
+    cudaFree(ctx->p_alt);
+    ctx->p_alt = nullptr;
+    ctx->p_alt_len = 0;
+    CUDA_TRY(cudaMalloc(&ctx->p_alt, sizeof(uint64_t) * npad_ext));
+    ctx->p_alt_len = npad_ext;
+  }
+  uint64_t* const P[2] = {reinterpret_cast<uint64_t*>(p->data), ctx->p_alt};
+
   CgState h{};
   h.tol = opts->tol;
   h.max_iters = opts->max_iters;
   h.abort_policy = opts->due_policy == 0 ? 1 : 0;
   h.dist = multi ? 1 : 0;
+  h.fused = fused ? 1 : 0;
   *ctx->h_state = h;
   CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
   CUDA_TRY(cudaMemsetAsync(ctx->due, 0, sizeof(int), s));
@@ -460,16 +501,28 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   if ((e = finish_dot(ctx, d, nrb, 1, s))) return e;
   CUDA_TRY(cudaGetLastError());
 
-  const int poll = opts->poll_every > 0 ? opts->poll_every : 16;
+  int poll = opts->poll_every > 0 ? opts->poll_every : 16;
+  if (fused && (poll & 1)) poll += 1;  // graph replays then always start at an odd iteration (buffer parity)
+  int64_t launched = 0;  // iterations issued so far (host); = device iterations until a stop
   // k iterations of (a3)..(a5) + the DUE/convergence logic, all device-side
   auto issue = [&](int64_t k, cudaStream_t s) -> int {
     prof.s = s;
     for (int64_t it = 0; it < k; it++) {
       int e2;
+      // fused: iteration kk's p lives in P[(kk-1) & 1], its predecessor in P[kk & 1]
+      const int64_t kk = launched + it + 1;
+      uint64_t* const pk = fused ? P[(kk - 1) & 1] : reinterpret_cast<uint64_t*>(p->data);
       if ((e2 = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e2;
       prof.begin(0);
-      e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2),
-                       MODE_CORRECT, interval);
+      if (fused) {
+        abft_vec pprev = *p;
+        pprev.data = reinterpret_cast<double*>(P[kk & 1]);
+        e2 = spmv_chunks(ctx, A, nchunks, &pprev, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2),
+                         MODE_CORRECT, interval, pk, reinterpret_cast<uint64_t*>(r->data));
+      } else {
+        e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2),
+                         MODE_CORRECT, interval);
+      }
       prof.end();
       if (e2) return e2;
       prof.begin(3);
@@ -477,15 +530,18 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       prof.end();
       prof.begin(1);
       VecArgs vu = va;
+      vu.p = pk + n_halo;
       vu.red = red_for(ctx, d, nrb, 3);
       count_launch(launch_calc_ur(vu, scheme, s));
       prof.end();
       prof.begin(3);
       if ((e2 = finish_dot(ctx, d, nrb, 3, s))) return e2;
       prof.end();
-      prof.begin(2);
-      count_launch(launch_calc_p(va, scheme, s));
-      prof.end();
+      if (!fused) {
+        prof.begin(2);
+        count_launch(launch_calc_p(va, scheme, s));
+        prof.end();
+      }
       if (multi && h.abort_policy) {
         count_launch(launch_pack_due(d->sendbuf, ctx->due, s));
         NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
@@ -504,7 +560,6 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   // graph replay: profiled solves launch kernels directly)
   const bool graphs = ctx->use_graphs && !multi && ctx->profile == 0;
   bool last_graph = false;
-  int64_t launched = 0;
   for (;;) {
     CUDA_TRY(cudaMemcpyAsync(ctx->h_state, ctx->state, sizeof(CgState), cudaMemcpyDeviceToHost, s));
     CUDA_TRY(cudaStreamSynchronize(s));
@@ -550,6 +605,25 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   }
   if (gexec) cudaGraphExecDestroy(gexec);
   const CgState& hs = *ctx->h_state;
+  if (fused) {
+    // the final p back into the caller's buffer, then the calc_p the unfused
+    // order runs before an abort / max_iters stop (state.pending_p)
+    if (hs.iters >= 1 && ((hs.iters - 1) & 1))
+      CUDA_TRY(cudaMemcpyAsync(p->data, ctx->p_alt, sizeof(uint64_t) * npad_ext, cudaMemcpyDeviceToDevice, s));
+    if (hs.pending_p) {
+      const CgState keep = hs;
+      CgState t{};
+      t.beta = keep.beta;
+      t.max_iters = 0x7FFFFFFF;
+      *ctx->h_state = t;
+      CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
+      VecArgs vp = va;
+      vp.red = RedArgs{};
+      count_launch(launch_calc_p(vp, scheme, s));
+      CUDA_TRY(cudaStreamSynchronize(s));
+      *ctx->h_state = keep;
+    }
+  }
   res->iters = hs.iters;
   res->rr0 = hs.rr0;
   res->rrn = hs.rrn;
@@ -708,6 +782,33 @@ int abft_calc_p(abft_ctx* ctx, abft_vec* p, abft_vec* r, double beta, abft_count
   va.r = reinterpret_cast<uint64_t*>(r->data);
   va.counts = reinterpret_cast<DevCounts*>(dcnt);
   count_launch(launch_calc_p(va, p->scheme, s));
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_calc_p_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* p_prev, abft_vec* r, double beta,
+                     abft_vec* p_out, abft_vec* out, double* dot_out, abft_counts* dcnt, void* stream) {
+  cudaStream_t s = (cudaStream_t)stream;
+  abft_vec* v[4] = {p_prev, r, p_out, out};
+  VecArgs va;
+  int e = check_chunks(A, nchunks);
+  if (e) return e;
+  if ((e = blas1_setup(ctx, v, 4, 0.0, beta, va, s))) return e;
+  const int vs = p_prev->scheme;
+  if (vec_padded_len(1, vs) != 1) return fail(ABFT_E_SHAPE, "fused calc_p + SpMV: vector scheme with group size > 1");
+  // the kernel takes the fused branch when state.iters > 0
+  ctx->h_state->iters = 1;
+  CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
+  DevCounts* cnt = reinterpret_cast<DevCounts*>(dcnt);
+  uint64_t* pc = reinterpret_cast<uint64_t*>(p_out->data);
+  uint64_t* rf = reinterpret_cast<uint64_t*>(r->data);
+  if (spmv_chunks(ctx, A, nchunks, p_prev, out, true, cnt, nullptr, s, nullptr, RedArgs{}, MODE_CORRECT, 0, pc, rf,
+                  true) != ABFT_OK)
+    return fail(ABFT_E_SHAPE, "fused calc_p + SpMV needs the tiled stencil path for every chunk");
+  int64_t nrb = 0;
+  e = spmv_chunks(ctx, A, nchunks, p_prev, out, true, cnt, ctx->state, s, &nrb, RedArgs{}, MODE_CORRECT, 0, pc, rf);
+  if (e) return e;
+  if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
   CUDA_TRY(cudaGetLastError());
   return ABFT_OK;
 }

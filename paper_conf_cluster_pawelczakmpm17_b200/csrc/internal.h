@@ -15,6 +15,11 @@ struct CgState {
   int32_t iters, max_iters, stop, status, abort_policy, converged;
   uint32_t ticket_p;   // calc_p last-block ticket
   int32_t dist;        // 1 = multi-GPU solve (abort decided after an all-gather)
+  // fused calc_p: calc_p of iteration k runs inside the SpMV
+  // of iteration k+1, so the stop decisions calc_p's last block takes move to
+  // the rrn reduction; a stop that the unfused order takes AFTER calc_p leaves
+  // pending_p = 1 and the host runs that calc_p on its own.
+  int32_t fused, pending_p;
 };
 
 struct DevCounts { unsigned long long v[3][5][4]; };
@@ -65,6 +70,17 @@ struct SpmvArgs {
   // iteration counter instead (access k = state->iters + 1, init = 0)
   int32_t check_mode, check_interval;
   const CrcTables* crc;   // device tables (CRC32C schemes only)
+  // fused calc_p (CG driver only, tiled path, G = 1 vector schemes,
+  // DESIGN.md §6.1): p is double-buffered.  Iteration k >= 2 reads
+  // p_{k-1} from `in` and r from r_f, computes p_k = enc(round(fma(beta,
+  // p_{k-1}, r))) into p_cur and multiplies by it; iteration 1 (state->iters
+  // == 0) multiplies by p_1 = p_cur as written by init.  The buffer roles
+  // alternate with the parity of k (host side).  fz / beta_f are filled in by
+  // the kernel (SMEM copy of the arguments).
+  uint64_t* p_cur;
+  uint64_t* r_f;
+  double beta_f;
+  int32_t fz;
 };
 enum { MODE_CORRECT = 0, MODE_DETECT = 1, MODE_RANGE = 2 };
 
@@ -82,6 +98,9 @@ struct VecArgs {
 
 // launchers (kernels.cu); each returns the number of kernels launched
 int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, bool dot, cudaStream_t s);
+// -1: a fused-calc_p launch (a.p_cur set) could not run
+// can this chunk take the fused-calc_p tiled SpMV (G = 1 vector scheme, stencil layout)?
+bool spmv_fusable(const SpmvArgs& a, int vs);
 int launch_calc_ur(const VecArgs& a, int vs, cudaStream_t s);
 int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s);
 int launch_init_r(const VecArgs& a, int vs, cudaStream_t s);

@@ -22,21 +22,22 @@
 namespace abft {
 
 // per-ES SpMV launchers live in spmv_es*.cu (parallel compilation)
-void spmv_es_none(const SpmvArgs&, int, int, bool, cudaStream_t);
-void spmv_es_sed(const SpmvArgs&, int, int, bool, cudaStream_t);
-void spmv_es_secded(const SpmvArgs&, int, int, bool, cudaStream_t);
-void spmv_es_crc(const SpmvArgs&, int, int, bool, cudaStream_t);
+bool spmv_es_none(const SpmvArgs&, int, int, bool, cudaStream_t);
+bool spmv_es_sed(const SpmvArgs&, int, int, bool, cudaStream_t);
+bool spmv_es_secded(const SpmvArgs&, int, int, bool, cudaStream_t);
+bool spmv_es_crc(const SpmvArgs&, int, int, bool, cudaStream_t);
 
 int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, bool dot, cudaStream_t s) {
   if (a.nrows <= 0) return 0;
+  bool ok;
   switch (es) {
-    case NONE: spmv_es_none(a, rs, vs, dot, s); break;
-    case SED: spmv_es_sed(a, rs, vs, dot, s); break;
+    case NONE: ok = spmv_es_none(a, rs, vs, dot, s); break;
+    case SED: ok = spmv_es_sed(a, rs, vs, dot, s); break;
     case SECDED64:
-    case SECDED128: spmv_es_secded(a, rs, vs, dot, s); break;  // R3: both map to E-SECDED
-    default: spmv_es_crc(a, rs, vs, dot, s); break;
+    case SECDED128: ok = spmv_es_secded(a, rs, vs, dot, s); break;  // R3: both map to E-SECDED
+    default: ok = spmv_es_crc(a, rs, vs, dot, s); break;
   }
-  return 1;
+  return ok ? 1 : -1;
 }
 
 // ================================================================ launchers

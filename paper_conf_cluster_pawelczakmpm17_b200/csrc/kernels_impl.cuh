@@ -283,6 +283,15 @@ __device__ __forceinline__ double gather_in(const uint64_t* in, int64_t idx) {
   }
 }
 
+// Fused calc_p (non-owner): p_k[idx] = round(fma(beta, p_{k-1}[idx], r[idx]))
+// from the checked (corrected in registers, not counted) operands — the
+// masked value of the word the unfused calc_p would have stored (G = 1).
+template <int VS>
+__device__ __forceinline__ double gather_fused(const uint64_t* pprev, const uint64_t* r, double beta, int64_t idx) {
+  const double pn = fma(beta, gather_in<VS>(pprev, idx), gather_in<VS>(r, idx));
+  return as_d(round_k(as_u(pn), vk(VS)));
+}
+
 // ============================================================ rowptr pass
 // Decode the rowptr groups covering entries [pb, pb+32] into srp (per warp),
 // checking them (owner = the pass holding row min(gG, nrows-1)), then return
@@ -571,7 +580,7 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
     else if (rel == -1) x = win[oslot - 1];
     else if (rel == n) x = win[oslot + TILE_WW];
     else if (rel == -n) x = win[oslot - TILE_WW];
-    else x = gather_in<VS>(a.in, own + rel);
+    else x = a.fz ? gather_fused<VS>(a.in, a.r_f, a.beta_f, own + rel) : gather_in<VS>(a.in, own + rel);
     acc = fma(as_d(v), x, acc);
   }
   if (ES == CRC32C && mode != MODE_RANGE) {
@@ -649,8 +658,9 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
   return acc;
 }
 
-template <int ES, int RS, int VS, bool DOT>
+template <int ES, int RS, int VS, bool DOT, bool FUSED = false>
 __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __grid_constant__ TileMaps tm) {
+  static_assert(!FUSED || (vgrp(VS) == 1 && DOT), "fused calc_p: G = 1 vector schemes, CG SpMV only");
   extern __shared__ uint8_t s_raw[];
   __shared__ __align__(16) uint8_t s_lut[128];
   // the cold row path takes the arguments by reference: give it a SMEM copy so
@@ -671,8 +681,17 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   const int64_t tx0 = (blockIdx.x % tiles_x) << 8;
   const int64_t ty0 = (int64_t)(blockIdx.x / tiles_x) * TILE_TY;
   // ---- 0. producer: barriers, then the first TILE_NST passes in flight
+  // fused calc_p: iteration 1 multiplies by p_cur as init
+  // wrote it; later iterations build p_cur from (in = p_{k-1}, r) in the window
+  const bool fz = FUSED && a.state->iters > 0;
+  uint64_t* const pin = (FUSED && !fz) ? a.p_cur : a.in;
   if (threadIdx.x == 0) {
     s_args = a;
+    if (FUSED) {
+      s_args.in = pin;
+      s_args.fz = fz ? 1 : 0;
+      s_args.beta_f = fz ? a.state->beta : 0.0;
+    }
 #pragma unroll
     for (int s = 0; s < TILE_NST; s++) {
       mbar_init(&full[s], 1);
@@ -780,7 +799,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       for (int q = 0; q < WPER; q++) {
         const int64_t idx = a0 + 32 * q + lane;
         ok[q] = idx >= 0 && idx < a.npad_in;   // identical across a group (npad_in is a multiple of G)
-        wv[q] = ok[q] ? ldg64(a.in + idx) : 0ull;
+        wv[q] = ok[q] ? ldg64(pin + idx) : 0ull;
       }
       bool bad = false;
       if (VS == SECDED128) {   // zero groups are clean
@@ -800,7 +819,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
         for (int q = 0; q < WPER; q++) {
           const int slot = 32 * q + lane - (VG - 1);
           const bool owner = row_own && slot >= 1 && slot <= 256;   // groups never straddle the tile edge
-          wv[q] = vg_check<VS>(wv[q], a.in + (a0 + 32 * q + (lane & ~(VG - 1))), lane, ok[q], owner && ok[q],
+          wv[q] = vg_check<VS>(wv[q], pin + (a0 + 32 * q + (lane & ~(VG - 1))), lane, ok[q], owner && ok[q],
                                a.counts, a.due);
         }
       }
@@ -810,12 +829,62 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
         if (slot >= 0 && slot < TILE_WW) dst[slot] = as_d(wv[q] & vkeep(VS));
       }
     }
+  } else if (FUSED && fz) {
+    // fused calc_p window (G = 1): every slot is p_k = round(fma(beta, p_{k-1},
+    // r)) of the checked operands (the masked value of the word calc_p would
+    // store); the tile's own cells (calc_p's owners) count and scrub, halo
+    // cells are recomputed without counting.  enc(p_k) of the own cells is
+    // stored to p_cur in the pass loop (off this latency-exposed phase).
+    const double beta = a.state->beta;
+    for (int wy = warp; wy < TILE_TY + 2; wy += 8) {
+      const int64_t rbase = win0 + (int64_t)wy * n;
+      const bool row_in = rbase >= 0 && rbase + TILE_WW <= a.npad_in;
+      double* dst = s_win + wy * TILE_WW;
+      uint64_t pv[WPER], rv[WPER];
+#pragma unroll
+      for (int q = 0; q < WPER; q++) {
+        const int wx = lane + 32 * q;
+        const int64_t idx = rbase + wx;
+        const bool ok = wx < TILE_WW && (row_in || (idx >= 0 && idx < a.npad_in));
+        pv[q] = ok ? ldg64(pin + idx) : 0ull;
+        rv[q] = ok ? ldg64(a.r_f + idx) : 0ull;
+      }
+      uint32_t acc_r = 0, acc_p = 0;
+#pragma unroll
+      for (int q = 0; q < WPER; q++) {   // OR-accumulated fast check; zero (out-of-range) words are clean
+        const int wx = lane + 32 * q;
+        if (VS == SED) acc_p |= (uint32_t)(popc64(pv[q]) | popc64(rv[q]));
+        if (VS == SECDED64) {
+          v64_acc(lo32(pv[q]), hi32(pv[q]), acc_r, acc_p);
+          v64_acc(lo32(rv[q]), hi32(rv[q]), acc_r, acc_p);
+        }
+        if (wx < TILE_WW) {
+          const int64_t idx = rbase + wx;
+          const bool ok = row_in || (idx >= 0 && idx < a.npad_in);
+          const double pn = fma(beta, as_d(pv[q] & vkeep(VS)), as_d(rv[q] & vkeep(VS)));
+          dst[wx] = ok ? as_d(round_k(as_u(pn), vk(VS))) : 0.0;
+        }
+      }
+      if (VS != NONE && syn_bad(acc_r, acc_p)) {  // cold: reload, correct (owner counts + scrubs), recompute
+        const bool row_own = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny;
+        for (int q = 0; q < WPER; q++) {
+          const int wx = lane + 32 * q;
+          const int64_t idx = rbase + wx;
+          if (wx >= TILE_WW || idx < 0 || idx >= a.npad_in) continue;
+          const bool owner = row_own && wx >= 1 && wx <= 256;
+          const uint64_t rw = v1_check<VS>(ldg64(a.r_f + idx), a.r_f + idx, owner, a.counts, a.due);
+          const uint64_t pw = v1_check<VS>(ldg64(pin + idx), pin + idx, owner, a.counts, a.due);
+          const double pn = fma(beta, as_d(pw & vkeep(VS)), as_d(rw & vkeep(VS)));
+          dst[wx] = as_d(round_k(as_u(pn), vk(VS)));
+        }
+      }
+    }
   } else
   for (int wy = warp; wy < TILE_TY + 2; wy += 8) {
     const int64_t rbase = win0 + (int64_t)wy * n;                 // in-index of (wy, 0)
     const bool row_in = rbase >= 0 && rbase + TILE_WW <= a.npad_in;  // uniform: no per-slot bounds
     const bool row_own = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny;
-    const uint64_t* src = a.in + rbase;
+    const uint64_t* src = pin + rbase;
     double* dst = s_win + wy * TILE_WW;
     uint64_t wv[WPER];
 #pragma unroll
@@ -840,7 +909,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
         const int64_t idx = rbase + wx;
         if (wx >= TILE_WW || idx < 0 || idx >= a.npad_in) continue;
         const bool owner = row_own && wx >= 1 && wx <= 256;
-        const uint64_t w = v1_check<VS>(ldg64(src + wx), a.in + idx, owner, a.counts, a.due);
+        const uint64_t w = v1_check<VS>(ldg64(src + wx), pin + idx, owner, a.counts, a.due);
         dst[wx] = as_d(w & vkeep(VS));
       }
     }
@@ -889,6 +958,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
         const uint64_t enc = (VS == CRC32C) ? vcrc_encode_lane(rounded, vcrc_tab(cs, lane), lane)
                                             : v_encode<VS>(rounded, lane, s_lut);
         a.out[own] = enc;
+        if (FUSED && fz) a.p_cur[own] = v_encode<VS>(as_u(p_own), lane, s_lut);   // enc(p_k), own cell
         if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
       }
     }
@@ -1242,6 +1312,11 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
       st->status = (st->abort_policy && dueflag) ? ABFT_E_DUE : ABFT_OK;
     } else {
       st->beta = res / st->rro;
+      if (st->fused) {  // calc_p's last-block logic (k_calc_p), taken here: calc_p runs in the next SpMV
+        st->rro = res;
+        if (!st->dist && st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; st->pending_p = 1; }
+        else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; st->pending_p = 1; }
+      }
     }
   }
 }

@@ -4,8 +4,8 @@
 
 namespace abft {
 
-void spmv_es_crc(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
-  spmv1<CRC32C>(a, rs, vs, dot, s);
+bool spmv_es_crc(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
+  return spmv1<CRC32C>(a, rs, vs, dot, s);
 }
 
 }  // namespace abft

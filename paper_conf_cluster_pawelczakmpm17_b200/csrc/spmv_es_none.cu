@@ -4,8 +4,12 @@
 
 namespace abft {
 
-void spmv_es_none(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
-  spmv1<NONE>(a, rs, vs, dot, s);
+bool spmv_es_none(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
+  return spmv1<NONE>(a, rs, vs, dot, s);
+}
+
+bool spmv_fusable(const SpmvArgs& a, int vs) {
+  return (vs == NONE || vs == SED || vs == SECDED64) && tile_ok(a, vs) && tmap_encoder() != nullptr;
 }
 
 }  // namespace abft

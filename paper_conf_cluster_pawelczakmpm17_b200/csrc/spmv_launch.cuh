@@ -47,52 +47,59 @@ static bool tile_maps(const SpmvArgs& a, TileMaps* m) {
                     CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   return r1 == CUDA_SUCCESS && r2 == CUDA_SUCCESS;
 }
-template <int ES, int RS, int VS, bool DOT>
+template <int ES, int RS, int VS, bool DOT, bool FUSED = false>
 static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   TileMaps tm;
   if (!tile_maps(a, &tm)) return false;
   const size_t smem = tile_smem<ES, RS, VS>();
   static bool attr = false;
-  if (!attr) {  // both variants at once: never inside a later CUDA-graph capture
-    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, true>, cudaFuncAttributePreferredSharedMemoryCarveout, 100);
-    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, false>, cudaFuncAttributePreferredSharedMemoryCarveout, 100);
+  if (!attr) {  // set before first use: never inside a later CUDA-graph capture
+    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, DOT, FUSED>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, DOT, FUSED>, cudaFuncAttributePreferredSharedMemoryCarveout, 100);
     attr = true;
   }
   const int64_t ny = a.nrows / a.stencil_n;
   const int64_t blocks = (a.stencil_n / 256) * ((ny + TILE_TY - 1) / TILE_TY);
-  k_spmv_tile<ES, RS, VS, DOT><<<(unsigned)blocks, 256, smem, s>>>(a, tm);
+  k_spmv_tile<ES, RS, VS, DOT, FUSED><<<(unsigned)blocks, 256, smem, s>>>(a, tm);
   return true;
 }
+// Returns false only when a fused-calc_p launch (a.p_cur set) was requested
+// and cannot run: the caller fails loudly, there is no unfused fallback here.
 template <int ES, int RS, int VS>
-static void spmv3(const SpmvArgs& a, bool dot, cudaStream_t s) {
+static bool spmv3(const SpmvArgs& a, bool dot, cudaStream_t s) {
+  if (a.p_cur) {
+    if constexpr (vgrp(VS) == 1) {
+      return dot && tile_ok(a, VS) && spmv_tile_launch<ES, RS, VS, true, true>(a, s);
+    }
+    return false;
+  }
   if (tile_ok(a, VS)) {
-    if (dot ? spmv_tile_launch<ES, RS, VS, true>(a, s) : spmv_tile_launch<ES, RS, VS, false>(a, s)) return;
+    if (dot ? spmv_tile_launch<ES, RS, VS, true>(a, s) : spmv_tile_launch<ES, RS, VS, false>(a, s)) return true;
   }
   const int64_t nrb = (a.nrows + 255) / 256;
   const int blocks = (int)((nrb + 7) / 8);
   if (dot) k_spmv<ES, RS, VS, true><<<blocks, 256, 0, s>>>(a);
   else k_spmv<ES, RS, VS, false><<<blocks, 256, 0, s>>>(a);
+  return true;
 }
 template <int ES, int RS>
-static void spmv2(const SpmvArgs& a, int vs, bool dot, cudaStream_t s) {
+static bool spmv2(const SpmvArgs& a, int vs, bool dot, cudaStream_t s) {
   switch (vs) {
-    case NONE: spmv3<ES, RS, NONE>(a, dot, s); break;
-    case SED: spmv3<ES, RS, SED>(a, dot, s); break;
-    case SECDED64: spmv3<ES, RS, SECDED64>(a, dot, s); break;
-    case SECDED128: spmv3<ES, RS, SECDED128>(a, dot, s); break;
-    default: spmv3<ES, RS, CRC32C>(a, dot, s); break;
+    case NONE: return spmv3<ES, RS, NONE>(a, dot, s);
+    case SED: return spmv3<ES, RS, SED>(a, dot, s);
+    case SECDED64: return spmv3<ES, RS, SECDED64>(a, dot, s);
+    case SECDED128: return spmv3<ES, RS, SECDED128>(a, dot, s);
+    default: return spmv3<ES, RS, CRC32C>(a, dot, s);
   }
 }
 template <int ES>
-static void spmv1(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
+static bool spmv1(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
   switch (rs) {
-    case NONE: spmv2<ES, NONE>(a, vs, dot, s); break;
-    case SED: spmv2<ES, SED>(a, vs, dot, s); break;
-    case SECDED64: spmv2<ES, SECDED64>(a, vs, dot, s); break;
-    case SECDED128: spmv2<ES, SECDED128>(a, vs, dot, s); break;
-    default: spmv2<ES, CRC32C>(a, vs, dot, s); break;
+    case NONE: return spmv2<ES, NONE>(a, vs, dot, s);
+    case SED: return spmv2<ES, SED>(a, vs, dot, s);
+    case SECDED64: return spmv2<ES, SECDED64>(a, vs, dot, s);
+    case SECDED128: return spmv2<ES, SECDED128>(a, vs, dot, s);
+    default: return spmv2<ES, CRC32C>(a, vs, dot, s);
   }
 }
 

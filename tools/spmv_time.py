@@ -51,6 +51,9 @@ def main():
             "calc_ur_ms": t(lambda: abft.calc_ur(ctx, x, p, r, w, 1e-30, rrn=dot, counts=cnt)),
             "calc_p_ms": t(lambda: abft.calc_p(ctx, p, r, 1e-30, counts=cnt)),
         }
+        p2 = abft.Vector.empty(P["N"], s)
+        res["fused_calc_p_spmv_ms"] = t(lambda: abft.calc_p_spmv(ctx, sol.A, p, r, 1e-30, p2, w, cnt, dot=dot))
+        res["fused_gbs"] = 96.0 * P["N"] / (res["fused_calc_p_spmv_ms"] * 1e-3) / 1e9
         res["spmv_gbs"] = 80.0 * P["N"] / (res["spmv_ms"] * 1e-3) / 1e9
         res["counts"] = int(cnt.read().sum())
         out[f"scheme{s}"] = res

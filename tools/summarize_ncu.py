@@ -80,7 +80,8 @@ def main():
                          f" {avg['dram%']:.1f} | {avg['sm%']:.1f} | {avg['issue%']:.1f} | {avg['alu%']:.1f} |"
                          f" {avg['fma%']:.1f} | {avg['lsu%']:.1f} | {avg['fp64%']:.1f} | {avg['occ%']:.1f} |"
                          f" {avg['regs']:.0f} | {avg['warp_inst'] / 1e6:.1f} |")
-            if "k_spmv<2, 2, 2, 1>" in k or k.endswith("k_spmv<2, 2, 2, 1>"):
+            # the protected CG SpMV of the bench (tiled path; the generic kernel in old reports)
+            if "k_spmv_tile<2, 2, 2, 1" in k or "k_spmv<2, 2, 2, 1>" in k:
                 json.dump({"kernel": k, "bytes_per_launch": avg["dram_rd"] + avg["dram_wr"],
                            "read": avg["dram_rd"], "write": avg["dram_wr"], "source": f"profiles/{tag}/ncu_full_raw.csv",
                            "dur_us_under_ncu": avg["dur"]},
