@@ -15,6 +15,9 @@
  *         CG         TeaLeaf CG (ref [19]), DESIGN.md §4
  *         interval   "less frequent correctness checking" P:398-425 (§VI-A.2),
  *                    DESIGN.md §3.9 (reading R27)
+ *         CRC fix    1EC4ED single-bit correction of a failing CRC32C codeword
+ *                    P:260-278 (§IV; HD 6 for 178..5243-bit codewords,
+ *                    P:268-271), DESIGN.md §3.5 (reading R9)
  *
  * Every computation is the plain definition: syndromes are XORs of H-columns
  * over a loop on every container bit, CRC32C is the bit-serial division,
@@ -262,6 +265,36 @@ static uint32_t vcrc(const uint64_t* d) {
   return or_crc32c(m, 32);
 }
 
+/* 1EC4ED: a failing CRC32C codeword that is one bit away from a
+ * valid codeword is corrected; the bit is found by flipping each stored bit
+ * in turn and re-checking (the plain definition).  Only within CRC32C's HD-6
+ * length range (message + 32 <= 5243 bits), where at most one
+ * single flip can succeed and 2..4 flips never look like one; anything else
+ * is a DUE.  ok(w, ctx) re-checks the words w[0 .. nbits/32). */
+#define CRC_HD6_MAX_BITS 5243
+static int crc_fix_brute(uint32_t* w, int nbits, int msg_bits, int (*ok)(const uint32_t*, const void*),
+                         const void* ctx) {
+  if (ok(w, ctx)) return OUT_CLEAN;
+  if (msg_bits + 32 > CRC_HD6_MAX_BITS) return OUT_DUE;
+  int found = -1, nfound = 0;
+  for (int b = 0; b < nbits; b++) {
+    flipbit(w, b);
+    if (ok(w, ctx)) { nfound++; found = b; }
+    flipbit(w, b);
+  }
+  if (nfound != 1) return OUT_DUE;
+  flipbit(w, found);
+  return OUT_CORRECTED;
+}
+static int vcrc_ok(const uint32_t* w, const void* ctx) {
+  (void)ctx;
+  uint64_t d[4];
+  for (int i = 0; i < 4; i++) d[i] = (uint64_t)w[2 * i] | ((uint64_t)w[2 * i + 1] << 32);
+  uint32_t c = 0;
+  for (int i = 0; i < 4; i++) c |= (uint32_t)(d[i] & 0xFF) << (8 * i);
+  return c == vcrc(d);
+}
+
 /* Encode one group of G already-rounded values (reserved bits are overwritten). */
 static void vec_encode_group(uint64_t* d, int scheme) {
   uint32_t w[4];
@@ -290,7 +323,7 @@ static void vec_encode_group(uint64_t* d, int scheme) {
 /* Check one group; corrects d in place; returns OUT_*; *word32 = index of the
  * 32-bit word holding the corrected bit (for scrub accounting). */
 static int vec_check_group(uint64_t* d, int scheme) {
-  uint32_t w[4];
+  uint32_t w[8];
   int out = OUT_CLEAN, bit;
   switch (scheme) {
     case S_SED:
@@ -303,12 +336,11 @@ static int vec_check_group(uint64_t* d, int scheme) {
     case S_SECDED128:
       u64_to_words(d, 2, w); out = secded_check(&INST[I_V_SECDED128], w, &bit); words_to_u64(w, 2, d);
       break;
-    case S_CRC32C: {
-      uint32_t c = 0;
-      for (int i = 0; i < 4; i++) c |= (uint32_t)(d[i] & 0xFF) << (8 * i);
-      out = (c == vcrc(d)) ? OUT_CLEAN : OUT_DUE;
+    case S_CRC32C:   /* V-CRC quad: 256 stored bits, 256-bit message */
+      u64_to_words(d, 4, w);
+      out = crc_fix_brute(w, 256, 256, vcrc_ok, NULL);
+      words_to_u64(w, 4, d);
       break;
-    }
     default: break;
   }
   return out;
@@ -382,17 +414,19 @@ static void rp_encode_group(uint32_t* e, int scheme) {
     default: break;
   }
 }
+static int rcrc_ok(const uint32_t* e, const void* ctx) {
+  (void)ctx;
+  uint32_t c = 0;
+  for (int i = 0; i < 8; i++) c |= (e[i] >> 28) << (4 * i);
+  return c == rcrc(e);
+}
 static int rp_check_group(uint32_t* e, int scheme) {
   int bit;
   switch (scheme) {
     case S_SED: return parity_words(e, 32) ? OUT_DUE : OUT_CLEAN;
     case S_SECDED64: return secded_check(&INST[I_R_SECDED64], e, &bit);
     case S_SECDED128: return secded_check(&INST[I_R_SECDED128], e, &bit);
-    case S_CRC32C: {
-      uint32_t c = 0;
-      for (int i = 0; i < 8; i++) c |= (e[i] >> 28) << (4 * i);
-      return c == rcrc(e) ? OUT_CLEAN : OUT_DUE;
-    }
+    case S_CRC32C: return crc_fix_brute(e, 256, 256, rcrc_ok, NULL);   /* R-CRC octet */
     default: return OUT_CLEAN;
   }
 }
@@ -423,6 +457,42 @@ static uint32_t ecrc_stored(const uint32_t* col, int64_t start) {
   uint32_t c = 0;
   for (int k = 0; k < 4; k++) c |= (col[start + k] >> 24) << (8 * k);
   return c;
+}
+/* E-CRC row check on the row's words w = [val lo, val hi, col] x L. */
+static int ecrc_ok(const uint32_t* w, const void* ctx) {
+  int64_t L = *(const int64_t*)ctx;
+  uint64_t* v = (uint64_t*)malloc(sizeof(uint64_t) * (size_t)L);
+  uint32_t* c = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)L);
+  for (int64_t k = 0; k < L; k++) {
+    v[k] = (uint64_t)w[3 * k] | ((uint64_t)w[3 * k + 1] << 32);
+    c[k] = w[3 * k + 2];
+  }
+  int ok = ecrc_stored(c, 0) == ecrc_row(v, c, 0, L);
+  free(v); free(c);
+  return ok;
+}
+/* Check the E-CRC codeword of row [s, t): rows with fewer than
+ * 4 entries are DUEs; a single flipped bit is located (crc_fix_brute) and, if
+ * fix, written back to val / col.  dec_col (may be NULL, L entries) receives
+ * the decoded column words: corrected when the outcome is CORRECTED (written
+ * back or not), the stored words otherwise. */
+static int ecrc_check_row(uint64_t* val, uint32_t* col, int64_t s, int64_t t, int fix, uint32_t* dec_col) {
+  int64_t L = t - s;
+  if (L < 4) {
+    if (dec_col) for (int64_t k = 0; k < L; k++) dec_col[k] = col[s + k];
+    return OUT_DUE;
+  }
+  uint32_t* w = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)(3 * L));
+  for (int64_t k = 0; k < L; k++) el_words(val[s + k], col[s + k], w + 3 * k);
+  int o = crc_fix_brute(w, (int)(96 * L), (int)(96 * L), ecrc_ok, &L);
+  if (o == OUT_CORRECTED && fix)
+    for (int64_t k = 0; k < L; k++) {
+      val[s + k] = (uint64_t)w[3 * k] | ((uint64_t)w[3 * k + 1] << 32);
+      col[s + k] = w[3 * k + 2];
+    }
+  if (dec_col) for (int64_t k = 0; k < L; k++) dec_col[k] = (o == OUT_CORRECTED) ? w[3 * k + 2] : col[s + k];
+  free(w);
+  return o;
 }
 
 /* Encode a CSR matrix in place (a0): col gets ECC in its spare bits, rowptr is
@@ -590,10 +660,9 @@ int64_t or_spmv_mode(or_csr* A, uint64_t* in, int64_t n_in, int vs, uint64_t* ou
       acc[i] = 0.0;
       continue;
     }
-    if (A->es == S_CRC32C && mode != M_RANGE) {   /* E-CRC: the row is the codeword */
-      int o;
-      if (t - s < 4) o = OUT_DUE;
-      else o = (ecrc_stored(A->col, s) == ecrc_row(A->val, A->col, s, t)) ? OUT_CLEAN : OUT_DUE;
+    if (A->es == S_CRC32C && mode != M_RANGE) {   /* E-CRC: the row is the codeword (corrected + scrubbed) */
+      int o = ecrc_check_row(A->val, A->col, s, t, mode == M_CORRECT, NULL);
+      if (o == OUT_CORRECTED && mode == M_DETECT) o = OUT_DUE;   /* detection only, stored bits */
       count_outcome(cnt, T_ELEM, S_CRC32C, o);
       if (o == OUT_DUE) dues++;
     }
@@ -674,7 +743,8 @@ static int64_t check_elements(or_csr* A, double* vd, uint32_t* cd, uint8_t* skip
     vd[e] = bits2d(v);
     cd[e] = w[2] & cm;
     skip[e] = 0;
-    if (A->es != S_NONE && (int64_t)cd[e] >= A->ncols) {
+    /* E-CRC columns are range-checked in the row pass, as decoded by their row codeword */
+    if (A->es != S_NONE && A->es != S_CRC32C && (int64_t)cd[e] >= A->ncols) {
       skip[e] = 1;
       if (cnt) (*cnt)[T_ELEM][A->es][C_RANGE]++;
       dues++;
@@ -705,9 +775,19 @@ int64_t or_check_csr(or_csr* A, counts_t* cnt, int scrub) {
       continue;
     }
     if (A->es == S_CRC32C) {
-      int o = (t - s < 4) ? OUT_DUE : (ecrc_stored(A->col, s) == ecrc_row(A->val, A->col, s, t) ? OUT_CLEAN : OUT_DUE);
+      /* the row is the codeword: range-check its columns as decoded by it */
+      uint32_t* dc = (uint32_t*)malloc(sizeof(uint32_t) * (size_t)(t - s + 1));
+      int o = ecrc_check_row(A->val, A->col, s, t, scrub && mode == M_CORRECT, mode == M_CORRECT ? dc : NULL);
+      if (mode != M_CORRECT) for (uint32_t j = s; j < t; j++) dc[j - s] = A->col[j];
+      if (o == OUT_CORRECTED && mode == M_DETECT) o = OUT_DUE;
       count_outcome(cnt, T_ELEM, S_CRC32C, o);
       if (o == OUT_DUE) dues++;
+      for (uint32_t j = s; j < t; j++)
+        if ((int64_t)(dc[j - s] & 0x00FFFFFFu) >= A->ncols) {
+          if (cnt) (*cnt)[T_ELEM][S_CRC32C][C_RANGE]++;
+          dues++;
+        }
+      free(dc);
     }
   }
   free(vd); free(cd); free(skip); free(rp);

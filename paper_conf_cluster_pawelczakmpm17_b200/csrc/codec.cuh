@@ -423,6 +423,56 @@ ABFT_HD bool vcrc_clean(const uint64_t* d) {
   return st == vcrc_compute(d);
 }
 
+// ---- CRC32C single-bit correction, 1EC4ED.
+// CRC32C is affine in the message, so a failing codeword's syndrome
+// syn = stored CRC ^ recomputed CRC depends only on the error pattern: a flip
+// of stored CRC bit t gives 1 << t; a flip of message bit i (bytes LSB-first,
+// i = 8 * byte + bit) of an M-bit message gives the register that a single 1
+// at position i leaves after the remaining M-1-i zero bits, i.e.
+// step0^(M-1-i)(poly).  Within CRC32C's HD-6 range (message + 32 <= 5243
+// bits) all these syndromes are distinct and no pattern of 2..4
+// flips shares one, so a match corrects exactly one bit and anything else is
+// a DUE (1EC4ED).  This runs only on the cold (failed-check) path.
+constexpr int CRC_NO_FIX = -1000;
+constexpr int CRC_HD6_MAX_BITS = 5243;
+ABFT_HD int ctz32(uint32_t x) {
+#if defined(__CUDA_ARCH__)
+  return __ffs((int)x) - 1;
+#else
+  return __builtin_ctz(x);
+#endif
+}
+// >= 0: message bit index; -1 - t: stored CRC bit t; CRC_NO_FIX: no single-bit explanation.
+ABFT_HD int crc_locate(uint32_t syn, int mbits) {
+  if (syn == 0u || mbits + 32 > CRC_HD6_MAX_BITS) return CRC_NO_FIX;
+  if ((syn & (syn - 1u)) == 0u) return -1 - ctz32(syn);
+  uint32_t v = 0x82F63B78u;   // syndrome of the last message bit
+  for (int i = mbits - 1; i >= 0; i--) {
+    if (v == syn) return i;
+    v = (v >> 1) ^ (0x82F63B78u & (0u - (v & 1u)));
+  }
+  return CRC_NO_FIX;
+}
+// V-CRC quad: check, locate and correct in place; *word = 32-bit word index in the group.
+ABFT_HD int vcrc_check_fix(uint64_t* d, int* word) {
+  uint32_t st = 0;
+  for (int i = 0; i < 4; i++) st |= (uint32_t)(d[i] & 0xFF) << (8 * i);
+  const uint32_t syn = st ^ vcrc_compute(d);
+  if (!syn) return CLEAN;
+  const int r = crc_locate(syn, 256);
+  if (r == CRC_NO_FIX) return DUE;
+  int bit;                                        // container bit: double bit / 64, bit % 64
+  if (r < 0) bit = 64 * ((-1 - r) >> 3) + ((-1 - r) & 7);   // CRC byte t/8 = low byte of double t/8
+  else {
+    const int byte = r >> 3, bb = byte & 7;
+    if (bb == 0) return DUE;                      // zeroed message byte: not a stored bit
+    bit = 64 * (byte >> 3) + 8 * bb + (r & 7);
+  }
+  d[bit >> 6] ^= 1ull << (bit & 63);
+  if (word) *word = bit >> 5;
+  return CORRECTED;
+}
+
 // Generic vector group encode / check (G = vec_group(S) consecutive values).
 template <int S>
 ABFT_HD void vec_encode_group(uint64_t* d, const uint8_t* v64lut) {
@@ -441,7 +491,7 @@ ABFT_HD int vec_check_group(uint64_t* d, int* word) {
     return v64_correct(d[0], word);
   }
   if (S == SECDED128) return v128_check(d, word);
-  if (S == CRC32C) return vcrc_clean(d) ? CLEAN : DUE;
+  if (S == CRC32C) return vcrc_check_fix(d, word);
   return CLEAN;
 }
 
@@ -619,10 +669,23 @@ ABFT_HD int rp_check_group(uint32_t* e, int* word) {
     if (!s && !q) return CLEAN;
     return secded_resolve<4>(ABFT_MAP(r128), e, s, q, word);
   }
-  if (RS == CRC32C) {
+  if (RS == CRC32C) {   // R-CRC octet, 1EC4ED (see crc_locate)
     uint32_t st = 0;
     for (int i = 0; i < 8; i++) st |= (e[i] >> 28) << (4 * i);
-    return st == rcrc_compute(e) ? CLEAN : DUE;
+    const uint32_t syn = st ^ rcrc_compute(e);
+    if (!syn) return CLEAN;
+    const int r = crc_locate(syn, 256);
+    if (r == CRC_NO_FIX) return DUE;
+    int ent, bit;
+    if (r < 0) { ent = (-1 - r) >> 2; bit = 28 + ((-1 - r) & 3); }   // CRC nibble t/4 = bits 28..31 of entry t/4
+    else {
+      ent = r >> 5;            // 4 message bytes per entry
+      bit = r & 31;
+      if (bit >= 28) return DUE;   // masked-out top nibble: not a message bit
+    }
+    e[ent] ^= 1u << bit;
+    if (word) *word = ent;
+    return CORRECTED;
   }
   return CLEAN;
 }

@@ -193,15 +193,15 @@ int launch_csr_encode(abft_csr* A, uint32_t* flags, cudaStream_t s) {
 }
 
 template <int ES>
-static int check_rows_es(const abft_csr* A, DevCounts* c, int* due, cudaStream_t s) {
+static int check_rows_es(const abft_csr* A, DevCounts* c, int* due, int scrub, cudaStream_t s) {
   int nb = grid_for(A->nrows, 256);
-  const uint64_t* val = reinterpret_cast<const uint64_t*>(A->val);
+  uint64_t* val = reinterpret_cast<uint64_t*>(A->val);
   switch (A->rowptr_scheme) {
-    case NONE: k_check_rows<ES, NONE><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, c, due); break;
-    case SED: k_check_rows<ES, SED><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, c, due); break;
-    case SECDED64: k_check_rows<ES, SECDED64><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, c, due); break;
-    case SECDED128: k_check_rows<ES, SECDED128><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, c, due); break;
-    default: k_check_rows<ES, CRC32C><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, c, due); break;
+    case NONE: k_check_rows<ES, NONE><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, A->ncols, c, due, scrub); break;
+    case SED: k_check_rows<ES, SED><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, A->ncols, c, due, scrub); break;
+    case SECDED64: k_check_rows<ES, SECDED64><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, A->ncols, c, due, scrub); break;
+    case SECDED128: k_check_rows<ES, SECDED128><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, A->ncols, c, due, scrub); break;
+    default: k_check_rows<ES, CRC32C><<<nb, 256, 0, s>>>(val, A->col, A->rowptr, A->nrows, A->nnz, A->ncols, c, due, scrub); break;
   }
   return 1;
 }
@@ -228,8 +228,8 @@ int launch_check_csr(const abft_csr* A, DevCounts* c, int* due, int scrub, cudaS
     launches++;
   }
   if (A->nrows > 0 && (rs != NONE || es == CRC32C)) {
-    if (es == CRC32C) launches += check_rows_es<CRC32C>(A, c, due, s);
-    else launches += check_rows_es<NONE>(A, c, due, s);
+    if (es == CRC32C) launches += check_rows_es<CRC32C>(A, c, due, scrub, s);
+    else launches += check_rows_es<NONE>(A, c, due, scrub, s);
   }
   return launches;
 }

@@ -370,6 +370,67 @@ __device__ __noinline__ int elem_fix(uint64_t& v, uint32_t& c, uint64_t* vaddr, 
   return o;
 }
 
+// E-CRC row codeword [start, start+len) failed its check:
+// recompute from global memory, locate a single flipped bit (1EC4ED,
+// crc_locate) and, per `how`: 1 scrub it (32-bit CAS; the winner counts the
+// correction), 0 count it without writing (check_all count-only), 2 report a
+// DUE (detection only: interval mode).  Anything else is a DUE
+// (counted at every access).  Returns CLEAN (someone else already scrubbed
+// it), CORRECTED (read the row from global memory again) or DUE (use the
+// stored bits).
+static __device__ __noinline__ int ecrc_fix(uint64_t* val, uint32_t* col, uint32_t start, uint32_t len, int how,
+                                            DevCounts* cnt, int* due, uint32_t** fix_addr = nullptr,
+                                            int* fix_bit = nullptr) {
+  int o = DUE;
+  uint32_t* addr = nullptr;
+  int bit = 0;
+  if (len >= 4) {
+    uint32_t crc = 0xFFFFFFFFu, st = 0;
+    for (uint32_t j = 0; j < len; j++) {
+      const uint32_t c = *(volatile uint32_t*)(col + start + j);
+      const uint64_t v = *(volatile uint64_t*)(val + start + j);
+      if (j < 4) st |= (c >> 24) << (8 * j);
+      crc = ecrc_update(crc, v, c, (int)j);
+    }
+    const uint32_t syn = st ^ crc ^ 0xFFFFFFFFu;
+    if (!syn) return CLEAN;
+    const int r = crc_locate(syn, 96 * (int)len);
+    if (r != CRC_NO_FIX) {
+      if (r < 0) {   // stored CRC byte t/8 = col[31:24] of entry t/8
+        addr = col + start + ((-1 - r) >> 3);
+        bit = 24 + ((-1 - r) & 7);
+        o = CORRECTED;
+      } else {       // message: per entry 8 bytes val LE, 4 bytes col LE (top byte zeroed for entries 0..3)
+        const int byte = r >> 3, k = byte / 12, bb = byte - 12 * k;
+        if (bb < 8) {
+          addr = reinterpret_cast<uint32_t*>(val + start + k) + (bb >> 2);
+          bit = 8 * (bb & 3) + (r & 7);
+          o = CORRECTED;
+        } else if (!(k < 4 && bb == 11)) {
+          addr = col + start + k;
+          bit = 8 * (bb - 8) + (r & 7);
+          o = CORRECTED;
+        }
+      }
+    }
+  }
+  if (o == CORRECTED && how == 2) o = DUE;
+  if (fix_addr) *fix_addr = (o == CORRECTED) ? addr : nullptr;   // the located bit (count-only callers apply it)
+  if (fix_bit) *fix_bit = bit;
+  if (o == CORRECTED) {
+    if (how == 1) {
+      const uint32_t w = *(volatile uint32_t*)addr;
+      if (scrub32(addr, w, w ^ (1u << bit))) cnt_add(cnt, T_ELEM, CRC32C, CORRECTED);
+    } else {
+      cnt_add(cnt, T_ELEM, CRC32C, CORRECTED);
+    }
+  } else {
+    cnt_add(cnt, T_ELEM, CRC32C, DUE);
+    *due = 1;
+  }
+  return o;
+}
+
 // ================================================================ SpMV (a3)
 template <int ES, int RS, int VS, bool DOT>
 __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
@@ -404,15 +465,21 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
         cnt_range(a.counts, T_ROWPTR, RS);
         *a.due = 1;
       } else {
-        uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
+        bool fixed = false;   // E-CRC row corrected in global memory: read it without the read-only path
+        if (ES == CRC32C && mode != MODE_RANGE) {   // the row is the codeword: check it first (1EC4ED)
+          uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
+          for (uint32_t j = start; j < end; j++) {
+            const uint32_t c = __ldg(a.col + j);
+            if (j - start < 4) crc_st |= (c >> 24) << (8 * (j - start));
+            crc = ecrc_update(crc, ldg64(a.val + j), c, (int)(j - start));
+          }
+          if (end - start < 4 || (crc ^ 0xFFFFFFFFu) != crc_st)
+            fixed = ecrc_fix(a.val, a.col, start, end - start, mode == MODE_DETECT ? 2 : 1, a.counts, a.due) != DUE;
+        }
         for (uint32_t j = start; j < end; j++) {
-          uint64_t v = ldg64(a.val + j);
-          uint32_t c = __ldg(a.col + j);
-          if (ES == CRC32C) {
-            int kk = (int)(j - start);
-            if (mode != MODE_RANGE) crc = ecrc_update(crc, v, c, kk);
-            if (kk < 4) crc_st |= (c >> 24) << (8 * kk);
-          } else if (ES != NONE && mode != MODE_RANGE) {
+          uint64_t v = fixed ? *(volatile uint64_t*)(a.val + j) : ldg64(a.val + j);
+          uint32_t c = fixed ? *(volatile uint32_t*)(a.col + j) : __ldg(a.col + j);
+          if (ES != NONE && ES != CRC32C && mode != MODE_RANGE) {
             bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
             if (bad) elem_fix<ES>(v, c, a.val + j, a.col + j, a.counts, a.due, mode);
           }
@@ -425,12 +492,6 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
           const int64_t idx = a.col_base + cm;
           const double x = (idx == own) ? p_own : gather_in<VS>(a.in, idx);
           acc = fma(as_d(v), x, acc);
-        }
-        if (ES == CRC32C && mode != MODE_RANGE) {
-          if (end - start < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
-            cnt_add(a.counts, T_ELEM, CRC32C, DUE);
-            *a.due = 1;
-          }
         }
       }
     }
@@ -548,22 +609,35 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
   }
   const uint32_t ckeep = col_keep(ES);
   const int64_t n = a.stencil_n;
-  uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
   const uint32_t len = end - start;
+  bool fixed = false;   // E-CRC row corrected in global memory: read it from there, past the read-only path
+  if (ES == CRC32C && mode != MODE_RANGE) {   // the row is the codeword: check it first (1EC4ED)
+    uint32_t crc = 0xFFFFFFFFu, crc_st = 0;
+    for (uint32_t j = 0; j < len; j++) {
+      const uint64_t v = staged ? sval[start + j - s0] : ldg64(a.val + start + j);
+      const uint32_t c = staged ? scol[start + j - s0] : __ldg(a.col + start + j);
+      if (j < 4) crc_st |= (c >> 24) << (8 * j);
+      crc = ecrc_update(crc, v, c, (int)j);
+    }
+    if (len < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
+      fixed = ecrc_fix(a.val, a.col, start, len, mode == MODE_DETECT ? 2 : 1, a.counts, a.due) != DUE;
+      staged = staged && !fixed;
+    }
+  }
   for (uint32_t j = 0; j < len; j++) {
     uint64_t v;
     uint32_t c;
     if (staged) {
       v = sval[start + j - s0];
       c = scol[start + j - s0];
+    } else if (fixed) {
+      v = *(volatile uint64_t*)(a.val + start + j);
+      c = *(volatile uint32_t*)(a.col + start + j);
     } else {
       v = ldg64(a.val + start + j);
       c = __ldg(a.col + start + j);
     }
-    if (ES == CRC32C) {
-      if (mode != MODE_RANGE) crc = ecrc_update(crc, v, c, (int)j);
-      if (j < 4) crc_st |= (c >> 24) << (8 * j);
-    } else if (ES != NONE && mode != MODE_RANGE) {
+    if (ES != NONE && ES != CRC32C && mode != MODE_RANGE) {
       bool bad = (ES == SED) ? !esed_clean(v, c) : (e96_bad(lo32(v), hi32(v), c) != 0);
       if (bad) elem_fix<ES>(v, c, a.val + start + j, a.col + start + j, a.counts, a.due, mode);
     }
@@ -582,12 +656,6 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
     else if (rel == -n) x = win[oslot - TILE_WW];
     else x = a.fz ? gather_fused<VS>(a.in, a.r_f, a.beta_f, own + rel) : gather_in<VS>(a.in, own + rel);
     acc = fma(as_d(v), x, acc);
-  }
-  if (ES == CRC32C && mode != MODE_RANGE) {
-    if (len < 4 || (crc ^ 0xFFFFFFFFu) != crc_st) {
-      cnt_add(a.counts, T_ELEM, CRC32C, DUE);
-      *a.due = 1;
-    }
   }
   return acc;
 }
@@ -1589,12 +1657,34 @@ __global__ void k_check_rowptr(uint32_t* rowptr, int64_t len, DevCounts* cnt, in
     }
   }
 }
+// rowptr entry idx, its group checked and corrected in registers (a DUE group
+// gives its stored bits), masked.
+template <int RS>
+__device__ uint32_t rp_decoded(const uint32_t* rowptr, int64_t idx, bool detect_only) {
+  constexpr int G = rgrp(RS);
+  uint32_t e[G];
+  const int64_t g0 = idx / G * G;
+#pragma unroll
+  for (int t = 0; t < G; t++) e[t] = rowptr[g0 + t];
+  const uint32_t raw = e[idx - g0];
+  uint32_t w = raw;
+  if (RS != NONE && !detect_only) {   // detection only: a correctable group is a DUE (stored bits)
+    int word = 0;
+    if (rp_check_group<RS>(e, &word) == CORRECTED) {
+#pragma unroll
+      for (int t = 0; t < G; t++) if (t == idx - g0) w = e[t];
+    }
+  }
+  return w & rp_keep(RS);
+}
 // Row pass of check_all: range check + E-CRC rows (after the rowptr pass scrubbed).
 template <int ES, int RS>
-__global__ void k_check_rows(const uint64_t* val, const uint32_t* col, const uint32_t* rowptr, int64_t nrows,
-                             int64_t nnz, DevCounts* cnt, int* due) {
+__global__ void k_check_rows(uint64_t* val, uint32_t* col, const uint32_t* rowptr, int64_t nrows,
+                             int64_t nnz, int64_t ncols, DevCounts* cnt, int* due, int scrub) {
   for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < nrows; i += (int64_t)gridDim.x * blockDim.x) {
-    uint32_t s = rowptr[i] & rp_keep(RS), t = rowptr[i + 1] & rp_keep(RS);
+    // decoded entries (corrected in registers, not counted: the rowptr pass
+    // counts), so count-only sweeps see the same ranges as scrubbing ones
+    const uint32_t s = rp_decoded<RS>(rowptr, i, scrub == 2), t = rp_decoded<RS>(rowptr, i + 1, scrub == 2);
     if (!(s <= t && (int64_t)t <= nnz)) {
       if (RS != NONE) { cnt_range(cnt, T_ROWPTR, RS); *due = 1; }
       continue;
@@ -1610,7 +1700,16 @@ __global__ void k_check_rows(const uint64_t* val, const uint32_t* col, const uin
         }
         bad = (crc ^ 0xFFFFFFFFu) != st;
       }
-      if (bad) { cnt_add(cnt, T_ELEM, CRC32C, DUE); *due = 1; }
+      // scrub: 0 count only, 1 count + correct in place, 2 detection only
+      uint32_t* fa = nullptr;
+      int fb = 0;
+      if (bad) ecrc_fix(val, col, s, t - s, scrub == 1 ? 1 : scrub == 2 ? 2 : 0, cnt, due, &fa, &fb);
+      // the row is the codeword: range-check its columns as decoded by it
+      for (uint32_t j = s; j < t; j++) {
+        uint32_t c = *(volatile uint32_t*)(col + j);
+        if (fa == col + j && scrub == 0) c ^= 1u << fb;
+        if ((int64_t)(c & 0x00FFFFFFu) >= ncols) { cnt_range(cnt, T_ELEM, CRC32C); *due = 1; }
+      }
     }
   }
 }
