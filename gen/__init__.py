@@ -7,3 +7,4 @@ schedules from a counter-based splitmix64.
 """
 from .tealeaf import (tealeaf_csr, tealeaf_rhs, const_k_csr, strip_csr, splitmix64, uniform_pm1, chunk_plan, chunk_csr,  # noqa: F401,E501
                       fault_positions)
+from .spd import random_spd_csr  # noqa: F401,E402
