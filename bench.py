@@ -88,6 +88,25 @@ class ClockSampler:
 
 
 # ------------------------------------------------------------------ problem
+def chunk_layout(grid: int, rank: int, world: int, chunk_rows=None):
+    """This rank's row-block chunks (no arrays): global grid rows, row_base /
+    col_base in the rank's halo-extended vector, rows and column-window width
+    (<= 2^24 for the 24-bit element index, reading R7)."""
+    import gen
+    n = grid
+    y0r, y1r = rank * grid, (rank + 1) * grid
+    halo = n if world > 1 else 0
+    out = []
+    for (c0, c1, cb) in gen.chunk_plan(n, y1r - y0r, chunk_rows=chunk_rows, halo=world > 1):
+        # local grid rows [c0, c1) of this rank's strip; vector index = halo + local row index
+        row_base = halo + c0 * n
+        col_base = max(0, row_base - n) if world > 1 or c0 > 0 else 0
+        ncols = min(halo + (y1r - y0r) * n + halo, row_base + (c1 - c0) * n + n) - col_base
+        out.append(dict(gy0=y0r + c0, gy1=y0r + c1, row_base=row_base, col_base=col_base, nrows=(c1 - c0) * n,
+                        ncols=ncols))
+    return out
+
+
 def build_problem(grid: int, rank: int, world: int, device, chunk_rows=None):
     """Raw (unencoded) device arrays of this rank's rows, as row-block chunks
     whose column windows fit the 24-bit element index (reading R7)."""
@@ -98,16 +117,12 @@ def build_problem(grid: int, rank: int, world: int, device, chunk_rows=None):
     y0r, y1r = rank * grid, (rank + 1) * grid
     halo = n if world > 1 else 0
     chunks = []
-    for (c0, c1, cb) in gen.chunk_plan(n, y1r - y0r, chunk_rows=chunk_rows):
-        # local grid rows [c0, c1) of this rank's strip; vector index = halo + local row index
-        gy0, gy1 = y0r + c0, y0r + c1
-        row_base = halo + c0 * n
-        col_base = max(0, row_base - n) if world > 1 or c0 > 0 else 0
-        val, col, rowptr = gen.strip_csr(n, gy0, gy1, ny=ny, device=device, col_offset=row_base - col_base)
-        ncols = min(halo + (y1r - y0r) * n + halo, row_base + (c1 - c0) * n + n) - col_base
+    for L in chunk_layout(grid, rank, world, chunk_rows):
+        val, col, rowptr = gen.strip_csr(n, L["gy0"], L["gy1"], ny=ny, device=device,
+                                         col_offset=L["row_base"] - L["col_base"])
         chunks.append(dict(val=val.contiguous(), col=col.to(torch.int32).contiguous(),
-                           rowptr=rowptr.to(torch.int32).contiguous(), row_base=row_base, col_base=col_base,
-                           nrows=(c1 - c0) * n, ncols=ncols))
+                           rowptr=rowptr.to(torch.int32).contiguous(), row_base=L["row_base"],
+                           col_base=L["col_base"], nrows=L["nrows"], ncols=L["ncols"]))
     b = gen.tealeaf_rhs(n, y0r, y1r, ny=ny, device=device)
     N = (y1r - y0r) * n
     return dict(chunks=chunks, b=b.contiguous(), N=N, n=n, halo=halo)

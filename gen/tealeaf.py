@@ -166,10 +166,13 @@ def fault_positions(seed: int, count: int, nbits_total: int) -> np.ndarray:
     return (r % np.uint64(nbits_total)).astype(np.int64)
 
 
-def chunk_plan(n: int, ny: int | None = None, max_cols: int = 1 << 24, chunk_rows: int | None = None):
+def chunk_plan(n: int, ny: int | None = None, max_cols: int = 1 << 24, chunk_rows: int | None = None,
+               halo: bool = False):
     """Row-block chunks (reading R7 / S§8(c) O11) of an n x ny grid so that each
     chunk's column window [(y0-1)*n, (y1+1)*n) fits the 24-bit element index and
-    its nnz fits 28-bit rowptr entries.  Returns [(y0, y1, col_base)]."""
+    its nnz fits 28-bit rowptr entries.  Returns [(y0, y1, col_base)].
+    halo=True: the grid is one rank's strip of a larger grid (multi-GPU), so
+    ghost rows exist above and below every chunk, also at the strip's edges."""
     ny = n if ny is None else ny
 
     def plan(rows):
@@ -180,15 +183,20 @@ def chunk_plan(n: int, ny: int | None = None, max_cols: int = 1 << 24, chunk_row
         return out
 
     def fits(pl):
-        return all((min(ny, y1 + 1) * n - cb) <= max_cols and 5 * (y1 - y0) * n <= (1 << 28) - 1
-                   for (y0, y1, cb) in pl)
+        def window(y0, y1, cb):
+            return (y1 - y0 + 2) * n if halo else min(ny, y1 + 1) * n - cb
+        return all(window(y0, y1, cb) <= max_cols and 5 * (y1 - y0) * n <= (1 << 28) - 1 for (y0, y1, cb) in pl)
 
     if chunk_rows is not None:
         return plan(chunk_rows)
-    rows = ny
-    while not fits(plan(rows)):
-        rows //= 2
-    return plan(rows)
+    # fewest chunks: an even split into multiples of 8 grid rows (the SpMV tile
+    # height), so the chunked SpMV pays the fewest launch tails
+    for k in range(1, ny + 1):
+        rows = -(-ny // k)
+        rows = min(ny, -(-rows // 8) * 8)
+        if fits(plan(rows)):
+            return plan(rows)
+    return plan(1)
 
 
 def chunk_csr(n: int, y0: int, y1: int, col_base: int, ny: int | None = None, device="cpu", kind: str = "tea"):
