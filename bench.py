@@ -317,6 +317,7 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--fuse", action="store_true", help="main line on the fused calc_p path (DESIGN.md §6.1)")
+    ap.add_argument("--no-pdl", action="store_true", help="plain launches in the CG loop (DESIGN.md §6.2)")
     ap.add_argument("--no-fused-extra", action="store_true", help="skip the fused-calc_p side measurement")
     args = ap.parse_args()
     if args.impl == "reference":
@@ -338,6 +339,7 @@ def main():
     # fused calc_p (opt-in) runs on the single-GPU tiled path (the dist path exchanges p halos unfused)
     fused = args.fuse and not dist_on
     ctx.set_fused_cg(fused)
+    ctx.set_pdl(not args.no_pdl)
     spmv_bpr = FUSED_SPMV_BYTES_PER_ROW if fused else SPMV_BYTES_PER_ROW
     cg_bpr = FUSED_CG_BYTES_PER_ROW if fused else CG_BYTES_PER_ROW
     dobj = abft.Dist(rank, world, local) if dist_on else None
@@ -428,7 +430,7 @@ def main():
                    "tol": args.tol, "iters_per_step": r_p["iters"] / args.steps,
                    "l2": "inputs larger than L2 (2.55 GB moved per CG iteration vs 126 MB L2)",
                    "parallelism": f"row-block strips x{world}" if world > 1 else "single GPU",
-                   "fused_calc_p": fused, "bytes_per_row_per_iter": cg_bpr},
+                   "fused_calc_p": fused, "pdl": not args.no_pdl and not dist_on, "bytes_per_row_per_iter": cg_bpr},
         "roofline": {"bound": "hbm",
                      "kernel": "k_spmv_tile (fused calc_p + protected SpMV + p.w)" if fused
                      else "k_spmv_tile (protected SpMV + p.w)",

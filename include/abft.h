@@ -83,6 +83,12 @@ int abft_ctx_destroy(abft_ctx* ctx);
  * iteration.  The context then owns a second p buffer (padded length of p).
  * enable = 0 runs the unfused sequence. */
 int abft_ctx_set_fused_cg(abft_ctx* ctx, int enable);
+/* Programmatic dependent launch between the kernels of abft_cg_solve's
+ * iterations (default on, single GPU): each kernel issues its
+ * loads of data the previous kernel does not write (the matrix, vectors from
+ * two kernels back) before waiting on it, hiding launch gaps and tails.
+ * Results are identical either way. */
+int abft_ctx_set_pdl(abft_ctx* ctx, int enable);
 
 int64_t abft_rowptr_padded_len(int64_t nrows, int32_t scheme);  /* pad with copies of nnz (R6) */
 int64_t abft_vec_padded_len(int64_t n, int32_t scheme);         /* pad with encoded +0.0 */

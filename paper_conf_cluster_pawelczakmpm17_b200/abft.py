@@ -49,6 +49,7 @@ _sig = {
     "abft_ctx_create": (C.c_int, [C.c_int, C.POINTER(C.c_void_p)]),
     "abft_ctx_destroy": (C.c_int, [_P]),
     "abft_ctx_set_fused_cg": (C.c_int, [_P, C.c_int]),
+    "abft_ctx_set_pdl": (C.c_int, [_P, C.c_int]),
     "abft_rowptr_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
     "abft_vec_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
     "abft_csr_encode": (C.c_int, [_P, C.POINTER(CSR), _P]),
@@ -150,6 +151,10 @@ class Context:
     def set_fused_cg(self, enable: bool):
         """Fused calc_p in the CG's SpMV (abft_ctx_set_fused_cg; default off)."""
         _check(_lib.abft_ctx_set_fused_cg(self.h, 1 if enable else 0), "abft_ctx_set_fused_cg")
+
+    def set_pdl(self, enable: bool):
+        """Programmatic dependent launch in the CG loop (abft_ctx_set_pdl; default on)."""
+        _check(_lib.abft_ctx_set_pdl(self.h, 1 if enable else 0), "abft_ctx_set_pdl")
 
     def close(self):
         if self.h:

@@ -59,6 +59,7 @@ struct abft_ctx {
   RedState* red = nullptr;   // fused-reduction counters/roots (zero between reductions)
   CrcTables* crc = nullptr;  // CRC32C lookup tables (device)
   bool fuse_p = false;       // fused calc_p in the CG's SpMV when eligible (opt-in)
+  bool pdl = true;           // programmatic dependent launch between the CG iteration kernels (§6.2)
   uint64_t* p_alt = nullptr; // second p buffer of the fused CG
   int64_t p_alt_len = 0;
 };
@@ -198,6 +199,12 @@ int abft_ctx_create(int device, abft_ctx** out) {
   int e = ensure_partials(c, 1024);
   if (e) return e;
   *out = c;
+  return ABFT_OK;
+}
+
+int abft_ctx_set_pdl(abft_ctx* c, int enable) {
+  if (!c) return fail(ABFT_E_INVALID, "null ctx");
+  c->pdl = enable != 0;
   return ABFT_OK;
 }
 
@@ -504,8 +511,16 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   int poll = opts->poll_every > 0 ? opts->poll_every : 16;
   if (fused && (poll & 1)) poll += 1;  // graph replays then always start at an odd iteration (buffer parity)
   int64_t launched = 0;  // iterations issued so far (host); = device iterations until a stop
+  // PDL between the iteration kernels (single GPU: the multi-GPU loop has NCCL
+  // kernels in between); off again on every exit from this function
+  struct PdlGuard {
+    explicit PdlGuard(bool on) { set_pdl(on); }
+    ~PdlGuard() { set_pdl(false); }
+  };
+  const bool pdl_on = ctx->pdl && !multi;
   // k iterations of (a3)..(a5) + the DUE/convergence logic, all device-side
   auto issue = [&](int64_t k, cudaStream_t s) -> int {
+    PdlGuard pg(pdl_on);
     prof.s = s;
     for (int64_t it = 0; it < k; it++) {
       int e2;

@@ -96,6 +96,8 @@ struct VecArgs {
   const CrcTables* crc;   // device tables (CRC32C schemes only)
 };
 
+// PDL for the CG driver's iteration launches
+void set_pdl(bool on);
 // launchers (kernels.cu); each returns the number of kernels launched
 int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, bool dot, cudaStream_t s);
 // -1: a fused-calc_p launch (a.p_cur set) could not run

@@ -21,6 +21,9 @@
 
 namespace abft {
 
+bool g_pdl = false;
+void set_pdl(bool on) { g_pdl = on; }
+
 // per-ES SpMV launchers live in spmv_es*.cu (parallel compilation)
 bool spmv_es_none(const SpmvArgs&, int, int, bool, cudaStream_t);
 bool spmv_es_sed(const SpmvArgs&, int, int, bool, cudaStream_t);
@@ -86,11 +89,11 @@ int launch_calc_ur(const VecArgs& a, int vs, cudaStream_t s) {
   if (a.n <= 0) return 0;
   int nb = blocks_rb(a.n);
   switch (vs) {
-    case NONE: k_calc_ur<NONE><<<nb, 256, 0, s>>>(a); break;
-    case SED: k_calc_ur<SED><<<nb, 256, 0, s>>>(a); break;
-    case SECDED64: k_calc_ur<SECDED64><<<nb, 256, 0, s>>>(a); break;
-    case SECDED128: k_calc_ur<SECDED128><<<nb, 256, 0, s>>>(a); break;
-    default: k_calc_ur<CRC32C><<<nb, 256, vec_dyn_smem<CRC32C>(), s>>>(a); break;
+    case NONE: launch_k(k_calc_ur<NONE>, nb, 256, 0, s, a); break;
+    case SED: launch_k(k_calc_ur<SED>, nb, 256, 0, s, a); break;
+    case SECDED64: launch_k(k_calc_ur<SECDED64>, nb, 256, 0, s, a); break;
+    case SECDED128: launch_k(k_calc_ur<SECDED128>, nb, 256, 0, s, a); break;
+    default: launch_k(k_calc_ur<CRC32C>, nb, 256, vec_dyn_smem<CRC32C>(), s, a); break;
   }
   return 1;
 }
@@ -98,11 +101,11 @@ int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s) {
   if (a.n <= 0) return 0;
   int nb = blocks_rb(a.n);
   switch (vs) {
-    case NONE: k_calc_p<NONE><<<nb, 256, 0, s>>>(a); break;
-    case SED: k_calc_p<SED><<<nb, 256, 0, s>>>(a); break;
-    case SECDED64: k_calc_p<SECDED64><<<nb, 256, 0, s>>>(a); break;
-    case SECDED128: k_calc_p<SECDED128><<<nb, 256, 0, s>>>(a); break;
-    default: k_calc_p<CRC32C><<<nb, 256, vec_dyn_smem<CRC32C>(), s>>>(a); break;
+    case NONE: launch_k(k_calc_p<NONE>, nb, 256, 0, s, a); break;
+    case SED: launch_k(k_calc_p<SED>, nb, 256, 0, s, a); break;
+    case SECDED64: launch_k(k_calc_p<SECDED64>, nb, 256, 0, s, a); break;
+    case SECDED128: launch_k(k_calc_p<SECDED128>, nb, 256, 0, s, a); break;
+    default: launch_k(k_calc_p<CRC32C>, nb, 256, vec_dyn_smem<CRC32C>(), s, a); break;
   }
   return 1;
 }
@@ -148,7 +151,7 @@ int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* 
   while (p2 < nrb) p2 <<= 1;
   int64_t leaves = p2 < 1024 ? p2 : 1024;
   int blocks = (int)(p2 / leaves);
-  k_reduce<<<blocks, 256, 0, s>>>(partials, nrb, leaves, roots, ticket, op, st, out, due);
+  launch_k(k_reduce, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, op, st, out, due);
   return 1;
 }
 

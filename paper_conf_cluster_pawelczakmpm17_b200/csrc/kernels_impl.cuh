@@ -10,6 +10,28 @@
 
 namespace abft {
 
+// Host: launch k with the programmatic-stream-serialization attribute when the
+// CG driver turned PDL on (set_pdl), else a plain launch.
+extern bool g_pdl;
+template <typename... KArgs, typename... Args>
+static inline void launch_k(void (*k)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t s, Args... args) {
+  if (!g_pdl) {
+    k<<<grid, block, smem, s>>>(args...);
+    return;
+  }
+  cudaLaunchConfig_t cfg{};
+  cfg.gridDim = grid;
+  cfg.blockDim = block;
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+  at[0].val.programmaticStreamSerializationAllowed = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  cudaLaunchKernelEx(&cfg, k, args...);
+}
+
 // --------------------------------------------------------------- helpers
 __host__ __device__ constexpr int vgrp(int s) { return s == SECDED128 ? 2 : s == CRC32C ? 4 : 1; }
 __host__ __device__ constexpr int rgrp(int s) { return s == SECDED64 ? 2 : s == SECDED128 ? 4 : s == CRC32C ? 8 : 1; }
@@ -23,6 +45,13 @@ static __device__ __forceinline__ uint64_t shfl64(uint64_t v, int src) {
   uint32_t hi = __shfl_sync(0xffffffffu, (uint32_t)(v >> 32), src);
   return mk64(lo, hi);
 }
+// Programmatic dependent launch (PDL): everything before
+// pdl_wait() may only read data no kernel of the previous two launches writes
+// (the matrix; vectors last written >= 2 kernels earlier); pdl_trigger() comes
+// right after the wait, so a kernel's pre-wait part overlaps only its direct
+// predecessor.  Both are no-ops for launches without the PDL attribute.
+static __device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+static __device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
 static __device__ __forceinline__ uint64_t ldg64(const uint64_t* p) { return (uint64_t)__ldg((const unsigned long long*)p); }
 
 static __device__ __forceinline__ void cnt_add(DevCounts* c, int t, int s, int o) {
@@ -438,6 +467,8 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
   __shared__ uint32_t s_rp[8][40];
   if (VS == SECDED64) load_lut(s_lut);
   __syncthreads();
+  pdl_wait();
+  pdl_trigger();
   if (a.state && a.state->stop) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
@@ -748,18 +779,9 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   const int64_t tiles_x = n >> 8;
   const int64_t tx0 = (blockIdx.x % tiles_x) << 8;
   const int64_t ty0 = (int64_t)(blockIdx.x / tiles_x) * TILE_TY;
-  // ---- 0. producer: barriers, then the first TILE_NST passes in flight
-  // fused calc_p (DESIGN.md §6.1): iteration 1 multiplies by p_cur as init
-  // wrote it; later iterations build p_cur from (in = p_{k-1}, r) in the window
-  const bool fz = FUSED && a.state->iters > 0;
-  uint64_t* const pin = (FUSED && !fz) ? a.p_cur : a.in;
+  // ---- 0. producer: barriers, then the first TILE_NST passes in flight (the
+  // matrix: loaded before the PDL grid dependency resolves)
   if (threadIdx.x == 0) {
-    s_args = a;
-    if (FUSED) {
-      s_args.in = pin;
-      s_args.fz = fz ? 1 : 0;
-      s_args.beta_f = fz ? a.state->beta : 0.0;
-    }
 #pragma unroll
     for (int s = 0; s < TILE_NST; s++) {
       mbar_init(&full[s], 1);
@@ -772,19 +794,17 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   if (VS == SECDED64) load_lut(s_lut);
   if (SLICE) smem_fill(s_slice, &a.crc->slice[0][0], CRC_SLICE_WORDS);
   if (VS == CRC32C) smem_fill(reinterpret_cast<uint32_t*>(s_vpos), &a.crc->vpos[0][0][0], CRC_VPOS_WORDS);
-  if (SLICE || VS == CRC32C) __syncthreads();
   const uint8_t* cs = (VS == CRC32C) ? s_vpos : s_lut;   // vector codec tables
-  const int stop_v = a.state ? a.state->stop : 0;  // checked after the prologue loads are in flight
-  const int mode = spmv_mode(a);
   const int64_t gy = ty0 + warp;
   const bool has_seg = gy < ny;
   const int64_t rowseg = gy * n + tx0;
-  // ---- 1. rowptr of the segment (entries rowseg .. rowseg+256)
+  // ---- 1. rowptr of the segment (entries rowseg .. rowseg+256): loads first
+  // (matrix, before the grid dependency), checks after it
+  constexpr int G = rgrp(RS);
+  constexpr int NG = 256 / G + 1;
+  constexpr int PER = (NG + 31) / 32;
+  uint32_t e[PER][G];
   if (has_seg) {
-    constexpr int G = rgrp(RS);
-    constexpr int NG = 256 / G + 1;
-    constexpr int PER = (NG + 31) / 32;
-    uint32_t e[PER][G];
 #pragma unroll
     for (int q = 0; q < PER; q++) {  // all loads first (latency overlapped)
       const int gl = lane + 32 * q;
@@ -801,6 +821,25 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
         }
       }
     }
+  }
+  pdl_wait();   // the previous kernel's writes (p / r, CG state, counters) are visible from here
+  pdl_trigger();
+  // fused calc_p (DESIGN.md §6.1): iteration 1 multiplies by p_cur as init
+  // wrote it; later iterations build p_cur from (in = p_{k-1}, r) in the window
+  const bool fz = FUSED && a.state->iters > 0;
+  uint64_t* const pin = (FUSED && !fz) ? a.p_cur : a.in;
+  if (threadIdx.x == 0) {
+    s_args = a;
+    if (FUSED) {
+      s_args.in = pin;
+      s_args.fz = fz ? 1 : 0;
+      s_args.beta_f = fz ? a.state->beta : 0.0;
+    }
+  }
+  if (SLICE || VS == CRC32C) __syncthreads();
+  const int stop_v = a.state ? a.state->stop : 0;
+  const int mode = spmv_mode(a);
+  if (has_seg) {
     if (!stop_v) {
       uint32_t acc = 0;
       if (mode != MODE_RANGE) {
@@ -1225,6 +1264,8 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 3 : 4) k_calc_ur(VecArgs a
   UrStep<VS> s0{};
   if (full)  // issue step 0 first: its latency overlaps the state loads and the barrier
     ur_load<VS>(a.x + rb * 256 + lane, a.p + rb * 256 + lane, a.r + rb * 256 + lane, a.w + rb * 256 + lane, 0, s0);
+  pdl_wait();   // alpha / stop from the pw reduction
+  pdl_trigger();
   const int stop = a.state->stop;
   const double alpha = a.state->alpha;
   const uint8_t* cs = vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
@@ -1272,6 +1313,8 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : 6) k_calc_p(VecArgs a)
     const uint64_t* P = a.p + rb * 256 + lane;
     r0 = ldg64(R); r1 = ldg64(R + 32); p0 = ldg64(P); p1 = ldg64(P + 32);
   }
+  pdl_wait();   // beta / stop from the rrn reduction
+  pdl_trigger();
   const int stop = a.state->stop;
   const double beta = a.state->beta;
   const uint8_t* cs = vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
@@ -1461,6 +1504,8 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
   // warp roots; the last block (ticket) combines the block roots.
   __shared__ double s_w[8];
   __shared__ bool s_last;
+  pdl_wait();   // partials of the producing kernel
+  pdl_trigger();
   if (st && op != 1 && st->stop) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t base = (int64_t)blockIdx.x * leaves;

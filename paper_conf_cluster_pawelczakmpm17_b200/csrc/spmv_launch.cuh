@@ -60,7 +60,7 @@ static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   }
   const int64_t ny = a.nrows / a.stencil_n;
   const int64_t blocks = (a.stencil_n / 256) * ((ny + TILE_TY - 1) / TILE_TY);
-  k_spmv_tile<ES, RS, VS, DOT, FUSED><<<(unsigned)blocks, 256, smem, s>>>(a, tm);
+  launch_k(k_spmv_tile<ES, RS, VS, DOT, FUSED>, (unsigned)blocks, 256, smem, s, a, tm);
   return true;
 }
 // Returns false only when a fused-calc_p launch (a.p_cur set) was requested
@@ -78,8 +78,8 @@ static bool spmv3(const SpmvArgs& a, bool dot, cudaStream_t s) {
   }
   const int64_t nrb = (a.nrows + 255) / 256;
   const int blocks = (int)((nrb + 7) / 8);
-  if (dot) k_spmv<ES, RS, VS, true><<<blocks, 256, 0, s>>>(a);
-  else k_spmv<ES, RS, VS, false><<<blocks, 256, 0, s>>>(a);
+  if (dot) launch_k(k_spmv<ES, RS, VS, true>, blocks, 256, 0, s, a);
+  else launch_k(k_spmv<ES, RS, VS, false>, blocks, 256, 0, s, a);
   return true;
 }
 template <int ES, int RS>
