@@ -59,7 +59,7 @@ struct abft_ctx {
   RedState* red = nullptr;   // fused-reduction counters/roots (zero between reductions)
   CrcTables* crc = nullptr;  // CRC32C lookup tables (device)
   bool fuse_p = false;       // fused calc_p in the CG's SpMV when eligible (opt-in)
-  bool pdl = true;           // programmatic dependent launch between the CG iteration kernels (§6.2)
+  bool pdl = false;          // programmatic dependent launch between the CG iteration kernels (opt-in, §6.2)
   uint64_t* p_alt = nullptr; // second p buffer of the fused CG
   int64_t p_alt_len = 0;
 };
