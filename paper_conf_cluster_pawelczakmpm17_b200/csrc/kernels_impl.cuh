@@ -854,25 +854,28 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
           if (gl >= NG) continue;
           const int64_t g = rowseg / G + gl;
           uint32_t* gp = a.rowptr + g * G;
-          uint32_t o0[G];
+          // the codec works on a copy: taking e[q]'s address would put the whole
+          // e[][] array (the hot prologue's rowptr loads) in local memory
+          uint32_t c[G];
 #pragma unroll
-          for (int t = 0; t < G; t++) o0[t] = e[q][t];
+          for (int t = 0; t < G; t++) c[t] = e[q][t];
           int word = 0;
-          int o = rp_check_group<RS>(e[q], &word);
+          int o = rp_check_group<RS>(c, &word);
           if (o == CORRECTED && mode == MODE_DETECT) o = DUE;   // interval mode: detection only
           if (o != CLEAN) {
             const int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
             const bool owner = own >= rowseg && own < rowseg + 256;
             if (o == CORRECTED) {
-              uint32_t ow = 0, nw = 0;   // select, not index: keeps e[][] out of local memory
+              uint32_t ow = 0, nw = 0;   // select, not index
 #pragma unroll
               for (int t = 0; t < G; t++)
-                if (t == word) { ow = o0[t]; nw = e[q][t]; }
+                if (t == word) { ow = e[q][t]; nw = c[t]; }
               if (owner && scrub32(gp + word, ow, nw)) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
-            } else {
 #pragma unroll
-              for (int t = 0; t < G; t++) e[q][t] = o0[t];
-              if (owner) { cnt_add(a.counts, T_ROWPTR, RS, DUE); *a.due = 1; }
+              for (int t = 0; t < G; t++) e[q][t] = c[t];
+            } else if (owner) {   // DUE: e keeps the stored bits
+              cnt_add(a.counts, T_ROWPTR, RS, DUE);
+              *a.due = 1;
             }
           }
         }
@@ -1255,7 +1258,13 @@ __device__ __forceinline__ const uint8_t* vec_codec_smem(uint8_t* s_lut, uint8_t
 }
 
 template <int VS>
-__global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 3 : 4) k_calc_ur(VecArgs a) {
+#ifndef ABFT_UR_MINB
+#define ABFT_UR_MINB 5
+#endif
+#ifndef ABFT_P_MINB
+#define ABFT_P_MINB 6
+#endif
+__global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 3 : ABFT_UR_MINB) k_calc_ur(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
   extern __shared__ __align__(16) uint8_t s_dyn_v[];
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -1300,7 +1309,7 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 3 : 4) k_calc_ur(VecArgs a
 }
 
 template <int VS>
-__global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : 6) k_calc_p(VecArgs a) {
+__global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : ABFT_P_MINB) k_calc_p(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
   extern __shared__ __align__(16) uint8_t s_dyn_v[];
   __shared__ bool s_last;
