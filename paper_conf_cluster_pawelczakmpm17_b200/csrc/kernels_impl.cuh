@@ -567,15 +567,21 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
 //     gathers neighbours from the window whenever col-row is one of {0, +-1,
 //     +-n} (anything else takes the global gather path, so results never
 //     depend on the stencil hint), encodes w, and releases the stage.
-struct TileMaps { CUtensorMap val, col; };
+// val / col element streams ([ny][5n] boxes); vin / vcur: the SpMV input
+// vector (and the fused path's p_cur) viewed as [rows][n/2][2] doubles, one
+// box = the tile's decoded-window rows (has_vmaps = 0: not built)
+struct TileMaps { CUtensorMap val, col, vin, vcur; int has_vmaps; };
 
 constexpr int TILE_TY = 8;
-constexpr int TILE_WW = 256 + 2;
+// window row: x = tx0-2 .. tx0+257 (one TMA box of 130 double pairs); the
+// tile's own cells sit at slots TILE_WX0 .. TILE_WX0+255
+constexpr int TILE_WX0 = 2;
+constexpr int TILE_WW = 256 + 4;
 constexpr int TILE_PE = 160;                                   // elements per warp per pass (32 rows x 5)
 constexpr int TILE_NST = 3;                                    // pipeline stages
 constexpr int TILE_STAGE_VAL = TILE_TY * TILE_PE * 8;          // 10240
 constexpr int TILE_STAGE = TILE_STAGE_VAL + TILE_TY * TILE_PE * 4;   // + 5120
-constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 20640
+constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 20800
 constexpr int TILE_RP = 264;                                   // rowptr entries staged per warp
 constexpr int TILE_OFF_WIN = TILE_NST * TILE_STAGE;            // stages first (128-B aligned)
 constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
@@ -610,6 +616,13 @@ static __device__ __forceinline__ void tma_2d(void* dst, const CUtensorMap* map,
       "cp.async.bulk.tensor.2d.shared::cluster.global.tile.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], [%4];" ::"r"(
           smem_u32(dst)),
       "l"(reinterpret_cast<uint64_t>(map)), "r"(x), "r"(y), "r"(smem_u32(bar))
+      : "memory");
+}
+static __device__ __forceinline__ void tma_3d(void* dst, const CUtensorMap* map, int x, int y, int z, uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3, %4}], [%5];" ::"r"(
+          smem_u32(dst)),
+      "l"(reinterpret_cast<uint64_t>(map)), "r"(x), "r"(y), "r"(z), "r"(smem_u32(bar))
       : "memory");
 }
 // Producer: the element boxes of pass k of the tile (tx0, ty0) into stage buffer `stage`.
@@ -769,6 +782,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   double* s_win = reinterpret_cast<double*>(s_dyn + TILE_OFF_WIN);
   uint64_t* full = reinterpret_cast<uint64_t*>(s_dyn + TILE_OFF_BAR);
   uint64_t* empty = full + TILE_NST;
+  uint64_t* winbar = empty + TILE_NST;   // the TMA-staged `in` window
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   uint32_t* srp = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_RP) + warp * TILE_RP;
   constexpr bool SLICE = (ES == CRC32C || RS == CRC32C);
@@ -787,6 +801,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       mbar_init(&full[s], 1);
       mbar_init(&empty[s], TILE_TY);
     }
+    mbar_init(winbar, 1);
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
 #pragma unroll
     for (int k = 0; k < TILE_NST; k++) tile_produce(tm, s_dyn + k * TILE_STAGE, &full[k], tx0, ty0, k);
@@ -839,6 +854,13 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
   if (SLICE || VS == CRC32C) __syncthreads();
   const int stop_v = a.state ? a.state->stop : 0;
   const int mode = spmv_mode(a);
+  // G = 1, not building p_k: the raw `in` window arrives by one TMA box
+  // (out-of-range rows / columns zero-filled = encoded +0.0) and is decoded in place
+  const bool tma_win = vgrp(VS) == 1 && !(FUSED && fz) && tm.has_vmaps;
+  if (tma_win && !stop_v && threadIdx.x == 0) {
+    mbar_expect_tx(winbar, TILE_WIN_BYTES);
+    tma_3d(s_win, (FUSED && !fz) ? &tm.vcur : &tm.vin, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 - 1), winbar);
+  }
   if (has_seg) {
     if (!stop_v) {
       uint32_t acc = 0;
@@ -894,13 +916,47 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       for (int s = 0; s < TILE_NST; s++) mbar_wait(&full[s], 0u);
     return;
   }
-  // ---- 2. decoded `in` window
-  const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - 1;   // in-index of slot (0,0)
-  constexpr int WPER = (TILE_WW + 31) / 32;                      // 9 slots per lane per window row
+  // ---- 2. decoded `in` window: rows ty0-1 .. ty0+TILE_TY, x = tx0-2 .. tx0+257
+  const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - TILE_WX0;   // in-index of slot (0,0)
+  constexpr int WPER = (TILE_WW + 31) / 32;                             // 9 slots per lane per window row
   constexpr int VG = vgrp(VS);
-  if (VG > 1) {  // G = 2 / 4: load aligned groups (win0 = -1 mod 256), lane-split fast check
+  if (tma_win) {
+    mbar_wait(winbar, 0);
+    // every codeword of the tile is checked ONCE here (owner: counted + scrubbed),
+    // halo codewords are checked without counting
+    constexpr int WS = (TILE_TY + 2) * TILE_WW;
+    const uint64_t* raw = reinterpret_cast<const uint64_t*>(s_win);
+    for (int sl = threadIdx.x; sl < WS; sl += 256) {
+      uint64_t w = raw[sl];
+      const bool bad = (VS == SED) ? !vsed_clean(w) : (VS == SECDED64) ? (v64_bad(lo32(w), hi32(w)) != 0u) : false;
+      if (VS != NONE && bad) {   // cold: only real codewords fail (zero fill is clean)
+        const int wy = sl / TILE_WW, j = sl - wy * TILE_WW;
+        const int64_t idx = win0 + (int64_t)wy * n + j;
+        const bool owner = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny && j >= TILE_WX0 && j < TILE_WX0 + 256;
+        w = v1_check<VS>(w, pin + idx, owner, a.counts, a.due);
+      }
+      s_win[sl] = as_d(w & vkeep(VS));
+    }
+    // grid-edge tiles: the x = -1 / x = n slots hold the linearly adjacent
+    // entries (in-index +-1: the previous row's last / next row's first cell),
+    // as the plain gather in[col] would read them for a column i -+ 1
+    const bool eL = tx0 == 0, eR = tx0 + 256 == n;
+    if (eL || eR) {
+      __syncthreads();
+      const int t = threadIdx.x;
+      int wy = -1, j = 0;
+      if (eL && t < TILE_TY + 2) { wy = t; j = TILE_WX0 - 1; }
+      else if (eR && t >= 32 && t < 32 + TILE_TY + 2) { wy = t - 32; j = TILE_WX0 + 256; }
+      if (wy >= 0) {
+        const int64_t idx = win0 + (int64_t)wy * n + j;
+        const uint64_t w = (idx >= 0 && idx < a.npad_in) ? v1_check<VS>(ldg64(pin + idx), pin + idx, false, a.counts, a.due)
+                                                         : 0ull;
+        s_win[wy * TILE_WW + j] = as_d(w & vkeep(VS));
+      }
+    }
+  } else if (VG > 1) {  // G = 2 / 4: load aligned groups (lane 0 at tx0 - G), lane-split fast check
     for (int wy = warp; wy < TILE_TY + 2; wy += 8) {
-      const int64_t a0 = win0 + (int64_t)wy * n - (VG - 1);      // in-index of lane 0's word, aligned to G
+      const int64_t a0 = win0 + (int64_t)wy * n + TILE_WX0 - VG;     // in-index of lane 0's word, aligned to G
       const bool row_own = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny;
       double* dst = s_win + wy * TILE_WW;
       uint64_t wv[WPER];
@@ -927,15 +983,15 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       if (__any_sync(0xffffffffu, bad)) {   // cold: locate / correct per group (owner counts + scrubs)
 #pragma unroll 1
         for (int q = 0; q < WPER; q++) {
-          const int slot = 32 * q + lane - (VG - 1);
-          const bool owner = row_own && slot >= 1 && slot <= 256;   // groups never straddle the tile edge
+          const int slot = 32 * q + lane + TILE_WX0 - VG;
+          const bool owner = row_own && slot >= TILE_WX0 && slot < TILE_WX0 + 256;   // groups never straddle the tile edge
           wv[q] = vg_check<VS>(wv[q], pin + (a0 + 32 * q + (lane & ~(VG - 1))), lane, ok[q], owner && ok[q],
                                a.counts, a.due);
         }
       }
 #pragma unroll
       for (int q = 0; q < WPER; q++) {
-        const int slot = 32 * q + lane - (VG - 1);
+        const int slot = 32 * q + lane + TILE_WX0 - VG;
         if (slot >= 0 && slot < TILE_WW) dst[slot] = as_d(wv[q] & vkeep(VS));
       }
     }
@@ -981,7 +1037,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
           const int wx = lane + 32 * q;
           const int64_t idx = rbase + wx;
           if (wx >= TILE_WW || idx < 0 || idx >= a.npad_in) continue;
-          const bool owner = row_own && wx >= 1 && wx <= 256;
+          const bool owner = row_own && wx >= TILE_WX0 && wx < TILE_WX0 + 256;
           const uint64_t rw = v1_check<VS>(ldg64(a.r_f + idx), a.r_f + idx, owner, a.counts, a.due);
           const uint64_t pw = v1_check<VS>(ldg64(pin + idx), pin + idx, owner, a.counts, a.due);
           const double pn = fma(beta, as_d(pw & vkeep(VS)), as_d(rw & vkeep(VS)));
@@ -990,7 +1046,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       }
     }
   } else
-  for (int wy = warp; wy < TILE_TY + 2; wy += 8) {
+  for (int wy = warp; wy < TILE_TY + 2; wy += 8) {   // G = 1 without vector tensor maps
     const int64_t rbase = win0 + (int64_t)wy * n;                 // in-index of (wy, 0)
     const bool row_in = rbase >= 0 && rbase + TILE_WW <= a.npad_in;  // uniform: no per-slot bounds
     const bool row_own = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny;
@@ -1018,7 +1074,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
         const int wx = lane + 32 * q;
         const int64_t idx = rbase + wx;
         if (wx >= TILE_WW || idx < 0 || idx >= a.npad_in) continue;
-        const bool owner = row_own && wx >= 1 && wx <= 256;
+        const bool owner = row_own && wx >= TILE_WX0 && wx < TILE_WX0 + 256;
         const uint64_t w = v1_check<VS>(ldg64(src + wx), pin + idx, owner, a.counts, a.due);
         dst[wx] = as_d(w & vkeep(VS));
       }
@@ -1044,7 +1100,7 @@ __global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __
       const uint64_t* sval = reinterpret_cast<const uint64_t*>(stage) + warp * TILE_PE;
       const uint32_t* scol = reinterpret_cast<const uint32_t*>(stage + TILE_STAGE_VAL) + warp * TILE_PE;
       const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
-      const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + 1;
+      const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + TILE_WX0;
       const double p_own = s_win[oslot];
       const int64_t own = a.row_base + rowseg + k * 32 + lane;
       const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s_win, oslot, p_own, own,

@@ -45,7 +45,26 @@ static bool tile_maps(const SpmvArgs& a, TileMaps* m) {
   CUresult r2 = enc(&m->col, CU_TENSOR_MAP_DATA_TYPE_UINT32, 2, a.col, dims, sc, box, estr,
                     CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
                     CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
-  return r1 == CUDA_SUCCESS && r2 == CUDA_SUCCESS;
+  if (r1 != CUDA_SUCCESS || r2 != CUDA_SUCCESS) return false;
+  // the input vector (and p_cur) as [rows][n/2][2] doubles: one box = the
+  // decoded window's TILE_TY+2 rows x 130 pairs (x = tx0-2 .. tx0+257)
+  m->has_vmaps = 0;
+  if ((a.npad_in % n) == 0 && (a.row_base % n) == 0 && (n % 2) == 0) {
+    cuuint64_t vd[3] = {2, (cuuint64_t)(n / 2), (cuuint64_t)(a.npad_in / n)};
+    cuuint64_t vs[2] = {16, (cuuint64_t)(n * 8)};
+    cuuint32_t vb[3] = {2, (cuuint32_t)(TILE_WW / 2), (cuuint32_t)(TILE_TY + 2)};
+    cuuint32_t ve[3] = {1, 1, 1};
+    CUresult r3 = enc(&m->vin, CU_TENSOR_MAP_DATA_TYPE_UINT64, 3, a.in, vd, vs, vb, ve, CU_TENSOR_MAP_INTERLEAVE_NONE,
+                      CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    CUresult r4 = CUDA_SUCCESS;
+    if (a.p_cur)
+      r4 = enc(&m->vcur, CU_TENSOR_MAP_DATA_TYPE_UINT64, 3, a.p_cur, vd, vs, vb, ve, CU_TENSOR_MAP_INTERLEAVE_NONE,
+               CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    else
+      m->vcur = m->vin;
+    m->has_vmaps = (r3 == CUDA_SUCCESS && r4 == CUDA_SUCCESS) ? 1 : 0;
+  }
+  return true;
 }
 template <int ES, int RS, int VS, bool DOT, bool FUSED = false>
 static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
