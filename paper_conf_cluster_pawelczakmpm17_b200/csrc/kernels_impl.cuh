@@ -770,8 +770,11 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
   return acc;
 }
 
+#ifndef ABFT_TILE_MINB
+#define ABFT_TILE_MINB 3
+#endif
 template <int ES, int RS, int VS, bool DOT, bool FUSED = false>
-__global__ void __launch_bounds__(256, 3) k_spmv_tile(const SpmvArgs a, const __grid_constant__ TileMaps tm) {
+__global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArgs a, const __grid_constant__ TileMaps tm) {
   static_assert(!FUSED || (vgrp(VS) == 1 && DOT), "fused calc_p: G = 1 vector schemes, CG SpMV only");
   extern __shared__ uint8_t s_raw[];
   __shared__ __align__(16) uint8_t s_lut[128];
