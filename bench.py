@@ -239,9 +239,13 @@ def read_traffic():
     p = os.path.join(ROOT, "profiles", "spmv_traffic.json")
     try:
         with open(p) as f:
-            return json.load(f)
+            t = json.load(f)
     except Exception:
         return None
+    b = t.get("bytes_per_launch")
+    if not isinstance(b, (int, float)) or b != b:   # a failed capture leaves NaN: report null
+        return None
+    return t
 
 
 # ------------------------------------------------------------------ oracle legs

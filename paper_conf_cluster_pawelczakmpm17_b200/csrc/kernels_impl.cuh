@@ -1289,6 +1289,9 @@ __device__ __forceinline__ void p_step(const VecArgs& a, uint64_t* P, uint64_t* 
   P[k] = e0;
   P[k + 32] = e1;
 }
+#ifndef ABFT_P_PREFETCH
+#define ABFT_P_PREFETCH 1
+#endif
 // Full RB of calc_p; step 0's words were loaded by the caller ahead of the
 // barrier / stop check.
 template <int VS>
@@ -1296,10 +1299,25 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
                                        uint64_t r0, uint64_t r1, uint64_t p0, uint64_t p1) {
   uint64_t* P = a.p + base + lane;
   uint64_t* R = a.r + base + lane;
+#if ABFT_P_PREFETCH
+  // Register double buffer: step k+64's four words are in flight while step k
+  // decodes / encodes (the codec ALU otherwise serialises with the next loads).
+#pragma unroll 1
+  for (int k = 0; k < 256; k += 64) {
+    uint64_t nr0 = 0, nr1 = 0, np0 = 0, np1 = 0;
+    if (k + 64 < 256) {
+      nr0 = ldg64(R + k + 64); nr1 = ldg64(R + k + 96);
+      np0 = ldg64(P + k + 64); np1 = ldg64(P + k + 96);
+    }
+    p_step<VS>(a, P, R, k, r0, r1, p0, p1, beta, lane, cs);
+    r0 = nr0; r1 = nr1; p0 = np0; p1 = np1;
+  }
+#else
   p_step<VS>(a, P, R, 0, r0, r1, p0, p1, beta, lane, cs);
 #pragma unroll 1
   for (int k = 64; k < 256; k += 64)
     p_step<VS>(a, P, R, k, ldg64(R + k), ldg64(R + k + 32), ldg64(P + k), ldg64(P + k + 32), beta, lane, cs);
+#endif
 }
 
 // Codec tables of the BLAS-1 / SpMV kernels in shared memory: the V-SECDED64

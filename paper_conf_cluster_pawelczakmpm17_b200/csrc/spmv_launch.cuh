@@ -2,6 +2,7 @@
 // generic CSR kernel), instantiated per element scheme in spmv_es_*.cu.
 #pragma once
 #include <cudaTypedefs.h>
+#include <cstdlib>
 
 #include "kernels_impl.cuh"
 
@@ -49,7 +50,8 @@ static bool tile_maps(const SpmvArgs& a, TileMaps* m) {
   // the input vector (and p_cur) as [rows][n/2][2] doubles: one box = the
   // decoded window's TILE_TY+2 rows x 130 pairs (x = tx0-2 .. tx0+257)
   m->has_vmaps = 0;
-  if ((a.npad_in % n) == 0 && (a.row_base % n) == 0 && (n % 2) == 0) {
+  static const bool no_vmaps = [] { const char* e = getenv("ABFT_NO_VMAPS"); return e && e[0] == '1'; }();
+  if (!no_vmaps && (a.npad_in % n) == 0 && (a.row_base % n) == 0 && (n % 2) == 0) {
     cuuint64_t vd[3] = {2, (cuuint64_t)(n / 2), (cuuint64_t)(a.npad_in / n)};
     cuuint64_t vs[2] = {16, (cuuint64_t)(n * 8)};
     cuuint32_t vb[3] = {2, (cuuint32_t)(TILE_WW / 2), (cuuint32_t)(TILE_TY + 2)};
