@@ -170,3 +170,20 @@ def test_bench_chunk_layout_fits_element_index(world, grid):
             # the window covers the chunk's rows and one grid row either side (ghost rows for world > 1)
             assert c["col_base"] <= max(0, c["row_base"] - grid)
             assert c["col_base"] + c["ncols"] >= min(c["row_base"] + c["nrows"] + grid, halo + grid * grid + halo)
+
+
+def test_bench_traffic_null_for_failed_capture(tmp_path, monkeypatch):
+    """bench.py's roofline `traffic` comes from profiles/spmv_traffic.json; a
+    failed ncu capture leaves NaN there, which must be reported as null (a NaN
+    would make the JSON line invalid)."""
+    import json
+    import bench
+    (tmp_path / "profiles").mkdir()
+    f = tmp_path / "profiles" / "spmv_traffic.json"
+    monkeypatch.setattr(bench, "ROOT", str(tmp_path))
+    f.write_text('{"bytes_per_launch": NaN}')
+    assert bench.read_traffic() is None
+    f.write_text(json.dumps({"bytes_per_launch": 1336580796.0}))
+    assert bench.read_traffic()["bytes_per_launch"] == 1336580796.0
+    f.unlink()
+    assert bench.read_traffic() is None
