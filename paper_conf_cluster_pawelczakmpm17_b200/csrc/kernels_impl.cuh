@@ -1289,6 +1289,9 @@ __device__ __forceinline__ void p_step(const VecArgs& a, uint64_t* P, uint64_t* 
   P[k] = e0;
   P[k + 32] = e1;
 }
+#ifndef ABFT_P_UNROLL
+#define ABFT_P_UNROLL 0
+#endif
 #ifndef ABFT_P_PREFETCH
 #define ABFT_P_PREFETCH 1
 #endif
@@ -1302,7 +1305,11 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
 #if ABFT_P_PREFETCH
   // Register double buffer: step k+64's four words are in flight while step k
   // decodes / encodes (the codec ALU otherwise serialises with the next loads).
+#if ABFT_P_UNROLL
+#pragma unroll
+#else
 #pragma unroll 1
+#endif
   for (int k = 0; k < 256; k += 64) {
     uint64_t nr0 = 0, nr1 = 0, np0 = 0, np1 = 0;
     if (k + 64 < 256) {

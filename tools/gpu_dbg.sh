@@ -1,6 +1,3 @@
-# r32: DRAM bytes of the default (3-D TMA window) k_spmv_tile from a single-pass
-# metric capture (no kernel replay), and application-replay attempt of the sections
+# same-box A/B of calc_p variants (tools/build_variant.sh): base, full unroll, full unroll + minb 5
 mkdir -p gpurun_out
-N="--steps 1 --warmup 0 --no-e2e --no-cpu-baseline --no-fused-extra --max-iters 4"
-timeout 400 ncu --metrics dram__bytes_read.sum,dram__bytes_write.sum,gpu__time_duration.sum --clock-control none -k regex:'k_spmv_tile|k_calc' -s 6 -c 6 --csv --log-file gpurun_out/dram_r32.csv python bench.py $N > gpurun_out/ncu_dram_r32.log 2>&1; tail -2 gpurun_out/ncu_dram_r32.log; cat gpurun_out/dram_r32.csv | cut -c1-220 | tail -20
-timeout 900 ncu --replay-mode application --section SpeedOfLight --section MemoryWorkloadAnalysis --section Occupancy --clock-control none -k regex:'k_spmv_tile' -s 6 -c 1 -o gpurun_out/prof_r32app -f python bench.py $N > gpurun_out/ncu_app_r32.log 2>&1; tail -3 gpurun_out/ncu_app_r32.log
+for rep in 1 2 3; do for v in base p1u p1u5; do echo "== $v"; ABFT_SO=variants/libabft_$v.so timeout 300 python tools/spmv_time.py --reps 200 2>&1 | tail -1 | python -c "import json,sys; d=json.loads(sys.stdin.read()); print(d['scheme2']['calc_p_ms'], d['scheme0']['calc_p_ms'])"; done; done
