@@ -248,6 +248,12 @@ def read_traffic():
     return t
 
 
+def traffic_matches(t, grid, world, fused):
+    """The stored capture is per SpMV launch of one workload (grid, ranks,
+    calc_p arrangement); another workload's line reports traffic null."""
+    return bool(t) and t.get("grid", 4096) == grid and t.get("n_gpus", 1) == world and t.get("fused", False) == fused
+
+
 # ------------------------------------------------------------------ oracle legs
 def oracle_sample(grid_sample=512, iters=3):
     """The CPU oracle (never tuned) on a bounded sample: `iters` protected CG
@@ -432,7 +438,7 @@ def main():
                    "chunks": len(P["chunks"]),
                    "schemes": {"elements": "E-SECDED", "rowptr": "R-SECDED64", "vectors": "V-SECDED64"},
                    "tol": args.tol, "iters_per_step": r_p["iters"] / args.steps,
-                   "l2": "inputs larger than L2 (2.55 GB moved per CG iteration vs 126 MB L2)",
+                   "l2": f"inputs larger than L2 ({cg_bpr * N / 1e9:.2f} GB moved per CG iteration vs 126 MB L2)",
                    "parallelism": f"row-block strips x{world}" if world > 1 else "single GPU",
                    "fused_calc_p": fused, "pdl": not args.no_pdl and not dist_on, "bytes_per_row_per_iter": cg_bpr},
         "roofline": {"bound": "hbm",
@@ -440,7 +446,7 @@ def main():
                      else "k_spmv_tile (protected SpMV + p.w)",
                      "achieved": spmv_gbs, "peak": peak, "unit": "GB/s",
                      "frac": (spmv_gbs / peak) if spmv_gbs else None,
-                     "traffic": traffic.get("bytes_per_launch") if traffic else None,
+                     "traffic": traffic.get("bytes_per_launch") if traffic_matches(traffic, args.grid, world, fused) else None,
                      "bytes_per_launch_algorithmic": spmv_bpr * N, "peak_source": peak_src,
                      "avg_launch_ms": spmv_ms},
         "cg_bandwidth": {"achieved_gbs": cg_bpr * N / (iter_ms_p / 1000.0) / 1e9,

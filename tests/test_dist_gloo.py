@@ -187,3 +187,15 @@ def test_bench_traffic_null_for_failed_capture(tmp_path, monkeypatch):
     assert bench.read_traffic()["bytes_per_launch"] == 1336580796.0
     f.unlink()
     assert bench.read_traffic() is None
+
+
+def test_bench_traffic_only_for_the_captured_workload():
+    """The stored DRAM bytes are per launch of one workload: other grids, rank
+    counts or the fused arrangement report traffic null."""
+    import bench
+    t = {"bytes_per_launch": 1.0, "grid": 4096, "n_gpus": 1, "fused": False}
+    assert bench.traffic_matches(t, 4096, 1, False)
+    assert not bench.traffic_matches(t, 16384, 1, False)
+    assert not bench.traffic_matches(t, 4096, 2, False)
+    assert not bench.traffic_matches(t, 4096, 1, True)
+    assert not bench.traffic_matches(None, 4096, 1, False)
