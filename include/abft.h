@@ -84,7 +84,7 @@ int abft_ctx_destroy(abft_ctx* ctx);
  * enable = 0 runs the unfused sequence. */
 int abft_ctx_set_fused_cg(abft_ctx* ctx, int enable);
 /* Programmatic dependent launch between the kernels of abft_cg_solve's
- * iterations (default on, single GPU): each kernel issues its
+ * iterations (library default off, single GPU): each kernel issues its
  * loads of data the previous kernel does not write (the matrix, vectors from
  * two kernels back) before waiting on it, hiding launch gaps and tails.
  * Results are identical either way. */
@@ -211,6 +211,23 @@ int abft_dist_destroy(abft_dist* d);
 int abft_cg_solve_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b,
                        abft_vec* x, abft_vec* r, abft_vec* p, abft_vec* w, const abft_cg_opts* opts,
                        abft_cg_result* res, abft_counts* dcnt, void* stream);
+/* In-process LOOPBACK transport (testing the P > 1 path on one device): nranks
+ * virtual ranks whose strips all live in this process on `device`.  The halo
+ * step becomes device-to-device copies between the ranks' extended vectors and
+ * the all-gather a shared device buffer; every other step (kernels, RED-1
+ * subtree roots, top-of-tree combine, DUE consensus, interior/boundary split,
+ * CUDA graph) is the code the NCCL transport runs.  Errors: ABFT_E_INVALID
+ * (nranks < 1 or > 1024), ABFT_E_CUDA. */
+int abft_dist_init_loopback(abft_dist** out, int nranks, int device);
+/* Distributed protected CG over a loopback transport: per rank q, ctxs[q] (one
+ * context per rank, all on the transport's device), its chunk array A[q] of
+ * nchunks[q] chunks, its halo-extended vectors vecs[5q .. 5q+4] = b, x, r, p, w,
+ * its counters dcnt[q] and its result res[q].  All ranks run in lockstep on
+ * `stream`; the return value is rank 0's status.  Same semantics and results as
+ * abft_cg_solve_dist on nranks processes (S§8(e), §V-A). */
+int abft_cg_solve_loopback(abft_dist* d, abft_ctx* const* ctxs, const abft_csr* const* A, const int* nchunks,
+                           int64_t n_halo, abft_vec* const* vecs, const abft_cg_opts* opts, abft_cg_result* res,
+                           abft_counts* const* dcnt, void* stream);
 
 /* Host-side codec hooks (no GPU needed): run the exact __host__ __device__
  * codec functions on the CPU for the unit tests.  inst: 0 E-SECDED, 1 V-SECDED64,

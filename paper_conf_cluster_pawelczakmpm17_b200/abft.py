@@ -78,6 +78,8 @@ _sig = {
     "abft_cg_solve_dist": (C.c_int, [_P, _P, C.POINTER(CSR), C.c_int, C.c_int64, C.POINTER(Vec), C.POINTER(Vec),
                                      C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts),
                                      C.POINTER(CGResult), _P, _P]),
+    "abft_dist_init_loopback": (C.c_int, [C.POINTER(C.c_void_p), C.c_int, C.c_int]),
+    "abft_cg_solve_loopback": (C.c_int, [_P, _P, _P, _P, C.c_int64, _P, C.POINTER(CGOpts), _P, _P, _P]),
     "abft_codec_host_check": (C.c_int, [C.c_int, _P]),
     "abft_codec_host_encode": (None, [C.c_int, _P]),
 }
@@ -153,7 +155,7 @@ class Context:
         _check(_lib.abft_ctx_set_fused_cg(self.h, 1 if enable else 0), "abft_ctx_set_fused_cg")
 
     def set_pdl(self, enable: bool):
-        """Programmatic dependent launch in the CG loop (abft_ctx_set_pdl; default on)."""
+        """Programmatic dependent launch in the CG loop (abft_ctx_set_pdl; library default off)."""
         _check(_lib.abft_ctx_set_pdl(self.h, 1 if enable else 0), "abft_ctx_set_pdl")
 
     def close(self):
@@ -378,3 +380,52 @@ class Dist:
                                        C.byref(res), counts.ptr if counts else None, _stream(stream))
         _check(code, "abft_cg_solve_dist", allow=(E_DUE, E_NOT_CONVERGED))
         return res
+
+
+class Loopback:
+    """abft_dist over the in-process loopback transport: `nranks` virtual ranks
+    on one device, each with its own Context, chunks and halo-extended vectors
+    (abft_dist_init_loopback / abft_cg_solve_loopback)."""
+
+    def __init__(self, nranks: int, device: int = 0):
+        h = C.c_void_p()
+        _check(_lib.abft_dist_init_loopback(C.byref(h), int(nranks), int(device)), "abft_dist_init_loopback")
+        self.h, self.nranks = h, int(nranks)
+
+    def close(self):
+        if self.h:
+            _lib.abft_dist_destroy(self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def cg_solve(self, ctxs, As, n_halo: int, vecs, tol=1e-10, max_iters=10000, due_policy=0, counts=None,
+                 poll_every=16, stream=None, check_interval=1):
+        """ctxs[q], As[q] (matrix or chunk list), vecs[q] = (b, x, r, p, w), counts[q]
+        for every rank q; returns the per-rank CGResult list."""
+        P = self.nranks
+        assert len(ctxs) == len(As) == len(vecs) == P
+        keep = []
+        arrs = []
+        nch = (C.c_int * P)()
+        for q in range(P):
+            arr, n = _chunks(As[q])
+            keep.append(arr)
+            arrs.append(C.cast(arr, C.c_void_p))
+            nch[q] = n
+        aptr = (C.c_void_p * P)(*arrs)
+        cptr = (C.c_void_p * P)(*[c.h for c in ctxs])
+        vstructs = [v.cstruct() for q in range(P) for v in vecs[q]]
+        vptr = (C.c_void_p * (5 * P))(*[C.cast(C.pointer(v), C.c_void_p) for v in vstructs])
+        cnts = counts if counts is not None else [None] * P
+        nptr = (C.c_void_p * P)(*[c.ptr if c is not None else None for c in cnts])
+        opts = CGOpts(tol, max_iters, due_policy, poll_every, check_interval)
+        res = (CGResult * P)()
+        code = _lib.abft_cg_solve_loopback(self.h, cptr, aptr, nch, int(n_halo), vptr, C.byref(opts),
+                                           C.cast(res, C.c_void_p), nptr, _stream(stream))
+        _check(code, "abft_cg_solve_loopback", allow=(E_DUE, E_NOT_CONVERGED))
+        return list(res)

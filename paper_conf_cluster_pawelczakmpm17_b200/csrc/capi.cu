@@ -104,7 +104,7 @@ int check_chunks(const abft_csr* A, int nchunks) {
 int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, bool dot,
                 DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total, RedArgs red = RedArgs{},
                 int check_mode = MODE_CORRECT, int check_interval = 0, uint64_t* p_cur = nullptr,
-                uint64_t* r_f = nullptr, bool probe = false) {
+                uint64_t* r_f = nullptr, bool probe = false, int part = 0) {
   const int64_t base0 = A[0].row_base;
   const int64_t npad_in = vec_padded_len(in->n, in->scheme);
   const int64_t npad_out = vec_padded_len(out->n, out->scheme);
@@ -123,6 +123,10 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
   for (int c = 0; c < nchunks; c++) {
     const abft_csr& M = A[c];
     if (M.row_base + M.nrows > out->n) return fail(ABFT_E_INVALID, "chunk %d rows exceed out", c);
+    // lane groups of G > 1 vector codecs (V-SECDED128 pairs, V-CRC quads) must
+    // line up with the stored codeword groups
+    if (M.row_base % vec_padded_len(1, out->scheme) != 0)
+      return fail(ABFT_E_SHAPE, "chunk %d: row_base not a multiple of the vector group size", c);
     if (M.col_base + M.ncols > npad_in) return fail(ABFT_E_INVALID, "chunk %d cols exceed in", c);
     SpmvArgs a{};
     a.nrows = M.nrows;
@@ -152,7 +156,28 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.p_cur = p_cur;
     a.r_f = r_f;
     if (probe) {
-      if (!spmv_fusable(a, in->scheme)) return ABFT_E_SHAPE;
+      // probe: p_cur set -> can the fused calc_p kernel run; else -> is every chunk tileable
+      if (p_cur ? !spmv_fusable(a, in->scheme) : !spmv_tileable(a, in->scheme)) return ABFT_E_SHAPE;
+      continue;
+    }
+    if (part != 0) {
+      // halo overlap (multi-rank, every chunk tileable): part 1 = the interior
+      // tile rows, whose windows never reach the ghost rows; part 2 = the first
+      // tile row of the first chunk and the last of the last chunk
+      const int64_t nty = spmv_tile_rows(a);
+      const int64_t lo = (c == 0) ? 1 : 0;
+      int64_t hi = (c == nchunks - 1) ? nty - 1 : nty;
+      if (hi < lo) hi = lo;
+      int64_t rng[2][2] = {{lo, hi}, {0, 0}};
+      if (part == 2) { rng[0][0] = 0; rng[0][1] = lo; rng[1][0] = hi; rng[1][1] = nty; }
+      for (int q = 0; q < 2; q++) {
+        if (rng[q][1] <= rng[q][0]) continue;
+        a.ty_lo = rng[q][0];
+        a.ty_hi = rng[q][1];
+        const int l = launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s);
+        if (l < 0) return fail(ABFT_E_CUDA, "chunk %d: SpMV part could not be launched", c);
+        count_launch(l);
+      }
       continue;
     }
     const int l = launch_spmv(a, M.elem_scheme, M.rowptr_scheme, in->scheme, dot, s);
@@ -365,11 +390,22 @@ struct Prof {
 
 }  // extern "C"
 
+// ------------------------------------------------------------ multi-rank plumbing
+// abft_dist is the transport of the row-block strips: NCCL with
+// one rank per process in production, or an in-process LOOPBACK of P virtual
+// ranks on one device (every rank's vectors in this process) that runs the same
+// per-rank kernel sequence, halo and all-gather points for testing the P > 1
+// path without a second GPU.  Both expose the two exchange steps the CG
+// iteration has: the p halo (one grid row each side) and the all-gather of one
+// (RED-1 subtree root, DUE flag) pair per rank.
 struct abft_dist {
+  int loopback = 0;
   ncclComm_t comm = nullptr;
   int rank = 0, nranks = 1, device = 0;
-  double* sendbuf = nullptr;   // [2]
-  double* gathered = nullptr;  // [2 * nranks]
+  double* sendbuf = nullptr;   // NCCL: this rank's pair [2]
+  double* gathered = nullptr;  // all ranks' pairs [2 * nranks] (loopback: rank r writes gathered + 2r directly)
+  cudaStream_t comm_stream = nullptr;   // halo exchange, overlapped with the interior SpMV
+  cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
 };
 
 namespace {
@@ -380,10 +416,85 @@ namespace {
     if (r_ != ncclSuccess) return fail(ABFT_E_NCCL, "%s: %s", #x, ncclGetErrorString(r_)); \
   } while (0)
 
-// Exchange the ghost rows of an extended vector (n_halo entries each side).
-int halo_exchange(abft_dist* d, uint64_t* ext, int64_t n_loc, int64_t n_halo, cudaStream_t s) {
+// One rank's share of a (possibly distributed) CG solve.
+struct RankRun {
+  abft_ctx* ctx = nullptr;
+  const abft_csr* A = nullptr;
+  int nchunks = 0;
+  abft_vec* v[5] = {};   // b x r p w
+  DevCounts* cnt = nullptr;
+  int64_t n = 0, nrb = 0, n_ext = 0;
+  VecArgs va{};
+  double* sendbuf = nullptr;
+  double* gathered = nullptr;
+  abft_vec* b() const { return v[0]; }
+  abft_vec* x() const { return v[1]; }
+  abft_vec* r() const { return v[2]; }
+  abft_vec* p() const { return v[3]; }
+  abft_vec* w() const { return v[4]; }
+};
+
+int validate_rank(RankRun& R, int64_t n_halo, const abft_cg_opts* opts) {
+  int e = check_chunks(R.A, R.nchunks);
+  if (e) return e;
+  const char* names[5] = {"b", "x", "r", "p", "w"};
+  for (int i = 0; i < 5; i++) if ((e = check_vec(R.v[i], names[i]))) return e;
+  const int scheme = R.x()->scheme;
+  R.n_ext = R.x()->n;
+  for (int i = 0; i < 5; i++) {
+    if (R.v[i]->scheme != scheme || R.v[i]->n != R.n_ext) return fail(ABFT_E_INVALID, "vector %s: scheme/length differ", names[i]);
+    for (int j = 0; j < i; j++) if (R.v[i]->data == R.v[j]->data) return fail(ABFT_E_INVALID, "vectors alias");
+  }
+  R.n = R.n_ext - 2 * n_halo;  // local rows
+  const int G = (int)vec_padded_len(1, scheme);
+  if (R.n <= 0 || n_halo < 0 || (n_halo % G) != 0) return fail(ABFT_E_SHAPE, "bad halo / local size");
+  if (n_halo > 0 && (R.n % G) != 0) return fail(ABFT_E_SHAPE, "local rows must be a multiple of the vector group");
+  int64_t rows = 0;
+  for (int c = 0; c < R.nchunks; c++) rows += R.A[c].nrows;
+  if (R.A[0].row_base != n_halo || rows != R.n) return fail(ABFT_E_SHAPE, "chunks must cover the local rows");
+  R.nrb = (R.n + 255) / 256;
+  if ((e = ensure_partials(R.ctx, R.nrb))) return e;
+  if (opts->check_interval < 0) return fail(ABFT_E_INVALID, "negative check interval");
+  if (R.nrb > (int64_t)1024 * 1024) return fail(ABFT_E_SHAPE, "more than 2^28 rows per GPU");
+  VecArgs& va = R.va;
+  va = VecArgs{};
+  va.n = R.n;
+  va.npad = vec_padded_len(R.n, scheme);
+  va.x = reinterpret_cast<uint64_t*>(R.x()->data) + n_halo;
+  va.p = reinterpret_cast<uint64_t*>(R.p()->data) + n_halo;
+  va.r = reinterpret_cast<uint64_t*>(R.r()->data) + n_halo;
+  va.w = reinterpret_cast<uint64_t*>(R.w()->data) + n_halo;
+  va.b = reinterpret_cast<uint64_t*>(R.b()->data) + n_halo;
+  va.partials = R.ctx->partials;
+  va.counts = R.cnt;
+  va.due = R.ctx->due;
+  va.state = R.ctx->state;
+  va.crc = R.ctx->crc;
+  return ABFT_OK;
+}
+
+// Exchange the ghost rows of vector `vi` (extended by n_halo entries each side)
+// of every local rank with its strip neighbours, on stream s.
+int halo_exchange(abft_dist* d, RankRun* R, int nl, int vi, int64_t n_halo, cudaStream_t s) {
   if (!d || d->nranks == 1 || n_halo == 0) return ABFT_OK;
   const size_t bytes = sizeof(uint64_t) * (size_t)n_halo;
+  if (d->loopback) {
+    // rank r's top ghost <- rank r-1's last local grid row; bottom ghost <- rank r+1's first
+    for (int q = 0; q < nl; q++) {
+      uint64_t* ext = reinterpret_cast<uint64_t*>(R[q].v[vi]->data);
+      if (q > 0) {
+        const uint64_t* up = reinterpret_cast<const uint64_t*>(R[q - 1].v[vi]->data);
+        CUDA_TRY(cudaMemcpyAsync(ext, up + R[q - 1].n, bytes, cudaMemcpyDeviceToDevice, s));
+      }
+      if (q < nl - 1) {
+        const uint64_t* dn = reinterpret_cast<const uint64_t*>(R[q + 1].v[vi]->data);
+        CUDA_TRY(cudaMemcpyAsync(ext + n_halo + R[q].n, dn + n_halo, bytes, cudaMemcpyDeviceToDevice, s));
+      }
+    }
+    return ABFT_OK;
+  }
+  uint64_t* ext = reinterpret_cast<uint64_t*>(R[0].v[vi]->data);
+  const int64_t n_loc = R[0].n;
   NCCL_TRY(ncclGroupStart());
   if (d->rank > 0) {
     NCCL_TRY(ncclSend(ext + n_halo, bytes, ncclChar, d->rank - 1, d->comm, s));
@@ -397,71 +508,72 @@ int halo_exchange(abft_dist* d, uint64_t* ext, int64_t n_loc, int64_t n_halo, cu
   return ABFT_OK;
 }
 
-// Fused dot-product finish: single GPU -> the producer kernel's
-// last warp applies `op`; multi-GPU -> it writes (subtree root, DUE flag) to
-// sendbuf, then all-gather + identical top-of-tree combine on every rank.
-RedArgs red_for(abft_ctx*, abft_dist*, int64_t, int) {
-  // Fused last-warp reductions (RedState) measured slower than a separate
-  // reduction kernel: the per-warp __threadfence before the group counter
-  // stalls every producer warp on its own outstanding stores (r14: SpMV
-  // 0.295 -> 0.327 ms).  Kept disabled; partials are reduced by k_reduce.
-  return RedArgs{};
-}
-// Dot-product finish: single GPU -> k_reduce applies `op`; multi-GPU -> subtree
-// root + DUE flag, all-gather, identical top-of-tree combine on every rank.
-int finish_dot(abft_ctx* ctx, abft_dist* d, int64_t nrb, int op, cudaStream_t s) {
-  if (!d) {
-    count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, op, ctx->state, nullptr, ctx->due, s));
-    return ABFT_OK;
-  }
-  count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 4, nullptr, d->sendbuf, ctx->due, s));
+// every rank's (root, due) pair -> every rank's `gathered`
+int allgather_pairs(abft_dist* d, cudaStream_t s) {
+  if (d->loopback) return ABFT_OK;   // the ranks wrote their pairs into the one shared buffer
   NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
-  count_launch(launch_combine(d->gathered, d->nranks, op, ctx->state, ctx->due, s));
   return ABFT_OK;
 }
 
-int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b, abft_vec* x,
-            abft_vec* r, abft_vec* p, abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt,
-            cudaStream_t s) {
-  if (!ctx || !opts || !res) return fail(ABFT_E_INVALID, "null ctx/opts/res");
-  int e = check_chunks(A, nchunks);
-  if (e) return e;
-  abft_vec* vs[5] = {b, x, r, p, w};
-  const char* names[5] = {"b", "x", "r", "p", "w"};
-  for (int i = 0; i < 5; i++) if ((e = check_vec(vs[i], names[i]))) return e;
-  const int scheme = x->scheme;
-  const int64_t n_ext = x->n;
-  for (int i = 0; i < 5; i++) {
-    if (vs[i]->scheme != scheme || vs[i]->n != n_ext) return fail(ABFT_E_INVALID, "vector %s: scheme/length differ", names[i]);
-    for (int j = 0; j < i; j++) if (vs[i]->data == vs[j]->data) return fail(ABFT_E_INVALID, "vectors alias");
+// Dot-product finish: single GPU -> k_reduce applies `op`;
+// multi-rank -> each rank's subtree root + DUE flag, all-gather, and the same
+// top-of-tree combine on every rank (bit-identical to one GPU for aligned
+// power-of-two subtrees).
+int finish_dot(RankRun* R, int nl, abft_dist* d, int op, cudaStream_t s) {
+  if (!d) {
+    abft_ctx* c = R[0].ctx;
+    count_launch(launch_reduce(c->partials, R[0].nrb, c->roots, c->ticket, op, c->state, nullptr, c->due, s));
+    return ABFT_OK;
   }
-  const int64_t n = n_ext - 2 * n_halo;  // local rows
-  const int G = (int)vec_padded_len(1, scheme);
-  if (n <= 0 || n_halo < 0 || (n_halo % G) != 0) return fail(ABFT_E_SHAPE, "bad halo / local size");
-  if (n_halo > 0 && (n % G) != 0) return fail(ABFT_E_SHAPE, "local rows must be a multiple of the vector group");
-  int64_t rows = 0;
-  for (int c = 0; c < nchunks; c++) rows += A[c].nrows;
-  if (A[0].row_base != n_halo || rows != n) return fail(ABFT_E_SHAPE, "chunks must cover the local rows");
+  for (int q = 0; q < nl; q++) {
+    abft_ctx* c = R[q].ctx;
+    count_launch(launch_reduce(c->partials, R[q].nrb, c->roots, c->ticket, 4, nullptr, R[q].sendbuf, c->due, s));
+  }
+  int e = allgather_pairs(d, s);
+  if (e) return e;
+  for (int q = 0; q < nl; q++)
+    count_launch(launch_combine(R[q].gathered, d->nranks, op, R[q].ctx->state, R[q].ctx->due, s));
+  return ABFT_OK;
+}
 
-  DevCounts* cnt = reinterpret_cast<DevCounts*>(dcnt);
-  const int64_t npad = vec_padded_len(n, scheme);
-  const int64_t nrb = (n + 255) / 256;
-  if ((e = ensure_partials(ctx, nrb))) return e;
-  if (opts->check_interval < 0) return fail(ABFT_E_INVALID, "negative check interval");
+// The CG driver for nl local ranks in lockstep (nl = 1: one GPU, or one NCCL
+// rank of a multi-process solve; nl = P: the loopback).  Every kernel runs on
+// stream s; all CG scalars live on the device.
+int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts* opts, abft_cg_result* res,
+           cudaStream_t s) {
+  if (!opts || !res) return fail(ABFT_E_INVALID, "null opts/res");
+  for (int q = 0; q < nl; q++) {
+    if (!R[q].ctx) return fail(ABFT_E_INVALID, "null ctx");
+    int e = validate_rank(R[q], n_halo, opts);
+    if (e) return e;
+    for (int j = 0; j < q; j++)
+      if (R[q].ctx == R[j].ctx) return fail(ABFT_E_INVALID, "loopback ranks need one context each");
+  }
+  abft_ctx* ctx = R[0].ctx;   // graphs, events, polling
+  const int scheme = R[0].x()->scheme;
+  const int G = (int)vec_padded_len(1, scheme);
   const int interval = opts->check_interval > 1 ? opts->check_interval : 0;
-  if (nrb > (int64_t)1024 * 1024) return fail(ABFT_E_SHAPE, "more than 2^28 rows per GPU");
-  // the dist path runs whenever a communicator is given (also with 1 rank, so the
+  // the dist path runs whenever a transport is given (also with 1 rank, so the
   // all-gather / top-of-tree combine code is exercised on a single GPU)
   const bool multi = d != nullptr;
-
+  if (multi) {
+    for (int q = 0; q < nl; q++) {
+      R[q].sendbuf = d->loopback ? d->gathered + 2 * q : d->sendbuf;
+      R[q].gathered = d->gathered;
+    }
+  }
+  int e;
   // fused calc_p: single GPU, every chunk on the tiled path,
   // G = 1 vector scheme; p is double-buffered with ctx->p_alt
-  const int64_t npad_ext = vec_padded_len(n_ext, scheme);
+  const int64_t npad_ext = vec_padded_len(R[0].n_ext, scheme);
   bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0;
+  abft_vec* const p = R[0].p();
+  abft_vec* const r = R[0].r();
   if (fused) {
     abft_vec ptmp = *p;
-    fused = spmv_chunks(ctx, A, nchunks, &ptmp, w, true, cnt, nullptr, s, nullptr, RedArgs{}, MODE_CORRECT, 0,
-                        reinterpret_cast<uint64_t*>(p->data), reinterpret_cast<uint64_t*>(r->data), true) == ABFT_OK;
+    fused = spmv_chunks(ctx, R[0].A, R[0].nchunks, &ptmp, R[0].w(), true, R[0].cnt, nullptr, s, nullptr, RedArgs{},
+                        MODE_CORRECT, 0, reinterpret_cast<uint64_t*>(p->data), reinterpret_cast<uint64_t*>(r->data),
+                        true) == ABFT_OK;
   }
   if (fused && ctx->p_alt_len < npad_ext) {
     cudaFree(ctx->p_alt);
@@ -471,6 +583,12 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
     ctx->p_alt_len = npad_ext;
   }
   uint64_t* const P[2] = {reinterpret_cast<uint64_t*>(p->data), ctx->p_alt};
+  // halo overlap: P > 1 and every chunk of every rank on the tiled kernel
+  bool overlap = multi && d->nranks > 1 && n_halo > 0;
+  for (int q = 0; q < nl && overlap; q++)
+    overlap = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].p(), R[q].w(), true, R[q].cnt, nullptr, s, nullptr,
+                          RedArgs{}, MODE_CORRECT, 0, nullptr, nullptr, true) == ABFT_OK;
+  (void)cudaGetLastError();
 
   CgState h{};
   h.tol = opts->tol;
@@ -478,102 +596,119 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
   h.abort_policy = opts->due_policy == 0 ? 1 : 0;
   h.dist = multi ? 1 : 0;
   h.fused = fused ? 1 : 0;
-  *ctx->h_state = h;
-  CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
-  CUDA_TRY(cudaMemsetAsync(ctx->due, 0, sizeof(int), s));
-
-  VecArgs va{};
-  va.n = n;
-  va.npad = npad;
-  va.x = reinterpret_cast<uint64_t*>(x->data) + n_halo;
-  va.p = reinterpret_cast<uint64_t*>(p->data) + n_halo;
-  va.r = reinterpret_cast<uint64_t*>(r->data) + n_halo;
-  va.w = reinterpret_cast<uint64_t*>(w->data) + n_halo;
-  va.b = reinterpret_cast<uint64_t*>(b->data) + n_halo;
-  va.partials = ctx->partials;
-  va.counts = cnt;
-  va.due = ctx->due;
-  va.state = ctx->state;
-  va.red = red_for(ctx, d, nrb, 1);
-  va.crc = ctx->crc;
+  for (int q = 0; q < nl; q++) {
+    count_launch(launch_set_state(h, R[q].ctx->state, s));
+    CUDA_TRY(cudaMemsetAsync(R[q].ctx->due, 0, sizeof(int), s));
+  }
 
   Prof prof{ctx, s};
   // init (a2): w = A x0 ; r = b - w ; p = r ; rr0
-  if ((e = halo_exchange(d, reinterpret_cast<uint64_t*>(x->data), n, n_halo, s))) return e;
+  if ((e = halo_exchange(d, R, nl, 1, n_halo, s))) return e;
   prof.begin(0);
-  e = spmv_chunks(ctx, A, nchunks, x, w, false, cnt, nullptr, s, nullptr, RedArgs{}, MODE_CORRECT, interval);
+  for (int q = 0; q < nl; q++) {
+    e = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].x(), R[q].w(), false, R[q].cnt, nullptr, s, nullptr,
+                    RedArgs{}, MODE_CORRECT, interval);
+    if (e) return e;
+  }
   prof.end();
-  if (e) return e;
-  count_launch(launch_init_r(va, scheme, s));
-  if ((e = finish_dot(ctx, d, nrb, 1, s))) return e;
+  for (int q = 0; q < nl; q++) count_launch(launch_init_r(R[q].va, scheme, s));
+  if ((e = finish_dot(R, nl, d, 1, s))) return e;
   CUDA_TRY(cudaGetLastError());
 
   int poll = opts->poll_every > 0 ? opts->poll_every : 16;
   if (fused && (poll & 1)) poll += 1;  // graph replays then always start at an odd iteration (buffer parity)
   int64_t launched = 0;  // iterations issued so far (host); = device iterations until a stop
-  // PDL between the iteration kernels (single GPU: the multi-GPU loop has NCCL
-  // kernels in between); off again on every exit from this function
+  // PDL between the iteration kernels (single GPU: the multi-rank loop has
+  // exchange steps in between); off again on every exit from this function
   struct PdlGuard {
     explicit PdlGuard(bool on) { set_pdl(on); }
     ~PdlGuard() { set_pdl(false); }
   };
   const bool pdl_on = ctx->pdl && !multi;
+  // the protected SpMV of one iteration, all ranks (halo first, or overlapped)
+  auto spmv_iter = [&](int64_t kk, cudaStream_t ss) -> int {
+    int e2;
+    if (fused) {
+      abft_vec pprev = *p;
+      pprev.data = reinterpret_cast<double*>(P[kk & 1]);
+      return spmv_chunks(ctx, R[0].A, R[0].nchunks, &pprev, R[0].w(), true, R[0].cnt, ctx->state, ss, nullptr,
+                         RedArgs{}, MODE_CORRECT, interval, P[(kk - 1) & 1], reinterpret_cast<uint64_t*>(r->data));
+    }
+    if (!overlap) {
+      if ((e2 = halo_exchange(d, R, nl, 3, n_halo, ss))) return e2;
+      for (int q = 0; q < nl; q++)
+        if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].p(), R[q].w(), true, R[q].cnt, R[q].ctx->state,
+                              ss, nullptr, RedArgs{}, MODE_CORRECT, interval)))
+          return e2;
+      return ABFT_OK;
+    }
+    // halo on the comm stream while the interior tile rows run on ss; then the boundary rows
+    CUDA_TRY(cudaEventRecord(d->ev_fork, ss));
+    CUDA_TRY(cudaStreamWaitEvent(d->comm_stream, d->ev_fork, 0));
+    if ((e2 = halo_exchange(d, R, nl, 3, n_halo, d->comm_stream))) return e2;
+    CUDA_TRY(cudaEventRecord(d->ev_join, d->comm_stream));
+    for (int part = 1; part <= 2; part++) {
+      if (part == 2) CUDA_TRY(cudaStreamWaitEvent(ss, d->ev_join, 0));
+      for (int q = 0; q < nl; q++)
+        if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].p(), R[q].w(), true, R[q].cnt, R[q].ctx->state,
+                              ss, nullptr, RedArgs{}, MODE_CORRECT, interval, nullptr, nullptr, false, part)))
+          return e2;
+    }
+    return ABFT_OK;
+  };
   // k iterations of (a3)..(a5) + the DUE/convergence logic, all device-side
-  auto issue = [&](int64_t k, cudaStream_t s) -> int {
+  auto issue = [&](int64_t k, cudaStream_t ss) -> int {
     PdlGuard pg(pdl_on);
-    prof.s = s;
+    prof.s = ss;
     for (int64_t it = 0; it < k; it++) {
       int e2;
       // fused: iteration kk's p lives in P[(kk-1) & 1], its predecessor in P[kk & 1]
       const int64_t kk = launched + it + 1;
-      uint64_t* const pk = fused ? P[(kk - 1) & 1] : reinterpret_cast<uint64_t*>(p->data);
-      if ((e2 = halo_exchange(d, reinterpret_cast<uint64_t*>(p->data), n, n_halo, s))) return e2;
       prof.begin(0);
-      if (fused) {
-        abft_vec pprev = *p;
-        pprev.data = reinterpret_cast<double*>(P[kk & 1]);
-        e2 = spmv_chunks(ctx, A, nchunks, &pprev, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2),
-                         MODE_CORRECT, interval, pk, reinterpret_cast<uint64_t*>(r->data));
-      } else {
-        e2 = spmv_chunks(ctx, A, nchunks, p, w, true, cnt, ctx->state, s, nullptr, red_for(ctx, d, nrb, 2),
-                         MODE_CORRECT, interval);
-      }
+      e2 = spmv_iter(kk, ss);
       prof.end();
       if (e2) return e2;
       prof.begin(3);
-      if ((e2 = finish_dot(ctx, d, nrb, 2, s))) return e2;
+      if ((e2 = finish_dot(R, nl, d, 2, ss))) return e2;
       prof.end();
       prof.begin(1);
-      VecArgs vu = va;
-      vu.p = pk + n_halo;
-      vu.red = red_for(ctx, d, nrb, 3);
-      count_launch(launch_calc_ur(vu, scheme, s));
+      for (int q = 0; q < nl; q++) {
+        VecArgs vu = R[q].va;
+        if (fused) vu.p = P[(kk - 1) & 1] + n_halo;
+        count_launch(launch_calc_ur(vu, scheme, ss));
+      }
       prof.end();
       prof.begin(3);
-      if ((e2 = finish_dot(ctx, d, nrb, 3, s))) return e2;
+      if ((e2 = finish_dot(R, nl, d, 3, ss))) return e2;
       prof.end();
       if (!fused) {
         prof.begin(2);
-        count_launch(launch_calc_p(va, scheme, s));
+        for (int q = 0; q < nl; q++) count_launch(launch_calc_p(R[q].va, scheme, ss));
         prof.end();
       }
-      if (multi && h.abort_policy) {
-        count_launch(launch_pack_due(d->sendbuf, ctx->due, s));
-        NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
-        count_launch(launch_due_combine(d->gathered, d->nranks, ctx->state, ctx->due, s));
+      if (multi && h.abort_policy) {   // DUE consensus: every rank stops after the same iteration
+        for (int q = 0; q < nl; q++) count_launch(launch_pack_due(R[q].sendbuf, R[q].ctx->due, ss));
+        if ((e2 = allgather_pairs(d, ss))) return e2;
+        for (int q = 0; q < nl; q++)
+          count_launch(launch_due_combine(R[q].gathered, d->nranks, R[q].ctx->state, R[q].ctx->due, ss));
       }
     }
     CUDA_TRY(cudaGetLastError());
     return ABFT_OK;
   };
-  // CUDA graph of `poll` iterations (single GPU): one launch per poll, no
-  // per-kernel CPU launch cost; kernels read alpha/beta/stop from device state.
+  // CUDA graph of `poll` iterations (all local ranks, exchange steps included):
+  // one launch per poll, no per-kernel CPU launch cost; kernels read
+  // alpha/beta/stop from device state.
   cudaGraphExec_t gexec = nullptr;
+  struct GraphGuard {
+    cudaGraphExec_t& g;
+    ~GraphGuard() { if (g) cudaGraphExecDestroy(g); }
+  } gguard{gexec};
   std::vector<std::pair<int, int>> gmarks;
   uint64_t glaunches = 0;
   // (profiling brackets kernels with events, which are not timeable inside a
   // graph replay: profiled solves launch kernels directly)
-  const bool graphs = ctx->use_graphs && !multi && ctx->profile == 0;
+  const bool graphs = ctx->use_graphs && ctx->profile == 0;
   bool last_graph = false;
   for (;;) {
     CUDA_TRY(cudaMemcpyAsync(ctx->h_state, ctx->state, sizeof(CgState), cudaMemcpyDeviceToHost, s));
@@ -601,10 +736,14 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
         e = issue(k, ctx->cap_stream);
         cudaError_t ce = cudaStreamEndCapture(ctx->cap_stream, &graph);
         prof.s = s;
-        if (e) return e;
+        if (e) {
+          if (graph) cudaGraphDestroy(graph);
+          return e;
+        }
         if (ce != cudaSuccess) return fail(ABFT_E_CUDA, "graph capture: %s", cudaGetErrorString(ce));
-        CUDA_TRY(cudaGraphInstantiate(&gexec, graph, 0));
+        cudaError_t ie = cudaGraphInstantiate(&gexec, graph, 0);
         cudaGraphDestroy(graph);
+        if (ie != cudaSuccess) return fail(ABFT_E_CUDA, "graph instantiate: %s", cudaGetErrorString(ie));
         glaunches = g_launches.load() - l0;
         g_launches.fetch_sub(glaunches);  // counted per replay below
         gmarks = prof.marks;
@@ -618,40 +757,48 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
     }
     launched += k;
   }
-  if (gexec) cudaGraphExecDestroy(gexec);
-  const CgState& hs = *ctx->h_state;
+  // per-rank states (identical control decisions on every rank)
+  std::vector<CgState> hs(nl);
+  hs[0] = *ctx->h_state;
+  for (int q = 1; q < nl; q++) {
+    CUDA_TRY(cudaMemcpyAsync(ctx->h_state, R[q].ctx->state, sizeof(CgState), cudaMemcpyDeviceToHost, s));
+    CUDA_TRY(cudaStreamSynchronize(s));
+    hs[q] = *ctx->h_state;
+  }
   if (fused) {
     // the final p back into the caller's buffer, then the calc_p the unfused
     // order runs before an abort / max_iters stop (state.pending_p)
-    if (hs.iters >= 1 && ((hs.iters - 1) & 1))
+    if (hs[0].iters >= 1 && ((hs[0].iters - 1) & 1))
       CUDA_TRY(cudaMemcpyAsync(p->data, ctx->p_alt, sizeof(uint64_t) * npad_ext, cudaMemcpyDeviceToDevice, s));
-    if (hs.pending_p) {
-      const CgState keep = hs;
+    if (hs[0].pending_p) {
       CgState t{};
-      t.beta = keep.beta;
+      t.beta = hs[0].beta;
       t.max_iters = 0x7FFFFFFF;
-      *ctx->h_state = t;
-      CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
-      VecArgs vp = va;
+      count_launch(launch_set_state(t, ctx->state, s));
+      VecArgs vp = R[0].va;
       vp.red = RedArgs{};
       count_launch(launch_calc_p(vp, scheme, s));
       CUDA_TRY(cudaStreamSynchronize(s));
-      *ctx->h_state = keep;
     }
   }
-  res->iters = hs.iters;
-  res->rr0 = hs.rr0;
-  res->rrn = hs.rrn;
-  res->status = hs.stop ? hs.status : (opts->max_iters > 0 ? ABFT_E_NOT_CONVERGED : ABFT_OK);
+  for (int q = 0; q < nl; q++) {
+    res[q].iters = hs[q].iters;
+    res[q].rr0 = hs[q].rr0;
+    res[q].rrn = hs[q].rrn;
+    res[q].status = hs[q].stop ? hs[q].status : (opts->max_iters > 0 ? ABFT_E_NOT_CONVERGED : ABFT_OK);
+  }
   // interval mode: detection-only integrity check of the whole matrix when the
   // last access (= iteration count) was not a checked one
-  if (interval && hs.iters % interval != 0) {
-    CUDA_TRY(cudaMemsetAsync(ctx->due, 0, sizeof(int), s));
-    for (int c = 0; c < nchunks; c++) count_launch(launch_check_csr(&A[c], cnt, ctx->due, 2, s));
+  if (interval && hs[0].iters % interval != 0) {
     int any = 0;
+    for (int q = 0; q < nl; q++) {
+      CUDA_TRY(cudaMemsetAsync(R[q].ctx->due, 0, sizeof(int), s));
+      for (int c = 0; c < R[q].nchunks; c++)
+        count_launch(launch_check_csr(&R[q].A[c], R[q].cnt, R[q].ctx->due, 2, s));
+    }
     if (multi) {
-      count_launch(launch_pack_due(d->sendbuf, ctx->due, s));
-      NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
+      for (int q = 0; q < nl; q++) count_launch(launch_pack_due(R[q].sendbuf, R[q].ctx->due, s));
+      if ((e = allgather_pairs(d, s))) return e;
       std::vector<double> g(2 * (size_t)d->nranks);
       CUDA_TRY(cudaMemcpyAsync(g.data(), d->gathered, sizeof(double) * g.size(), cudaMemcpyDeviceToHost, s));
       CUDA_TRY(cudaStreamSynchronize(s));
@@ -661,10 +808,30 @@ int cg_core(abft_ctx* ctx, abft_dist* d, const abft_csr* A, int nchunks, int64_t
       CUDA_TRY(cudaStreamSynchronize(s));
       any = ctx->h_flags[0] != 0;
     }
-    if (any && h.abort_policy && res->status != ABFT_E_DUE) res->status = ABFT_E_DUE;
+    if (any && h.abort_policy)
+      for (int q = 0; q < nl; q++) if (res[q].status != ABFT_E_DUE) res[q].status = ABFT_E_DUE;
   }
-  if (res->status != ABFT_OK) fail(res->status, "CG finished with status %d after %d iterations", res->status, res->iters);
-  return res->status;
+  if (res[0].status != ABFT_OK)
+    fail(res[0].status, "CG finished with status %d after %d iterations", res[0].status, res[0].iters);
+  return res[0].status;
+}
+
+RankRun make_rank(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                  abft_vec* w, abft_counts* dcnt) {
+  RankRun R;
+  R.ctx = ctx;
+  R.A = A;
+  R.nchunks = nchunks;
+  R.v[0] = b; R.v[1] = x; R.v[2] = r; R.v[3] = p; R.v[4] = w;
+  R.cnt = reinterpret_cast<DevCounts*>(dcnt);
+  return R;
+}
+
+int dist_streams(abft_dist* d) {
+  CUDA_TRY(cudaStreamCreateWithFlags(&d->comm_stream, cudaStreamNonBlocking));
+  CUDA_TRY(cudaEventCreateWithFlags(&d->ev_fork, cudaEventDisableTiming));
+  CUDA_TRY(cudaEventCreateWithFlags(&d->ev_join, cudaEventDisableTiming));
+  return ABFT_OK;
 }
 
 }  // namespace
@@ -673,7 +840,9 @@ extern "C" {
 
 int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
                   abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream) {
-  return cg_core(ctx, nullptr, A, nchunks, 0, b, x, r, p, w, opts, res, dcnt, (cudaStream_t)stream);
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  return cg_run(&R, 1, nullptr, 0, opts, res, (cudaStream_t)stream);
 }
 
 int abft_dist_get_unique_id(void* out128) {
@@ -693,9 +862,35 @@ int abft_dist_init(abft_dist** out, const void* uid, int rank, int nranks, int d
   d->device = device;
   ncclUniqueId id;
   memcpy(&id, uid, sizeof(id));
-  NCCL_TRY(ncclCommInitRank(&d->comm, nranks, id, rank));
-  CUDA_TRY(cudaMalloc(&d->sendbuf, sizeof(double) * 2));
-  CUDA_TRY(cudaMalloc(&d->gathered, sizeof(double) * 2 * nranks));
+  ncclResult_t nr = ncclCommInitRank(&d->comm, nranks, id, rank);
+  if (nr != ncclSuccess) {
+    delete d;
+    return fail(ABFT_E_NCCL, "ncclCommInitRank: %s", ncclGetErrorString(nr));
+  }
+  int e = dist_streams(d);
+  if (!e && cudaMalloc(&d->sendbuf, sizeof(double) * 2) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc sendbuf");
+  if (!e && cudaMalloc(&d->gathered, sizeof(double) * 2 * nranks) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
+  if (e) {
+    abft_dist_destroy(d);
+    return e;
+  }
+  *out = d;
+  return ABFT_OK;
+}
+
+int abft_dist_init_loopback(abft_dist** out, int nranks, int device) {
+  if (!out || nranks < 1 || nranks > 1024) return fail(ABFT_E_INVALID, "bad loopback args");
+  CUDA_TRY(cudaSetDevice(device));
+  abft_dist* d = new abft_dist();
+  d->loopback = 1;
+  d->nranks = nranks;
+  d->device = device;
+  int e = dist_streams(d);
+  if (!e && cudaMalloc(&d->gathered, sizeof(double) * 2 * nranks) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
+  if (e) {
+    abft_dist_destroy(d);
+    return e;
+  }
   *out = d;
   return ABFT_OK;
 }
@@ -705,6 +900,9 @@ int abft_dist_destroy(abft_dist* d) {
   if (d->comm) ncclCommDestroy(d->comm);
   cudaFree(d->sendbuf);
   cudaFree(d->gathered);
+  if (d->ev_fork) cudaEventDestroy(d->ev_fork);
+  if (d->ev_join) cudaEventDestroy(d->ev_join);
+  if (d->comm_stream) cudaStreamDestroy(d->comm_stream);
   delete d;
   return ABFT_OK;
 }
@@ -712,8 +910,23 @@ int abft_dist_destroy(abft_dist* d) {
 int abft_cg_solve_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b,
                        abft_vec* x, abft_vec* r, abft_vec* p, abft_vec* w, const abft_cg_opts* opts,
                        abft_cg_result* res, abft_counts* dcnt, void* stream) {
-  if (!d) return fail(ABFT_E_INVALID, "null dist");
-  return cg_core(ctx, d, A, nchunks, n_halo, b, x, r, p, w, opts, res, dcnt, (cudaStream_t)stream);
+  if (!d || !ctx) return fail(ABFT_E_INVALID, "null dist/ctx");
+  if (d->loopback) return fail(ABFT_E_INVALID, "loopback transport: use abft_cg_solve_loopback");
+  RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  return cg_run(&R, 1, d, n_halo, opts, res, (cudaStream_t)stream);
+}
+
+int abft_cg_solve_loopback(abft_dist* d, abft_ctx* const* ctxs, const abft_csr* const* A, const int* nchunks,
+                           int64_t n_halo, abft_vec* const* vecs, const abft_cg_opts* opts, abft_cg_result* res,
+                           abft_counts* const* dcnt, void* stream) {
+  if (!d || !d->loopback) return fail(ABFT_E_INVALID, "abft_cg_solve_loopback needs a loopback transport");
+  if (!ctxs || !A || !nchunks || !vecs || !dcnt) return fail(ABFT_E_INVALID, "null per-rank arrays");
+  std::vector<RankRun> R(d->nranks);
+  for (int q = 0; q < d->nranks; q++) {
+    abft_vec* const* v = vecs + 5 * q;
+    R[q] = make_rank(ctxs[q], A[q], nchunks[q], v[0], v[1], v[2], v[3], v[4], dcnt[q]);
+  }
+  return cg_run(R.data(), d->nranks, d, n_halo, opts, res, (cudaStream_t)stream);
 }
 
 int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs, int nvec, int scrub,
@@ -739,7 +952,7 @@ int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs
 
 // a4 / a5 as single calls: a scratch CG state carries alpha / beta (never stops)
 static int blas1_setup(abft_ctx* ctx, abft_vec* const* v, int nv, double alpha, double beta, VecArgs& va,
-                       cudaStream_t s) {
+                       cudaStream_t s, int32_t iters = 0) {
   if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
   const char* names[4] = {"x", "p", "r", "w"};
   for (int i = 0; i < nv; i++) {
@@ -755,8 +968,8 @@ static int blas1_setup(abft_ctx* ctx, abft_vec* const* v, int nv, double alpha, 
   h.alpha = alpha;
   h.beta = beta;
   h.max_iters = 0x7FFFFFFF;
-  *ctx->h_state = h;
-  CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
+  h.iters = iters;
+  count_launch(launch_set_state(h, ctx->state, s));
   va = VecArgs{};
   va.n = n;
   va.npad = vec_padded_len(n, v[0]->scheme);
@@ -808,12 +1021,10 @@ int abft_calc_p_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* p_
   VecArgs va;
   int e = check_chunks(A, nchunks);
   if (e) return e;
-  if ((e = blas1_setup(ctx, v, 4, 0.0, beta, va, s))) return e;
   const int vs = p_prev->scheme;
   if (vec_padded_len(1, vs) != 1) return fail(ABFT_E_SHAPE, "fused calc_p + SpMV: vector scheme with group size > 1");
   // the kernel takes the fused branch when state.iters > 0
-  ctx->h_state->iters = 1;
-  CUDA_TRY(cudaMemcpyAsync(ctx->state, ctx->h_state, sizeof(CgState), cudaMemcpyHostToDevice, s));
+  if ((e = blas1_setup(ctx, v, 4, 0.0, beta, va, s, 1))) return e;
   DevCounts* cnt = reinterpret_cast<DevCounts*>(dcnt);
   uint64_t* pc = reinterpret_cast<uint64_t*>(p_out->data);
   uint64_t* rf = reinterpret_cast<uint64_t*>(r->data);

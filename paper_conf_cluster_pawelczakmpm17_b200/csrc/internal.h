@@ -55,6 +55,9 @@ struct RedArgs {
 struct SpmvArgs {
   int64_t nrows, ncols, nnz, row_base, col_base, n_in, npad_in, npad_out, rb_offset;
   int64_t stencil_n;  // > 0: 5-point stencil row stride (tiled fast path)
+  // tiled path only: launch the tile rows [ty_lo, ty_hi) of the chunk (ty_hi =
+  // 0: all) — the interior / boundary split that overlaps the halo exchange
+  int64_t ty_lo, ty_hi;
   uint64_t* val;
   uint32_t* col;
   uint32_t* rowptr;
@@ -98,11 +101,16 @@ struct VecArgs {
 
 // PDL for the CG driver's iteration launches
 void set_pdl(bool on);
+// write the device CG state from a by-value launch argument (no host staging buffer)
+int launch_set_state(const CgState& h, CgState* dst, cudaStream_t s);
 // launchers (kernels.cu); each returns the number of kernels launched
 int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, bool dot, cudaStream_t s);
 // -1: a fused-calc_p launch (a.p_cur set) could not run
 // can this chunk take the fused-calc_p tiled SpMV (G = 1 vector scheme, stencil layout)?
 bool spmv_fusable(const SpmvArgs& a, int vs);
+// will this chunk run on the tiled stencil kernel (so a tile-row split is possible)?
+bool spmv_tileable(const SpmvArgs& a, int vs);
+int64_t spmv_tile_rows(const SpmvArgs& a);   // tile rows of a tileable chunk
 int launch_calc_ur(const VecArgs& a, int vs, cudaStream_t s);
 int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s);
 int launch_init_r(const VecArgs& a, int vs, cudaStream_t s);

@@ -21,8 +21,16 @@
 
 namespace abft {
 
-bool g_pdl = false;
+thread_local bool g_pdl = false;
 void set_pdl(bool on) { g_pdl = on; }
+
+// CG scalars written by a kernel (arguments captured at launch), never by an
+// async copy of a host buffer that a later call could overwrite first.
+static __global__ void k_set_state(CgState h, CgState* dst) { *dst = h; }
+int launch_set_state(const CgState& h, CgState* dst, cudaStream_t s) {
+  k_set_state<<<1, 1, 0, s>>>(h, dst);
+  return 1;
+}
 
 // per-ES SpMV launchers live in spmv_es*.cu (parallel compilation)
 bool spmv_es_none(const SpmvArgs&, int, int, bool, cudaStream_t);

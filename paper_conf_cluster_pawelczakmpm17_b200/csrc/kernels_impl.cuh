@@ -12,7 +12,7 @@ namespace abft {
 
 // Host: launch k with the programmatic-stream-serialization attribute when the
 // CG driver turned PDL on (set_pdl), else a plain launch.
-extern bool g_pdl;
+extern thread_local bool g_pdl;   // per host thread: one solve's PdlGuard never leaks into another thread's launches
 template <typename... KArgs, typename... Args>
 static inline void launch_k(void (*k)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t s, Args... args) {
   if (!g_pdl) {
@@ -795,7 +795,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   const int64_t ny = a.nrows / n;
   const int64_t tiles_x = n >> 8;
   const int64_t tx0 = (blockIdx.x % tiles_x) << 8;
-  const int64_t ty0 = (int64_t)(blockIdx.x / tiles_x) * TILE_TY;
+  const int64_t ty0 = ((int64_t)(blockIdx.x / tiles_x) + a.ty_lo) * TILE_TY;
   // ---- 0. producer: barriers, then the first TILE_NST passes in flight (the
   // matrix: loaded before the PDL grid dependency resolves)
   if (threadIdx.x == 0) {
@@ -854,7 +854,9 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
       s_args.beta_f = fz ? a.state->beta : 0.0;
     }
   }
-  if (SLICE || VS == CRC32C) __syncthreads();
+  // every warp waits on winbar / the stage barriers below: thread 0's
+  // mbarrier.init (and the SMEM tables) must be visible to the whole CTA first
+  __syncthreads();
   const int stop_v = a.state ? a.state->stop : 0;
   const int mode = spmv_mode(a);
   // G = 1, not building p_k: the raw `in` window arrives by one TMA box

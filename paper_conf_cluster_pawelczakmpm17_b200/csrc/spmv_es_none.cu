@@ -12,4 +12,7 @@ bool spmv_fusable(const SpmvArgs& a, int vs) {
   return (vs == NONE || vs == SED || vs == SECDED64) && tile_ok(a, vs) && tmap_encoder() != nullptr;
 }
 
+bool spmv_tileable(const SpmvArgs& a, int vs) { return tile_ok(a, vs) && tmap_encoder() != nullptr; }
+int64_t spmv_tile_rows(const SpmvArgs& a) { return (a.nrows / a.stencil_n + TILE_TY - 1) / TILE_TY; }
+
 }  // namespace abft

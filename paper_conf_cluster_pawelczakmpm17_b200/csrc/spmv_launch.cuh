@@ -2,6 +2,7 @@
 // generic CSR kernel), instantiated per element scheme in spmv_es_*.cu.
 #pragma once
 #include <cudaTypedefs.h>
+#include <atomic>
 #include <cstdlib>
 
 #include "kernels_impl.cuh"
@@ -18,16 +19,14 @@ static bool tile_ok(const SpmvArgs& a, int vs) {
 }
 // The driver's tensor-map encoder, resolved once through the runtime (no -lcuda).
 static PFN_cuTensorMapEncodeTiled_v12000 tmap_encoder() {
-  static PFN_cuTensorMapEncodeTiled_v12000 fn = nullptr;
-  static bool tried = false;
-  if (!tried) {
-    tried = true;
+  static const PFN_cuTensorMapEncodeTiled_v12000 fn = [] {   // thread-safe one-time lookup
     void* p = nullptr;
     cudaDriverEntryPointQueryResult q;
     if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &p, cudaEnableDefault, &q) == cudaSuccess &&
         q == cudaDriverEntryPointSuccess)
-      fn = reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(p);
-  }
+      return reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(p);
+    return static_cast<PFN_cuTensorMapEncodeTiled_v12000>(nullptr);
+  }();
   return fn;
 }
 // The chunk's element arrays viewed as [ny grid rows][5n elements]; box = one
@@ -73,14 +72,22 @@ static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   TileMaps tm;
   if (!tile_maps(a, &tm)) return false;
   const size_t smem = tile_smem<ES, RS, VS>();
-  static bool attr = false;
-  if (!attr) {  // set before first use: never inside a later CUDA-graph capture
+  // function attributes are per device: set them once per device (thread
+  // safe), before first use there, so never inside a later CUDA-graph capture
+  static std::atomic<uint64_t> attr_devs{0};
+  int dev = 0;
+  cudaGetDevice(&dev);
+  const uint64_t bit = 1ull << (dev & 63);
+  if (!(attr_devs.load(std::memory_order_acquire) & bit)) {
     cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, DOT, FUSED>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     cudaFuncSetAttribute(k_spmv_tile<ES, RS, VS, DOT, FUSED>, cudaFuncAttributePreferredSharedMemoryCarveout, 100);
-    attr = true;
+    attr_devs.fetch_or(bit, std::memory_order_release);
   }
   const int64_t ny = a.nrows / a.stencil_n;
-  const int64_t blocks = (a.stencil_n / 256) * ((ny + TILE_TY - 1) / TILE_TY);
+  const int64_t nty = (ny + TILE_TY - 1) / TILE_TY;
+  const int64_t lo = a.ty_lo, hi = a.ty_hi > 0 ? a.ty_hi : nty;
+  const int64_t blocks = (a.stencil_n / 256) * (hi - lo);
+  if (blocks <= 0) return true;
   launch_k(k_spmv_tile<ES, RS, VS, DOT, FUSED>, (unsigned)blocks, 256, smem, s, a, tm);
   return true;
 }

@@ -9,7 +9,7 @@ python -c "import __graft_entry__ as g; g.build()" > gpurun_out/build_$TAG.log 2
 for w in $WHAT; do
   case $w in
   tests)
-    timeout 1200 python -m pytest tests -m gpu -q --tb=short --maxfail=30 > gpurun_out/tests_$TAG.log 2>&1
+    timeout 2400 python -m pytest tests -m gpu -q --tb=short --maxfail=30 --durations=25 > gpurun_out/tests_$TAG.log 2>&1
     tail -30 gpurun_out/tests_$TAG.log ;;
   smoke)
     timeout 300 python __graft_entry__.py --smoke > gpurun_out/smoke_$TAG.log 2>&1; tail -5 gpurun_out/smoke_$TAG.log ;;
@@ -27,6 +27,20 @@ for w in $WHAT; do
     timeout 900 ncu --set full --clock-control none --import-source on -k regex:'k_spmv' -s 2 -c 4 \
       -o gpurun_out/prof_$TAG -f python bench.py --steps 1 --warmup 0 --no-e2e --no-cpu-baseline --max-iters 3 > gpurun_out/ncu_full_$TAG.log 2>&1
     tail -3 gpurun_out/ncu_full_$TAG.log ;;
+  sanitize)
+    for tool in memcheck racecheck synccheck initcheck; do
+      timeout 1500 compute-sanitizer --tool $tool --print-limit 20 --error-exitcode 9 python tools/sanitize_run.py \
+        > gpurun_out/sanitize_${tool}_$TAG.log 2>&1
+      echo "$tool rc=$?"; tail -4 gpurun_out/sanitize_${tool}_$TAG.log
+    done ;;
+  ncutma)
+    # kernel-replay capture of the DEFAULT (3-D TMA window) protected SpMV and its unprotected twin
+    timeout 900 ncu --set full --clock-control none --import-source on -k regex:'k_spmv_tile' -s 3 -c 1 \
+      -o gpurun_out/prof_tma_prot_$TAG -f python tools/spmv_time.py --reps 2 --schemes 2 > gpurun_out/ncu_tma_prot_$TAG.log 2>&1
+    tail -3 gpurun_out/ncu_tma_prot_$TAG.log
+    timeout 900 ncu --set full --clock-control none --import-source on -k regex:'k_spmv_tile' -s 3 -c 1 \
+      -o gpurun_out/prof_tma_twin_$TAG -f python tools/spmv_time.py --reps 2 --schemes 0 > gpurun_out/ncu_tma_twin_$TAG.log 2>&1
+    tail -3 gpurun_out/ncu_tma_twin_$TAG.log ;;
   sweep)
     timeout 1500 python tools/sweep.py --out gpurun_out/sweep_$TAG.json > gpurun_out/sweep_$TAG.log 2>&1; tail -4 gpurun_out/sweep_$TAG.log ;;
   big)
