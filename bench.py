@@ -88,13 +88,14 @@ class ClockSampler:
 
 
 # ------------------------------------------------------------------ problem
-def chunk_layout(grid: int, rank: int, world: int, chunk_rows=None):
-    """This rank's row-block chunks (no arrays): global grid rows, row_base /
-    col_base in the rank's halo-extended vector, rows and column-window width
-    (<= 2^24 for the 24-bit element index, reading R7)."""
+def chunk_layout(n: int, ny: int, rank: int, world: int, chunk_rows=None):
+    """This rank's row-block chunks (no arrays) of an n x ny grid split into
+    `world` strips of ny/world grid rows: global grid rows, row_base / col_base
+    in the rank's halo-extended vector, rows and column-window width (<= 2^24
+    for the 24-bit element index, reading R7)."""
     import gen
-    n = grid
-    y0r, y1r = rank * grid, (rank + 1) * grid
+    rows = ny // world
+    y0r, y1r = rank * rows, (rank + 1) * rows
     halo = n if world > 1 else 0
     out = []
     for (c0, c1, cb) in gen.chunk_plan(n, y1r - y0r, chunk_rows=chunk_rows, halo=world > 1):
@@ -107,17 +108,19 @@ def chunk_layout(grid: int, rank: int, world: int, chunk_rows=None):
     return out
 
 
-def build_problem(grid: int, rank: int, world: int, device, chunk_rows=None):
-    """Raw (unencoded) device arrays of this rank's rows, as row-block chunks
-    whose column windows fit the 24-bit element index (reading R7)."""
+def build_problem(n: int, ny: int, rank: int, world: int, device, chunk_rows=None):
+    """Raw (unencoded) device arrays of this rank's strip of the n x ny G-TEA
+    grid, as row-block chunks whose column windows fit the 24-bit element index
+    (reading R7)."""
     import torch
     import gen
-    n = grid
-    ny = grid * world
-    y0r, y1r = rank * grid, (rank + 1) * grid
+    if ny % world:
+        raise ValueError(f"{ny} grid rows do not split into {world} equal strips")
+    rows = ny // world
+    y0r, y1r = rank * rows, (rank + 1) * rows
     halo = n if world > 1 else 0
     chunks = []
-    for L in chunk_layout(grid, rank, world, chunk_rows):
+    for L in chunk_layout(n, ny, rank, world, chunk_rows):
         val, col, rowptr = gen.strip_csr(n, L["gy0"], L["gy1"], ny=ny, device=device,
                                          col_offset=L["row_base"] - L["col_base"])
         chunks.append(dict(val=val.contiguous(), col=col.to(torch.int32).contiguous(),
@@ -255,35 +258,67 @@ def traffic_matches(t, grid, world, fused):
 
 
 # ------------------------------------------------------------------ oracle legs
-def oracle_sample(grid_sample=512, iters=3):
-    """The CPU oracle (never tuned) on a bounded sample: `iters` protected CG
-    iterations on a grid_sample^2 G-TEA problem with the config-2 schemes,
-    single-threaded; scaled to the 4096^2 workload by row count."""
+UNIT = "CG it/s (4096^2-equivalent)"
+
+
+def cpu_info():
+    model = None
+    try:
+        with open("/proc/cpuinfo") as f:
+            for line in f:
+                if line.startswith("model name"):
+                    model = line.split(":", 1)[1].strip()
+                    break
+    except Exception:
+        pass
+    return {"model": model, "nproc": os.cpu_count()}
+
+
+def oracle_sample(strip_rows=128, iters=3, grid=4096):
+    """The CPU oracle (never tuned) on a bounded sample of the 4096^2 workload
+    itself: the grid rows [grid/2, grid/2 + strip_rows) of the 4096^2 G-TEA
+    matrix (config-2 schemes, read from their own input window), through `iters`
+    CG iterations' worth of the oracle's hot-path calls (protected SpMV + p.w,
+    calc_ur, calc_p), single-threaded and pinned to one host core; scaled to the
+    whole 4096^2 iteration by rows.  Returns (it/s, cores, sample text)."""
     import numpy as np
     import gen
     import oracle as orc
-    n = grid_sample
-    v, c, r = gen.tealeaf_csr(n)
-    N = n * n
-    A = orc.Matrix(v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32), N, N, orc.SECDED64,
-                   orc.SECDED64)
+    n = grid
+    y0, y1 = n // 2, n // 2 + strip_rows
+    w0, w1 = y0 - 1, y1 + 1
+    rows = strip_rows * n
+    v, c, r = gen.strip_csr(n, y0, y1, ny=n, col_offset=n)
+    S = orc.SECDED64
+    A = orc.Matrix(v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32), rows, (w1 - w0) * n, S, S,
+                   row_base=n, col_base=0)
     A.encode()
-    b = gen.tealeaf_rhs(n).numpy()
-    B = orc.vec_encode(b, orc.SECDED64)
-    X = B.copy()
-    R, Pv, W = (np.zeros_like(B) for _ in range(3))
-    # init (untimed) then time `iters` iterations: the oracle has no per-iteration
-    # entry, so time init+k and init+0 and take the difference
-    t0 = time.perf_counter()
-    orc.cg_solve(A, B.copy(), X.copy(), R, Pv, W, orc.SECDED64, 0.0, 0, 1, None)
-    t1 = time.perf_counter()
-    orc.cg_solve(A, B.copy(), X.copy(), R, Pv, W, orc.SECDED64, 0.0, iters, 1, None)
-    t2 = time.perf_counter()
-    per_iter = ((t2 - t1) - (t1 - t0)) / iters
-    scale = (4096 * 4096) / N
-    its = 1.0 / (per_iter * scale)
-    return its, f"{iters} protected CG iterations (E-SECDED+R-SECDED64+V-SECDED64) on a {n}^2 G-TEA grid, " \
-                f"per-iteration time scaled by rows to 4096^2 ({per_iter:.3f} s/iter at {n}^2)"
+    W = (w1 - w0) * n
+    p = orc.vec_encode(gen.uniform_pm1(W, 5), S)
+    x = orc.vec_encode(gen.uniform_pm1(rows, 6), S)
+    rv = orc.vec_encode(gen.uniform_pm1(rows, 7), S)
+    out = np.zeros(W, dtype=np.uint64)
+    old = os.sched_getaffinity(0)
+    core = min(old)
+    try:
+        os.sched_setaffinity(0, {core})
+        t0 = time.perf_counter()
+        for _ in range(iters):
+            orc.spmv(A, p, W, S, out, W, None, want_dot=True)
+            w = out[n:n + rows].copy()
+            pl = p[n:n + rows].copy()
+            orc.calc_ur(x, pl, rv, w, rows, S, 1e-3, None)
+            orc.calc_p(pl, rv, rows, S, 0.5, None)
+        per_iter = (time.perf_counter() - t0) / iters
+    finally:
+        os.sched_setaffinity(0, old)
+    its = 1.0 / (per_iter * (n * n) / rows)
+    ci = cpu_info()
+    sample = (f"{iters} CG iterations of the oracle's hot-path calls (protected SpMV + p.w, calc_ur, calc_p; "
+              f"E-SECDED + R-SECDED64 + V-SECDED64) on grid rows [{y0}, {y1}) of the {n}^2 G-TEA matrix "
+              f"({rows} of {n * n} rows), {per_iter:.3f} s per sampled iteration, scaled by rows to the whole "
+              f"{n}^2 iteration; pinned to host core {core} ({ci['model']}, nproc {ci['nproc']})")
+    return its, 1, sample
 
 
 def run_reference(args):
@@ -293,22 +328,21 @@ def run_reference(args):
     vals = []
     sample = ""
     for _ in range(args.warmup):
-        oracle_sample(args.oracle_grid, 1)
+        oracle_sample(32, 1)
     t0 = time.perf_counter()
     for _ in range(args.steps):
-        v, sample = oracle_sample(args.oracle_grid, 2)
+        v, cores, sample = oracle_sample(args.oracle_rows, 1)
         vals.append(v)
     wall = time.perf_counter() - t0
     val = statistics.median(vals)
-    line = {"impl": "reference", "metric": METRIC, "value": val, "unit": "CG it/s (4096^2, protected)",
+    line = {"impl": "reference", "metric": METRIC, "value": val, "unit": UNIT,
             "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
             "ms_per_step": 1000.0 * wall / max(args.steps, 1), "higher_is_better": True, "scaling": "weak",
             "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-            "config": {"workload": "tealeaf-4096x4096-cg-full-ecc", "grid": 4096, "sample_grid": args.oracle_grid},
-            "cpu_baseline": {"value": val, "unit": "CG it/s (4096^2, protected)", "cores": 1, "kind": "oracle",
-                             "sample": sample},
-            "e2e": {"value": val, "unit": "CG it/s (4096^2, protected)", "h2d_bytes_per_step": 0,
-                    "d2h_bytes_per_step": 0}}
+            "config": {"workload": "tealeaf-4096x4096-cg-full-ecc", "grid": 4096, "sample_strip_rows": args.oracle_rows},
+            "cpu_baseline": {"value": val, "unit": UNIT, "cores": cores, "kind": "oracle", "sample": sample,
+                             "cpu": cpu_info()},
+            "e2e": {"value": val, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
 
 
@@ -319,10 +353,13 @@ def main():
     ap.add_argument("--steps", type=int, default=3)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
-    ap.add_argument("--grid", type=int, default=4096)
+    ap.add_argument("--grid", type=int, default=None, help="grid side (default 4096; 16384 with --mode strong)")
     ap.add_argument("--tol", type=float, default=1e-10)
     ap.add_argument("--max-iters", type=int, default=20000)
-    ap.add_argument("--oracle-grid", type=int, default=512)
+    ap.add_argument("--oracle-rows", type=int, default=64, help="grid rows of the 4096^2 strip the oracle legs time")
+    ap.add_argument("--mode", default="weak", choices=["weak", "strong"],
+                    help="N > 1: weak = a grid x grid strip per GPU (config 2 per GPU); strong = config 4, one "
+                         "fixed grid x grid problem (default grid 16384) split into N strips")
     ap.add_argument("--chunk-rows", type=int, default=None, help="grid rows per row-block chunk (default: fit 2^24 cols)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
@@ -332,6 +369,8 @@ def main():
     args = ap.parse_args()
     if args.impl == "reference":
         return run_reference(args)
+    if args.grid is None:
+        args.grid = 16384 if args.mode == "strong" else 4096
 
     import torch
     import torch.distributed as dist
@@ -344,7 +383,8 @@ def main():
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     from paper_conf_cluster_pawelczakmpm17_b200 import abft
 
-    P = build_problem(args.grid, rank, world, torch.device("cuda", local), args.chunk_rows)
+    ny = args.grid * world if args.mode == "weak" else args.grid
+    P = build_problem(args.grid, ny, rank, world, torch.device("cuda", local), args.chunk_rows)
     ctx = abft.Context(local)
     # fused calc_p (opt-in) runs on the single-GPU tiled path (the dist path exchanges p halos unfused)
     fused = args.fuse and not dist_on
@@ -399,7 +439,7 @@ def main():
         r_e = timed(prot, args.steps, 1, args.tol, args.max_iters, dist_on, host=host, out_host=out_host)
         h2d = sum(t.numel() * t.element_size() for c in host["chunks"] for t in c) + host["b"].numel() * 8
         e2e = {"value": world * r_e["iters"] / (r_e["ms"] / 1000.0) * P["N"] / float(4096 * 4096),
-               "unit": "CG it/s (4096^2-equivalent)",
+               "unit": UNIT,
                "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": P["N"] * 8}
         del prot
 
@@ -424,17 +464,18 @@ def main():
     line = {
         "metric": METRIC,
         "value": world * its,
-        "unit": "CG it/s (4096^2-equivalent)",
+        "unit": UNIT,
         "n_gpus": world,
         "steps": args.steps,
         "warmup": args.warmup,
         "ms_per_step": r_p["ms"] / args.steps,
         "higher_is_better": True,
-        "scaling": "weak",
+        "scaling": args.mode if world > 1 else "weak",
         "vs_baseline": None,
         "dtype": "f64",
         "data": "synthetic",
-        "config": {"workload": f"tealeaf-{args.grid}x{args.grid}-cg-full-ecc", "grid": args.grid, "rows_per_gpu": N,
+        "config": {"workload": f"tealeaf-{args.grid}x{ny}-cg-full-ecc", "grid": args.grid, "grid_rows": ny,
+                   "rows_per_gpu": N,
                    "chunks": len(P["chunks"]),
                    "schemes": {"elements": "E-SECDED", "rowptr": "R-SECDED64", "vectors": "V-SECDED64"},
                    "tol": args.tol, "iters_per_step": r_p["iters"] / args.steps,
@@ -466,9 +507,9 @@ def main():
         "e2e": e2e,
     }
     if world == 1 and not args.no_cpu_baseline:
-        v, sample = oracle_sample(args.oracle_grid, 3)
-        line["cpu_baseline"] = {"value": v, "unit": "CG it/s (4096^2, protected)", "cores": 1, "kind": "oracle",
-                                "sample": sample}
+        v, cores, sample = oracle_sample(2 * args.oracle_rows, 3)
+        line["cpu_baseline"] = {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle", "sample": sample,
+                                "cpu": cpu_info()}
     print(json.dumps(line), flush=True)
     if dist_on:
         dist.destroy_process_group()

@@ -79,6 +79,8 @@ def lib():
                                   C.c_int, C.c_void_p, C.c_void_p]
         L.or_cg_solve_ex.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
                                      C.c_int, C.c_void_p, C.c_void_p, C.c_int]
+        L.or_cg_solve_sched.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
+                                        C.c_int, C.c_void_p, C.c_void_p, C.c_int, C.c_void_p, C.c_int]
         L.or_vec_masked.argtypes = [u64p, C.c_int64, C.c_int, dp]
         L.or_round_k.restype = C.c_uint64
         L.or_round_k.argtypes = [C.c_uint64, C.c_int]
@@ -279,4 +281,33 @@ def cg_solve(A: Matrix, b, x, r, p, w, scheme, tol=1e-10, max_iters=10000, due_p
     st = lib().or_cg_solve_ex(C.byref(s), _p(b, C.c_uint64), _p(x, C.c_uint64), _p(r, C.c_uint64),
                               _p(p, C.c_uint64), _p(w, C.c_uint64), scheme, tol, max_iters, due_policy, C.byref(res),
                               counts.ctypes.data if counts is not None else None, int(check_interval))
+    return st, res
+
+
+# O10 fault targets (S§8(c) O10): storage words of val (64-bit), col, rowptr
+# (32-bit) and the CG vectors b, x, r, p, w (64-bit)
+F_VAL, F_COL, F_ROWPTR, F_B, F_X, F_R, F_P, F_W = range(8)
+FAULT_DTYPE = np.dtype([("iter", "<i4"), ("target", "<i4"), ("word", "<i8"), ("bit", "<i4"), ("pad", "<i4")])
+
+
+def fault_schedule(entries) -> np.ndarray:
+    """[(iteration k, target, storage-word index, bit), ...] -> packed schedule."""
+    out = np.zeros(len(entries), dtype=FAULT_DTYPE)
+    for i, (k, t, w, b) in enumerate(entries):
+        out[i] = (k, t, w, b, 0)
+    return out
+
+
+def cg_solve_sched(A: Matrix, b, x, r, p, w, scheme, tol=1e-10, max_iters=10000, due_policy=1, counts=None,
+                   check_interval=1, faults=None):
+    """Protected CG with an O10 fault schedule: fault (k, target, word, bit) is
+    XOR-ed into the stored bits before init (k = 0) or before iteration k's
+    SpMV (S§8(c) O10)."""
+    s = A.cstruct()
+    res = CGResult()
+    f = faults if faults is not None else np.zeros(0, dtype=FAULT_DTYPE)
+    st = lib().or_cg_solve_sched(C.byref(s), _p(b, C.c_uint64), _p(x, C.c_uint64), _p(r, C.c_uint64),
+                                 _p(p, C.c_uint64), _p(w, C.c_uint64), scheme, tol, max_iters, due_policy,
+                                 C.byref(res), counts.ctypes.data if counts is not None else None,
+                                 int(check_interval), f.ctypes.data if len(f) else None, len(f))
     return st, res

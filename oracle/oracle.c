@@ -15,6 +15,8 @@
  *         CG         TeaLeaf CG (ref [19]), DESIGN.md §4
  *         interval   "less frequent correctness checking" P:398-425 (§VI-A.2),
  *                    DESIGN.md §3.9 (reading R27)
+ *         faults     O10 scheduled bit flips (S§8(c) O10): XOR before init /
+ *                    before iteration k's SpMV, or_cg_solve_sched
  *         CRC fix    1EC4ED single-bit correction of a failing CRC32C codeword
  *                    P:260-278 (§IV; HD 6 for 178..5243-bit codewords,
  *                    P:268-271), DESIGN.md §3.5 (reading R9)
@@ -878,11 +880,33 @@ static int access_mode(int64_t a, int interval) {
   return (a % interval == 0) ? M_DETECT : M_RANGE;
 }
 
+/* ---------------------------------------------------------- O10 injection
+ * S§8(c) O10: a fault is (target, storage-word index, bit), applied as an XOR
+ * to the stored bits; a schedule is a list of (iteration k, fault): k = 0 is
+ * applied before init, k >= 1 before iteration k's SpMV.  Targets: 0 val
+ * (64-bit words), 1 col, 2 rowptr (32-bit words), 3 b, 4 x, 5 r, 6 p, 7 w
+ * (64-bit words). */
+typedef struct { int32_t iter; int32_t target; int64_t word; int32_t bit; int32_t pad; } or_fault;
+
+static void apply_faults(or_csr* A, uint64_t* v[5], const or_fault* f, int nf, int k) {
+  for (int i = 0; i < nf; i++) {
+    if (f[i].iter != k) continue;
+    int t = f[i].target;
+    if (t == 0) A->val[f[i].word] ^= 1ull << f[i].bit;
+    else if (t == 1) A->col[f[i].word] ^= 1u << f[i].bit;
+    else if (t == 2) A->rowptr[f[i].word] ^= 1u << f[i].bit;
+    else if (t >= 3 && t <= 7) v[t - 3][f[i].word] ^= 1ull << f[i].bit;
+  }
+}
+
 static int cg_run(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
-                  int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval) {
+                  int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval,
+                  const or_fault* faults, int nfaults) {
   int64_t n = A->nrows;
   double rr0, rro, rrn = 0.0, pw;
+  uint64_t* vecs[5] = {b, x, r, p, w};
   res->iters = 0; res->status = OK; res->rr0 = 0.0; res->rrn = 0.0;
+  apply_faults(A, vecs, faults, nfaults, 0);
   int64_t dues = or_spmv_mode(A, x, n, vs, w, n, cnt, NULL, access_mode(0, interval));
   dues += or_cg_init_r(b, w, r, p, n, vs, cnt, &rr0);
   res->rr0 = rr0; res->rrn = rr0;
@@ -890,6 +914,7 @@ static int cg_run(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p,
   if (rr0 == 0.0) return OK;
   rro = rr0;
   for (int k = 1; k <= max_iters; k++) {
+    apply_faults(A, vecs, faults, nfaults, k);
     dues = or_spmv_mode(A, p, n, vs, w, n, cnt, &pw, access_mode(k, interval));
     double alpha = rro / pw;
     dues += or_calc_ur(x, p, r, w, n, vs, alpha, cnt, &rrn);
@@ -912,15 +937,20 @@ static int cg_run(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p,
  * matrix "just in case N does not divide the number of iterations performed"
  * (P:418-421); a DUE found there turns OK / NOT_CONVERGED into E_DUE under
  * policy abort. */
-int or_cg_solve_ex(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
-                   int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval) {
+int or_cg_solve_sched(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs,
+                      double tol, int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval,
+                      const or_fault* faults, int nfaults) {
   init_instances();
-  int st = cg_run(A, b, x, r, p, w, vs, tol, max_iters, due_policy, res, cnt, interval);
+  int st = cg_run(A, b, x, r, p, w, vs, tol, max_iters, due_policy, res, cnt, interval, faults, nfaults);
   if (interval > 1 && res->iters % interval != 0) {
     int64_t dues = or_check_csr(A, cnt, 2);
     if (dues && due_policy == 0 && st != E_DUE) { res->status = E_DUE; st = E_DUE; }
   }
   return st;
+}
+int or_cg_solve_ex(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
+                   int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval) {
+  return or_cg_solve_sched(A, b, x, r, p, w, vs, tol, max_iters, due_policy, res, cnt, interval, NULL, 0);
 }
 int or_cg_solve(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
                 int max_iters, int due_policy, or_cg_result* res, counts_t* cnt) {

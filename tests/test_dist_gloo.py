@@ -152,16 +152,20 @@ def test_distributed_cg_matches_single_process(world, scheme_name):
 
 @pytest.mark.parametrize("world", [1, 2, 4, 8])
 @pytest.mark.parametrize("grid", [4096, 8192, 16384])
-def test_bench_chunk_layout_fits_element_index(world, grid):
-    """bench.py's per-rank chunks (weak scaling: a grid-row strip per rank plus
-    ghost rows) cover the strip and keep every column window within E-SECDED's
-    24-bit index and R-SECDED's 28-bit nnz (reading R7), at the sizes the driver
-    runs (no arrays are built)."""
+@pytest.mark.parametrize("mode", ["weak", "strong"])
+def test_bench_chunk_layout_fits_element_index(world, grid, mode):
+    """bench.py's per-rank chunks (weak scaling: a grid x grid strip per rank of
+    a grid x grid*world grid; strong scaling, config 4: grid/world rows of a
+    fixed grid x grid grid) cover the strip and keep every column window within
+    E-SECDED's 24-bit index and R-SECDED's 28-bit nnz (reading R7), at the
+    sizes the driver runs (no arrays are built)."""
     import bench
+    ny = grid * world if mode == "weak" else grid
+    rows = ny // world
     for rank in {0, world // 2, world - 1}:
-        L = bench.chunk_layout(grid, rank, world)
+        L = bench.chunk_layout(grid, ny, rank, world)
         halo = grid if world > 1 else 0
-        assert L[0]["row_base"] == halo and L[0]["gy0"] == rank * grid and L[-1]["gy1"] == (rank + 1) * grid
+        assert L[0]["row_base"] == halo and L[0]["gy0"] == rank * rows and L[-1]["gy1"] == (rank + 1) * rows
         for a, b in zip(L[:-1], L[1:]):
             assert a["gy1"] == b["gy0"] and b["row_base"] == a["row_base"] + a["nrows"]
         for c in L:
@@ -169,7 +173,7 @@ def test_bench_chunk_layout_fits_element_index(world, grid):
             assert c["nrows"] % 256 == 0 and (c["row_base"] - halo) % 256 == 0
             # the window covers the chunk's rows and one grid row either side (ghost rows for world > 1)
             assert c["col_base"] <= max(0, c["row_base"] - grid)
-            assert c["col_base"] + c["ncols"] >= min(c["row_base"] + c["nrows"] + grid, halo + grid * grid + halo)
+            assert c["col_base"] + c["ncols"] >= min(c["row_base"] + c["nrows"] + grid, halo + grid * rows + halo)
 
 
 def test_bench_traffic_null_for_failed_capture(tmp_path, monkeypatch):

@@ -40,7 +40,7 @@ def main():
     import bench
     from paper_conf_cluster_pawelczakmpm17_b200 import abft
     torch.cuda.set_device(0)
-    P = bench.build_problem(a.grid, 0, 1, torch.device("cuda", 0))
+    P = bench.build_problem(a.grid, a.grid, 0, 1, torch.device("cuda", 0))
     ctx = abft.Context(0)
     names = ["NONE", "SED", "SECDED64", "SECDED128", "CRC32C"]
     configs = [("all", "NONE", ("NONE", "NONE", "NONE"), 1)]
