@@ -348,7 +348,8 @@ def test_8192_five_chunk_spmv_sampled(abft, ctx):
     rng = np.random.default_rng(8192)
     xo = periodic_encoded(N, S, 81)
     # sampled strips: 3 grid rows each side of every chunk boundary, the first and last rows
-    strips = [(0, 3), (n - 3, n)] + [(y0 - 3, y0 + 3) for (y0, _, _) in plan[1:]]
+    # (each strip lies inside one chunk: the rows on both sides of a boundary are two strips)
+    strips = [(0, 3), (n - 3, n)] + [s for (y0, _, _) in plan[1:] for s in ((y0 - 3, y0), (y0, y0 + 3))]
     cells = []
     for (y0, y1) in strips:
         for y in range(y0, y1):
