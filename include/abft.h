@@ -179,6 +179,21 @@ int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs
 /* Fault injection (not in the paper; the harness of S§3.4): XOR one stored bit
  * at bit_offset of the device buffer dev_base.  Stream-ordered. */
 int abft_inject_bitflip(abft_ctx* ctx, void* dev_base, uint64_t bit_offset, void* stream);
+/* Scheduled fault injection (S§8(c) O10, the harness of BASELINE configs 1 and
+ * 5): fault i XORs bit `bit` of storage word `word` of `target` — matrix chunk
+ * `chunk`'s val (64-bit words), col or rowptr (32-bit words), or the CG vector
+ * b, x, r, p, w (64-bit words, vecs[target - ABFT_F_B]) — before init (iter 0)
+ * or before iteration `iter`'s SpMV, inside the solve (a device-side kernel
+ * reads the iteration counter, so CUDA-graph replays apply it too).  The
+ * schedule (device copy owned by ctx) applies to every later abft_cg_solve /
+ * abft_cg_solve_dist on ctx with the SAME matrix and vector buffers, until
+ * replaced; nfaults = 0 clears it.  A schedule turns the fused calc_p off.
+ * Errors: ABFT_E_INVALID (bad target / chunk / word / bit), ABFT_E_CUDA. */
+typedef enum { ABFT_F_VAL = 0, ABFT_F_COL = 1, ABFT_F_ROWPTR = 2, ABFT_F_B = 3, ABFT_F_X = 4, ABFT_F_R = 5,
+               ABFT_F_P = 6, ABFT_F_W = 7 } abft_fault_target;
+typedef struct { int32_t iter; int32_t target; int64_t word; int32_t bit; int32_t chunk; } abft_fault;
+int abft_ctx_set_faults(abft_ctx* ctx, const abft_fault* faults, int nfaults, const abft_csr* A, int nchunks,
+                        abft_vec* const* vecs /* [5]: b, x, r, p, w */);
 
 /* Copy the device counters to host_out[ABFT_T_COUNT*ABFT_SCHEME_COUNT].  Syncs. */
 int abft_counts_read(const abft_counts* dcnt, abft_counts* host_out, void* stream);

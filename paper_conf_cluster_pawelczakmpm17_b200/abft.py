@@ -39,6 +39,15 @@ class CGOpts(C.Structure):
                 ("check_interval", C.c_int32)]
 
 
+class Fault(C.Structure):
+    _fields_ = [("iter", C.c_int32), ("target", C.c_int32), ("word", C.c_int64), ("bit", C.c_int32),
+                ("chunk", C.c_int32)]
+
+
+# abft_fault_target (S§8(c) O10)
+F_VAL, F_COL, F_ROWPTR, F_B, F_X, F_R, F_P, F_W = range(8)
+
+
 class CGResult(C.Structure):
     _fields_ = [("iters", C.c_int32), ("status", C.c_int32), ("rr0", C.c_double), ("rrn", C.c_double)]
 
@@ -66,6 +75,7 @@ _sig = {
     "abft_calc_p_spmv": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.c_double,
                                    C.POINTER(Vec), C.POINTER(Vec), _P, _P, _P]),
     "abft_inject_bitflip": (C.c_int, [_P, _P, C.c_uint64, _P]),
+    "abft_ctx_set_faults": (C.c_int, [_P, _P, C.c_int, C.POINTER(CSR), C.c_int, _P]),
     "abft_counts_read": (C.c_int, [_P, _P, _P]),
     "abft_counts_reset": (C.c_int, [_P, _P]),
     "abft_launch_count": (C.c_uint64, []),
@@ -157,6 +167,25 @@ class Context:
     def set_pdl(self, enable: bool):
         """Programmatic dependent launch in the CG loop (abft_ctx_set_pdl; library default off)."""
         _check(_lib.abft_ctx_set_pdl(self.h, 1 if enable else 0), "abft_ctx_set_pdl")
+
+    def set_faults(self, faults, A=None, vecs=None):
+        """O10 fault schedule for the next CG solves on this context:
+        faults = [(iter, target, word, bit[, chunk]), ...] (targets F_VAL ..
+        F_W), A = the matrix / chunk list and vecs = (b, x, r, p, w) that the
+        solve will be given.  An empty list clears it (abft_ctx_set_faults)."""
+        fl = list(faults or [])
+        arr = (Fault * max(len(fl), 1))()
+        for i, f in enumerate(fl):
+            k, t, w, b = f[:4]
+            arr[i] = Fault(int(k), int(t), int(w), int(b), int(f[4]) if len(f) > 4 else 0)
+        if fl:
+            carr, nch = _chunks(A)
+            vstructs = [v.cstruct() for v in vecs]
+            vptr = (C.c_void_p * 5)(*[C.cast(C.pointer(v), C.c_void_p) for v in vstructs])
+        else:
+            carr, nch, vptr = None, 0, None
+        _check(_lib.abft_ctx_set_faults(self.h, C.cast(arr, C.c_void_p), len(fl), carr, nch, vptr),
+               "abft_ctx_set_faults")
 
     def close(self):
         if self.h:

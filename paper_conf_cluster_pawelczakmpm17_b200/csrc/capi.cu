@@ -62,6 +62,8 @@ struct abft_ctx {
   bool pdl = false;          // programmatic dependent launch between the CG iteration kernels (opt-in, §6.2)
   uint64_t* p_alt = nullptr; // second p buffer of the fused CG
   int64_t p_alt_len = 0;
+  DevFault* faults = nullptr; // O10 fault schedule applied by the next CG solves (abft_ctx_set_faults)
+  int nfaults = 0;
 };
 
 namespace {
@@ -249,6 +251,7 @@ int abft_ctx_destroy(abft_ctx* c) {
   cudaFree(c->due);
   cudaFree(c->flags);
   cudaFree(c->p_alt);
+  cudaFree(c->faults);
   cudaFree(c->red);
   cudaFree(c->crc);
   cudaFreeHost(c->h_state);
@@ -566,7 +569,8 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   // fused calc_p: single GPU, every chunk on the tiled path,
   // G = 1 vector scheme; p is double-buffered with ctx->p_alt
   const int64_t npad_ext = vec_padded_len(R[0].n_ext, scheme);
-  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0;
+  // (a fault schedule addresses the caller's p: the double-buffered fused CG is off then)
+  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0 && ctx->nfaults == 0;
   abft_vec* const p = R[0].p();
   abft_vec* const r = R[0].r();
   if (fused) {
@@ -602,6 +606,9 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   }
 
   Prof prof{ctx, s};
+  // O10 fault schedule: iteration-0 faults before init
+  for (int q = 0; q < nl; q++)
+    count_launch(launch_inject_sched(R[q].ctx->faults, R[q].ctx->nfaults, R[q].ctx->state, 0, s));
   // init (a2): w = A x0 ; r = b - w ; p = r ; rr0
   if ((e = halo_exchange(d, R, nl, 1, n_halo, s))) return e;
   prof.begin(0);
@@ -664,6 +671,8 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
       int e2;
       // fused: iteration kk's p lives in P[(kk-1) & 1], its predecessor in P[kk & 1]
       const int64_t kk = launched + it + 1;
+      for (int q = 0; q < nl; q++)   // O10: faults of this iteration, before its SpMV
+        count_launch(launch_inject_sched(R[q].ctx->faults, R[q].ctx->nfaults, R[q].ctx->state, 1, ss));
       prof.begin(0);
       e2 = spmv_iter(kk, ss);
       prof.end();
@@ -1036,6 +1045,49 @@ int abft_calc_p_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* p_
   if (e) return e;
   if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
   CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
+int abft_ctx_set_faults(abft_ctx* ctx, const abft_fault* faults, int nfaults, const abft_csr* A, int nchunks,
+                        abft_vec* const* vecs) {
+  if (!ctx || nfaults < 0 || (nfaults > 0 && (!faults || !A || nchunks <= 0 || !vecs)))
+    return fail(ABFT_E_INVALID, "bad fault schedule arguments");
+  std::vector<DevFault> h((size_t)nfaults);
+  for (int i = 0; i < nfaults; i++) {
+    const abft_fault& f = faults[i];
+    if (f.iter < 0 || f.word < 0) return fail(ABFT_E_INVALID, "fault %d: negative iteration / word", i);
+    const int wbits = (f.target == ABFT_F_COL || f.target == ABFT_F_ROWPTR) ? 32 : 64;
+    if (f.bit < 0 || f.bit >= wbits) return fail(ABFT_E_INVALID, "fault %d: bit out of range", i);
+    uint8_t* base = nullptr;
+    int64_t limit = 0;
+    if (f.target <= ABFT_F_ROWPTR) {
+      if (f.chunk < 0 || f.chunk >= nchunks) return fail(ABFT_E_INVALID, "fault %d: bad chunk", i);
+      const abft_csr& M = A[f.chunk];
+      if (f.target == ABFT_F_VAL) { base = reinterpret_cast<uint8_t*>(M.val); limit = M.nnz; }
+      else if (f.target == ABFT_F_COL) { base = reinterpret_cast<uint8_t*>(M.col); limit = M.nnz; }
+      else { base = reinterpret_cast<uint8_t*>(M.rowptr); limit = rowptr_padded_len(M.nrows, M.rowptr_scheme); }
+    } else if (f.target <= ABFT_F_W) {
+      abft_vec* v = vecs[f.target - ABFT_F_B];
+      if (!v || !v->data) return fail(ABFT_E_INVALID, "fault %d: null vector", i);
+      base = reinterpret_cast<uint8_t*>(v->data);
+      limit = vec_padded_len(v->n, v->scheme);
+    } else {
+      return fail(ABFT_E_INVALID, "fault %d: bad target", i);
+    }
+    if (f.word >= limit) return fail(ABFT_E_INVALID, "fault %d: word beyond the target", i);
+    const int64_t byte = f.word * (wbits / 8) + (f.bit / 32) * 4;
+    h[i].addr = reinterpret_cast<uint32_t*>(base + byte);
+    h[i].mask = 1u << (f.bit % 32);
+    h[i].iter = f.iter;
+  }
+  cudaFree(ctx->faults);
+  ctx->faults = nullptr;
+  ctx->nfaults = 0;
+  if (nfaults > 0) {
+    CUDA_TRY(cudaMalloc(&ctx->faults, sizeof(DevFault) * (size_t)nfaults));
+    CUDA_TRY(cudaMemcpy(ctx->faults, h.data(), sizeof(DevFault) * (size_t)nfaults, cudaMemcpyHostToDevice));
+  }
+  ctx->nfaults = nfaults;
   return ABFT_OK;
 }
 

@@ -24,6 +24,10 @@ struct CgState {
 
 struct DevCounts { unsigned long long v[3][5][4]; };
 
+// One scheduled fault (S§8(c) O10) resolved to a device word: XOR `mask` into
+// the 32-bit word at `addr` before iteration `iter`'s SpMV (0 = before init).
+struct DevFault { uint32_t* addr; uint32_t mask; int32_t iter; };
+
 // CRC32C lookup tables (reflected 0x82F63B78), built once per
 // context on the host and copied to shared memory by the kernels that use them.
 struct CrcTables {
@@ -127,6 +131,9 @@ int launch_pack_due(double* out, const int* due, cudaStream_t s);
 int launch_csr_encode(abft_csr* A, uint32_t* flags, cudaStream_t s);
 int launch_check_csr(const abft_csr* A, DevCounts* c, int* due, int scrub, cudaStream_t s);
 int launch_inject(void* base, uint64_t bit, cudaStream_t s);
+// phase 0: the faults of iteration 0 (before init); phase 1: those of
+// iteration state->iters + 1 (skipped once the solve stopped)
+int launch_inject_sched(const DevFault* f, int n, const CgState* st, int phase, cudaStream_t s);
 
 int64_t rowptr_padded_len(int64_t nrows, int scheme);
 int64_t vec_padded_len(int64_t n, int scheme);

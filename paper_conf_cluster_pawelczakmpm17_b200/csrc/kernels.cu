@@ -245,6 +245,18 @@ int launch_check_csr(const abft_csr* A, DevCounts* c, int* due, int scrub, cudaS
   return launches;
 }
 
+static __global__ void k_inject_sched(const DevFault* f, int n, const CgState* st, int phase) {
+  if (phase && st->stop) return;
+  const int k = phase ? st->iters + 1 : 0;
+  for (int i = threadIdx.x; i < n; i += blockDim.x)
+    if (f[i].iter == k) atomicXor(f[i].addr, f[i].mask);
+}
+int launch_inject_sched(const DevFault* f, int n, const CgState* st, int phase, cudaStream_t s) {
+  if (n <= 0) return 0;
+  k_inject_sched<<<1, 256, 0, s>>>(f, n, st, phase);
+  return 1;
+}
+
 int launch_inject(void* base, uint64_t bit, cudaStream_t s) {
   k_inject<<<1, 1, 0, s>>>(reinterpret_cast<uint32_t*>(base), bit);
   return 1;

@@ -578,11 +578,20 @@ constexpr int TILE_TY = 8;
 constexpr int TILE_WX0 = 2;
 constexpr int TILE_WW = 256 + 4;
 constexpr int TILE_PE = 160;                                   // elements per warp per pass (32 rows x 5)
-constexpr int TILE_NST = 3;                                    // pipeline stages
+#ifndef ABFT_TILE_NST
+#define ABFT_TILE_NST 3
+#endif
+// ABFT_RP_FLAGS = 1: the prologue keeps only a per-row "row pointers are the
+// stencil layout" bit per warp instead of 257 decoded entries (SMEM for a 4th
+// CTA per SM); rows without the bit re-decode their entries from global memory
+#ifndef ABFT_RP_FLAGS
+#define ABFT_RP_FLAGS 0
+#endif
+constexpr int TILE_NST = ABFT_TILE_NST;                        // pipeline stages
 constexpr int TILE_STAGE_VAL = TILE_TY * TILE_PE * 8;          // 10240
 constexpr int TILE_STAGE = TILE_STAGE_VAL + TILE_TY * TILE_PE * 4;   // + 5120
 constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 20800
-constexpr int TILE_RP = 264;                                   // rowptr entries staged per warp
+constexpr int TILE_RP = ABFT_RP_FLAGS ? 9 : 264;               // rowptr entries (flag words) staged per warp
 constexpr int TILE_OFF_WIN = TILE_NST * TILE_STAGE;            // stages first (128-B aligned)
 constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
 constexpr int TILE_OFF_BAR = TILE_OFF_RP + TILE_TY * TILE_RP * 4;
@@ -770,6 +779,31 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
   return acc;
 }
 
+// Row pointer entry idx of a chunk as the SpMV uses it (cold path of
+// ABFT_RP_FLAGS): its group checked and corrected in registers (no count, no
+// scrub: the prologue's owner did both), a DUE group's stored bits, masked;
+// detection-only accesses use stored bits for correctable groups too, range-only
+// accesses skip the codec.
+template <int RS>
+__device__ __noinline__ uint32_t rp_entry(const uint32_t* rowptr, int64_t idx, int mode) {
+  constexpr int G = rgrp(RS);
+  uint32_t e[G];
+  const int64_t g0 = idx / G * G;
+#pragma unroll
+  for (int t = 0; t < G; t++) e[t] = *(volatile const uint32_t*)(rowptr + g0 + t);
+  uint32_t w = 0;
+#pragma unroll
+  for (int t = 0; t < G; t++) if (t == idx - g0) w = e[t];
+  if (RS != NONE && mode == MODE_CORRECT) {
+    int word = 0;
+    if (rp_check_group<RS>(e, &word) == CORRECTED) {
+#pragma unroll
+      for (int t = 0; t < G; t++) if (t == idx - g0) w = e[t];
+    }
+  }
+  return w & rp_keep(RS);
+}
+
 #ifndef ABFT_TILE_MINB
 #define ABFT_TILE_MINB 3
 #endif
@@ -907,6 +941,22 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
           }
         }
       }
+#if ABFT_RP_FLAGS
+      // bit j of the warp's flag words: decoded entry j == the stencil layout's 5 (rowseg + j)
+      if (lane < TILE_RP) srp[lane] = 0u;
+      __syncwarp();
+      const uint32_t seg_e0 = (uint32_t)(5 * rowseg);
+#pragma unroll
+      for (int q = 0; q < PER; q++) {
+        const int gl = lane + 32 * q;
+        if (gl >= NG) continue;
+#pragma unroll
+        for (int t = 0; t < G; t++) {
+          const int j = gl * G + t;
+          if (j <= 256 && (e[q][t] & rp_keep(RS)) == seg_e0 + 5u * (uint32_t)j) atomicOr(&srp[j >> 5], 1u << (j & 31));
+        }
+      }
+#else
 #pragma unroll
       for (int q = 0; q < PER; q++) {
         const int gl = lane + 32 * q;
@@ -914,6 +964,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
 #pragma unroll
         for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[q][t] & rp_keep(RS);
       }
+#endif
     }
   }
   if (stop_v) {  // uniform per grid: drain the producer's copies before the CTA exits
@@ -1104,7 +1155,23 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
     if (has_seg) {
       const uint64_t* sval = reinterpret_cast<const uint64_t*>(stage) + warp * TILE_PE;
       const uint32_t* scol = reinterpret_cast<const uint32_t*>(stage + TILE_STAGE_VAL) + warp * TILE_PE;
+#if ABFT_RP_FLAGS
+      uint32_t start, end;
+      {
+        const uint32_t w0 = srp[k], w1 = srp[k + 1];
+        const uint32_t canon = w0 & ((w0 >> 1) | (w1 << 31));
+        if ((canon >> lane) & 1u) {
+          start = seg_e + 160u * k + 5u * (uint32_t)lane;
+          end = start + 5u;
+        } else {   // cold: this row's entries, decoded again from global memory (not counted)
+          const int64_t i = rowseg + 32 * k + lane;
+          start = rp_entry<RS>(a.rowptr, i, mode);
+          end = rp_entry<RS>(a.rowptr, i + 1, mode);
+        }
+      }
+#else
       const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
+#endif
       const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + TILE_WX0;
       const double p_own = s_win[oslot];
       const int64_t own = a.row_base + rowseg + k * 32 + lane;
