@@ -81,6 +81,11 @@ def lib():
                                      C.c_int, C.c_void_p, C.c_void_p, C.c_int]
         L.or_cg_solve_sched.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
                                         C.c_int, C.c_void_p, C.c_void_p, C.c_int, C.c_void_p, C.c_int]
+        L.or_calc_sr.restype = C.c_int64
+        L.or_calc_sr.argtypes = [u64p, u64p, u64p, u64p, u64p, C.c_int64, C.c_int, C.c_double, C.c_double,
+                                 C.c_void_p]
+        L.or_cg_solve_sr.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
+                                     C.c_int, C.c_void_p, C.c_void_p, C.c_void_p, C.c_int]
         L.or_vec_masked.argtypes = [u64p, C.c_int64, C.c_int, dp]
         L.or_round_k.restype = C.c_uint64
         L.or_round_k.argtypes = [C.c_uint64, C.c_int]
@@ -311,3 +316,25 @@ def cg_solve_sched(A: Matrix, b, x, r, p, w, scheme, tol=1e-10, max_iters=10000,
                                  C.byref(res), counts.ctypes.data if counts is not None else None,
                                  int(check_interval), f.ctypes.data if len(f) else None, len(f))
     return st, res
+
+F_S = 8   # the single-reduction CG's extra vector s (or_cg_solve_sr)
+
+
+def calc_sr(x, p, s, r, w, n, scheme, alpha, beta, counts=None):
+    """Single-reduction CG update: p, s, x, r in place."""
+    return lib().or_calc_sr(_p(x, C.c_uint64), _p(p, C.c_uint64), _p(s, C.c_uint64), _p(r, C.c_uint64),
+                            _p(w, C.c_uint64), n, scheme, alpha, beta,
+                            counts.ctypes.data if counts is not None else None)
+
+
+def cg_solve_sr(A: Matrix, b, x, r, p, w, s, scheme, tol=1e-10, max_iters=10000, due_policy=1, counts=None,
+                faults=None):
+    """Protected single-reduction CG (Chronopoulos-Gear; S§8(f) f3)."""
+    st = A.cstruct()
+    res = CGResult()
+    f = faults if faults is not None else np.zeros(0, dtype=FAULT_DTYPE)
+    code = lib().or_cg_solve_sr(C.byref(st), _p(b, C.c_uint64), _p(x, C.c_uint64), _p(r, C.c_uint64),
+                                _p(p, C.c_uint64), _p(w, C.c_uint64), _p(s, C.c_uint64), scheme, tol, max_iters,
+                                due_policy, C.byref(res), counts.ctypes.data if counts is not None else None,
+                                f.ctypes.data if len(f) else None, len(f))
+    return code, res

@@ -15,6 +15,8 @@
  *         CG         TeaLeaf CG (ref [19]), DESIGN.md §4
  *         interval   "less frequent correctness checking" P:398-425 (§VI-A.2),
  *                    DESIGN.md §3.9 (reading R27)
+ *         single-reduction CG (S§8(f) f3): Chronopoulos-Gear recurrences,
+ *                    DESIGN.md §4.1 (reading R28), or_cg_solve_sr
  *         faults     O10 scheduled bit flips (S§8(c) O10): XOR before init /
  *                    before iteration k's SpMV, or_cg_solve_sched
  *         CRC fix    1EC4ED single-bit correction of a failing CRC32C codeword
@@ -955,6 +957,110 @@ int or_cg_solve_ex(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p
 int or_cg_solve(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
                 int max_iters, int due_policy, or_cg_result* res, counts_t* cnt) {
   return or_cg_solve_ex(A, b, x, r, p, w, vs, tol, max_iters, due_policy, res, cnt, 1);
+}
+
+/* ---------------------------------------------------------- single-reduction CG
+ * S§8(f) f3 "single-reduction CG": the Chronopoulos-Gear recurrences
+ * (Chronopoulos & Gear, "s-step iterative methods for symmetric linear
+ * systems", J. Comput. Appl. Math. 25 (1989); unpreconditioned, s = 1) as
+ * restated in DESIGN.md §4.1 (reading R28).  One SpMV per iteration, w = A r,
+ * carries BOTH dot products (gamma = r.r, delta = w.r; RED-1 each), followed by
+ * one fused vector update; PAPER.md's protection applies unchanged:
+ * every vector read is checked, every write re-encodes.
+ *
+ * calc_sr: p = enc(fma(beta, p, r)); s = enc(fma(beta, s, w));
+ *          x = enc(fma(alpha, p', x)); r = enc(fma(-alpha, s', r))
+ * where p', s' are the masked values of the NEW stored p, s.  Checks x, p, s, r, w. */
+int64_t or_calc_sr(uint64_t* x, uint64_t* p, uint64_t* s, uint64_t* r, uint64_t* w, int64_t n, int vs,
+                   double alpha, double beta, counts_t* cnt) {
+  init_instances();
+  double* X = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* P = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* S = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* R = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* W = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  int64_t dues = vdec(x, n, vs, X, cnt) + vdec(p, n, vs, P, cnt) + vdec(s, n, vs, S, cnt) + vdec(r, n, vs, R, cnt) +
+                 vdec(w, n, vs, W, cnt);
+  for (int64_t i = 0; i < n; i++) {
+    P[i] = fma(beta, P[i], R[i]);
+    S[i] = fma(beta, S[i], W[i]);
+  }
+  venc(p, P, n, vs);
+  venc(s, S, n, vs);
+  vmasked(p, n, vs, P);
+  vmasked(s, n, vs, S);
+  for (int64_t i = 0; i < n; i++) {
+    X[i] = fma(alpha, P[i], X[i]);
+    R[i] = fma(-alpha, S[i], R[i]);
+  }
+  venc(x, X, n, vs);
+  venc(r, R, n, vs);
+  free(X); free(P); free(S); free(R); free(W);
+  return dues;
+}
+
+/* w = A r with both dots: returns the SpMV's DUE count; *delta = r.w, *gamma = r.r (RED-1). */
+static int64_t spmv_sr(or_csr* A, uint64_t* r, uint64_t* w, int64_t n, int vs, counts_t* cnt, int mode,
+                       double* gamma, double* delta) {
+  int64_t dues = or_spmv_mode(A, r, n, vs, w, n, cnt, delta, mode);
+  double* R = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  vmasked(r, n, vs, R);
+  *gamma = or_dot_red1(R, R, n);
+  free(R);
+  return dues;
+}
+
+/* Protected single-reduction CG (targets of the O10 schedule: 0..7 as in
+ * or_cg_solve_sched, 8 = s; iteration k's faults are applied before its
+ * vector update, i.e. at the start of the iteration).
+ * Init: w = A x0; r = enc(b - w); p = s = enc(+0.0); w = A r, gamma = r.r,
+ * delta = w.r; rr0 = gamma (0 -> 0 iterations); alpha = gamma/delta, beta = 0.
+ * Iteration k: calc_sr; w = A r, gamma' = r.r, delta = w.r; converged when
+ * sqrt(gamma') <= tol sqrt(rr0) -> k; else beta = gamma'/gamma,
+ * alpha = gamma'/(delta - beta gamma'/alpha), gamma = gamma'. */
+int or_cg_solve_sr(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, uint64_t* s, int vs,
+                   double tol, int max_iters, int due_policy, or_cg_result* res, counts_t* cnt,
+                   const or_fault* faults, int nfaults) {
+  init_instances();
+  int64_t n = A->nrows;
+  uint64_t* vecs[5] = {b, x, r, p, w};
+  double gamma, delta, gnew, rr0, alpha, beta = 0.0;
+  res->iters = 0; res->status = OK; res->rr0 = 0.0; res->rrn = 0.0;
+  for (int i = 0; i < nfaults; i++)
+    if (faults[i].iter == 0 && faults[i].target == 8) s[faults[i].word] ^= 1ull << faults[i].bit;
+  apply_faults(A, vecs, faults, nfaults, 0);
+  int64_t dues = or_spmv_mode(A, x, n, vs, w, n, cnt, NULL, M_CORRECT);
+  double tmp;
+  dues += or_cg_init_r(b, w, r, p, n, vs, cnt, &tmp);
+  int64_t npad = or_vec_padded_len(n, vs);
+  double* Z = (double*)calloc((size_t)(npad + 1), sizeof(double));
+  venc(p, Z, npad, vs);   /* p = s = encoded +0.0 (padding included) */
+  venc(s, Z, npad, vs);
+  free(Z);
+  dues += spmv_sr(A, r, w, n, vs, cnt, M_CORRECT, &gamma, &delta);
+  rr0 = gamma;
+  res->rr0 = rr0; res->rrn = rr0;
+  if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+  if (rr0 == 0.0) return OK;
+  alpha = gamma / delta;
+  for (int k = 1; k <= max_iters; k++) {
+    for (int i = 0; i < nfaults; i++)
+      if (faults[i].iter == k && faults[i].target == 8) s[faults[i].word] ^= 1ull << faults[i].bit;
+    apply_faults(A, vecs, faults, nfaults, k);
+    dues = or_calc_sr(x, p, s, r, w, n, vs, alpha, beta, cnt);
+    dues += spmv_sr(A, r, w, n, vs, cnt, M_CORRECT, &gnew, &delta);
+    res->iters = k; res->rrn = gnew;
+    int conv = sqrt(gnew) <= tol * sqrt(rr0);
+    if (!conv) {
+      beta = gnew / gamma;
+      alpha = gnew / (delta - beta * gnew / alpha);
+      gamma = gnew;
+    }
+    if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+    if (conv) return OK;
+  }
+  res->status = (max_iters > 0) ? E_NOT_CONVERGED : OK;
+  return res->status;
 }
 
 /* Masked-value helper for tests: clear the k reserved LSBs of each entry. */

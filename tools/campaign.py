@@ -264,6 +264,7 @@ def _clone(orc, Ac):
     """An oracle matrix holding exactly Ac's stored words (padding included)."""
     M = orc.Matrix(Ac.val.view(np.float64).copy(), Ac.col.copy(), Ac.rowptr.copy(), Ac.nrows, Ac.ncols, Ac.es, Ac.rs)
     M.rowptr[:] = Ac.rowptr
+    M.nnz = Ac.nnz    # (the constructor read nnz from rowptr[nrows], which now carries ECC bits)
     return M
 
 

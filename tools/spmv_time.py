@@ -55,6 +55,16 @@ def main():
         res["fused_calc_p_spmv_ms"] = t(lambda: abft.calc_p_spmv(ctx, sol.A, p, r, 1e-30, p2, w, cnt, dot=dot))
         res["fused_gbs"] = 96.0 * P["N"] / (res["fused_calc_p_spmv_ms"] * 1e-3) / 1e9
         res["spmv_gbs"] = 80.0 * P["N"] / (res["spmv_ms"] * 1e-3) / 1e9
+        # one protected CG iteration inside the graph-replayed solve loop (tol 0: no convergence stop)
+        iters = 200
+        sol.step(0.0, 8)
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        torch.cuda.synchronize()
+        e0.record()
+        sol.step(0.0, iters)
+        e1.record()
+        torch.cuda.synchronize()
+        res["cg_step_ms_200it"] = e0.elapsed_time(e1)
         res["counts"] = int(cnt.read().sum())
         out[f"scheme{s}"] = res
         del sol
