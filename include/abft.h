@@ -148,6 +148,18 @@ typedef struct { int32_t iters; int32_t status; double rr0, rrn; } abft_cg_resul
 int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
                   abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream);
 
+/* Single-reduction protected CG (S§8(f) f3, reading R28): the
+ * Chronopoulos-Gear recurrences — per iteration one fused update
+ * (p = r + beta p, s = w + beta s, x += alpha p, r -= alpha s; every operand
+ * checked, every result re-encoded) and one protected SpMV w = A r
+ * carrying BOTH dot products (r.r, w.r) into ONE reduction, instead of two.
+ * Same matrix / vector conventions, options, counters and statuses as
+ * abft_cg_solve; s is a sixth vector like the others (scheme, length).
+ * Single GPU, every access checked (check_interval <= 1, else ABFT_E_SHAPE). */
+int abft_cg_solve_sr(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r,
+                     abft_vec* p, abft_vec* w, abft_vec* s, const abft_cg_opts* opts, abft_cg_result* res,
+                     abft_counts* dcnt, void* stream);
+
 /* a4 / a5 as single calls (the CG driver fuses them into its device-side loop):
  * calc_ur  x = enc(fma(alpha, p, x)); r = enc(fma(-alpha, w, r)); rrn_out = r.r (RED-1)
  * calc_p   p = enc(fma(beta, p, r))

@@ -68,6 +68,9 @@ _sig = {
     "abft_spmv_ex": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), _P, _P, C.c_int32, _P]),
     "abft_cg_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                 C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
+    "abft_cg_solve_sr": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
+                                   C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts),
+                                   C.POINTER(CGResult), _P, _P]),
     "abft_check_all": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.c_int, C.c_int, _P, _P]),
     "abft_calc_ur": (C.c_int, [_P, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.c_double, _P, _P,
                                _P]),
@@ -316,6 +319,19 @@ def cg_solve(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vec
     code = _lib.abft_cg_solve(ctx.h, arr, n, *[C.byref(v) for v in vs], C.byref(opts), C.byref(res),
                               counts.ptr if counts else None, _stream(stream))
     _check(code, "abft_cg_solve", allow=(E_DUE, E_NOT_CONVERGED))
+    return res
+
+
+def cg_solve_sr(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vector, s: Vector, tol=1e-10,
+                max_iters=10000, due_policy=0, counts: Counters | None = None, poll_every=16, stream=None) -> CGResult:
+    """Single-reduction protected CG (Chronopoulos-Gear; abft_cg_solve_sr)."""
+    arr, n = _chunks(A)
+    opts = CGOpts(tol, max_iters, due_policy, poll_every, 1)
+    res = CGResult()
+    vs = [v.cstruct() for v in (b, x, r, p, w, s)]
+    code = _lib.abft_cg_solve_sr(ctx.h, arr, n, *[C.byref(v) for v in vs], C.byref(opts), C.byref(res),
+                                 counts.ptr if counts else None, _stream(stream))
+    _check(code, "abft_cg_solve_sr", allow=(E_DUE, E_NOT_CONVERGED))
     return res
 
 

@@ -42,7 +42,9 @@ static inline void count_launch(int n) { g_launches.fetch_add((uint64_t)n, std::
 struct abft_ctx {
   int device = 0;
   double* partials = nullptr;
+  double* partials2 = nullptr;  // second dot of the single-reduction CG's SpMV (same capacity)
   int64_t partials_cap = 0;
+  double* roots2 = nullptr;
   double* roots = nullptr;
   uint32_t* ticket = nullptr;
   CgState* state = nullptr;
@@ -71,9 +73,12 @@ namespace {
 int ensure_partials(abft_ctx* c, int64_t nrb) {
   if (nrb <= c->partials_cap) return ABFT_OK;
   if (c->partials) cudaFree(c->partials);
-  c->partials = nullptr;
+  if (c->partials2) cudaFree(c->partials2);
+  c->partials = c->partials2 = nullptr;
+  c->partials_cap = 0;
   int64_t cap = nrb < 1024 ? 1024 : nrb;
   CUDA_TRY(cudaMalloc(&c->partials, sizeof(double) * cap));
+  CUDA_TRY(cudaMalloc(&c->partials2, sizeof(double) * cap));
   c->partials_cap = cap;
   return ABFT_OK;
 }
@@ -103,7 +108,7 @@ int check_chunks(const abft_csr* A, int nchunks) {
 // fused calc_p (CG driver): p_cur != null => in = p_{k-1}, r_f = r;
 // probe = true only builds the arguments and reports whether every chunk can
 // take the fused tiled kernel (nothing is launched).
-int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, bool dot,
+int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, int dot,
                 DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total, RedArgs red = RedArgs{},
                 int check_mode = MODE_CORRECT, int check_interval = 0, uint64_t* p_cur = nullptr,
                 uint64_t* r_f = nullptr, bool probe = false, int part = 0) {
@@ -147,6 +152,7 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.in = reinterpret_cast<uint64_t*>(in->data);
     a.out = reinterpret_cast<uint64_t*>(out->data);
     a.partials = dot ? ctx->partials : nullptr;
+    a.partials2 = dot == 2 ? ctx->partials2 : nullptr;
     a.counts = cnt;
     a.due = ctx->due;
     a.state = st;
@@ -206,6 +212,7 @@ int abft_ctx_create(int device, abft_ctx** out) {
   abft_ctx* c = new abft_ctx();
   c->device = device;
   CUDA_TRY(cudaMalloc(&c->roots, sizeof(double) * 1024));
+  CUDA_TRY(cudaMalloc(&c->roots2, sizeof(double) * 1024));
   CUDA_TRY(cudaMalloc(&c->ticket, sizeof(uint32_t) * 4));
   CUDA_TRY(cudaMemset(c->ticket, 0, sizeof(uint32_t) * 4));
   CUDA_TRY(cudaMalloc(&c->state, sizeof(CgState)));
@@ -245,7 +252,9 @@ int abft_ctx_destroy(abft_ctx* c) {
   if (!c) return ABFT_OK;
   cudaSetDevice(c->device);
   cudaFree(c->partials);
+  cudaFree(c->partials2);
   cudaFree(c->roots);
+  cudaFree(c->roots2);
   cudaFree(c->ticket);
   cudaFree(c->state);
   cudaFree(c->due);
@@ -425,6 +434,7 @@ struct RankRun {
   const abft_csr* A = nullptr;
   int nchunks = 0;
   abft_vec* v[5] = {};   // b x r p w
+  abft_vec* s_vec = nullptr;   // single-reduction CG: its extra vector s
   DevCounts* cnt = nullptr;
   int64_t n = 0, nrb = 0, n_ext = 0;
   VecArgs va{};
@@ -554,6 +564,17 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   }
   abft_ctx* ctx = R[0].ctx;   // graphs, events, polling
   const int scheme = R[0].x()->scheme;
+  // single-reduction CG (Chronopoulos-Gear, S§8(f) f3): one GPU, every access checked
+  const bool sr = R[0].s_vec != nullptr;
+  if (sr) {
+    if (d || nl != 1) return fail(ABFT_E_SHAPE, "single-reduction CG runs on one GPU");
+    if (opts->check_interval > 1) return fail(ABFT_E_SHAPE, "single-reduction CG checks every access");
+    int e0 = check_vec(R[0].s_vec, "s");
+    if (e0) return e0;
+    if (R[0].s_vec->scheme != scheme || R[0].s_vec->n != R[0].n_ext)
+      return fail(ABFT_E_INVALID, "vector s: scheme/length differ");
+    for (int j = 0; j < 5; j++) if (R[0].v[j]->data == R[0].s_vec->data) return fail(ABFT_E_INVALID, "vectors alias");
+  }
   const int G = (int)vec_padded_len(1, scheme);
   const int interval = opts->check_interval > 1 ? opts->check_interval : 0;
   // the dist path runs whenever a transport is given (also with 1 rank, so the
@@ -570,7 +591,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   // G = 1 vector scheme; p is double-buffered with ctx->p_alt
   const int64_t npad_ext = vec_padded_len(R[0].n_ext, scheme);
   // (a fault schedule addresses the caller's p: the double-buffered fused CG is off then)
-  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0 && ctx->nfaults == 0;
+  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0 && ctx->nfaults == 0 && !sr;
   abft_vec* const p = R[0].p();
   abft_vec* const r = R[0].r();
   if (fused) {
@@ -619,7 +640,21 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   }
   prof.end();
   for (int q = 0; q < nl; q++) count_launch(launch_init_r(R[q].va, scheme, s));
-  if ((e = finish_dot(R, nl, d, 1, s))) return e;
+  VecArgs vsr = R[0].va;   // single-reduction update: VecArgs.b carries s
+  if (sr) {
+    vsr.b = reinterpret_cast<uint64_t*>(R[0].s_vec->data) + n_halo;
+    // p = s = encoded +0.0, then w = A r with both dots (gamma = r.r, delta = w.r)
+    for (abft_vec* v : {R[0].p(), R[0].s_vec}) {
+      CUDA_TRY(cudaMemsetAsync(v->data, 0, sizeof(uint64_t) * npad_ext, s));
+      count_launch(launch_vec_encode(reinterpret_cast<uint64_t*>(v->data), v->n, npad_ext, scheme, s));
+    }
+    if ((e = spmv_chunks(ctx, R[0].A, R[0].nchunks, R[0].r(), R[0].w(), 2, R[0].cnt, nullptr, s, nullptr)))
+      return e;
+    count_launch(launch_reduce_sr(ctx->partials, ctx->partials2, R[0].nrb, ctx->roots, ctx->roots2, ctx->ticket, 7,
+                                  ctx->state, ctx->due, s));
+  } else if ((e = finish_dot(R, nl, d, 1, s))) {
+    return e;
+  }
   CUDA_TRY(cudaGetLastError());
 
   int poll = opts->poll_every > 0 ? opts->poll_every : 16;
@@ -673,6 +708,20 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
       const int64_t kk = launched + it + 1;
       for (int q = 0; q < nl; q++)   // O10: faults of this iteration, before its SpMV
         count_launch(launch_inject_sched(R[q].ctx->faults, R[q].ctx->nfaults, R[q].ctx->state, 1, ss));
+      if (sr) {   // update, then w = A r with both dots, then the one reduction
+        prof.begin(1);
+        count_launch(launch_calc_sr(vsr, scheme, ss));
+        prof.end();
+        prof.begin(0);
+        e2 = spmv_chunks(ctx, R[0].A, R[0].nchunks, R[0].r(), R[0].w(), 2, R[0].cnt, ctx->state, ss, nullptr);
+        prof.end();
+        if (e2) return e2;
+        prof.begin(3);
+        count_launch(launch_reduce_sr(ctx->partials, ctx->partials2, R[0].nrb, ctx->roots, ctx->roots2, ctx->ticket,
+                                      6, ctx->state, ctx->due, ss));
+        prof.end();
+        continue;
+      }
       prof.begin(0);
       e2 = spmv_iter(kk, ss);
       prof.end();
@@ -851,6 +900,16 @@ int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, ab
                   abft_vec* w, const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream) {
   if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
   RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  return cg_run(&R, 1, nullptr, 0, opts, res, (cudaStream_t)stream);
+}
+
+int abft_cg_solve_sr(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r,
+                     abft_vec* p, abft_vec* w, abft_vec* sv, const abft_cg_opts* opts, abft_cg_result* res,
+                     abft_counts* dcnt, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  if (!sv) return fail(ABFT_E_INVALID, "null vector s");
+  RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  R.s_vec = sv;
   return cg_run(&R, 1, nullptr, 0, opts, res, (cudaStream_t)stream);
 }
 

@@ -68,6 +68,7 @@ struct SpmvArgs {
   uint64_t* in;
   uint64_t* out;
   double* partials;  // indexed rb_offset + local RB (may be null)
+  double* partials2; // DOT 2 (single-reduction CG): in.in partials, same indexing
   DevCounts* counts; // may be null
   int* due;          // DUE / range flag (never null)
   const CgState* state;  // may be null
@@ -108,7 +109,8 @@ void set_pdl(bool on);
 // write the device CG state from a by-value launch argument (no host staging buffer)
 int launch_set_state(const CgState& h, CgState* dst, cudaStream_t s);
 // launchers (kernels.cu); each returns the number of kernels launched
-int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, bool dot, cudaStream_t s);
+// dot: 0 none, 1 in.out -> partials, 2 also in.in -> partials2
+int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, int dot, cudaStream_t s);
 // -1: a fused-calc_p launch (a.p_cur set) could not run
 // can this chunk take the fused-calc_p tiled SpMV (G = 1 vector scheme, stencil layout)?
 bool spmv_fusable(const SpmvArgs& a, int vs);
@@ -125,6 +127,12 @@ int launch_vec_check(uint64_t* data, int64_t n, int64_t npad, int vs, double* ou
 //     4 subtree root + DUE flag -> out[0..2) (multi-GPU all-gather payload)
 int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* ticket, int op, CgState* st,
                   double* out, const int* due, cudaStream_t s);
+// single-reduction CG: reduce partials (w.r) and partials2
+// (r.r) in RED-1 order and apply op 7 (init) / 6 (iteration)
+int launch_reduce_sr(const double* partials, const double* partials2, int64_t nrb, double* roots, double* roots2,
+                     uint32_t* ticket, int op, CgState* st, const int* due, cudaStream_t s);
+// single-reduction CG update: p, s, x, r (VecArgs.b carries s)
+int launch_calc_sr(const VecArgs& a, int vs, cudaStream_t s);
 int launch_combine(const double* gathered, int P, int op, CgState* st, int* due, cudaStream_t s);
 int launch_due_combine(const double* gathered, int P, CgState* st, int* due, cudaStream_t s);
 int launch_pack_due(double* out, const int* due, cudaStream_t s);

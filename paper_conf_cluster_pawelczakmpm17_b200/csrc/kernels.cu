@@ -33,12 +33,12 @@ int launch_set_state(const CgState& h, CgState* dst, cudaStream_t s) {
 }
 
 // per-ES SpMV launchers live in spmv_es*.cu (parallel compilation)
-bool spmv_es_none(const SpmvArgs&, int, int, bool, cudaStream_t);
-bool spmv_es_sed(const SpmvArgs&, int, int, bool, cudaStream_t);
-bool spmv_es_secded(const SpmvArgs&, int, int, bool, cudaStream_t);
-bool spmv_es_crc(const SpmvArgs&, int, int, bool, cudaStream_t);
+bool spmv_es_none(const SpmvArgs&, int, int, int, cudaStream_t);
+bool spmv_es_sed(const SpmvArgs&, int, int, int, cudaStream_t);
+bool spmv_es_secded(const SpmvArgs&, int, int, int, cudaStream_t);
+bool spmv_es_crc(const SpmvArgs&, int, int, int, cudaStream_t);
 
-int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, bool dot, cudaStream_t s) {
+int launch_spmv(const SpmvArgs& a, int es, int rs, int vs, int dot, cudaStream_t s) {
   if (a.nrows <= 0) return 0;
   bool ok;
   switch (es) {
@@ -115,6 +115,23 @@ int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s) {
     case SECDED128: launch_k(k_calc_p<SECDED128>, nb, 256, 0, s, a); break;
     default: launch_k(k_calc_p<CRC32C>, nb, 256, vec_dyn_smem<CRC32C>(), s, a); break;
   }
+#if ABFT_P_TICKET
+  return 1;
+#else
+  launch_k(k_post_p, 1, 1, 0, s, a.state, (const int*)a.due);
+  return 2;
+#endif
+}
+int launch_calc_sr(const VecArgs& a, int vs, cudaStream_t s) {
+  if (a.n <= 0) return 0;
+  int nb = blocks_rb(a.n);
+  switch (vs) {
+    case NONE: launch_k(k_calc_sr<NONE>, nb, 256, 0, s, a); break;
+    case SED: launch_k(k_calc_sr<SED>, nb, 256, 0, s, a); break;
+    case SECDED64: launch_k(k_calc_sr<SECDED64>, nb, 256, 0, s, a); break;
+    case SECDED128: launch_k(k_calc_sr<SECDED128>, nb, 256, 0, s, a); break;
+    default: launch_k(k_calc_sr<CRC32C>, nb, 256, vec_dyn_smem<CRC32C>(), s, a); break;
+  }
   return 1;
 }
 int launch_init_r(const VecArgs& a, int vs, cudaStream_t s) {
@@ -159,7 +176,18 @@ int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* 
   while (p2 < nrb) p2 <<= 1;
   int64_t leaves = p2 < 1024 ? p2 : 1024;
   int blocks = (int)(p2 / leaves);
-  launch_k(k_reduce, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, op, st, out, due);
+  launch_k(k_reduce<false>, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, op, st, out, due,
+           (const double*)nullptr, (double*)nullptr);
+  return 1;
+}
+int launch_reduce_sr(const double* partials, const double* partials2, int64_t nrb, double* roots, double* roots2,
+                     uint32_t* ticket, int op, CgState* st, const int* due, cudaStream_t s) {
+  int64_t p2 = 1;
+  while (p2 < nrb) p2 <<= 1;
+  int64_t leaves = p2 < 1024 ? p2 : 1024;
+  int blocks = (int)(p2 / leaves);
+  launch_k(k_reduce<true>, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, op, st, (double*)nullptr, due,
+           partials2, roots2);
   return 1;
 }
 

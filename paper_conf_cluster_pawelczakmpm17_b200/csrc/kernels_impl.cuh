@@ -461,7 +461,8 @@ static __device__ __noinline__ int ecrc_fix(uint64_t* val, uint32_t* col, uint32
 }
 
 // ================================================================ SpMV (a3)
-template <int ES, int RS, int VS, bool DOT>
+// DOT: 0 no dot, 1 in.out, 2 in.out and in.in (single-reduction CG)
+template <int ES, int RS, int VS, int DOT>
 __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
   __shared__ uint32_t s_rp[8][40];
@@ -474,7 +475,7 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
   const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
   const int64_t nrb = (a.nrows + 255) >> 8;
   if (rb >= nrb) return;
-  double dot = 0.0;
+  double dot = 0.0, dot2 = 0.0;
   const uint32_t ckeep = col_keep(ES);
   const int mode = spmv_mode(a);
   for (int k = 0; k < 8; k++) {
@@ -532,12 +533,18 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
     const uint64_t enc = v_encode<VS>(rounded, lane, s_lut);
     if (i < a.npad_out) a.out[own] = enc;
     if (DOT && valid) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+    if (DOT == 2 && valid) dot2 = fma(p_own, p_own, dot2);
   }
   if (DOT) {
 #pragma unroll
     for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
     if (a.red.rs) red_push(a.partials, a.rb_offset + rb, dot, a.red, lane);
     else if (lane == 0) a.partials[a.rb_offset + rb] = dot;
+  }
+  if (DOT == 2) {
+#pragma unroll
+    for (int off = 16; off >= 1; off >>= 1) dot2 = dot2 + __shfl_xor_sync(0xffffffffu, dot2, off);
+    if (lane == 0) a.partials2[a.rb_offset + rb] = dot2;
   }
 }
 
@@ -581,17 +588,11 @@ constexpr int TILE_PE = 160;                                   // elements per w
 #ifndef ABFT_TILE_NST
 #define ABFT_TILE_NST 3
 #endif
-// ABFT_RP_FLAGS = 1: the prologue keeps only a per-row "row pointers are the
-// stencil layout" bit per warp instead of 257 decoded entries (SMEM for a 4th
-// CTA per SM); rows without the bit re-decode their entries from global memory
-#ifndef ABFT_RP_FLAGS
-#define ABFT_RP_FLAGS 0
-#endif
 constexpr int TILE_NST = ABFT_TILE_NST;                        // pipeline stages
 constexpr int TILE_STAGE_VAL = TILE_TY * TILE_PE * 8;          // 10240
 constexpr int TILE_STAGE = TILE_STAGE_VAL + TILE_TY * TILE_PE * 4;   // + 5120
 constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 20800
-constexpr int TILE_RP = ABFT_RP_FLAGS ? 9 : 264;               // rowptr entries (flag words) staged per warp
+constexpr int TILE_RP = 264;                                   // rowptr entries staged per warp
 constexpr int TILE_OFF_WIN = TILE_NST * TILE_STAGE;            // stages first (128-B aligned)
 constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
 constexpr int TILE_OFF_BAR = TILE_OFF_RP + TILE_TY * TILE_RP * 4;
@@ -779,35 +780,10 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
   return acc;
 }
 
-// Row pointer entry idx of a chunk as the SpMV uses it (cold path of
-// ABFT_RP_FLAGS): its group checked and corrected in registers (no count, no
-// scrub: the prologue's owner did both), a DUE group's stored bits, masked;
-// detection-only accesses use stored bits for correctable groups too, range-only
-// accesses skip the codec.
-template <int RS>
-__device__ __noinline__ uint32_t rp_entry(const uint32_t* rowptr, int64_t idx, int mode) {
-  constexpr int G = rgrp(RS);
-  uint32_t e[G];
-  const int64_t g0 = idx / G * G;
-#pragma unroll
-  for (int t = 0; t < G; t++) e[t] = *(volatile const uint32_t*)(rowptr + g0 + t);
-  uint32_t w = 0;
-#pragma unroll
-  for (int t = 0; t < G; t++) if (t == idx - g0) w = e[t];
-  if (RS != NONE && mode == MODE_CORRECT) {
-    int word = 0;
-    if (rp_check_group<RS>(e, &word) == CORRECTED) {
-#pragma unroll
-      for (int t = 0; t < G; t++) if (t == idx - g0) w = e[t];
-    }
-  }
-  return w & rp_keep(RS);
-}
-
 #ifndef ABFT_TILE_MINB
 #define ABFT_TILE_MINB 3
 #endif
-template <int ES, int RS, int VS, bool DOT, bool FUSED = false>
+template <int ES, int RS, int VS, int DOT, bool FUSED = false>
 __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArgs a, const __grid_constant__ TileMaps tm) {
   static_assert(!FUSED || (vgrp(VS) == 1 && DOT), "fused calc_p: G = 1 vector schemes, CG SpMV only");
   extern __shared__ uint8_t s_raw[];
@@ -880,6 +856,15 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   // wrote it; later iterations build p_cur from (in = p_{k-1}, r) in the window
   const bool fz = FUSED && a.state->iters > 0;
   uint64_t* const pin = (FUSED && !fz) ? a.p_cur : a.in;
+  // G = 1, not building p_k: the raw `in` window arrives by one TMA box
+  // (out-of-range rows / columns zero-filled = encoded +0.0) and is decoded in
+  // place.  Unfused, it is issued right here, before the CG-state load below,
+  // so the window's latency overlaps it (a stopped solve drains it).
+  const bool tma_win = vgrp(VS) == 1 && !(FUSED && fz) && tm.has_vmaps;
+  if (tma_win && threadIdx.x == 0) {
+    mbar_expect_tx(winbar, TILE_WIN_BYTES);
+    tma_3d(s_win, (FUSED && !fz) ? &tm.vcur : &tm.vin, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 - 1), winbar);
+  }
   if (threadIdx.x == 0) {
     s_args = a;
     if (FUSED) {
@@ -893,13 +878,6 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   __syncthreads();
   const int stop_v = a.state ? a.state->stop : 0;
   const int mode = spmv_mode(a);
-  // G = 1, not building p_k: the raw `in` window arrives by one TMA box
-  // (out-of-range rows / columns zero-filled = encoded +0.0) and is decoded in place
-  const bool tma_win = vgrp(VS) == 1 && !(FUSED && fz) && tm.has_vmaps;
-  if (tma_win && !stop_v && threadIdx.x == 0) {
-    mbar_expect_tx(winbar, TILE_WIN_BYTES);
-    tma_3d(s_win, (FUSED && !fz) ? &tm.vcur : &tm.vin, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 - 1), winbar);
-  }
   if (has_seg) {
     if (!stop_v) {
       uint32_t acc = 0;
@@ -941,22 +919,6 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
           }
         }
       }
-#if ABFT_RP_FLAGS
-      // bit j of the warp's flag words: decoded entry j == the stencil layout's 5 (rowseg + j)
-      if (lane < TILE_RP) srp[lane] = 0u;
-      __syncwarp();
-      const uint32_t seg_e0 = (uint32_t)(5 * rowseg);
-#pragma unroll
-      for (int q = 0; q < PER; q++) {
-        const int gl = lane + 32 * q;
-        if (gl >= NG) continue;
-#pragma unroll
-        for (int t = 0; t < G; t++) {
-          const int j = gl * G + t;
-          if (j <= 256 && (e[q][t] & rp_keep(RS)) == seg_e0 + 5u * (uint32_t)j) atomicOr(&srp[j >> 5], 1u << (j & 31));
-        }
-      }
-#else
 #pragma unroll
       for (int q = 0; q < PER; q++) {
         const int gl = lane + 32 * q;
@@ -964,12 +926,13 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
 #pragma unroll
         for (int t = 0; t < G; t++) if (gl * G + t < TILE_RP) srp[gl * G + t] = e[q][t] & rp_keep(RS);
       }
-#endif
     }
   }
   if (stop_v) {  // uniform per grid: drain the producer's copies before the CTA exits
-    if (threadIdx.x == 0)
+    if (threadIdx.x == 0) {
       for (int s = 0; s < TILE_NST; s++) mbar_wait(&full[s], 0u);
+      if (tma_win) mbar_wait(winbar, 0u);
+    }
     return;
   }
   // ---- 2. decoded `in` window: rows ty0-1 .. ty0+TILE_TY, x = tx0-2 .. tx0+257
@@ -1138,7 +1101,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   }
   __syncthreads();
   // ---- 3. passes (every warp takes part in the stage protocol)
-  double dot = 0.0;
+  double dot = 0.0, dot2 = 0.0;
   uint64_t acc_prev = 0;   // SECDED128: rounded result of the even pass awaiting its pair
   double p_prev = 0.0;
   const uint32_t seg_e = (uint32_t)(5 * rowseg);   // assumed element start of the segment
@@ -1155,23 +1118,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
     if (has_seg) {
       const uint64_t* sval = reinterpret_cast<const uint64_t*>(stage) + warp * TILE_PE;
       const uint32_t* scol = reinterpret_cast<const uint32_t*>(stage + TILE_STAGE_VAL) + warp * TILE_PE;
-#if ABFT_RP_FLAGS
-      uint32_t start, end;
-      {
-        const uint32_t w0 = srp[k], w1 = srp[k + 1];
-        const uint32_t canon = w0 & ((w0 >> 1) | (w1 << 31));
-        if ((canon >> lane) & 1u) {
-          start = seg_e + 160u * k + 5u * (uint32_t)lane;
-          end = start + 5u;
-        } else {   // cold: this row's entries, decoded again from global memory (not counted)
-          const int64_t i = rowseg + 32 * k + lane;
-          start = rp_entry<RS>(a.rowptr, i, mode);
-          end = rp_entry<RS>(a.rowptr, i + 1, mode);
-        }
-      }
-#else
       const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
-#endif
       const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + TILE_WX0;
       const double p_own = s_win[oslot];
       const int64_t own = a.row_base + rowseg + k * 32 + lane;
@@ -1191,6 +1138,10 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
             dot = fma(p_prev, as_d(e0 & vkeep(VS)), dot);
             dot = fma(p_own, as_d(e1 & vkeep(VS)), dot);
           }
+          if (DOT == 2) {
+            dot2 = fma(p_prev, p_prev, dot2);
+            dot2 = fma(p_own, p_own, dot2);
+          }
         }
       } else {
         const uint64_t enc = (VS == CRC32C) ? vcrc_encode_lane(rounded, vcrc_tab(cs, lane), lane)
@@ -1198,6 +1149,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
         a.out[own] = enc;
         if (FUSED && fz) a.p_cur[own] = v_encode<VS>(as_u(p_own), lane, s_lut);   // enc(p_k), own cell
         if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+        if (DOT == 2) dot2 = fma(p_own, p_own, dot2);
       }
     }
     __syncwarp();
@@ -1212,6 +1164,11 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
     for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
     if (a.red.rs) red_push(a.partials, a.rb_offset + (rowseg >> 8), dot, a.red, lane);
     else if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
+  }
+  if (DOT == 2 && has_seg) {
+#pragma unroll
+    for (int off = 16; off >= 1; off >>= 1) dot2 = dot2 + __shfl_xor_sync(0xffffffffu, dot2, off);
+    if (lane == 0) a.partials2[a.rb_offset + (rowseg >> 8)] = dot2;
   }
 }
 
@@ -1358,6 +1315,12 @@ __device__ __forceinline__ void p_step(const VecArgs& a, uint64_t* P, uint64_t* 
   P[k] = e0;
   P[k + 32] = e1;
 }
+// 0 (default): calc_p's end-of-iteration logic runs in a one-thread kernel
+// after it (measured r2c: protected calc_p 0.0758 -> 0.0723 ms at 4096^2);
+// 1: in calc_p's last CTA (per-CTA fence + ticket)
+#ifndef ABFT_P_TICKET
+#define ABFT_P_TICKET 0
+#endif
 #ifndef ABFT_P_UNROLL
 #define ABFT_P_UNROLL 0
 #endif
@@ -1465,7 +1428,9 @@ template <int VS>
 __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : ABFT_P_MINB) k_calc_p(VecArgs a) {
   __shared__ __align__(16) uint8_t s_lut[128];
   extern __shared__ __align__(16) uint8_t s_dyn_v[];
+#if ABFT_P_TICKET
   __shared__ bool s_last;
+#endif
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
   const bool full = rb * 256 + 256 <= a.n;
@@ -1499,6 +1464,7 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : ABFT_P_MINB) k_calc_p(
       if (i < a.npad) a.p[i] = pe;
     }
   }
+#if ABFT_P_TICKET
   // last block finishes the iteration: DUE policy and max_iters
   __syncthreads();
   if (threadIdx.x == 0) {
@@ -1516,6 +1482,60 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : ABFT_P_MINB) k_calc_p(
     if (!st->dist && st->abort_policy && *due) { st->stop = 1; st->status = ABFT_E_DUE; }
     else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
     st->rro = st->rrn;
+  }
+#endif
+}
+// ABFT_P_TICKET = 0: the end-of-iteration logic runs in this one-thread kernel
+// after calc_p instead of in calc_p's last block (no per-CTA fence + ticket).
+static __global__ void k_post_p(CgState* st, const int* due) {
+  pdl_wait();
+  pdl_trigger();
+  if (st->stop) return;
+  if (!st->dist && st->abort_policy && *((volatile const int*)due)) { st->stop = 1; st->status = ABFT_E_DUE; }
+  else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
+  st->rro = st->rrn;
+}
+
+// Single-reduction CG update (S§8(f) f3): p = enc(fma(beta,
+// p, r)); s = enc(fma(beta, s, w)); x = enc(fma(alpha, p', x)); r =
+// enc(fma(-alpha, s', r)) with p', s' the masked NEW stored values.  Checks
+// (owner: counts + scrubs) x, p, s, r, w; VecArgs.b carries s.
+template <int VS>
+__global__ void __launch_bounds__(256) k_calc_sr(VecArgs a) {
+  __shared__ __align__(16) uint8_t s_lut[128];
+  extern __shared__ __align__(16) uint8_t s_dyn_v[];
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  pdl_wait();   // alpha / beta / stop from the reduction
+  pdl_trigger();
+  const int stop = a.state->stop;
+  const double alpha = a.state->alpha, beta = a.state->beta;
+  const uint8_t* cs = vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
+  (void)cs;
+  __syncthreads();
+  if (stop || rb * 256 >= a.n) return;
+  uint64_t* const S = a.b;
+  const uint64_t keep = vkeep(VS);
+  for (int k = 0; k < 8; k++) {
+    const int64_t pb = rb * 256 + k * 32;
+    if (pb >= a.n) break;
+    const int64_t i = pb + lane;
+    const bool valid = i < a.n;
+    const int64_t lim = a.npad;
+    const uint64_t xw = v_load_check<VS>(a.x, i, lim, lane, true, a.counts, a.due);
+    const uint64_t pw = v_load_check<VS>(a.p, i, lim, lane, true, a.counts, a.due);
+    const uint64_t sw = v_load_check<VS>(S, i, lim, lane, true, a.counts, a.due);
+    const uint64_t rw = v_load_check<VS>(a.r, i, lim, lane, true, a.counts, a.due);
+    const uint64_t ww = v_load_check<VS>(a.w, i, lim, lane, true, a.counts, a.due);
+    const uint64_t pr = valid ? round_k(as_u(fma(beta, as_d(pw & keep), as_d(rw & keep))), vk(VS)) : 0ull;
+    const uint64_t sr = valid ? round_k(as_u(fma(beta, as_d(sw & keep), as_d(ww & keep))), vk(VS)) : 0ull;
+    const uint64_t pe = v_encode<VS>(pr, lane, s_lut);
+    const uint64_t se = v_encode<VS>(sr, lane, s_lut);
+    const uint64_t xr = valid ? round_k(as_u(fma(alpha, as_d(pe & keep), as_d(xw & keep))), vk(VS)) : 0ull;
+    const uint64_t rr = valid ? round_k(as_u(fma(-alpha, as_d(se & keep), as_d(rw & keep))), vk(VS)) : 0ull;
+    const uint64_t xe = v_encode<VS>(xr, lane, s_lut);
+    const uint64_t re = v_encode<VS>(rr, lane, s_lut);
+    if (i < a.npad) { a.p[i] = pe; S[i] = se; a.x[i] = xe; a.r[i] = re; }
   }
 }
 
@@ -1659,16 +1679,48 @@ static __device__ void red_push(double* partials, int64_t rb, double val, const 
   else apply_op(r.op, res, r.st, dueflag != 0);
 }
 
-static __global__ void __launch_bounds__(256) k_reduce(const double* partials, int64_t nrb, int64_t leaves, double* roots,
-                                                uint32_t* ticket, int op, CgState* st, double* out, const int* due) {
+// Single-reduction CG scalar logic: g = r.r, d = w.r of the
+// SpMV w = A r.  op 7: init (rr0); op 6: end of an iteration.
+static __device__ void apply_op_sr(int op, double g, double d, CgState* st, bool dueflag) {
+  if (op == 7) {
+    st->rr0 = st->rro = st->rrn = g;
+    st->pw = d;
+    if (st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; }
+    else if (g == 0.0) { st->stop = 1; st->status = ABFT_OK; st->converged = 1; }
+    else if (st->max_iters <= 0) { st->stop = 1; st->status = ABFT_OK; }
+    else { st->alpha = g / d; st->beta = 0.0; }
+    return;
+  }
+  st->iters += 1;
+  st->rrn = g;
+  st->pw = d;
+  const bool conv = sqrt(g) <= st->tol * sqrt(st->rr0);
+  if (!conv) {
+    const double beta = g / st->rro;
+    st->alpha = g / (d - beta * g / st->alpha);
+    st->beta = beta;
+    st->rro = g;
+  }
+  if (st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; }
+  else if (conv) { st->stop = 1; st->status = ABFT_OK; st->converged = 1; }
+  else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
+}
+
+// TWO: also reduce partials2 (second tree, same order) and apply the
+// single-reduction CG logic (op 6 / 7) to both results.
+template <bool TWO>
+static __global__ void __launch_bounds__(256) k_reduce(const double* partials, int64_t nrb, int64_t leaves,
+                                                       double* roots, uint32_t* ticket, int op, CgState* st,
+                                                       double* out, const int* due, const double* partials2,
+                                                       double* roots2) {
   // Block b reduces leaves [b*L, b*L+L): warp w the aligned sub-range of L/8
   // leaves (warp trees keep the pairwise order), then warp 0 combines the 8
   // warp roots; the last block (ticket) combines the block roots.
-  __shared__ double s_w[8];
+  __shared__ double s_w[8], s_w2[8];
   __shared__ bool s_last;
   pdl_wait();   // partials of the producing kernel
   pdl_trigger();
-  if (st && op != 1 && st->stop) return;
+  if (st && op != 1 && op != 7 && st->stop) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t base = (int64_t)blockIdx.x * leaves;
   const int nw = leaves >= 8 ? 8 : 1;
@@ -1676,16 +1728,21 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
   if (warp < nw) {
     const double r = warp_subtree(partials + base + warp * per, per, nrb - base - warp * per, lane);
     if (lane == 0) s_w[warp] = r;
+    if (TWO) {
+      const double r2 = warp_subtree(partials2 + base + warp * per, per, nrb - base - warp * per, lane);
+      if (lane == 0) s_w2[warp] = r2;
+    }
   }
   __syncthreads();
-  double root = 0.0;
+  double root = 0.0, root2 = 0.0;
   if (warp == 0) {
-    const double v = (lane < nw) ? s_w[lane] : 0.0;
-    root = warp_tree(v, nw);
+    root = warp_tree((lane < nw) ? s_w[lane] : 0.0, nw);
+    if (TWO) root2 = warp_tree((lane < nw) ? s_w2[lane] : 0.0, nw);
   }
   if (gridDim.x > 1) {
     if (threadIdx.x == 0) {
       roots[blockIdx.x] = root;
+      if (TWO) roots2[blockIdx.x] = root2;
       __threadfence();
       s_last = (atomicAdd(ticket, 1u) == gridDim.x - 1);
     }
@@ -1693,12 +1750,15 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
     if (!s_last || warp != 0) return;
     __threadfence();
     root = warp_subtree(roots, gridDim.x, gridDim.x, lane);
+    if (TWO) root2 = warp_subtree(roots2, gridDim.x, gridDim.x, lane);
   }
   if (threadIdx.x != 0) return;
   if (gridDim.x > 1) *ticket = 0;
+  const bool dueflag = *((volatile const int*)due) != 0;
+  if (TWO) { apply_op_sr(op, root2, root, st, dueflag); return; }
   if (op == 0) { *out = root; return; }
-  if (op == 4) { out[0] = root; out[1] = (double)(*((volatile const int*)due)); return; }
-  apply_op(op, root, st, *((volatile const int*)due) != 0);
+  if (op == 4) { out[0] = root; out[1] = (double)(dueflag ? 1 : 0); return; }
+  apply_op(op, root, st, dueflag);
 }
 
 // Multi-GPU: combine the all-gathered (root, due) pairs of P ranks with the top

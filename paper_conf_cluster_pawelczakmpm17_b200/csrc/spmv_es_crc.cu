@@ -4,7 +4,7 @@
 
 namespace abft {
 
-bool spmv_es_crc(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
+bool spmv_es_crc(const SpmvArgs& a, int rs, int vs, int dot, cudaStream_t s) {
   return spmv1<CRC32C>(a, rs, vs, dot, s);
 }
 

@@ -67,7 +67,7 @@ static bool tile_maps(const SpmvArgs& a, TileMaps* m) {
   }
   return true;
 }
-template <int ES, int RS, int VS, bool DOT, bool FUSED = false>
+template <int ES, int RS, int VS, int DOT, bool FUSED = false>
 static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   TileMaps tm;
   if (!tile_maps(a, &tm)) return false;
@@ -94,24 +94,28 @@ static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
 // Returns false only when a fused-calc_p launch (a.p_cur set) was requested
 // and cannot run: the caller fails loudly, there is no unfused fallback here.
 template <int ES, int RS, int VS>
-static bool spmv3(const SpmvArgs& a, bool dot, cudaStream_t s) {
+static bool spmv3(const SpmvArgs& a, int dot, cudaStream_t s) {
   if (a.p_cur) {
     if constexpr (vgrp(VS) == 1) {
-      return dot && tile_ok(a, VS) && spmv_tile_launch<ES, RS, VS, true, true>(a, s);
+      return dot == 1 && tile_ok(a, VS) && spmv_tile_launch<ES, RS, VS, 1, true>(a, s);
     }
     return false;
   }
   if (tile_ok(a, VS)) {
-    if (dot ? spmv_tile_launch<ES, RS, VS, true>(a, s) : spmv_tile_launch<ES, RS, VS, false>(a, s)) return true;
+    const bool ok = dot == 2   ? spmv_tile_launch<ES, RS, VS, 2>(a, s)
+                    : dot == 1 ? spmv_tile_launch<ES, RS, VS, 1>(a, s)
+                               : spmv_tile_launch<ES, RS, VS, 0>(a, s);
+    if (ok) return true;
   }
   const int64_t nrb = (a.nrows + 255) / 256;
   const int blocks = (int)((nrb + 7) / 8);
-  if (dot) launch_k(k_spmv<ES, RS, VS, true>, blocks, 256, 0, s, a);
-  else launch_k(k_spmv<ES, RS, VS, false>, blocks, 256, 0, s, a);
+  if (dot == 2) launch_k(k_spmv<ES, RS, VS, 2>, blocks, 256, 0, s, a);
+  else if (dot == 1) launch_k(k_spmv<ES, RS, VS, 1>, blocks, 256, 0, s, a);
+  else launch_k(k_spmv<ES, RS, VS, 0>, blocks, 256, 0, s, a);
   return true;
 }
 template <int ES, int RS>
-static bool spmv2(const SpmvArgs& a, int vs, bool dot, cudaStream_t s) {
+static bool spmv2(const SpmvArgs& a, int vs, int dot, cudaStream_t s) {
   switch (vs) {
     case NONE: return spmv3<ES, RS, NONE>(a, dot, s);
     case SED: return spmv3<ES, RS, SED>(a, dot, s);
@@ -121,7 +125,7 @@ static bool spmv2(const SpmvArgs& a, int vs, bool dot, cudaStream_t s) {
   }
 }
 template <int ES>
-static bool spmv1(const SpmvArgs& a, int rs, int vs, bool dot, cudaStream_t s) {
+static bool spmv1(const SpmvArgs& a, int rs, int vs, int dot, cudaStream_t s) {
   switch (rs) {
     case NONE: return spmv2<ES, NONE>(a, vs, dot, s);
     case SED: return spmv2<ES, SED>(a, vs, dot, s);

@@ -300,6 +300,9 @@ def _touched_counts(orc, flips, Ac, vc, ES, RS, VS, N, nnz):
                         c[0] ^= np.uint32(1 << b)
             st = _codeword_state(orc, "val", 0, v, c, None, None, ES, RS, VS, N)
             t, s = orc.ELEM, ES
+            # a DUE element keeps its stored bits: check_all range-checks the masked stored column
+            if st == orc.DUE and (int(c[0]) & (0x7FFFFFFF if ES == orc.SED else 0x00FFFFFF)) >= N:
+                exp[orc.ELEM, ES, orc.RANGE] += 1
         elif key[0] == "rp":
             g0 = key[1] * G
             ents = Ac.rowptr[g0:g0 + G].copy()
