@@ -311,7 +311,7 @@ def _touched_counts(orc, flips, Ac, vc, ES, RS, VS, N, nnz):
                     ents[wi - g0] ^= np.uint32(1 << b)
             st = _codeword_state(orc, "rowptr", 0, None, None, ents, None, ES, RS, VS, N)
             t, s = orc.ROWPTR, RS
-            if st == orc.DUE:
+            if st != orc.CORRECTED:   # DUE, or an undetected (even-weight SED) change: stored bits are used
                 for q in range(G):
                     dues_rp[g0 + q] = int(ents[q]) & (0x7FFFFFFF if RS == orc.SED else 0x0FFFFFFF)
         else:
@@ -325,7 +325,7 @@ def _touched_counts(orc, flips, Ac, vc, ES, RS, VS, N, nnz):
         if st != orc.CLEAN:
             exp[t, s, orc.DET] += 1
             exp[t, s, orc.COR if st == orc.CORRECTED else orc.UNC] += 1
-    # check_all's row pass: the range rule on the masked stored entries of DUE'd row pointers
+    # check_all's row pass: the range rule on the masked stored entries of row pointers left corrupted
     rows = set()
     for i in dues_rp:
         rows.update(r_ for r_ in (i - 1, i) if 0 <= r_ < N)
