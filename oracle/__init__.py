@@ -86,6 +86,10 @@ def lib():
                                  C.c_void_p]
         L.or_cg_solve_sr.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
                                      C.c_int, C.c_void_p, C.c_void_p, C.c_void_p, C.c_int]
+        L.or_cg_solve_log.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_int,
+                                      C.c_int, C.c_void_p, C.c_void_p, dp, dp]
+        L.or_cheby_solve.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_double,
+                                     C.c_double, C.c_int, C.c_int, C.c_void_p, C.c_void_p]
         L.or_vec_masked.argtypes = [u64p, C.c_int64, C.c_int, dp]
         L.or_round_k.restype = C.c_uint64
         L.or_round_k.argtypes = [C.c_uint64, C.c_int]
@@ -338,3 +342,42 @@ def cg_solve_sr(A: Matrix, b, x, r, p, w, s, scheme, tol=1e-10, max_iters=10000,
                                 due_policy, C.byref(res), counts.ctypes.data if counts is not None else None,
                                 f.ctypes.data if len(f) else None, len(f))
     return code, res
+
+
+def cg_solve_log(A: Matrix, b, x, r, p, w, scheme, tol=1e-10, max_iters=30, due_policy=1, counts=None):
+    """Protected CG that also returns its step coefficients alpha_k, beta_k
+    (the Lanczos data of TeaLeaf's spectrum estimate)."""
+    s = A.cstruct()
+    res = CGResult()
+    al = np.zeros(max(max_iters, 1))
+    bl = np.zeros(max(max_iters, 1))
+    st = lib().or_cg_solve_log(C.byref(s), _p(b, C.c_uint64), _p(x, C.c_uint64), _p(r, C.c_uint64),
+                               _p(p, C.c_uint64), _p(w, C.c_uint64), scheme, tol, max_iters, due_policy, C.byref(res),
+                               counts.ctypes.data if counts is not None else None, _p(al, C.c_double),
+                               _p(bl, C.c_double))
+    return st, res, al[:res.iters], bl[:max(res.iters - 1, 0)] if res.iters else bl[:0]
+
+
+def lanczos_bounds(alphas, betas):
+    """Extreme eigenvalues of the Lanczos tridiagonal built from CG's step
+    coefficients (T_jj = 1/a_j + b_{j-1}/a_{j-1}, T_{j,j+1} = sqrt(b_j)/a_j),
+    by numpy.linalg.eigvalsh (library routine) — TeaLeaf's eigenvalue estimate."""
+    k = len(alphas)
+    T = np.zeros((k, k))
+    for j in range(k):
+        T[j, j] = 1.0 / alphas[j] + (betas[j - 1] / alphas[j - 1] if j > 0 else 0.0)
+        if j + 1 < k:
+            T[j, j + 1] = T[j + 1, j] = np.sqrt(betas[j]) / alphas[j]
+    ev = np.linalg.eigvalsh(T)
+    return float(ev[0]), float(ev[-1])
+
+
+def cheby_solve(A: Matrix, b, u, r, p, w, scheme, eigmin, eigmax, tol=1e-10, max_iters=10000, due_policy=1,
+                counts=None):
+    """Protected Chebyshev iteration (TeaLeaf) with spectrum bounds [eigmin, eigmax]."""
+    s = A.cstruct()
+    res = CGResult()
+    st = lib().or_cheby_solve(C.byref(s), _p(b, C.c_uint64), _p(u, C.c_uint64), _p(r, C.c_uint64),
+                              _p(p, C.c_uint64), _p(w, C.c_uint64), scheme, float(eigmin), float(eigmax), tol,
+                              max_iters, due_policy, C.byref(res), counts.ctypes.data if counts is not None else None)
+    return st, res

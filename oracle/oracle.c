@@ -17,6 +17,9 @@
  *                    DESIGN.md §3.9 (reading R27)
  *         single-reduction CG (S§8(f) f3): Chronopoulos-Gear recurrences,
  *                    DESIGN.md §4.1 (reading R28), or_cg_solve_sr
+ *         Chebyshev  TeaLeaf's Chebyshev iteration (S§8(f) f4), DESIGN.md §4.3
+ *                    (reading R32), or_cheby_solve; CG coefficient log
+ *                    or_cg_solve_log for the spectrum estimate
  *         faults     O10 scheduled bit flips (S§8(c) O10): XOR before init /
  *                    before iteration k's SpMV, or_cg_solve_sched
  *         CRC fix    1EC4ED single-bit correction of a failing CRC32C codeword
@@ -901,6 +904,10 @@ static void apply_faults(or_csr* A, uint64_t* v[5], const or_fault* f, int nf, i
   }
 }
 
+/* optional CG coefficient log (or_cg_solve_log): alpha_k, beta_k of every iteration */
+static double* g_alog = NULL;
+static double* g_blog = NULL;
+
 static int cg_run(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
                   int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, int interval,
                   const or_fault* faults, int nfaults) {
@@ -919,11 +926,13 @@ static int cg_run(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p,
     apply_faults(A, vecs, faults, nfaults, k);
     dues = or_spmv_mode(A, p, n, vs, w, n, cnt, &pw, access_mode(k, interval));
     double alpha = rro / pw;
+    if (g_alog) g_alog[k - 1] = alpha;
     dues += or_calc_ur(x, p, r, w, n, vs, alpha, cnt, &rrn);
     res->iters = k; res->rrn = rrn;
     int conv = sqrt(rrn) <= tol * sqrt(rr0);
     if (!conv) {
       double beta = rrn / rro;
+      if (g_blog) g_blog[k - 1] = beta;
       dues += or_calc_p(p, r, n, vs, beta, cnt);
       rro = rrn;
     }
@@ -1056,6 +1065,83 @@ int or_cg_solve_sr(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p
       alpha = gnew / (delta - beta * gnew / alpha);
       gamma = gnew;
     }
+    if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+    if (conv) return OK;
+  }
+  res->status = (max_iters > 0) ? E_NOT_CONVERGED : OK;
+  return res->status;
+}
+
+/* CG with its step coefficients logged: alog[k-1] = alpha_k, blog[k-1] =
+ * beta_k (iterations that computed one) — the Lanczos data TeaLeaf's
+ * Chebyshev / PPCG solvers estimate the spectrum from. */
+int or_cg_solve_log(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, int vs, double tol,
+                    int max_iters, int due_policy, or_cg_result* res, counts_t* cnt, double* alog, double* blog) {
+  g_alog = alog;
+  g_blog = blog;
+  int st = or_cg_solve_sched(A, b, x, r, p, w, vs, tol, max_iters, due_policy, res, cnt, 1, NULL, 0);
+  g_alog = g_blog = NULL;
+  return st;
+}
+
+/* ---------------------------------------------------------- Chebyshev iteration
+ * S§8(f) f4: TeaLeaf's Chebyshev solver (ref [19]; reading R32,
+ * DESIGN.md §4.3) with the paper's protection: every vector read
+ * checked, every write re-encoded.  Spectrum bounds [eigmin, eigmax] given.
+ * theta = (eigmax + eigmin)/2, delta = (eigmax - eigmin)/2, sigma = theta/delta,
+ * rho_0 = 1/sigma; step k: rho_k = 1/(2 sigma - rho_{k-1}), alpha_k = rho_k
+ * rho_{k-1}, beta_k = (2 rho_k)/delta.
+ * Init:  w = A u; r = enc(b - w); rr0 = r.r; p = enc(r'/theta); u = enc(u' + p').
+ * Iter k: w = A u; r = enc(b - w); rr = r.r; p = enc(fma(alpha_k, p', beta_k * r'));
+ *         u = enc(u' + p'); converged when sqrt(rr) <= tol sqrt(rr0) -> k. */
+static int64_t cheb_update(uint64_t* b, uint64_t* w, uint64_t* p, uint64_t* u, uint64_t* r, int64_t n, int vs,
+                           int init, double theta, double alpha, double beta, counts_t* cnt, double* rr) {
+  double* B = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* W = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* P = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* U = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  int64_t dues = vdec(b, n, vs, B, cnt) + vdec(w, n, vs, W, cnt) + (init ? 0 : vdec(p, n, vs, P, cnt)) +
+                 vdec(u, n, vs, U, cnt);
+  for (int64_t i = 0; i < n; i++) B[i] = B[i] - W[i];
+  venc(r, B, n, vs);
+  vmasked(r, n, vs, B);                       /* B = r' */
+  *rr = or_dot_red1(B, B, n);
+  for (int64_t i = 0; i < n; i++) {
+    if (init) P[i] = B[i] / theta;
+    else {
+      double t = beta * B[i];
+      P[i] = fma(alpha, P[i], t);
+    }
+  }
+  venc(p, P, n, vs);
+  vmasked(p, n, vs, P);
+  for (int64_t i = 0; i < n; i++) U[i] = U[i] + P[i];
+  venc(u, U, n, vs);
+  free(B); free(W); free(P); free(U);
+  return dues;
+}
+
+int or_cheby_solve(or_csr* A, uint64_t* b, uint64_t* u, uint64_t* r, uint64_t* p, uint64_t* w, int vs,
+                   double eigmin, double eigmax, double tol, int max_iters, int due_policy, or_cg_result* res,
+                   counts_t* cnt) {
+  init_instances();
+  int64_t n = A->nrows;
+  double theta = (eigmax + eigmin) / 2.0, delta = (eigmax - eigmin) / 2.0;
+  double sigma = theta / delta, rho = 1.0 / sigma, rr0, rr;
+  res->iters = 0; res->status = OK; res->rr0 = 0.0; res->rrn = 0.0;
+  int64_t dues = or_spmv_mode(A, u, n, vs, w, n, cnt, NULL, M_CORRECT);
+  dues += cheb_update(b, w, p, u, r, n, vs, 1, theta, 0.0, 0.0, cnt, &rr0);
+  res->rr0 = rr0; res->rrn = rr0;
+  if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+  if (rr0 == 0.0) return OK;
+  for (int k = 1; k <= max_iters; k++) {
+    double rho_new = 1.0 / (2.0 * sigma - rho);
+    double alpha = rho_new * rho, beta = (2.0 * rho_new) / delta;
+    rho = rho_new;
+    dues = or_spmv_mode(A, u, n, vs, w, n, cnt, NULL, M_CORRECT);
+    dues += cheb_update(b, w, p, u, r, n, vs, 0, theta, alpha, beta, cnt, &rr);
+    res->iters = k; res->rrn = rr;
+    int conv = sqrt(rr) <= tol * sqrt(rr0);
     if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
     if (conv) return OK;
   }

@@ -580,10 +580,13 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
 struct TileMaps { CUtensorMap val, col, vin, vcur, vin8; int has_vmaps; };
 
 constexpr int TILE_TY = 8;
-// window row: x = tx0-2 .. tx0+257 (one TMA box of 130 double pairs); the
+// window row: x = tx0-2 .. tx0+261 (one TMA box of 132 double pairs); the
 // tile's own cells sit at slots TILE_WX0 .. TILE_WX0+255
 constexpr int TILE_WX0 = 2;
-constexpr int TILE_WW = 256 + 4;
+// (x = tx0-2 .. tx0+261: 132 double pairs per row, so every row starts on a
+// 64-byte boundary and any two rows on a 128-byte one — TMA destinations must
+// be 128-byte aligned; the persistent kernel lands 8 rows at row 2)
+constexpr int TILE_WW = 256 + 8;
 constexpr int TILE_PE = 160;                                   // elements per warp per pass (32 rows x 5)
 #ifndef ABFT_TILE_NST
 #define ABFT_TILE_NST 3
@@ -591,7 +594,7 @@ constexpr int TILE_PE = 160;                                   // elements per w
 constexpr int TILE_NST = ABFT_TILE_NST;                        // pipeline stages
 constexpr int TILE_STAGE_VAL = TILE_TY * TILE_PE * 8;          // 10240
 constexpr int TILE_STAGE = TILE_STAGE_VAL + TILE_TY * TILE_PE * 4;   // + 5120
-constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 20800
+constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 21120
 constexpr int TILE_RP = 264;                                   // rowptr entries staged per warp
 constexpr int TILE_OFF_WIN = TILE_NST * TILE_STAGE;            // stages first (128-B aligned)
 constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
@@ -935,7 +938,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
     }
     return;
   }
-  // ---- 2. decoded `in` window: rows ty0-1 .. ty0+TILE_TY, x = tx0-2 .. tx0+257
+  // ---- 2. decoded `in` window: rows ty0-1 .. ty0+TILE_TY, x = tx0-2 .. tx0+261
   const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - TILE_WX0;   // in-index of slot (0,0)
   constexpr int WPER = (TILE_WW + 31) / 32;                             // 9 slots per lane per window row
   constexpr int VG = vgrp(VS);

@@ -47,7 +47,7 @@ static bool tile_maps(const SpmvArgs& a, TileMaps* m) {
                     CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   if (r1 != CUDA_SUCCESS || r2 != CUDA_SUCCESS) return false;
   // the input vector (and p_cur) as [rows][n/2][2] doubles: one box = the
-  // decoded window's TILE_TY+2 rows x 130 pairs (x = tx0-2 .. tx0+257)
+  // decoded window's TILE_TY+2 rows x 132 pairs (x = tx0-2 .. tx0+261)
   m->has_vmaps = 0;
   static const bool no_vmaps = [] { const char* e = getenv("ABFT_NO_VMAPS"); return e && e[0] == '1'; }();
   if (!no_vmaps && (a.npad_in % n) == 0 && (a.row_base % n) == 0 && (n % 2) == 0) {
