@@ -156,6 +156,27 @@ int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, ab
  * Same matrix / vector conventions, options, counters and statuses as
  * abft_cg_solve; s is a sixth vector like the others (scheme, length).
  * Single GPU, every access checked (check_interval <= 1, else ABFT_E_SHAPE). */
+/* Protected Chebyshev iteration (S§8(f) f4: TeaLeaf's Chebyshev solver,
+ * ref [19] P:778-781, reading R32) for an SPD matrix with
+ * spectrum inside [eigmin, eigmax]: per step one protected SpMV w = A u and one
+ * fused update r = b - w, p = alpha_k p + beta_k r (first step p = r/theta),
+ * u += p with r.r, every operand checked and every result re-encoded as in the
+ * paper's CG.  x holds u (in: u0, out: u); stops when
+ * sqrt(r.r) <= tol sqrt(r0.r0).  Same conventions, counters and statuses as
+ * abft_cg_solve; single GPU, every access checked.  Errors: ABFT_E_INVALID
+ * (eigmax <= eigmin), ABFT_E_SHAPE. */
+int abft_cheby_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                     abft_vec* w, double eigmin, double eigmax, const abft_cg_opts* opts, abft_cg_result* res,
+                     abft_counts* dcnt, void* stream);
+/* TeaLeaf's spectrum estimate (reading R33): `steps` (2..128)
+ * protected CG iterations from x (opts supply the policy; tol is ignored),
+ * then the extreme eigenvalues of the Lanczos tridiagonal built from the CG
+ * step coefficients (T_jj = 1/alpha_j + beta_{j-1}/alpha_{j-1},
+ * T_{j,j+1} = sqrt(beta_j)/alpha_j) by Sturm bisection.  x is left at the CG
+ * iterate.  The caller applies any safety margin. */
+int abft_cg_spectrum(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                     abft_vec* w, int steps, const abft_cg_opts* opts, double* eigmin, double* eigmax,
+                     abft_cg_result* res, abft_counts* dcnt, void* stream);
 int abft_cg_solve_sr(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r,
                      abft_vec* p, abft_vec* w, abft_vec* s, const abft_cg_opts* opts, abft_cg_result* res,
                      abft_counts* dcnt, void* stream);

@@ -71,6 +71,12 @@ _sig = {
     "abft_cg_solve_sr": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                    C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts),
                                    C.POINTER(CGResult), _P, _P]),
+    "abft_cheby_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
+                                   C.POINTER(Vec), C.POINTER(Vec), C.c_double, C.c_double, C.POINTER(CGOpts),
+                                   C.POINTER(CGResult), _P, _P]),
+    "abft_cg_spectrum": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
+                                   C.POINTER(Vec), C.POINTER(Vec), C.c_int, C.POINTER(CGOpts),
+                                   C.POINTER(C.c_double), C.POINTER(C.c_double), C.POINTER(CGResult), _P, _P]),
     "abft_check_all": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.c_int, C.c_int, _P, _P]),
     "abft_calc_ur": (C.c_int, [_P, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.c_double, _P, _P,
                                _P]),
@@ -333,6 +339,35 @@ def cg_solve_sr(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: 
                                  counts.ptr if counts else None, _stream(stream))
     _check(code, "abft_cg_solve_sr", allow=(E_DUE, E_NOT_CONVERGED))
     return res
+
+
+def cheby_solve(ctx: Context, A, b: Vector, u: Vector, r: Vector, p: Vector, w: Vector, eigmin: float, eigmax: float,
+                tol=1e-10, max_iters=10000, due_policy=0, counts: Counters | None = None, poll_every=16,
+                stream=None) -> CGResult:
+    """Protected Chebyshev iteration with spectrum bounds (abft_cheby_solve)."""
+    arr, n = _chunks(A)
+    opts = CGOpts(tol, max_iters, due_policy, poll_every, 1)
+    res = CGResult()
+    vs = [v.cstruct() for v in (b, u, r, p, w)]
+    code = _lib.abft_cheby_solve(ctx.h, arr, n, *[C.byref(v) for v in vs], float(eigmin), float(eigmax),
+                                 C.byref(opts), C.byref(res), counts.ptr if counts else None, _stream(stream))
+    _check(code, "abft_cheby_solve", allow=(E_DUE, E_NOT_CONVERGED))
+    return res
+
+
+def cg_spectrum(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vector, steps=30, due_policy=1,
+                counts: Counters | None = None, poll_every=16, stream=None):
+    """TeaLeaf's Lanczos spectrum estimate from `steps` protected CG steps
+    (abft_cg_spectrum): returns (eigmin, eigmax, CGResult)."""
+    arr, n = _chunks(A)
+    opts = CGOpts(0.0, steps, due_policy, poll_every, 1)
+    res = CGResult()
+    lo, hi = C.c_double(), C.c_double()
+    vs = [v.cstruct() for v in (b, x, r, p, w)]
+    _check(_lib.abft_cg_spectrum(ctx.h, arr, n, *[C.byref(v) for v in vs], int(steps), C.byref(opts), C.byref(lo),
+                                 C.byref(hi), C.byref(res), counts.ptr if counts else None, _stream(stream)),
+           "abft_cg_spectrum")
+    return lo.value, hi.value, res
 
 
 def calc_ur(ctx: Context, x: Vector, p: Vector, r: Vector, w: Vector, alpha: float,

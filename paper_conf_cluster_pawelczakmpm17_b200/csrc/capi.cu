@@ -435,6 +435,8 @@ struct RankRun {
   int nchunks = 0;
   abft_vec* v[5] = {};   // b x r p w
   abft_vec* s_vec = nullptr;   // single-reduction CG: its extra vector s
+  bool cheb = false;           // Chebyshev iteration with bounds [eigmin, eigmax]; x is u
+  double eigmin = 0.0, eigmax = 0.0;
   DevCounts* cnt = nullptr;
   int64_t n = 0, nrb = 0, n_ext = 0;
   VecArgs va{};
@@ -566,6 +568,12 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   const int scheme = R[0].x()->scheme;
   // single-reduction CG (Chronopoulos-Gear, S§8(f) f3): one GPU, every access checked
   const bool sr = R[0].s_vec != nullptr;
+  const bool cheb = R[0].cheb;
+  if (cheb) {
+    if (d || nl != 1) return fail(ABFT_E_SHAPE, "Chebyshev iteration runs on one GPU");
+    if (opts->check_interval > 1) return fail(ABFT_E_SHAPE, "Chebyshev iteration checks every access");
+    if (!(R[0].eigmax > R[0].eigmin)) return fail(ABFT_E_INVALID, "Chebyshev bounds need eigmax > eigmin");
+  }
   if (sr) {
     if (d || nl != 1) return fail(ABFT_E_SHAPE, "single-reduction CG runs on one GPU");
     if (opts->check_interval > 1) return fail(ABFT_E_SHAPE, "single-reduction CG checks every access");
@@ -591,7 +599,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   // G = 1 vector scheme; p is double-buffered with ctx->p_alt
   const int64_t npad_ext = vec_padded_len(R[0].n_ext, scheme);
   // (a fault schedule addresses the caller's p: the double-buffered fused CG is off then)
-  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0 && ctx->nfaults == 0 && !sr;
+  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0 && ctx->nfaults == 0 && !sr && !cheb;
   abft_vec* const p = R[0].p();
   abft_vec* const r = R[0].r();
   if (fused) {
@@ -621,6 +629,12 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   h.abort_policy = opts->due_policy == 0 ? 1 : 0;
   h.dist = multi ? 1 : 0;
   h.fused = fused ? 1 : 0;
+  if (cheb) {   // host arithmetic, rounded as written
+    h.ch_theta = (R[0].eigmax + R[0].eigmin) / 2.0;
+    h.ch_delta = (R[0].eigmax - R[0].eigmin) / 2.0;
+    h.ch_sigma = h.ch_theta / h.ch_delta;
+    h.ch_rho = 1.0 / h.ch_sigma;
+  }
   for (int q = 0; q < nl; q++) {
     count_launch(launch_set_state(h, R[q].ctx->state, s));
     CUDA_TRY(cudaMemsetAsync(R[q].ctx->due, 0, sizeof(int), s));
@@ -639,9 +653,13 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     if (e) return e;
   }
   prof.end();
-  for (int q = 0; q < nl; q++) count_launch(launch_init_r(R[q].va, scheme, s));
+  if (!cheb)
+    for (int q = 0; q < nl; q++) count_launch(launch_init_r(R[q].va, scheme, s));
   VecArgs vsr = R[0].va;   // single-reduction update: VecArgs.b carries s
-  if (sr) {
+  if (cheb) {   // r = b - A u0; p = r/theta; u += p; rr0
+    count_launch(launch_cheb(R[0].va, scheme, 1, s));
+    if ((e = finish_dot(R, nl, d, 8, s))) return e;
+  } else if (sr) {
     vsr.b = reinterpret_cast<uint64_t*>(R[0].s_vec->data) + n_halo;
     // p = s = encoded +0.0, then w = A r with both dots (gamma = r.r, delta = w.r)
     for (abft_vec* v : {R[0].p(), R[0].s_vec}) {
@@ -708,6 +726,19 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
       const int64_t kk = launched + it + 1;
       for (int q = 0; q < nl; q++)   // O10: faults of this iteration, before its SpMV
         count_launch(launch_inject_sched(R[q].ctx->faults, R[q].ctx->nfaults, R[q].ctx->state, 1, ss));
+      if (cheb) {   // w = A u; r = b - w, p, u; r.r and the step coefficients
+        prof.begin(0);
+        e2 = spmv_chunks(ctx, R[0].A, R[0].nchunks, R[0].x(), R[0].w(), 0, R[0].cnt, ctx->state, ss, nullptr);
+        prof.end();
+        if (e2) return e2;
+        prof.begin(1);
+        count_launch(launch_cheb(R[0].va, scheme, 0, ss));
+        prof.end();
+        prof.begin(3);
+        if ((e2 = finish_dot(R, nl, d, 9, ss))) return e2;
+        prof.end();
+        continue;
+      }
       if (sr) {   // update, then w = A r with both dots, then the one reduction
         prof.begin(1);
         count_launch(launch_calc_sr(vsr, scheme, ss));
@@ -911,6 +942,71 @@ int abft_cg_solve_sr(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b,
   RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
   R.s_vec = sv;
   return cg_run(&R, 1, nullptr, 0, opts, res, (cudaStream_t)stream);
+}
+
+int abft_cheby_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                     abft_vec* w, double eigmin, double eigmax, const abft_cg_opts* opts, abft_cg_result* res,
+                     abft_counts* dcnt, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  R.cheb = true;
+  R.eigmin = eigmin;
+  R.eigmax = eigmax;
+  return cg_run(&R, 1, nullptr, 0, opts, res, (cudaStream_t)stream);
+}
+
+// Extreme eigenvalues of the symmetric tridiagonal (diag a[0..k), off-diagonal
+// e[0..k-1)) by Sturm-sequence bisection (host, 64 halvings from the
+// Gershgorin interval): TeaLeaf's Lanczos spectrum estimate.
+static int sturm_count(const double* a, const double* e, int k, double x) {
+  int neg = 0;
+  double q = a[0] - x;
+  if (q < 0) neg++;
+  for (int i = 1; i < k; i++) {
+    if (q == 0.0) q = 1e-300;
+    q = (a[i] - x) - e[i - 1] * e[i - 1] / q;
+    if (q < 0) neg++;
+  }
+  return neg;   // eigenvalues < x
+}
+static double tridiag_eig(const double* a, const double* e, int k, int which /* 0 min, 1 max */) {
+  double lo = a[0], hi = a[0];
+  for (int i = 0; i < k; i++) {
+    const double rad = (i > 0 ? fabs(e[i - 1]) : 0.0) + (i + 1 < k ? fabs(e[i]) : 0.0);
+    lo = fmin(lo, a[i] - rad);
+    hi = fmax(hi, a[i] + rad);
+  }
+  const int target = which ? k - 1 : 0;   // index of the wanted eigenvalue
+  for (int it = 0; it < 64; it++) {
+    const double mid = 0.5 * (lo + hi);
+    if (sturm_count(a, e, k, mid) > target) hi = mid;
+    else lo = mid;
+  }
+  return 0.5 * (lo + hi);
+}
+
+int abft_cg_spectrum(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                     abft_vec* w, int steps, const abft_cg_opts* opts, double* eigmin, double* eigmax,
+                     abft_cg_result* res, abft_counts* dcnt, void* stream) {
+  if (!ctx || !opts || !eigmin || !eigmax || !res) return fail(ABFT_E_INVALID, "null argument");
+  if (steps < 2 || steps > CG_LOG) return fail(ABFT_E_INVALID, "steps must be in [2, %d]", CG_LOG);
+  abft_cg_opts o = *opts;
+  o.max_iters = steps;
+  o.tol = 0.0;
+  RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  int e = cg_run(&R, 1, nullptr, 0, &o, res, (cudaStream_t)stream);
+  if (e != ABFT_OK && e != ABFT_E_NOT_CONVERGED) return e;
+  const CgState& h = *ctx->h_state;   // the solve's final state (read back by cg_run)
+  const int k = h.iters;
+  if (k < 2) return fail(ABFT_E_SHAPE, "spectrum estimate needs >= 2 CG steps (got %d)", k);
+  std::vector<double> a(k), off(k);
+  for (int j = 0; j < k; j++) {
+    a[j] = 1.0 / h.alpha_log[j] + (j > 0 ? h.beta_log[j - 1] / h.alpha_log[j - 1] : 0.0);
+    if (j + 1 < k) off[j] = sqrt(h.beta_log[j]) / h.alpha_log[j];
+  }
+  *eigmin = tridiag_eig(a.data(), off.data(), k, 0);
+  *eigmax = tridiag_eig(a.data(), off.data(), k, 1);
+  return ABFT_OK;
 }
 
 int abft_dist_get_unique_id(void* out128) {

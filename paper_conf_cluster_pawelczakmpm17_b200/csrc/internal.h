@@ -20,7 +20,15 @@ struct CgState {
   // the rrn reduction; a stop that the unfused order takes AFTER calc_p leaves
   // pending_p = 1 and the host runs that calc_p on its own.
   int32_t fused, pending_p;
+  // Chebyshev iteration: theta, delta, sigma of the spectrum
+  // bounds and the recurrence's rho (alpha / beta above hold its step
+  // coefficients)
+  double ch_theta, ch_delta, ch_sigma, ch_rho;
+  // CG step coefficients of the first CG_LOG iterations (Lanczos data of the
+  // spectrum estimate, abft_cg_spectrum)
+  double alpha_log[128], beta_log[128];
 };
+constexpr int CG_LOG = 128;
 
 struct DevCounts { unsigned long long v[3][5][4]; };
 
@@ -131,6 +139,8 @@ int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* 
 // (r.r) in RED-1 order and apply op 7 (init) / 6 (iteration)
 int launch_reduce_sr(const double* partials, const double* partials2, int64_t nrb, double* roots, double* roots2,
                      uint32_t* ticket, int op, CgState* st, const int* due, cudaStream_t s);
+// Chebyshev update: init = 1 -> the first step (p = r/theta)
+int launch_cheb(const VecArgs& a, int vs, int init, cudaStream_t s);
 // single-reduction CG update: p, s, x, r (VecArgs.b carries s)
 int launch_calc_sr(const VecArgs& a, int vs, cudaStream_t s);
 int launch_combine(const double* gathered, int P, int op, CgState* st, int* due, cudaStream_t s);

@@ -134,6 +134,23 @@ int launch_calc_sr(const VecArgs& a, int vs, cudaStream_t s) {
   }
   return 1;
 }
+template <bool INIT>
+static void launch_cheb_t(const VecArgs& a, int vs, cudaStream_t s) {
+  int nb = blocks_rb(a.n);
+  switch (vs) {
+    case NONE: launch_k(k_cheb<NONE, INIT>, nb, 256, 0, s, a); break;
+    case SED: launch_k(k_cheb<SED, INIT>, nb, 256, 0, s, a); break;
+    case SECDED64: launch_k(k_cheb<SECDED64, INIT>, nb, 256, 0, s, a); break;
+    case SECDED128: launch_k(k_cheb<SECDED128, INIT>, nb, 256, 0, s, a); break;
+    default: launch_k(k_cheb<CRC32C, INIT>, nb, 256, vec_dyn_smem<CRC32C>(), s, a); break;
+  }
+}
+int launch_cheb(const VecArgs& a, int vs, int init, cudaStream_t s) {
+  if (a.n <= 0) return 0;
+  if (init) launch_cheb_t<true>(a, vs, s);
+  else launch_cheb_t<false>(a, vs, s);
+  return 1;
+}
 int launch_init_r(const VecArgs& a, int vs, cudaStream_t s) {
   if (a.n <= 0) return 0;
   int nb = blocks_rb(a.n);

@@ -577,15 +577,14 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
 // val / col element streams ([ny][5n] boxes); vin / vcur: the SpMV input
 // vector (and the fused path's p_cur) viewed as [rows][n/2][2] doubles, one
 // box = the tile's decoded-window rows (has_vmaps = 0: not built)
-struct TileMaps { CUtensorMap val, col, vin, vcur, vin8; int has_vmaps; };
+struct TileMaps { CUtensorMap val, col, vin, vcur; int has_vmaps; };
 
 constexpr int TILE_TY = 8;
 // window row: x = tx0-2 .. tx0+261 (one TMA box of 132 double pairs); the
 // tile's own cells sit at slots TILE_WX0 .. TILE_WX0+255
 constexpr int TILE_WX0 = 2;
-// (x = tx0-2 .. tx0+261: 132 double pairs per row, so every row starts on a
-// 64-byte boundary and any two rows on a 128-byte one — TMA destinations must
-// be 128-byte aligned; the persistent kernel lands 8 rows at row 2)
+// (x = tx0-2 .. tx0+261: 132 double pairs per row, so any two rows start on a
+// 128-byte boundary, as TMA destinations must)
 constexpr int TILE_WW = 256 + 8;
 constexpr int TILE_PE = 160;                                   // elements per warp per pass (32 rows x 5)
 #ifndef ABFT_TILE_NST
@@ -1175,274 +1174,6 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   }
 }
 
-// ================================================ persistent tiled SpMV (a3)
-// Same per-row work, codec and counting as k_spmv_tile, for G = 1 vector
-// schemes with the TMA window (the production configuration), but each CTA
-// walks a contiguous run of tiles down a tile column (tiles in column-major
-// order, runs balanced across a grid of (SMs x resident CTAs)):
-//  * the element-stage ring keeps running across tile boundaries (the next
-//    tile's first passes are in flight while the current tile finishes), and
-//    the barrier set-up / CG-state load / PDL wait happen once per CTA;
-//  * consecutive tiles share two window rows (grid rows ty0 + 7 and ty0 + 8):
-//    they are moved in SMEM and only 8 new rows arrive by TMA and are decoded
-//    (1.02 instead of 1.27 decodes per row).  The shared halo row below the
-//    previous tile becomes an own row of the next one: it was checked there
-//    without counting, so if that check failed anywhere the row is checked
-//    again from global memory with owner semantics (count + scrub) — the same
-//    counts as k_spmv_tile.
-struct TileRun { int64_t n, ny, tiles_x, lo, nty; };
-static __device__ __forceinline__ void tile_of(const TileRun& R, int64_t t, int64_t& tx0, int64_t& ty0) {
-  tx0 = (t / R.nty) << 8;
-  ty0 = (R.lo + t % R.nty) * TILE_TY;
-}
-// Producer: pass g of this CTA's tile run (tile t0 + g / 8, pass g % 8).
-static __device__ __forceinline__ void pers_produce(const TileMaps& tm, uint8_t* s_dyn, uint64_t* full,
-                                                    const TileRun& R, int64_t t0, int64_t t1, int64_t g) {
-  const int64_t t = t0 + g / 8;
-  if (t >= t1) return;
-  int64_t tx0, ty0;
-  tile_of(R, t, tx0, ty0);
-  const int st = (int)(g % TILE_NST);
-  tile_produce(tm, s_dyn + st * TILE_STAGE, &full[st], tx0, ty0, (int)(g % 8));
-}
-
-template <int ES, int RS, int VS, int DOT>
-__global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_pers(const SpmvArgs a, const __grid_constant__ TileMaps tm) {
-  static_assert(vgrp(VS) == 1, "persistent tiled SpMV: G = 1 vector schemes");
-  extern __shared__ uint8_t s_raw[];
-  __shared__ __align__(16) uint8_t s_lut[128];
-  __shared__ SpmvArgs s_args;
-  __shared__ int s_bad_below;   // the halo-below row of the current window failed a (non-owner) check
-  uint8_t* s_dyn = s_raw + ((128u - (smem_u32(s_raw) & 127u)) & 127u);
-  double* s_win = reinterpret_cast<double*>(s_dyn + TILE_OFF_WIN);
-  uint64_t* full = reinterpret_cast<uint64_t*>(s_dyn + TILE_OFF_BAR);
-  uint64_t* empty = full + TILE_NST;
-  uint64_t* winbar = empty + TILE_NST;
-  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  uint32_t* srp = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_RP) + warp * TILE_RP;
-  constexpr bool SLICE = (ES == CRC32C || RS == CRC32C);
-  uint32_t* s_slice = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_CRC);
-  TileRun R;
-  R.n = a.stencil_n;
-  R.ny = a.nrows / R.n;
-  R.tiles_x = R.n >> 8;
-  R.lo = a.ty_lo;
-  R.nty = (a.ty_hi > 0 ? a.ty_hi : (R.ny + TILE_TY - 1) / TILE_TY) - a.ty_lo;
-  const int64_t T = R.tiles_x * R.nty;
-  const int64_t t0 = (int64_t)blockIdx.x * T / gridDim.x, t1 = ((int64_t)blockIdx.x + 1) * T / gridDim.x;
-  if (t0 >= t1) return;
-  const int64_t n = R.n, ny = R.ny;
-  // ---- producer set-up: barriers, the first TILE_NST passes (matrix: before the PDL wait)
-  if (threadIdx.x == 0) {
-#pragma unroll
-    for (int s = 0; s < TILE_NST; s++) {
-      mbar_init(&full[s], 1);
-      mbar_init(&empty[s], TILE_TY);
-    }
-    mbar_init(winbar, 1);
-    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-    for (int g = 0; g < TILE_NST; g++) pers_produce(tm, s_dyn, full, R, t0, t1, g);
-    s_bad_below = 0;
-  }
-  if (VS == SECDED64) load_lut(s_lut);
-  if (SLICE) smem_fill(s_slice, &a.crc->slice[0][0], CRC_SLICE_WORDS);
-  pdl_wait();   // the previous kernel's writes (p, CG state, counters) are visible from here
-  pdl_trigger();
-  if (threadIdx.x == 0) s_args = a;
-  __syncthreads();
-  const int stop_v = a.state ? a.state->stop : 0;
-  const int mode = spmv_mode(a);
-  if (stop_v) {   // uniform per grid: drain the producer's copies before the CTA exits
-    if (threadIdx.x == 0)
-      for (int g = 0; g < TILE_NST; g++)
-        if (t0 + g / 8 < t1) mbar_wait(&full[g % TILE_NST], 0u);
-    return;
-  }
-  constexpr int G = rgrp(RS);
-  constexpr int NG = 256 / G + 1;
-  constexpr int PER = (NG + 31) / 32;
-  constexpr int WS = (TILE_TY + 2) * TILE_WW;
-  const uint64_t* raw = reinterpret_cast<const uint64_t*>(s_win);
-  int64_t g = 0;           // this CTA's pass counter (element-stage ring position)
-  uint32_t wph = 0;        // window barrier phase
-  int64_t ptx0 = -1, pty0 = -1;
-  for (int64_t t = t0; t < t1; t++) {
-    int64_t tx0, ty0;
-    tile_of(R, t, tx0, ty0);
-    const bool reuse = tx0 == ptx0 && ty0 == pty0 + TILE_TY;
-    const int64_t gy = ty0 + warp;
-    const bool has_seg = gy < ny;
-    const int64_t rowseg = gy * n + tx0;
-    // ---- rowptr loads of the tile's segments (latency overlaps the window set-up)
-    uint32_t e[PER][G];
-    if (has_seg) {
-#pragma unroll
-      for (int q = 0; q < PER; q++) {
-        const int gl = lane + 32 * q;
-        const uint32_t* gp = a.rowptr + (rowseg / G + gl) * G;
-        if (gl < NG) {
-          if (G == 1) e[q][0] = __ldg(gp);
-          else if (G == 2) { uint2 u = __ldg(reinterpret_cast<const uint2*>(gp)); e[q][0] = u.x; e[q][1 % G] = u.y; }
-          else {
-#pragma unroll
-            for (int tt = 0; tt < G; tt += 4) {
-              uint4 u = __ldg(reinterpret_cast<const uint4*>(gp + tt));
-              e[q][tt] = u.x; e[q][(tt + 1) % G] = u.y; e[q][(tt + 2) % G] = u.z; e[q][(tt + 3) % G] = u.w;
-            }
-          }
-        }
-      }
-    }
-    // ---- window: previous tile's passes are done (window, srp free)
-    if (t != t0) __syncthreads();
-    const int bad_prev = s_bad_below;
-    if (reuse) {   // grid rows ty0-1, ty0 (old rows 8, 9) -> rows 0, 1; TMA the 8 rows ty0+1 .. ty0+8
-      for (int sl = threadIdx.x; sl < 2 * TILE_WW; sl += 256) s_win[sl] = s_win[TILE_TY * TILE_WW + sl];
-      __syncthreads();
-      if (threadIdx.x == 0) {
-        s_bad_below = 0;
-        mbar_expect_tx(winbar, TILE_TY * TILE_WW * 8);
-        tma_3d(s_win + 2 * TILE_WW, &tm.vin8, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 + 1), winbar);
-      }
-    } else if (threadIdx.x == 0) {
-      s_bad_below = 0;
-      mbar_expect_tx(winbar, TILE_WIN_BYTES);
-      tma_3d(s_win, &tm.vin, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 - 1), winbar);
-    }
-    // ---- rowptr checks (owner counts), decoded entries into srp
-    if (has_seg) {
-      uint32_t acc = 0;
-      if (mode != MODE_RANGE) {
-#pragma unroll
-        for (int q = 0; q < PER; q++)
-          if (RS != NONE && lane + 32 * q < NG) acc |= (RS == CRC32C) ? rcrc_acc_tab(e[q], s_slice) : rp_acc<RS>(e[q]);
-      }
-      if (RS != NONE && (acc & 1u)) {  // cold: locate, correct, count (owner), per group
-#pragma unroll
-        for (int q = 0; q < PER; q++) {
-          const int gl = lane + 32 * q;
-          if (gl >= NG) continue;
-          const int64_t gg = rowseg / G + gl;
-          uint32_t* gp = a.rowptr + gg * G;
-          uint32_t c[G];
-#pragma unroll
-          for (int tt = 0; tt < G; tt++) c[tt] = e[q][tt];
-          int word = 0;
-          int o = rp_check_group<RS>(c, &word);
-          if (o == CORRECTED && mode == MODE_DETECT) o = DUE;
-          if (o != CLEAN) {
-            const int64_t own = gg * G < a.nrows ? gg * G : a.nrows - 1;
-            const bool owner = own >= rowseg && own < rowseg + 256;
-            if (o == CORRECTED) {
-              uint32_t ow = 0, nw = 0;
-#pragma unroll
-              for (int tt = 0; tt < G; tt++)
-                if (tt == word) { ow = e[q][tt]; nw = c[tt]; }
-              if (owner && scrub32(gp + word, ow, nw)) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
-#pragma unroll
-              for (int tt = 0; tt < G; tt++) e[q][tt] = c[tt];
-            } else if (owner) {
-              cnt_add(a.counts, T_ROWPTR, RS, DUE);
-              *a.due = 1;
-            }
-          }
-        }
-      }
-#pragma unroll
-      for (int q = 0; q < PER; q++) {
-        const int gl = lane + 32 * q;
-        if (gl >= NG) continue;
-#pragma unroll
-        for (int tt = 0; tt < G; tt++) if (gl * G + tt < TILE_RP) srp[gl * G + tt] = e[q][tt] & rp_keep(RS);
-      }
-    }
-    // ---- decode the new window rows in place (tile codewords: owner counts + scrubs)
-    const int64_t win0 = a.row_base + (ty0 - 1) * n + tx0 - TILE_WX0;   // in-index of slot (0,0)
-    mbar_wait(winbar, wph);
-    wph ^= 1u;
-    const int sl0 = reuse ? 2 * TILE_WW : 0;
-    for (int sl = sl0 + threadIdx.x; sl < WS; sl += 256) {
-      uint64_t w = raw[sl];
-      const bool bad = (VS == SED) ? !vsed_clean(w) : (VS == SECDED64) ? (v64_bad(lo32(w), hi32(w)) != 0u) : false;
-      if (VS != NONE && bad) {   // cold: only real codewords fail (zero fill is clean)
-        const int wy = sl / TILE_WW, j = sl - wy * TILE_WW;
-        const int64_t idx = win0 + (int64_t)wy * n + j;
-        const bool owner = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny && j >= TILE_WX0 && j < TILE_WX0 + 256;
-        if (wy == TILE_TY + 1) s_bad_below = 1;
-        w = v1_check<VS>(w, a.in + idx, owner, a.counts, a.due);
-      }
-      s_win[sl] = as_d(w & vkeep(VS));
-    }
-    if (reuse && bad_prev && VS != NONE) {
-      // the row that was the previous tile's halo below is an own row now: check it as its owner
-      for (int j = TILE_WX0 + threadIdx.x; j < TILE_WX0 + 256; j += 256) {
-        const int64_t idx = win0 + n + j;
-        const uint64_t w = ldg64(a.in + idx);
-        const bool bad = (VS == SED) ? !vsed_clean(w) : (v64_bad(lo32(w), hi32(w)) != 0u);
-        if (bad && ty0 < ny) v1_check<VS>(w, a.in + idx, true, a.counts, a.due);
-      }
-    }
-    const bool eL = tx0 == 0, eR = tx0 + 256 == n;
-    if (eL || eR) {   // grid-edge tiles: x = -1 / x = n slots of the newly loaded rows (see k_spmv_tile)
-      __syncthreads();
-      const int tt = threadIdx.x;
-      const int wy0 = reuse ? 2 : 0;
-      int wy = -1, j = 0;
-      if (eL && tt < TILE_TY + 2) { wy = tt; j = TILE_WX0 - 1; }
-      else if (eR && tt >= 32 && tt < 32 + TILE_TY + 2) { wy = tt - 32; j = TILE_WX0 + 256; }
-      if (wy >= wy0) {
-        const int64_t idx = win0 + (int64_t)wy * n + j;
-        const uint64_t w = (idx >= 0 && idx < a.npad_in) ? v1_check<VS>(ldg64(a.in + idx), a.in + idx, false, a.counts, a.due)
-                                                         : 0ull;
-        s_win[wy * TILE_WW + j] = as_d(w & vkeep(VS));
-      }
-    }
-    __syncthreads();
-    // ---- 8 passes (the element-stage ring continues across tiles)
-    double dot = 0.0, dot2 = 0.0;
-    const uint32_t seg_e = (uint32_t)(5 * rowseg);
-    for (int k = 0; k < 8; k++, g++) {
-      const int st = (int)(g % TILE_NST);
-      const uint32_t ph = (uint32_t)((g / TILE_NST) & 1);
-      uint8_t* stage = s_dyn + st * TILE_STAGE;
-      mbar_wait(&full[st], ph);
-      if (has_seg) {
-        const uint64_t* sval = reinterpret_cast<const uint64_t*>(stage) + warp * TILE_PE;
-        const uint32_t* scol = reinterpret_cast<const uint32_t*>(stage + TILE_STAGE_VAL) + warp * TILE_PE;
-        const uint32_t start = srp[32 * k + lane], end = srp[32 * k + lane + 1];
-        const int oslot = (warp + 1) * TILE_WW + k * 32 + lane + TILE_WX0;
-        const double p_own = s_win[oslot];
-        const int64_t own = a.row_base + rowseg + k * 32 + lane;
-        const double acc = tile_row5<ES, RS, VS>(a, s_args, start, end, sval, scol, s_win, oslot, p_own, own,
-                                                 seg_e + 160u * k, lane, mode, s_slice);
-        const uint64_t rounded = round_k(as_u(acc), vk(VS));
-        const uint64_t enc = v_encode<VS>(rounded, lane, s_lut);
-        a.out[own] = enc;
-        if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
-        if (DOT == 2) dot2 = fma(p_own, p_own, dot2);
-      }
-      __syncwarp();
-      if (lane == 0) mbar_arrive(&empty[st]);
-      if (threadIdx.x == 0 && t0 + (g + TILE_NST) / 8 < t1) {  // refill once every warp released the stage
-        mbar_wait(&empty[st], ph);
-        pers_produce(tm, s_dyn, full, R, t0, t1, g + TILE_NST);
-      }
-    }
-    if (DOT && has_seg) {
-#pragma unroll
-      for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-      if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
-    }
-    if (DOT == 2 && has_seg) {
-#pragma unroll
-      for (int off = 16; off >= 1; off >>= 1) dot2 = dot2 + __shfl_xor_sync(0xffffffffu, dot2, off);
-      if (lane == 0) a.partials2[a.rb_offset + (rowseg >> 8)] = dot2;
-    }
-    ptx0 = tx0;
-    pty0 = ty0;
-  }
-}
-
 // ============================================================= BLAS-1 (a4, a5, a2)
 // Full-RB fast paths: two passes per step, so each lane has 8 (calc_ur) / 4
 // (calc_p) independent 8-byte loads in flight, and all addressing is pointer +
@@ -1810,6 +1541,50 @@ __global__ void __launch_bounds__(256) k_calc_sr(VecArgs a) {
   }
 }
 
+// Chebyshev update (TeaLeaf tea_leaf_cheby, reading R32):
+// r = enc(b - w); p = enc(r'/theta) (INIT) or enc(fma(alpha, p', beta r'));
+// u = enc(u' + p'); RED-1 partials of r'.r'.  Checks b, w, (p), u; VecArgs.x is u.
+template <int VS, bool INIT>
+__global__ void __launch_bounds__(256) k_cheb(VecArgs a) {
+  __shared__ __align__(16) uint8_t s_lut[128];
+  extern __shared__ __align__(16) uint8_t s_dyn_v[];
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  pdl_wait();
+  pdl_trigger();
+  const int stop = a.state->stop;
+  const double alpha = a.state->alpha, beta = a.state->beta, theta = a.state->ch_theta;
+  const uint8_t* cs = vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
+  (void)cs;
+  __syncthreads();
+  if ((!INIT && stop) || rb * 256 >= a.n) return;
+  const uint64_t keep = vkeep(VS);
+  double dot = 0.0;
+  for (int k = 0; k < 8; k++) {
+    const int64_t pb = rb * 256 + k * 32;
+    if (pb >= a.n) break;
+    const int64_t i = pb + lane;
+    const bool valid = i < a.n;
+    const int64_t lim = a.npad;
+    const uint64_t bw = v_load_check<VS>(a.b, i, lim, lane, true, a.counts, a.due);
+    const uint64_t ww = v_load_check<VS>(a.w, i, lim, lane, true, a.counts, a.due);
+    const uint64_t pw = INIT ? 0ull : v_load_check<VS>(a.p, i, lim, lane, true, a.counts, a.due);
+    const uint64_t uw = v_load_check<VS>(a.x, i, lim, lane, true, a.counts, a.due);
+    const uint64_t rr = valid ? round_k(as_u(__dsub_rn(as_d(bw & keep), as_d(ww & keep))), vk(VS)) : 0ull;
+    const uint64_t re = v_encode<VS>(rr, lane, s_lut);
+    const double rm = as_d(re & keep);
+    const double pn = INIT ? rm / theta : fma(alpha, as_d(pw & keep), __dmul_rn(beta, rm));
+    const uint64_t pe = v_encode<VS>(valid ? round_k(as_u(pn), vk(VS)) : 0ull, lane, s_lut);
+    const uint64_t ue =
+        v_encode<VS>(valid ? round_k(as_u(__dadd_rn(as_d(uw & keep), as_d(pe & keep))), vk(VS)) : 0ull, lane, s_lut);
+    if (i < a.npad) { a.r[i] = re; a.p[i] = pe; a.x[i] = ue; }
+    if (valid) dot = fma(rm, rm, dot);
+  }
+#pragma unroll
+  for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
+  if (lane == 0) a.partials[rb] = dot;
+}
+
 // init (a2): r = enc(round(b - w)), p = r, rr0 partials
 template <int VS>
 __global__ void __launch_bounds__(256) k_init_r(VecArgs a) {
@@ -1858,7 +1633,33 @@ static __device__ __forceinline__ double tree_smem(double* s, int m) {
 }
 
 // CG scalar logic applied by exactly one thread.
+// Chebyshev step coefficients for the next step, rounded as
+// written: no contraction into FMAs
+static __device__ __forceinline__ void cheb_next(CgState* st) {
+  const double rho_new = __ddiv_rn(1.0, __dsub_rn(__dmul_rn(2.0, st->ch_sigma), st->ch_rho));
+  st->alpha = __dmul_rn(rho_new, st->ch_rho);
+  st->beta = __ddiv_rn(__dmul_rn(2.0, rho_new), st->ch_delta);
+  st->ch_rho = rho_new;
+}
 static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
+  if (op == 8) {  // Chebyshev init: rr0 of r = b - A u0
+    st->rr0 = st->rro = st->rrn = res;
+    if (st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; }
+    else if (res == 0.0) { st->stop = 1; st->status = ABFT_OK; st->converged = 1; }
+    else if (st->max_iters <= 0) { st->stop = 1; st->status = ABFT_OK; }
+    else cheb_next(st);
+    return;
+  }
+  if (op == 9) {  // Chebyshev step
+    st->iters += 1;
+    st->rrn = res;
+    const bool conv = sqrt(res) <= st->tol * sqrt(st->rr0);
+    if (st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; }
+    else if (conv) { st->stop = 1; st->status = ABFT_OK; st->converged = 1; }
+    else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
+    else cheb_next(st);
+    return;
+  }
   if (op == 1) {  // rr0
     st->rr0 = st->rro = st->rrn = res;
     if (st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; }
@@ -1868,6 +1669,7 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
     st->pw = res;
     st->alpha = st->rro / res;
     st->iters += 1;
+    if (st->iters <= CG_LOG) st->alpha_log[st->iters - 1] = st->alpha;
   } else if (op == 3) {  // rrn -> convergence, beta
     st->rrn = res;
     if (sqrt(res) <= st->tol * sqrt(st->rr0)) {
@@ -1876,6 +1678,7 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
       st->status = (st->abort_policy && dueflag) ? ABFT_E_DUE : ABFT_OK;
     } else {
       st->beta = res / st->rro;
+      if (st->iters <= CG_LOG) st->beta_log[st->iters - 1] = st->beta;
       if (st->fused) {  // calc_p's last-block logic (k_calc_p), taken here: calc_p runs in the next SpMV
         st->rro = res;
         if (!st->dist && st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; st->pending_p = 1; }
@@ -1991,7 +1794,7 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
   __shared__ bool s_last;
   pdl_wait();   // partials of the producing kernel
   pdl_trigger();
-  if (st && op != 1 && op != 7 && st->stop) return;
+  if (st && op != 1 && op != 7 && op != 8 && st->stop) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t base = (int64_t)blockIdx.x * leaves;
   const int nw = leaves >= 8 ? 8 : 1;

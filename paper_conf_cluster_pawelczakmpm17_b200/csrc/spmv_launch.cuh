@@ -57,10 +57,7 @@ static bool tile_maps(const SpmvArgs& a, TileMaps* m) {
     cuuint32_t ve[3] = {1, 1, 1};
     CUresult r3 = enc(&m->vin, CU_TENSOR_MAP_DATA_TYPE_UINT64, 3, a.in, vd, vs, vb, ve, CU_TENSOR_MAP_INTERLEAVE_NONE,
                       CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
-    cuuint32_t vb8[3] = {2, (cuuint32_t)(TILE_WW / 2), (cuuint32_t)TILE_TY};
-    CUresult r5 = enc(&m->vin8, CU_TENSOR_MAP_DATA_TYPE_UINT64, 3, a.in, vd, vs, vb8, ve, CU_TENSOR_MAP_INTERLEAVE_NONE,
-                      CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
-    CUresult r4 = (r5 == CUDA_SUCCESS) ? CUDA_SUCCESS : r5;
+    CUresult r4 = CUDA_SUCCESS;
     if (a.p_cur)
       r4 = enc(&m->vcur, CU_TENSOR_MAP_DATA_TYPE_UINT64, 3, a.p_cur, vd, vs, vb, ve, CU_TENSOR_MAP_INTERLEAVE_NONE,
                CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
@@ -94,42 +91,6 @@ static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   launch_k(k_spmv_tile<ES, RS, VS, DOT, FUSED>, (unsigned)blocks, 256, smem, s, a, tm);
   return true;
 }
-// Persistent tiled SpMV (k_spmv_pers): G = 1 vector schemes with the TMA
-// window.  ABFT_NO_PERSIST=1 in the environment selects the one-tile-per-CTA
-// kernel instead (A/B timing; identical results).
-static bool persist_enabled() {
-  static const bool on = [] { const char* e = getenv("ABFT_NO_PERSIST"); return !(e && e[0] == '1'); }();
-  return on;
-}
-template <int ES, int RS, int VS, int DOT>
-static bool spmv_pers_launch(const SpmvArgs& a, cudaStream_t s) {
-  TileMaps tm;
-  if (!tile_maps(a, &tm) || !tm.has_vmaps) return false;
-  const size_t smem = tile_smem<ES, RS, VS>();
-  static std::atomic<uint64_t> attr_devs{0};
-  static std::atomic<int> occ_cache[64];
-  int dev = 0;
-  cudaGetDevice(&dev);
-  const uint64_t bit = 1ull << (dev & 63);
-  if (!(attr_devs.load(std::memory_order_acquire) & bit)) {
-    cudaFuncSetAttribute(k_spmv_pers<ES, RS, VS, DOT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    cudaFuncSetAttribute(k_spmv_pers<ES, RS, VS, DOT>, cudaFuncAttributePreferredSharedMemoryCarveout, 100);
-    int per_sm = 0, sms = 0;
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_spmv_pers<ES, RS, VS, DOT>, 256, smem);
-    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-    occ_cache[dev & 63].store(per_sm * sms > 0 ? per_sm * sms : 1);
-    attr_devs.fetch_or(bit, std::memory_order_release);
-  }
-  const int64_t ny = a.nrows / a.stencil_n;
-  const int64_t nty = (ny + TILE_TY - 1) / TILE_TY;
-  const int64_t lo = a.ty_lo, hi = a.ty_hi > 0 ? a.ty_hi : nty;
-  const int64_t tiles = (a.stencil_n / 256) * (hi - lo);
-  if (tiles <= 0) return true;
-  const int64_t slots = occ_cache[dev & 63].load();
-  const int64_t blocks = tiles < slots ? tiles : slots;
-  launch_k(k_spmv_pers<ES, RS, VS, DOT>, (unsigned)blocks, 256, smem, s, a, tm);
-  return true;
-}
 // Returns false only when a fused-calc_p launch (a.p_cur set) was requested
 // and cannot run: the caller fails loudly, there is no unfused fallback here.
 template <int ES, int RS, int VS>
@@ -139,14 +100,6 @@ static bool spmv3(const SpmvArgs& a, int dot, cudaStream_t s) {
       return dot == 1 && tile_ok(a, VS) && spmv_tile_launch<ES, RS, VS, 1, true>(a, s);
     }
     return false;
-  }
-  if constexpr (vgrp(VS) == 1) {
-    if (persist_enabled() && tile_ok(a, VS)) {
-      const bool ok = dot == 2   ? spmv_pers_launch<ES, RS, VS, 2>(a, s)
-                      : dot == 1 ? spmv_pers_launch<ES, RS, VS, 1>(a, s)
-                                 : spmv_pers_launch<ES, RS, VS, 0>(a, s);
-      if (ok) return true;
-    }
   }
   if (tile_ok(a, VS)) {
     const bool ok = dot == 2   ? spmv_tile_launch<ES, RS, VS, 2>(a, s)
