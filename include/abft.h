@@ -276,6 +276,18 @@ int abft_dist_init_loopback(abft_dist** out, int nranks, int device);
 int abft_cg_solve_loopback(abft_dist* d, abft_ctx* const* ctxs, const abft_csr* const* A, const int* nchunks,
                            int64_t n_halo, abft_vec* const* vecs, const abft_cg_opts* opts, abft_cg_result* res,
                            abft_counts* const* dcnt, void* stream);
+/* Single-reduction CG on row-block strips (S§8(e) + f3): the halo exchanged
+ * before each SpMV is r's (the SpMV's input), and the ONE all-gather per
+ * iteration carries (w.r root, DUE flag, r.r root) per rank.  Same strip
+ * conventions as abft_cg_solve_dist / abft_cg_solve_loopback; the loopback
+ * variant takes vecs[6q .. 6q+5] = b, x, r, p, w, s per rank. */
+int abft_cg_solve_sr_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b,
+                          abft_vec* x, abft_vec* r, abft_vec* p, abft_vec* w, abft_vec* s, const abft_cg_opts* opts,
+                          abft_cg_result* res, abft_counts* dcnt, void* stream);
+int abft_cg_solve_loopback_sr(abft_dist* d, abft_ctx* const* ctxs, const abft_csr* const* A, const int* nchunks,
+                              int64_t n_halo, abft_vec* const* vecs, const abft_cg_opts* opts, abft_cg_result* res,
+                              abft_counts* const* dcnt, void* stream);
+
 
 /* Host-side codec hooks (no GPU needed): run the exact __host__ __device__
  * codec functions on the CPU for the unit tests.  inst: 0 E-SECDED, 1 V-SECDED64,

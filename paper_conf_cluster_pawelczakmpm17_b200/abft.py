@@ -98,6 +98,10 @@ _sig = {
                                      C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts),
                                      C.POINTER(CGResult), _P, _P]),
     "abft_dist_init_loopback": (C.c_int, [C.POINTER(C.c_void_p), C.c_int, C.c_int]),
+    "abft_cg_solve_sr_dist": (C.c_int, [_P, _P, C.POINTER(CSR), C.c_int, C.c_int64, C.POINTER(Vec), C.POINTER(Vec),
+                                        C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
+                                        C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
+    "abft_cg_solve_loopback_sr": (C.c_int, [_P, _P, _P, _P, C.c_int64, _P, C.POINTER(CGOpts), _P, _P, _P]),
     "abft_cg_solve_loopback": (C.c_int, [_P, _P, _P, _P, C.c_int64, _P, C.POINTER(CGOpts), _P, _P, _P]),
     "abft_codec_host_check": (C.c_int, [C.c_int, _P]),
     "abft_codec_host_encode": (None, [C.c_int, _P]),
@@ -461,6 +465,18 @@ class Dist:
         _check(code, "abft_cg_solve_dist", allow=(E_DUE, E_NOT_CONVERGED))
         return res
 
+    def cg_solve_sr(self, ctx: Context, A, n_halo: int, b, x, r, p, w, s, tol=1e-10, max_iters=10000, due_policy=0,
+                    counts: Counters | None = None, poll_every=16, stream=None) -> CGResult:
+        """Single-reduction CG on this rank's strip (abft_cg_solve_sr_dist)."""
+        arr, n = _chunks(A)
+        opts = CGOpts(tol, max_iters, due_policy, poll_every, 1)
+        res = CGResult()
+        vs = [v.cstruct() for v in (b, x, r, p, w, s)]
+        code = _lib.abft_cg_solve_sr_dist(self.h, ctx.h, arr, n, int(n_halo), *[C.byref(v) for v in vs],
+                                          C.byref(opts), C.byref(res), counts.ptr if counts else None, _stream(stream))
+        _check(code, "abft_cg_solve_sr_dist", allow=(E_DUE, E_NOT_CONVERGED))
+        return res
+
 
 class Loopback:
     """abft_dist over the in-process loopback transport: `nranks` virtual ranks
@@ -487,6 +503,17 @@ class Loopback:
                  poll_every=16, stream=None, check_interval=1):
         """ctxs[q], As[q] (matrix or chunk list), vecs[q] = (b, x, r, p, w), counts[q]
         for every rank q; returns the per-rank CGResult list."""
+        return self._solve(_lib.abft_cg_solve_loopback, 5, ctxs, As, n_halo, vecs, tol, max_iters, due_policy,
+                           counts, poll_every, stream, check_interval)
+
+    def cg_solve_sr(self, ctxs, As, n_halo: int, vecs, tol=1e-10, max_iters=10000, due_policy=0, counts=None,
+                    poll_every=16, stream=None):
+        """Single-reduction CG on the loopback strips: vecs[q] = (b, x, r, p, w, s)."""
+        return self._solve(_lib.abft_cg_solve_loopback_sr, 6, ctxs, As, n_halo, vecs, tol, max_iters, due_policy,
+                           counts, poll_every, stream, 1)
+
+    def _solve(self, fn, nv, ctxs, As, n_halo, vecs, tol, max_iters, due_policy, counts, poll_every, stream,
+               check_interval):
         P = self.nranks
         assert len(ctxs) == len(As) == len(vecs) == P
         keep = []
@@ -499,13 +526,14 @@ class Loopback:
             nch[q] = n
         aptr = (C.c_void_p * P)(*arrs)
         cptr = (C.c_void_p * P)(*[c.h for c in ctxs])
+        assert all(len(vecs[q]) == nv for q in range(P))
         vstructs = [v.cstruct() for q in range(P) for v in vecs[q]]
-        vptr = (C.c_void_p * (5 * P))(*[C.cast(C.pointer(v), C.c_void_p) for v in vstructs])
+        vptr = (C.c_void_p * (nv * P))(*[C.cast(C.pointer(v), C.c_void_p) for v in vstructs])
         cnts = counts if counts is not None else [None] * P
         nptr = (C.c_void_p * P)(*[c.ptr if c is not None else None for c in cnts])
         opts = CGOpts(tol, max_iters, due_policy, poll_every, check_interval)
         res = (CGResult * P)()
-        code = _lib.abft_cg_solve_loopback(self.h, cptr, aptr, nch, int(n_halo), vptr, C.byref(opts),
-                                           C.cast(res, C.c_void_p), nptr, _stream(stream))
-        _check(code, "abft_cg_solve_loopback", allow=(E_DUE, E_NOT_CONVERGED))
+        code = fn(self.h, cptr, aptr, nch, int(n_halo), vptr, C.byref(opts), C.cast(res, C.c_void_p), nptr,
+                  _stream(stream))
+        _check(code, fn.__name__, allow=(E_DUE, E_NOT_CONVERGED))
         return list(res)

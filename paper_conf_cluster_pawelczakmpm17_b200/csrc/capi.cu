@@ -64,6 +64,7 @@ struct abft_ctx {
   bool pdl = false;          // programmatic dependent launch between the CG iteration kernels (opt-in, §6.2)
   uint64_t* p_alt = nullptr; // second p buffer of the fused CG
   int64_t p_alt_len = 0;
+  double* cg_log = nullptr;   // [2 * CG_LOG]: CG alpha / beta of the first iterations (abft_cg_spectrum)
   DevFault* faults = nullptr; // O10 fault schedule applied by the next CG solves (abft_ctx_set_faults)
   int nfaults = 0;
 };
@@ -213,6 +214,7 @@ int abft_ctx_create(int device, abft_ctx** out) {
   c->device = device;
   CUDA_TRY(cudaMalloc(&c->roots, sizeof(double) * 1024));
   CUDA_TRY(cudaMalloc(&c->roots2, sizeof(double) * 1024));
+  CUDA_TRY(cudaMalloc(&c->cg_log, sizeof(double) * 2 * CG_LOG));
   CUDA_TRY(cudaMalloc(&c->ticket, sizeof(uint32_t) * 4));
   CUDA_TRY(cudaMemset(c->ticket, 0, sizeof(uint32_t) * 4));
   CUDA_TRY(cudaMalloc(&c->state, sizeof(CgState)));
@@ -261,6 +263,7 @@ int abft_ctx_destroy(abft_ctx* c) {
   cudaFree(c->flags);
   cudaFree(c->p_alt);
   cudaFree(c->faults);
+  cudaFree(c->cg_log);
   cudaFree(c->red);
   cudaFree(c->crc);
   cudaFreeHost(c->h_state);
@@ -415,7 +418,7 @@ struct abft_dist {
   ncclComm_t comm = nullptr;
   int rank = 0, nranks = 1, device = 0;
   double* sendbuf = nullptr;   // NCCL: this rank's pair [2]
-  double* gathered = nullptr;  // all ranks' pairs [2 * nranks] (loopback: rank r writes gathered + 2r directly)
+  double* gathered = nullptr;  // all ranks' payloads [GATHER_W * nranks] (loopback: rank r writes its own slot)
   cudaStream_t comm_stream = nullptr;   // halo exchange, overlapped with the interior SpMV
   cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
 };
@@ -435,6 +438,7 @@ struct RankRun {
   int nchunks = 0;
   abft_vec* v[5] = {};   // b x r p w
   abft_vec* s_vec = nullptr;   // single-reduction CG: its extra vector s
+  VecArgs va_sr{};
   bool cheb = false;           // Chebyshev iteration with bounds [eigmin, eigmax]; x is u
   double eigmin = 0.0, eigmax = 0.0;
   DevCounts* cnt = nullptr;
@@ -526,7 +530,7 @@ int halo_exchange(abft_dist* d, RankRun* R, int nl, int vi, int64_t n_halo, cuda
 // every rank's (root, due) pair -> every rank's `gathered`
 int allgather_pairs(abft_dist* d, cudaStream_t s) {
   if (d->loopback) return ABFT_OK;   // the ranks wrote their pairs into the one shared buffer
-  NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, 2, ncclDouble, d->comm, s));
+  NCCL_TRY(ncclAllGather(d->sendbuf, d->gathered, GATHER_W, ncclDouble, d->comm, s));
   return ABFT_OK;
 }
 
@@ -548,6 +552,28 @@ int finish_dot(RankRun* R, int nl, abft_dist* d, int op, cudaStream_t s) {
   if (e) return e;
   for (int q = 0; q < nl; q++)
     count_launch(launch_combine(R[q].gathered, d->nranks, op, R[q].ctx->state, R[q].ctx->due, s));
+  return ABFT_OK;
+}
+
+// Single-reduction CG's one reduction: both RED-1 trees;
+// multi-rank -> (w.r root, DUE flag, r.r root) all-gathered, both tops of the
+// tree combined identically on every rank.
+int finish_sr(RankRun* R, int nl, abft_dist* d, int op, cudaStream_t s) {
+  if (!d) {
+    abft_ctx* c = R[0].ctx;
+    count_launch(launch_reduce_sr(c->partials, c->partials2, R[0].nrb, c->roots, c->roots2, c->ticket, op, c->state,
+                                  c->due, s));
+    return ABFT_OK;
+  }
+  for (int q = 0; q < nl; q++) {
+    abft_ctx* c = R[q].ctx;
+    count_launch(launch_reduce_sr_root(c->partials, c->partials2, R[q].nrb, c->roots, c->roots2, c->ticket,
+                                       R[q].sendbuf, c->due, s));
+  }
+  int e = allgather_pairs(d, s);
+  if (e) return e;
+  for (int q = 0; q < nl; q++)
+    count_launch(launch_combine_sr(R[q].gathered, d->nranks, op, R[q].ctx->state, R[q].ctx->due, s));
   return ABFT_OK;
 }
 
@@ -575,13 +601,18 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     if (!(R[0].eigmax > R[0].eigmin)) return fail(ABFT_E_INVALID, "Chebyshev bounds need eigmax > eigmin");
   }
   if (sr) {
-    if (d || nl != 1) return fail(ABFT_E_SHAPE, "single-reduction CG runs on one GPU");
     if (opts->check_interval > 1) return fail(ABFT_E_SHAPE, "single-reduction CG checks every access");
-    int e0 = check_vec(R[0].s_vec, "s");
-    if (e0) return e0;
-    if (R[0].s_vec->scheme != scheme || R[0].s_vec->n != R[0].n_ext)
-      return fail(ABFT_E_INVALID, "vector s: scheme/length differ");
-    for (int j = 0; j < 5; j++) if (R[0].v[j]->data == R[0].s_vec->data) return fail(ABFT_E_INVALID, "vectors alias");
+    for (int q = 0; q < nl; q++) {
+      if (!R[q].s_vec) return fail(ABFT_E_INVALID, "rank %d: null vector s", q);
+      int e0 = check_vec(R[q].s_vec, "s");
+      if (e0) return e0;
+      if (R[q].s_vec->scheme != scheme || R[q].s_vec->n != R[q].n_ext)
+        return fail(ABFT_E_INVALID, "vector s: scheme/length differ");
+      for (int j = 0; j < 5; j++)
+        if (R[q].v[j]->data == R[q].s_vec->data) return fail(ABFT_E_INVALID, "vectors alias");
+      R[q].va_sr = R[q].va;   // the update's VecArgs.b carries s
+      R[q].va_sr.b = reinterpret_cast<uint64_t*>(R[q].s_vec->data) + n_halo;
+    }
   }
   const int G = (int)vec_padded_len(1, scheme);
   const int interval = opts->check_interval > 1 ? opts->check_interval : 0;
@@ -590,7 +621,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   const bool multi = d != nullptr;
   if (multi) {
     for (int q = 0; q < nl; q++) {
-      R[q].sendbuf = d->loopback ? d->gathered + 2 * q : d->sendbuf;
+      R[q].sendbuf = d->loopback ? d->gathered + GATHER_W * q : d->sendbuf;
       R[q].gathered = d->gathered;
     }
   }
@@ -629,6 +660,8 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   h.abort_policy = opts->due_policy == 0 ? 1 : 0;
   h.dist = multi ? 1 : 0;
   h.fused = fused ? 1 : 0;
+  h.alpha_log = ctx->cg_log;
+  h.beta_log = ctx->cg_log + CG_LOG;
   if (cheb) {   // host arithmetic, rounded as written
     h.ch_theta = (R[0].eigmax + R[0].eigmin) / 2.0;
     h.ch_delta = (R[0].eigmax - R[0].eigmin) / 2.0;
@@ -655,21 +688,22 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   prof.end();
   if (!cheb)
     for (int q = 0; q < nl; q++) count_launch(launch_init_r(R[q].va, scheme, s));
-  VecArgs vsr = R[0].va;   // single-reduction update: VecArgs.b carries s
   if (cheb) {   // r = b - A u0; p = r/theta; u += p; rr0
     count_launch(launch_cheb(R[0].va, scheme, 1, s));
     if ((e = finish_dot(R, nl, d, 8, s))) return e;
   } else if (sr) {
-    vsr.b = reinterpret_cast<uint64_t*>(R[0].s_vec->data) + n_halo;
     // p = s = encoded +0.0, then w = A r with both dots (gamma = r.r, delta = w.r)
-    for (abft_vec* v : {R[0].p(), R[0].s_vec}) {
-      CUDA_TRY(cudaMemsetAsync(v->data, 0, sizeof(uint64_t) * npad_ext, s));
-      count_launch(launch_vec_encode(reinterpret_cast<uint64_t*>(v->data), v->n, npad_ext, scheme, s));
-    }
-    if ((e = spmv_chunks(ctx, R[0].A, R[0].nchunks, R[0].r(), R[0].w(), 2, R[0].cnt, nullptr, s, nullptr)))
-      return e;
-    count_launch(launch_reduce_sr(ctx->partials, ctx->partials2, R[0].nrb, ctx->roots, ctx->roots2, ctx->ticket, 7,
-                                  ctx->state, ctx->due, s));
+    for (int q = 0; q < nl; q++)
+      for (abft_vec* v : {R[q].p(), R[q].s_vec}) {
+        const int64_t np = vec_padded_len(v->n, scheme);
+        CUDA_TRY(cudaMemsetAsync(v->data, 0, sizeof(uint64_t) * np, s));
+        count_launch(launch_vec_encode(reinterpret_cast<uint64_t*>(v->data), v->n, np, scheme, s));
+      }
+    if ((e = halo_exchange(d, R, nl, 2, n_halo, s))) return e;
+    for (int q = 0; q < nl; q++)
+      if ((e = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].r(), R[q].w(), 2, R[q].cnt, nullptr, s, nullptr)))
+        return e;
+    if ((e = finish_sr(R, nl, d, 7, s))) return e;
   } else if ((e = finish_dot(R, nl, d, 1, s))) {
     return e;
   }
@@ -686,7 +720,8 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   };
   const bool pdl_on = ctx->pdl && !multi;
   // the protected SpMV of one iteration, all ranks (halo first, or overlapped)
-  auto spmv_iter = [&](int64_t kk, cudaStream_t ss) -> int {
+  // vi: the SpMV's input vector (3 = p; 2 = r for the single-reduction CG), dots 1 or 2
+  auto spmv_iter = [&](int64_t kk, cudaStream_t ss, int vi, int dots) -> int {
     int e2;
     if (fused) {
       abft_vec pprev = *p;
@@ -695,9 +730,9 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
                          RedArgs{}, MODE_CORRECT, interval, P[(kk - 1) & 1], reinterpret_cast<uint64_t*>(r->data));
     }
     if (!overlap) {
-      if ((e2 = halo_exchange(d, R, nl, 3, n_halo, ss))) return e2;
+      if ((e2 = halo_exchange(d, R, nl, vi, n_halo, ss))) return e2;
       for (int q = 0; q < nl; q++)
-        if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].p(), R[q].w(), true, R[q].cnt, R[q].ctx->state,
+        if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].v[vi], R[q].w(), dots, R[q].cnt, R[q].ctx->state,
                               ss, nullptr, RedArgs{}, MODE_CORRECT, interval)))
           return e2;
       return ABFT_OK;
@@ -705,12 +740,12 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     // halo on the comm stream while the interior tile rows run on ss; then the boundary rows
     CUDA_TRY(cudaEventRecord(d->ev_fork, ss));
     CUDA_TRY(cudaStreamWaitEvent(d->comm_stream, d->ev_fork, 0));
-    if ((e2 = halo_exchange(d, R, nl, 3, n_halo, d->comm_stream))) return e2;
+    if ((e2 = halo_exchange(d, R, nl, vi, n_halo, d->comm_stream))) return e2;
     CUDA_TRY(cudaEventRecord(d->ev_join, d->comm_stream));
     for (int part = 1; part <= 2; part++) {
       if (part == 2) CUDA_TRY(cudaStreamWaitEvent(ss, d->ev_join, 0));
       for (int q = 0; q < nl; q++)
-        if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].p(), R[q].w(), true, R[q].cnt, R[q].ctx->state,
+        if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].v[vi], R[q].w(), dots, R[q].cnt, R[q].ctx->state,
                               ss, nullptr, RedArgs{}, MODE_CORRECT, interval, nullptr, nullptr, false, part)))
           return e2;
     }
@@ -739,22 +774,21 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
         prof.end();
         continue;
       }
-      if (sr) {   // update, then w = A r with both dots, then the one reduction
+      if (sr) {   // update, then w = A r with both dots, then the one reduction (+ all-gather)
         prof.begin(1);
-        count_launch(launch_calc_sr(vsr, scheme, ss));
+        for (int q = 0; q < nl; q++) count_launch(launch_calc_sr(R[q].va_sr, scheme, ss));
         prof.end();
         prof.begin(0);
-        e2 = spmv_chunks(ctx, R[0].A, R[0].nchunks, R[0].r(), R[0].w(), 2, R[0].cnt, ctx->state, ss, nullptr);
+        e2 = spmv_iter(kk, ss, 2, 2);
         prof.end();
         if (e2) return e2;
         prof.begin(3);
-        count_launch(launch_reduce_sr(ctx->partials, ctx->partials2, R[0].nrb, ctx->roots, ctx->roots2, ctx->ticket,
-                                      6, ctx->state, ctx->due, ss));
+        if ((e2 = finish_sr(R, nl, d, 6, ss))) return e2;
         prof.end();
         continue;
       }
       prof.begin(0);
-      e2 = spmv_iter(kk, ss);
+      e2 = spmv_iter(kk, ss, 3, 1);
       prof.end();
       if (e2) return e2;
       prof.begin(3);
@@ -888,10 +922,10 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     if (multi) {
       for (int q = 0; q < nl; q++) count_launch(launch_pack_due(R[q].sendbuf, R[q].ctx->due, s));
       if ((e = allgather_pairs(d, s))) return e;
-      std::vector<double> g(2 * (size_t)d->nranks);
+      std::vector<double> g(GATHER_W * (size_t)d->nranks);
       CUDA_TRY(cudaMemcpyAsync(g.data(), d->gathered, sizeof(double) * g.size(), cudaMemcpyDeviceToHost, s));
       CUDA_TRY(cudaStreamSynchronize(s));
-      for (int rk = 0; rk < d->nranks; rk++) any |= g[2 * rk + 1] != 0.0;
+      for (int rk = 0; rk < d->nranks; rk++) any |= g[GATHER_W * rk + 1] != 0.0;
     } else {
       CUDA_TRY(cudaMemcpyAsync(ctx->h_flags, ctx->due, sizeof(int), cudaMemcpyDeviceToHost, s));
       CUDA_TRY(cudaStreamSynchronize(s));
@@ -996,13 +1030,16 @@ int abft_cg_spectrum(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b,
   RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
   int e = cg_run(&R, 1, nullptr, 0, &o, res, (cudaStream_t)stream);
   if (e != ABFT_OK && e != ABFT_E_NOT_CONVERGED) return e;
-  const CgState& h = *ctx->h_state;   // the solve's final state (read back by cg_run)
-  const int k = h.iters;
+  const int k = ctx->h_state->iters;   // the solve's final state (read back by cg_run)
   if (k < 2) return fail(ABFT_E_SHAPE, "spectrum estimate needs >= 2 CG steps (got %d)", k);
+  std::vector<double> lg(2 * CG_LOG);
+  CUDA_TRY(cudaMemcpy(lg.data(), ctx->cg_log, sizeof(double) * 2 * CG_LOG, cudaMemcpyDeviceToHost));
+  const double* al = lg.data();
+  const double* bl = lg.data() + CG_LOG;
   std::vector<double> a(k), off(k);
   for (int j = 0; j < k; j++) {
-    a[j] = 1.0 / h.alpha_log[j] + (j > 0 ? h.beta_log[j - 1] / h.alpha_log[j - 1] : 0.0);
-    if (j + 1 < k) off[j] = sqrt(h.beta_log[j]) / h.alpha_log[j];
+    a[j] = 1.0 / al[j] + (j > 0 ? bl[j - 1] / al[j - 1] : 0.0);
+    if (j + 1 < k) off[j] = sqrt(bl[j]) / al[j];
   }
   *eigmin = tridiag_eig(a.data(), off.data(), k, 0);
   *eigmax = tridiag_eig(a.data(), off.data(), k, 1);
@@ -1032,8 +1069,9 @@ int abft_dist_init(abft_dist** out, const void* uid, int rank, int nranks, int d
     return fail(ABFT_E_NCCL, "ncclCommInitRank: %s", ncclGetErrorString(nr));
   }
   int e = dist_streams(d);
-  if (!e && cudaMalloc(&d->sendbuf, sizeof(double) * 2) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc sendbuf");
-  if (!e && cudaMalloc(&d->gathered, sizeof(double) * 2 * nranks) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
+  if (!e && cudaMalloc(&d->sendbuf, sizeof(double) * GATHER_W) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc sendbuf");
+  if (!e && cudaMalloc(&d->gathered, sizeof(double) * GATHER_W * nranks) != cudaSuccess)
+    e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
   if (e) {
     abft_dist_destroy(d);
     return e;
@@ -1050,7 +1088,8 @@ int abft_dist_init_loopback(abft_dist** out, int nranks, int device) {
   d->nranks = nranks;
   d->device = device;
   int e = dist_streams(d);
-  if (!e && cudaMalloc(&d->gathered, sizeof(double) * 2 * nranks) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
+  if (!e && cudaMalloc(&d->gathered, sizeof(double) * GATHER_W * nranks) != cudaSuccess)
+    e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
   if (e) {
     abft_dist_destroy(d);
     return e;
@@ -1078,6 +1117,30 @@ int abft_cg_solve_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchun
   if (d->loopback) return fail(ABFT_E_INVALID, "loopback transport: use abft_cg_solve_loopback");
   RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
   return cg_run(&R, 1, d, n_halo, opts, res, (cudaStream_t)stream);
+}
+
+int abft_cg_solve_sr_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchunks, int64_t n_halo, abft_vec* b,
+                          abft_vec* x, abft_vec* r, abft_vec* p, abft_vec* w, abft_vec* sv, const abft_cg_opts* opts,
+                          abft_cg_result* res, abft_counts* dcnt, void* stream) {
+  if (!d || !ctx) return fail(ABFT_E_INVALID, "null dist/ctx");
+  if (d->loopback) return fail(ABFT_E_INVALID, "loopback transport: use abft_cg_solve_loopback_sr");
+  RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  R.s_vec = sv;
+  return cg_run(&R, 1, d, n_halo, opts, res, (cudaStream_t)stream);
+}
+
+int abft_cg_solve_loopback_sr(abft_dist* d, abft_ctx* const* ctxs, const abft_csr* const* A, const int* nchunks,
+                              int64_t n_halo, abft_vec* const* vecs, const abft_cg_opts* opts, abft_cg_result* res,
+                              abft_counts* const* dcnt, void* stream) {
+  if (!d || !d->loopback) return fail(ABFT_E_INVALID, "abft_cg_solve_loopback_sr needs a loopback transport");
+  if (!ctxs || !A || !nchunks || !vecs || !dcnt) return fail(ABFT_E_INVALID, "null per-rank arrays");
+  std::vector<RankRun> R(d->nranks);
+  for (int q = 0; q < d->nranks; q++) {
+    abft_vec* const* v = vecs + 6 * q;
+    R[q] = make_rank(ctxs[q], A[q], nchunks[q], v[0], v[1], v[2], v[3], v[4], dcnt[q]);
+    R[q].s_vec = v[5];
+  }
+  return cg_run(R.data(), d->nranks, d, n_halo, opts, res, (cudaStream_t)stream);
 }
 
 int abft_cg_solve_loopback(abft_dist* d, abft_ctx* const* ctxs, const abft_csr* const* A, const int* nchunks,

@@ -25,10 +25,14 @@ struct CgState {
   // coefficients)
   double ch_theta, ch_delta, ch_sigma, ch_rho;
   // CG step coefficients of the first CG_LOG iterations (Lanczos data of the
-  // spectrum estimate, abft_cg_spectrum)
-  double alpha_log[128], beta_log[128];
+  // spectrum estimate, abft_cg_spectrum): ctx-owned device arrays [CG_LOG]
+  double* alpha_log;
+  double* beta_log;
 };
 constexpr int CG_LOG = 128;
+// multi-rank all-gather payload per rank: (RED-1 subtree root, DUE flag,
+// second root — the single-reduction CG's r.r)
+constexpr int GATHER_W = 3;
 
 struct DevCounts { unsigned long long v[3][5][4]; };
 
@@ -143,6 +147,10 @@ int launch_reduce_sr(const double* partials, const double* partials2, int64_t nr
 int launch_cheb(const VecArgs& a, int vs, int init, cudaStream_t s);
 // single-reduction CG update: p, s, x, r (VecArgs.b carries s)
 int launch_calc_sr(const VecArgs& a, int vs, cudaStream_t s);
+// single-reduction CG, multi-rank: op 10 -> out[0..3) = (w.r root, DUE flag, r.r root)
+int launch_reduce_sr_root(const double* partials, const double* partials2, int64_t nrb, double* roots, double* roots2,
+                          uint32_t* ticket, double* out, const int* due, cudaStream_t s);
+int launch_combine_sr(const double* gathered, int P, int op, CgState* st, int* due, cudaStream_t s);
 int launch_combine(const double* gathered, int P, int op, CgState* st, int* due, cudaStream_t s);
 int launch_due_combine(const double* gathered, int P, CgState* st, int* due, cudaStream_t s);
 int launch_pack_due(double* out, const int* due, cudaStream_t s);

@@ -208,6 +208,20 @@ int launch_reduce_sr(const double* partials, const double* partials2, int64_t nr
   return 1;
 }
 
+int launch_reduce_sr_root(const double* partials, const double* partials2, int64_t nrb, double* roots, double* roots2,
+                          uint32_t* ticket, double* out, const int* due, cudaStream_t s) {
+  int64_t p2 = 1;
+  while (p2 < nrb) p2 <<= 1;
+  int64_t leaves = p2 < 1024 ? p2 : 1024;
+  int blocks = (int)(p2 / leaves);
+  launch_k(k_reduce<true>, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, 10, (CgState*)nullptr, out, due,
+           partials2, roots2);
+  return 1;
+}
+int launch_combine_sr(const double* gathered, int P, int op, CgState* st, int* due, cudaStream_t s) {
+  k_combine_sr<<<1, 512, 0, s>>>(gathered, P, op, st, due);
+  return 1;
+}
 int launch_combine(const double* gathered, int P, int op, CgState* st, int* due, cudaStream_t s) {
   k_combine<<<1, 512, 0, s>>>(gathered, P, op, st, due);
   return 1;

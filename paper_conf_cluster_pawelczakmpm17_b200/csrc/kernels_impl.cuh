@@ -1669,7 +1669,7 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
     st->pw = res;
     st->alpha = st->rro / res;
     st->iters += 1;
-    if (st->iters <= CG_LOG) st->alpha_log[st->iters - 1] = st->alpha;
+    if (st->alpha_log && st->iters <= CG_LOG) st->alpha_log[st->iters - 1] = st->alpha;
   } else if (op == 3) {  // rrn -> convergence, beta
     st->rrn = res;
     if (sqrt(res) <= st->tol * sqrt(st->rr0)) {
@@ -1678,7 +1678,7 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
       st->status = (st->abort_policy && dueflag) ? ABFT_E_DUE : ABFT_OK;
     } else {
       st->beta = res / st->rro;
-      if (st->iters <= CG_LOG) st->beta_log[st->iters - 1] = st->beta;
+      if (st->beta_log && st->iters <= CG_LOG) st->beta_log[st->iters - 1] = st->beta;
       if (st->fused) {  // calc_p's last-block logic (k_calc_p), taken here: calc_p runs in the next SpMV
         st->rro = res;
         if (!st->dist && st->abort_policy && dueflag) { st->stop = 1; st->status = ABFT_E_DUE; st->pending_p = 1; }
@@ -1794,7 +1794,7 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
   __shared__ bool s_last;
   pdl_wait();   // partials of the producing kernel
   pdl_trigger();
-  if (st && op != 1 && op != 7 && op != 8 && st->stop) return;
+  if (st && op != 1 && op != 7 && op != 8 && op != 10 && st->stop) return;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t base = (int64_t)blockIdx.x * leaves;
   const int nw = leaves >= 8 ? 8 : 1;
@@ -1829,9 +1829,10 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
   if (threadIdx.x != 0) return;
   if (gridDim.x > 1) *ticket = 0;
   const bool dueflag = *((volatile const int*)due) != 0;
+  if (TWO && op == 10) { out[0] = root; out[1] = (double)(dueflag ? 1 : 0); out[2] = root2; return; }
   if (TWO) { apply_op_sr(op, root2, root, st, dueflag); return; }
   if (op == 0) { *out = root; return; }
-  if (op == 4) { out[0] = root; out[1] = (double)(dueflag ? 1 : 0); return; }
+  if (op == 4) { out[0] = root; out[1] = (double)(dueflag ? 1 : 0); out[2] = 0.0; return; }
   apply_op(op, root, st, dueflag);
 }
 
@@ -1842,24 +1843,48 @@ static __global__ void k_combine(const double* gathered, int P, int op, CgState*
   if (op != 1 && st->stop) return;
   int m = 1;
   while (m < P) m <<= 1;
-  for (int t = threadIdx.x; t < m; t += blockDim.x) s[t] = (t < P) ? gathered[2 * t] : 0.0;
+  for (int t = threadIdx.x; t < m; t += blockDim.x) s[t] = (t < P) ? gathered[GATHER_W * t] : 0.0;
   __syncthreads();
   double root = tree_smem(s, m);
   if (threadIdx.x != 0) return;
   int any = 0;
-  for (int t = 0; t < P; t++) any |= gathered[2 * t + 1] != 0.0;
+  for (int t = 0; t < P; t++) any |= gathered[GATHER_W * t + 1] != 0.0;
   if (any) *due = 1;
   apply_op(op, root, st, any != 0);
+}
+// Single-reduction CG, multi-rank: both roots' top of the tree (same order on
+// every rank), then the SR scalar logic (op 6 / 7).
+static __global__ void k_combine_sr(const double* gathered, int P, int op, CgState* st, int* due) {
+  __shared__ double s[1024], s2[1024];
+  if (op != 7 && st->stop) return;
+  int m = 1;
+  while (m < P) m <<= 1;
+  for (int t = threadIdx.x; t < m; t += blockDim.x) {
+    s[t] = (t < P) ? gathered[GATHER_W * t] : 0.0;
+    s2[t] = (t < P) ? gathered[GATHER_W * t + 2] : 0.0;
+  }
+  __syncthreads();
+  const double d = tree_smem(s, m);
+  const double g = tree_smem(s2, m);
+  if (threadIdx.x != 0) return;
+  int any = 0;
+  for (int t = 0; t < P; t++) any |= gathered[GATHER_W * t + 1] != 0.0;
+  if (any) *due = 1;
+  apply_op_sr(op, g, d, st, any != 0);
 }
 // Multi-GPU abort check after calc_p (policy abort only): gathered due flags.
 static __global__ void k_due_combine(const double* gathered, int P, CgState* st, int* due) {
   int any = 0;
-  for (int t = 0; t < P; t++) any |= gathered[2 * t + 1] != 0.0;
+  for (int t = 0; t < P; t++) any |= gathered[GATHER_W * t + 1] != 0.0;
   if (any) *due = 1;
   if (st->stop && st->status != ABFT_E_NOT_CONVERGED) return;
   if (st->abort_policy && any) { st->stop = 1; st->status = ABFT_E_DUE; }
 }
-static __global__ void k_pack_due(double* out, const int* due) { out[1] = (double)(*((volatile const int*)due)); out[0] = 0.0; }
+static __global__ void k_pack_due(double* out, const int* due) {
+  out[1] = (double)(*((volatile const int*)due));
+  out[0] = 0.0;
+  out[2] = 0.0;
+}
 
 // ========================================================== vector encode / check
 template <int VS>

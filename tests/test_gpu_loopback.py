@@ -50,7 +50,7 @@ def _oracle(n, S, vflips, eflips, policy, max_iters, interval=1):
     return st, res, xo[:N], cnt
 
 
-def _loopback(abft, n, P, S, stencil, vflips, eflips, policy, max_iters, interval=1, poll=8):
+def _loopback(abft, n, P, S, stencil, vflips, eflips, policy, max_iters, interval=1, poll=8, sr=False):
     rows = n // P
     h = n
     ctxs, As, vecs, cnts = [], [], [], []
@@ -77,14 +77,18 @@ def _loopback(abft, n, P, S, stencil, vflips, eflips, policy, max_iters, interva
                 for bit in bits:
                     xe[h + i - y0 * n] ^= np.uint64(1 << bit)
         vs = [gpu_vec_from_words(abft, a, Nl + 2 * h, S) for a in (be, xe)]
-        vs += [abft.Vector.empty(Nl + 2 * h, S) for _ in range(3)]
+        vs += [abft.Vector.empty(Nl + 2 * h, S) for _ in range(4 if sr else 3)]
         ctxs.append(ctx)
         As.append(A)
         vecs.append(vs)
         cnts.append(abft.Counters())
     d = abft.Loopback(P, 0)
-    res = d.cg_solve(ctxs, As, h, vecs, tol=1e-10, max_iters=max_iters, due_policy=policy, counts=cnts,
-                     poll_every=poll, check_interval=interval)
+    if sr:
+        res = d.cg_solve_sr(ctxs, As, h, vecs, tol=1e-10, max_iters=max_iters, due_policy=policy, counts=cnts,
+                            poll_every=poll)
+    else:
+        res = d.cg_solve(ctxs, As, h, vecs, tol=1e-10, max_iters=max_iters, due_policy=policy, counts=cnts,
+                         poll_every=poll, check_interval=interval)
     torch.cuda.synchronize()
     x = np.concatenate([words_of(vecs[q][1])[h:h + rows * n] for q in range(P)])
     cnt = sum(c.read() for c in cnts)
@@ -157,3 +161,31 @@ def test_loopback_graph_vs_direct(abft):
     r2, x2, c2 = _loopback(abft, n, P, S, n, [], [], 1, 60, poll=4)
     assert [r.iters for r in r1] == [r.iters for r in r2]
     assert np.array_equal(x1, x2) and np.array_equal(c1, c2)
+
+
+@pytest.mark.parametrize("n,stencil,P", [(64, 0, 4), (256, 256, 2), (256, 256, 8)])
+@pytest.mark.parametrize("policy", [0, 1])
+def test_loopback_single_reduction_cg(abft, n, stencil, P, policy):
+    """Single-reduction CG on P strips: r's halo before the
+    SpMV, ONE all-gather of (w.r root, DUE flag, r.r root) per iteration;
+    bit-identical to the single-process oracle or_cg_solve_sr."""
+    S = orc.SECDED64
+    N = n * n
+    rows = n // P
+    vflips = [((rows - 1) * n + 5, [9]), (rows * n + 7, [40])]
+    v, c, r = gen.tealeaf_csr(n)
+    Ao = orc.Matrix(v.numpy(), c.numpy().astype(np.uint32), r.numpy().astype(np.uint32), N, N, S, S)
+    assert Ao.encode() == 0
+    bo = orc.vec_encode(gen.tealeaf_rhs(n).numpy(), S)
+    xo = bo.copy()
+    for (i, bits) in vflips:
+        for bit in bits:
+            xo[i] ^= np.uint64(1 << bit)
+    ro, po, wo, so = (np.zeros_like(bo) for _ in range(4))
+    cnt_o = orc.new_counts()
+    st, res_o = orc.cg_solve_sr(Ao, bo.copy(), xo, ro, po, wo, so, S, 1e-10, 400, policy, cnt_o)
+    res, x, cnt = _loopback(abft, n, P, S, stencil, vflips, [], policy, 400, sr=True)
+    for q in range(P):
+        assert res[q].iters == res_o.iters and res[q].status == st and res[q].rrn == res_o.rrn
+    assert np.array_equal(x, xo[:N])
+    assert np.array_equal(cnt, cnt_o)
