@@ -90,6 +90,7 @@ def lib():
                                       C.c_int, C.c_void_p, C.c_void_p, dp, dp]
         L.or_cheby_solve.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_double,
                                      C.c_double, C.c_int, C.c_int, C.c_void_p, C.c_void_p]
+        L.or_set_crc_correct.argtypes = [C.c_int]
         L.or_vec_masked.argtypes = [u64p, C.c_int64, C.c_int, dp]
         L.or_round_k.restype = C.c_uint64
         L.or_round_k.argtypes = [C.c_uint64, C.c_int]
@@ -381,3 +382,8 @@ def cheby_solve(A: Matrix, b, u, r, p, w, scheme, eigmin, eigmax, tol=1e-10, max
                               _p(p, C.c_uint64), _p(w, C.c_uint64), scheme, float(eigmin), float(eigmax), tol,
                               max_iters, due_policy, C.byref(res), counts.ctypes.data if counts is not None else None)
     return st, res
+
+
+def set_crc_correct(t: int):
+    """CRC32C correction capability: 1 = 1EC4ED (default), 2 = 2EC3ED."""
+    lib().or_set_crc_correct(int(t))

@@ -22,7 +22,8 @@
  *                    or_cg_solve_log for the spectrum estimate
  *         faults     O10 scheduled bit flips (S§8(c) O10): XOR before init /
  *                    before iteration k's SpMV, or_cg_solve_sched
- *         CRC fix    1EC4ED single-bit correction of a failing CRC32C codeword
+ *         CRC fix    1EC4ED single-bit correction (2EC3ED pair correction with
+ *                    or_set_crc_correct(2), reading R9b) of a failing CRC32C codeword
  *                    P:260-278 (§IV; HD 6 for 178..5243-bit codewords,
  *                    P:268-271), DESIGN.md §3.5 (reading R9)
  *
@@ -279,6 +280,13 @@ static uint32_t vcrc(const uint64_t* d) {
  * single flip can succeed and 2..4 flips never look like one; anything else
  * is a DUE.  ok(w, ctx) re-checks the words w[0 .. nbits/32). */
 #define CRC_HD6_MAX_BITS 5243
+/* 2EC3ED (reading R9b, or_set_crc_correct(2)): when no single
+ * flip explains the failure, every pair of stored bits is tried; exactly one
+ * pair that makes the codeword valid is corrected (with HD 6 a weight-2 error
+ * is unique and a weight-3 one is never one or two flips away from another
+ * codeword), anything else is a DUE. */
+static int g_crc_t = 1;
+void or_set_crc_correct(int t) { g_crc_t = (t == 2) ? 2 : 1; }
 static int crc_fix_brute(uint32_t* w, int nbits, int msg_bits, int (*ok)(const uint32_t*, const void*),
                          const void* ctx) {
   if (ok(w, ctx)) return OUT_CLEAN;
@@ -289,8 +297,25 @@ static int crc_fix_brute(uint32_t* w, int nbits, int msg_bits, int (*ok)(const u
     if (ok(w, ctx)) { nfound++; found = b; }
     flipbit(w, b);
   }
+  if (nfound == 1) {
+    flipbit(w, found);
+    return OUT_CORRECTED;
+  }
+  if (nfound != 0 || g_crc_t < 2) return OUT_DUE;
+  int f1 = -1, f2 = -1;
+  nfound = 0;
+  for (int b1 = 0; b1 < nbits; b1++) {
+    flipbit(w, b1);
+    for (int b2 = b1 + 1; b2 < nbits; b2++) {
+      flipbit(w, b2);
+      if (ok(w, ctx)) { nfound++; f1 = b1; f2 = b2; }
+      flipbit(w, b2);
+    }
+    flipbit(w, b1);
+  }
   if (nfound != 1) return OUT_DUE;
-  flipbit(w, found);
+  flipbit(w, f1);
+  flipbit(w, f2);
   return OUT_CORRECTED;
 }
 static int vcrc_ok(const uint32_t* w, const void* ctx) {

@@ -169,3 +169,56 @@ def test_spmv_uses_the_corrected_row():
     assert np.array_equal(ya, yb)
     assert cnt[orc.ELEM, orc.CRC32C, COR] == 4 and cnt[orc.ROWPTR, orc.CRC32C, COR] == 1
     assert np.array_equal(A.val, B.val) and np.array_equal(A.col, B.col) and np.array_equal(A.rowptr, B.rowptr)
+
+
+# ---------------------------------------------------------------- 2EC3ED (reading R9b)
+@pytest.fixture
+def two_ec():
+    orc.set_crc_correct(2)
+    yield
+    orc.set_crc_correct(1)
+
+
+def test_2ec_vcrc_double_flips_corrected_triples_due(two_ec):
+    """With HD 6, every double flip is the unique weight-2 explanation: corrected
+    back exactly; a triple flip is never within distance 2 of another codeword:
+    DUE, nothing written; singles stay corrected."""
+    rng = np.random.default_rng(41)
+    base = _vcrc_words(1, 8)
+    for k, trials in ((1, 20), (2, 60), (3, 30)):
+        w = np.tile(base, trials)
+        for t in range(trials):
+            for b in rng.choice(256, k, replace=False):
+                w[4 * t + b // 64] ^= np.uint64(1 << int(b % 64))
+        before = w.copy()
+        cnt = orc.new_counts()
+        orc.vec_check(w, len(w), orc.CRC32C, cnt, scrub=True)
+        if k <= 2:
+            assert cnt[orc.VEC, orc.CRC32C, COR] == trials and cnt[orc.VEC, orc.CRC32C, UNC] == 0
+            assert np.array_equal(w, np.tile(base, trials))
+        else:
+            assert cnt[orc.VEC, orc.CRC32C, UNC] == trials and cnt[orc.VEC, orc.CRC32C, COR] == 0
+            assert np.array_equal(w, before)
+
+
+def test_2ec_rcrc_and_ecrc_double_flips_corrected(two_ec):
+    rng = np.random.default_rng(42)
+    A = _rcrc_matrix(40 * 8 - 1)
+    ref = A.rowptr.copy()
+    for g in range(40):
+        for b in rng.choice(256, 2, replace=False):
+            A.rowptr[8 * g + b // 32] ^= np.uint32(1 << int(b % 32))
+    cnt = orc.new_counts()
+    A.check(cnt, scrub=True)
+    assert cnt[orc.ROWPTR, orc.CRC32C, COR] == 40 and cnt[orc.ROWPTR, orc.CRC32C, UNC] == 0
+    assert np.array_equal(A.rowptr, ref)
+    L = 5
+    E = _ecrc_rows(12, L, 13)
+    rv, rc = E.val.copy(), E.col.copy()
+    for r in range(12):
+        for b in rng.choice(96 * L, 2, replace=False):
+            _flip_elem_bit(E, L * r + int(b) // 96, int(b) % 96)
+    cnt = orc.new_counts()
+    E.check(cnt, scrub=True)
+    assert cnt[orc.ELEM, orc.CRC32C, COR] == 12 and cnt[orc.ELEM, orc.CRC32C, UNC] == 0
+    assert np.array_equal(E.val, rv) and np.array_equal(E.col, rc)
