@@ -83,6 +83,13 @@ int abft_ctx_destroy(abft_ctx* ctx);
  * iteration.  The context then owns a second p buffer (padded length of p).
  * enable = 0 runs the unfused sequence. */
 int abft_ctx_set_fused_cg(abft_ctx* ctx, int enable);
+/* CRC32C correction capability of every later call on ctx (reading
+ * R9b): bits = 1 (default) 1EC4ED — a failing CRC32C codeword is corrected when
+ * one stored bit explains it, 2..4 flips are DUEs; bits = 2 2EC3ED — also the
+ * unique stored-bit pair (cold path, O(M^2) syndrome search), 3 flips are DUEs.
+ * Only within CRC32C's HD-6 length (message + 32 <= 5243 bits).  Errors:
+ * ABFT_E_INVALID (bits not 1 or 2). */
+int abft_ctx_set_crc_correction(abft_ctx* ctx, int bits);
 /* Programmatic dependent launch between the kernels of abft_cg_solve's
  * iterations (library default off, single GPU): each kernel issues its
  * loads of data the previous kernel does not write (the matrix, vectors from

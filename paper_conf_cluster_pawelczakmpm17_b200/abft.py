@@ -59,6 +59,7 @@ _sig = {
     "abft_ctx_destroy": (C.c_int, [_P]),
     "abft_ctx_set_fused_cg": (C.c_int, [_P, C.c_int]),
     "abft_ctx_set_pdl": (C.c_int, [_P, C.c_int]),
+    "abft_ctx_set_crc_correction": (C.c_int, [_P, C.c_int]),
     "abft_rowptr_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
     "abft_vec_padded_len": (C.c_int64, [C.c_int64, C.c_int32]),
     "abft_csr_encode": (C.c_int, [_P, C.POINTER(CSR), _P]),
@@ -176,6 +177,10 @@ class Context:
     def set_fused_cg(self, enable: bool):
         """Fused calc_p in the CG's SpMV (abft_ctx_set_fused_cg; default off)."""
         _check(_lib.abft_ctx_set_fused_cg(self.h, 1 if enable else 0), "abft_ctx_set_fused_cg")
+
+    def set_crc_correction(self, bits: int):
+        """CRC32C correction: 1 = 1EC4ED (default), 2 = 2EC3ED (abft_ctx_set_crc_correction)."""
+        _check(_lib.abft_ctx_set_crc_correction(self.h, int(bits)), "abft_ctx_set_crc_correction")
 
     def set_pdl(self, enable: bool):
         """Programmatic dependent launch in the CG loop (abft_ctx_set_pdl; library default off)."""

@@ -244,6 +244,13 @@ int abft_ctx_set_pdl(abft_ctx* c, int enable) {
   return ABFT_OK;
 }
 
+int abft_ctx_set_crc_correction(abft_ctx* c, int bits) {
+  if (!c || (bits != 1 && bits != 2)) return fail(ABFT_E_INVALID, "CRC32C correction: 1 (1EC4ED) or 2 (2EC3ED)");
+  CUDA_TRY(cudaSetDevice(c->device));
+  CUDA_TRY(cudaMemcpy(c->due + 1, &bits, sizeof(int), cudaMemcpyHostToDevice));   // cfg[1] (crc_t_of)
+  return ABFT_OK;
+}
+
 int abft_ctx_set_fused_cg(abft_ctx* c, int enable) {
   if (!c) return fail(ABFT_E_INVALID, "null ctx");
   c->fuse_p = enable != 0;

@@ -423,7 +423,8 @@ ABFT_HD bool vcrc_clean(const uint64_t* d) {
   return st == vcrc_compute(d);
 }
 
-// ---- CRC32C single-bit correction, 1EC4ED.
+// ---- CRC32C single-bit correction, 1EC4ED;
+// optional pair correction, 2EC3ED (crc_locate2 below).
 // CRC32C is affine in the message, so a failing codeword's syndrome
 // syn = stored CRC ^ recomputed CRC depends only on the error pattern: a flip
 // of stored CRC bit t gives 1 << t; a flip of message bit i (bytes LSB-first,
@@ -453,23 +454,69 @@ ABFT_HD int crc_locate(uint32_t syn, int mbits) {
   }
   return CRC_NO_FIX;
 }
-// V-CRC quad: check, locate and correct in place; *word = 32-bit word index in the group.
-ABFT_HD int vcrc_check_fix(uint64_t* d, int* word) {
+// 2EC3ED (reading R9b): when no single flip explains syn, the
+// unique pair of positions (message bits and / or stored CRC bits) whose
+// syndromes XOR to syn; with HD 6 a weight-2 error is unique and a weight-3
+// one never matches.  Returns 2 with pos[0..1] (encoded as crc_locate) or 0.
+// O(M^2) register steps: cold path only.
+ABFT_HD int crc_locate2(uint32_t syn, int mbits, int* pos) {
+  if (syn == 0u || mbits + 32 > CRC_HD6_MAX_BITS) return 0;
+  const uint32_t P = 0x82F63B78u;
+  if (popc32(syn) == 2) {   // two stored CRC bits
+    pos[0] = -1 - ctz32(syn);
+    pos[1] = -1 - ctz32(syn & (syn - 1u));
+    return 2;
+  }
+  uint32_t vi = P;   // S(i) for i = mbits-1 .. 0
+  for (int i = mbits - 1; i >= 0; i--) {
+    const uint32_t t = syn ^ vi;
+    if ((t & (t - 1u)) == 0u) {   // message bit i + stored CRC bit
+      pos[0] = i;
+      pos[1] = -1 - ctz32(t);
+      return 2;
+    }
+    uint32_t vj = vi;
+    for (int j = i - 1; j >= 0; j--) {
+      vj = (vj >> 1) ^ (P & (0u - (vj & 1u)));
+      if (vj == t) { pos[0] = i; pos[1] = j; return 2; }
+    }
+    vi = (vi >> 1) ^ (P & (0u - (vi & 1u)));
+  }
+  return 0;
+}
+// CRC32C correction capability of a launch (1 = 1EC4ED, 2 = 2EC3ED): cfg is
+// the context's device int[4] flag block (cfg[1], set by
+// abft_ctx_set_crc_correction); read only on the cold path.
+ABFT_HD int crc_t_of(const int* cfg) { return (cfg && cfg[1] == 2) ? 2 : 1; }
+// Positions of a failing CRC codeword to flip: 1 (1EC), 2 (2EC) or 0 (DUE).
+ABFT_HD int crc_fix_positions(uint32_t syn, int mbits, const int* cfg, int* pos) {
+  const int r = crc_locate(syn, mbits);
+  if (r != CRC_NO_FIX) { pos[0] = r; return 1; }
+  if (crc_t_of(cfg) == 2) return crc_locate2(syn, mbits, pos);
+  return 0;
+}
+// V-CRC quad: check, locate and correct in place (1 or 2 bits); *word = 32-bit
+// word index of the (first) corrected bit in the group.
+ABFT_HD int vcrc_check_fix(uint64_t* d, int* word, const int* cfg = nullptr) {
   uint32_t st = 0;
   for (int i = 0; i < 4; i++) st |= (uint32_t)(d[i] & 0xFF) << (8 * i);
   const uint32_t syn = st ^ vcrc_compute(d);
   if (!syn) return CLEAN;
-  const int r = crc_locate(syn, 256);
-  if (r == CRC_NO_FIX) return DUE;
-  int bit;                                        // container bit: double bit / 64, bit % 64
-  if (r < 0) bit = 64 * ((-1 - r) >> 3) + ((-1 - r) & 7);   // CRC byte t/8 = low byte of double t/8
-  else {
-    const int byte = r >> 3, bb = byte & 7;
-    if (bb == 0) return DUE;                      // zeroed message byte: not a stored bit
-    bit = 64 * (byte >> 3) + 8 * bb + (r & 7);
+  int pos[2];
+  const int np = crc_fix_positions(syn, 256, cfg, pos);
+  if (np == 0) return DUE;
+  int bits[2];
+  for (int q = 0; q < np; q++) {
+    const int r = pos[q];
+    if (r < 0) bits[q] = 64 * ((-1 - r) >> 3) + ((-1 - r) & 7);   // CRC byte t/8 = low byte of double t/8
+    else {
+      const int byte = r >> 3, bb = byte & 7;
+      if (bb == 0) return DUE;                    // zeroed message byte: not a stored bit
+      bits[q] = 64 * (byte >> 3) + 8 * bb + (r & 7);
+    }
   }
-  d[bit >> 6] ^= 1ull << (bit & 63);
-  if (word) *word = bit >> 5;
+  for (int q = 0; q < np; q++) d[bits[q] >> 6] ^= 1ull << (bits[q] & 63);
+  if (word) *word = bits[0] >> 5;
   return CORRECTED;
 }
 
@@ -484,14 +531,14 @@ ABFT_HD void vec_encode_group(uint64_t* d, const uint8_t* v64lut) {
 // Returns outcome; corrects d in place; *word = 32-bit word (within the group)
 // that was corrected.
 template <int S>
-ABFT_HD int vec_check_group(uint64_t* d, int* word) {
+ABFT_HD int vec_check_group(uint64_t* d, int* word, const int* cfg = nullptr) {
   if (S == SED) return vsed_clean(d[0]) ? CLEAN : DUE;
   if (S == SECDED64) {
     if (!v64_bad(lo32(d[0]), hi32(d[0]))) return CLEAN;
     return v64_correct(d[0], word);
   }
   if (S == SECDED128) return v128_check(d, word);
-  if (S == CRC32C) return vcrc_check_fix(d, word);
+  if (S == CRC32C) return vcrc_check_fix(d, word, cfg);
   return CLEAN;
 }
 
@@ -655,7 +702,7 @@ ABFT_HD uint32_t rp_acc(const uint32_t* e) {
 
 // Fast-path check of a rowptr group; corrects in place.
 template <int RS>
-ABFT_HD int rp_check_group(uint32_t* e, int* word) {
+ABFT_HD int rp_check_group(uint32_t* e, int* word, const int* cfg = nullptr) {
   if (RS == SED) return (popc32(e[0]) & 1) ? DUE : CLEAN;
   if (RS == SECDED64) {
     int s, q;
@@ -674,17 +721,21 @@ ABFT_HD int rp_check_group(uint32_t* e, int* word) {
     for (int i = 0; i < 8; i++) st |= (e[i] >> 28) << (4 * i);
     const uint32_t syn = st ^ rcrc_compute(e);
     if (!syn) return CLEAN;
-    const int r = crc_locate(syn, 256);
-    if (r == CRC_NO_FIX) return DUE;
-    int ent, bit;
-    if (r < 0) { ent = (-1 - r) >> 2; bit = 28 + ((-1 - r) & 3); }   // CRC nibble t/4 = bits 28..31 of entry t/4
-    else {
-      ent = r >> 5;            // 4 message bytes per entry
-      bit = r & 31;
-      if (bit >= 28) return DUE;   // masked-out top nibble: not a message bit
+    int pos[2];
+    const int np = crc_fix_positions(syn, 256, cfg, pos);
+    if (np == 0) return DUE;
+    int ent[2], bit[2];
+    for (int q = 0; q < np; q++) {
+      const int r = pos[q];
+      if (r < 0) { ent[q] = (-1 - r) >> 2; bit[q] = 28 + ((-1 - r) & 3); }   // CRC nibble t/4 = bits 28..31 of entry t/4
+      else {
+        ent[q] = r >> 5;            // 4 message bytes per entry
+        bit[q] = r & 31;
+        if (bit[q] >= 28) return DUE;   // masked-out top nibble: not a message bit
+      }
     }
-    e[ent] ^= 1u << bit;
-    if (word) *word = ent;
+    for (int q = 0; q < np; q++) e[ent[q]] ^= 1u << bit[q];
+    if (word) *word = ent[0];
     return CORRECTED;
   }
   return CLEAN;

@@ -67,6 +67,30 @@ static __device__ __forceinline__ void cnt_range(DevCounts* c, int t, int s) {
 static __device__ __forceinline__ bool scrub32(uint32_t* addr, uint32_t oldw, uint32_t neww) {
   return atomicCAS((unsigned int*)addr, oldw, neww) == oldw;
 }
+// Scrub every 32-bit word of a corrected group that changed (one for a single
+// flip, up to two for a CRC32C 2EC3ED pair); the winner of the first CAS counts.
+static __device__ __noinline__ bool scrub_group32(uint32_t* a32, const uint64_t* oldv, const uint64_t* newv, int G) {
+  bool first = true, won = false;
+  for (int w = 0; w < 2 * G; w++) {
+    const uint32_t ow = (w & 1) ? hi32(oldv[w >> 1]) : lo32(oldv[w >> 1]);
+    const uint32_t nw = (w & 1) ? hi32(newv[w >> 1]) : lo32(newv[w >> 1]);
+    if (ow == nw) continue;
+    const bool ok = scrub32(a32 + w, ow, nw);
+    if (first) won = ok;
+    first = false;
+  }
+  return won;
+}
+static __device__ __noinline__ bool scrub_entries32(uint32_t* a32, const uint32_t* oldv, const uint32_t* newv, int G) {
+  bool first = true, won = false;
+  for (int w = 0; w < G; w++) {
+    if (oldv[w] == newv[w]) continue;
+    const bool ok = scrub32(a32 + w, oldv[w], newv[w]);
+    if (first) won = ok;
+    first = false;
+  }
+  return won;
+}
 
 static __device__ __forceinline__ void load_lut(uint8_t* s_lut) {
   if (threadIdx.x < 32) reinterpret_cast<uint32_t*>(s_lut)[threadIdx.x] = reinterpret_cast<const uint32_t*>(&c_v64_lut)[threadIdx.x];
@@ -225,14 +249,10 @@ __device__ uint64_t vg_check(uint64_t my, uint64_t* group_addr, int lane, bool a
 #pragma unroll
     for (int t = 0; t < G; t++) o0[t] = d[t];
     int word = 0;
-    int o = vec_check_group<VS>(d, &word);
+    int o = vec_check_group<VS>(d, &word, due);
     if (o == CORRECTED) {
-      if (owner) {
-        uint32_t* a32 = reinterpret_cast<uint32_t*>(group_addr) + word;
-        uint64_t ow = o0[word >> 1], nw = d[word >> 1];
-        uint32_t oldw = (word & 1) ? hi32(ow) : lo32(ow), neww = (word & 1) ? hi32(nw) : lo32(nw);
-        if (scrub32(a32, oldw, neww)) cnt_add(cnt, T_VEC, VS, CORRECTED);
-      }
+      if (owner && scrub_group32(reinterpret_cast<uint32_t*>(group_addr), o0, d, G))
+        cnt_add(cnt, T_VEC, VS, CORRECTED);
     } else if (o == DUE) {
 #pragma unroll
       for (int t = 0; t < G; t++) d[t] = o0[t];
@@ -288,7 +308,7 @@ __device__ __forceinline__ uint64_t v_load_check(uint64_t* v, int64_t idx, int64
 
 // Non-owner gather of in[idx] (any lane, no shuffles): returns the masked value.
 template <int VS>
-__device__ __forceinline__ double gather_in(const uint64_t* in, int64_t idx) {
+__device__ __forceinline__ double gather_in(const uint64_t* in, int64_t idx, const int* cfg = nullptr) {
   constexpr int G = vgrp(VS);
   if (G == 1) {
     uint64_t w = ldg64(in + idx);
@@ -306,7 +326,7 @@ __device__ __forceinline__ double gather_in(const uint64_t* in, int64_t idx) {
 #pragma unroll
     for (int t = 0; t < G; t++) d[t] = ldg64(in + g + t);
     uint64_t o0 = d[idx - g];
-    int o = vec_check_group<VS>(d, nullptr);
+    int o = vec_check_group<VS>(d, nullptr, cfg);
     uint64_t w = (o == CORRECTED) ? d[idx - g] : o0;
     return as_d(w & vkeep(VS));
   }
@@ -354,13 +374,13 @@ __device__ __forceinline__ void rowptr_pass(const SpmvArgs& a, int64_t pb, int l
 #pragma unroll
     for (int t = 0; t < G; t++) o0[t] = e[t];
     int word = 0;
-    int o = (mode == MODE_RANGE) ? CLEAN : rp_check_group<RS>(e, &word);
+    int o = (mode == MODE_RANGE) ? CLEAN : rp_check_group<RS>(e, &word, a.due);
     if (o == CORRECTED && mode == MODE_DETECT) o = DUE;   // interval mode: detection only
     if (o != CLEAN) {
       int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
       bool owner = own >= pb && own < pb + 32;
       if (o == CORRECTED) {
-        if (owner && scrub32(gp + word, o0[word], e[word])) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
+        if (owner && scrub_entries32(gp, o0, e, G)) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
       } else {
 #pragma unroll
         for (int t = 0; t < G; t++) e[t] = o0[t];
@@ -401,18 +421,20 @@ __device__ __noinline__ int elem_fix(uint64_t& v, uint32_t& c, uint64_t* vaddr, 
 
 // E-CRC row codeword [start, start+len) failed its check:
 // recompute from global memory, locate a single flipped bit (1EC4ED,
-// crc_locate) and, per `how`: 1 scrub it (32-bit CAS; the winner counts the
-// correction), 0 count it without writing (check_all count-only), 2 report a
-// DUE (detection only: interval mode).  Anything else is a DUE
-// (counted at every access).  Returns CLEAN (someone else already scrubbed
-// it), CORRECTED (read the row from global memory again) or DUE (use the
-// stored bits).
+// crc_locate) or, with 2EC3ED enabled (cfg, reading R9b), a flipped pair, and,
+// per `how`: 1 scrub it (32-bit CAS per changed word; the first CAS's winner
+// counts the correction), 0 count it without writing (check_all count-only),
+// 2 report a DUE (detection only: interval mode).  Anything else is
+// a DUE (counted at every access).  Returns CLEAN (someone else already
+// scrubbed it), CORRECTED (read the row from global memory again) or DUE (use
+// the stored bits).  fix_addr / fix_bit [2] receive the located bits (null
+// when none) for count-only callers to apply.
 static __device__ __noinline__ int ecrc_fix(uint64_t* val, uint32_t* col, uint32_t start, uint32_t len, int how,
                                             DevCounts* cnt, int* due, uint32_t** fix_addr = nullptr,
                                             int* fix_bit = nullptr) {
   int o = DUE;
-  uint32_t* addr = nullptr;
-  int bit = 0;
+  uint32_t* addr[2] = {nullptr, nullptr};
+  int bit[2] = {0, 0}, np = 0;
   if (len >= 4) {
     uint32_t crc = 0xFFFFFFFFu, st = 0;
     for (uint32_t j = 0; j < len; j++) {
@@ -423,33 +445,43 @@ static __device__ __noinline__ int ecrc_fix(uint64_t* val, uint32_t* col, uint32
     }
     const uint32_t syn = st ^ crc ^ 0xFFFFFFFFu;
     if (!syn) return CLEAN;
-    const int r = crc_locate(syn, 96 * (int)len);
-    if (r != CRC_NO_FIX) {
+    int pos[2];
+    np = crc_fix_positions(syn, 96 * (int)len, due, pos);
+    o = np ? CORRECTED : DUE;
+    for (int q = 0; q < np && o == CORRECTED; q++) {
+      const int r = pos[q];
       if (r < 0) {   // stored CRC byte t/8 = col[31:24] of entry t/8
-        addr = col + start + ((-1 - r) >> 3);
-        bit = 24 + ((-1 - r) & 7);
-        o = CORRECTED;
+        addr[q] = col + start + ((-1 - r) >> 3);
+        bit[q] = 24 + ((-1 - r) & 7);
       } else {       // message: per entry 8 bytes val LE, 4 bytes col LE (top byte zeroed for entries 0..3)
         const int byte = r >> 3, k = byte / 12, bb = byte - 12 * k;
         if (bb < 8) {
-          addr = reinterpret_cast<uint32_t*>(val + start + k) + (bb >> 2);
-          bit = 8 * (bb & 3) + (r & 7);
-          o = CORRECTED;
+          addr[q] = reinterpret_cast<uint32_t*>(val + start + k) + (bb >> 2);
+          bit[q] = 8 * (bb & 3) + (r & 7);
         } else if (!(k < 4 && bb == 11)) {
-          addr = col + start + k;
-          bit = 8 * (bb - 8) + (r & 7);
-          o = CORRECTED;
+          addr[q] = col + start + k;
+          bit[q] = 8 * (bb - 8) + (r & 7);
+        } else {
+          o = DUE;   // a zeroed message byte: not a stored bit
         }
       }
     }
   }
   if (o == CORRECTED && how == 2) o = DUE;
-  if (fix_addr) *fix_addr = (o == CORRECTED) ? addr : nullptr;   // the located bit (count-only callers apply it)
-  if (fix_bit) *fix_bit = bit;
+  if (fix_addr)
+    for (int q = 0; q < 2; q++) {
+      fix_addr[q] = (o == CORRECTED && q < np) ? addr[q] : nullptr;
+      fix_bit[q] = bit[q];
+    }
   if (o == CORRECTED) {
     if (how == 1) {
-      const uint32_t w = *(volatile uint32_t*)addr;
-      if (scrub32(addr, w, w ^ (1u << bit))) cnt_add(cnt, T_ELEM, CRC32C, CORRECTED);
+      bool won = false;
+      for (int q = 0; q < np; q++) {
+        const uint32_t w = *(volatile uint32_t*)addr[q];
+        const bool ok = scrub32(addr[q], w, w ^ (1u << bit[q]));
+        if (q == 0) won = ok;
+      }
+      if (won) cnt_add(cnt, T_ELEM, CRC32C, CORRECTED);
     } else {
       cnt_add(cnt, T_ELEM, CRC32C, CORRECTED);
     }
@@ -522,7 +554,7 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
             continue;
           }
           const int64_t idx = a.col_base + cm;
-          const double x = (idx == own) ? p_own : gather_in<VS>(a.in, idx);
+          const double x = (idx == own) ? p_own : gather_in<VS>(a.in, idx, a.due);
           acc = fma(as_d(v), x, acc);
         }
       }
@@ -710,7 +742,7 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
     else if (rel == -1) x = win[oslot - 1];
     else if (rel == n) x = win[oslot + TILE_WW];
     else if (rel == -n) x = win[oslot - TILE_WW];
-    else x = a.fz ? gather_fused<VS>(a.in, a.r_f, a.beta_f, own + rel) : gather_in<VS>(a.in, own + rel);
+    else x = a.fz ? gather_fused<VS>(a.in, a.r_f, a.beta_f, own + rel) : gather_in<VS>(a.in, own + rel, a.due);
     acc = fma(as_d(v), x, acc);
   }
   return acc;
@@ -901,17 +933,16 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
 #pragma unroll
           for (int t = 0; t < G; t++) c[t] = e[q][t];
           int word = 0;
-          int o = rp_check_group<RS>(c, &word);
+          int o = rp_check_group<RS>(c, &word, a.due);
           if (o == CORRECTED && mode == MODE_DETECT) o = DUE;   // interval mode: detection only
           if (o != CLEAN) {
             const int64_t own = g * G < a.nrows ? g * G : a.nrows - 1;
             const bool owner = own >= rowseg && own < rowseg + 256;
             if (o == CORRECTED) {
-              uint32_t ow = 0, nw = 0;   // select, not index
+              uint32_t ov[G];   // (a copy: indexing e[q] would move it to local memory)
 #pragma unroll
-              for (int t = 0; t < G; t++)
-                if (t == word) { ow = e[q][t]; nw = c[t]; }
-              if (owner && scrub32(gp + word, ow, nw)) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
+              for (int t = 0; t < G; t++) ov[t] = e[q][t];
+              if (owner && scrub_entries32(gp, ov, c, G)) cnt_add(a.counts, T_ROWPTR, RS, CORRECTED);
 #pragma unroll
               for (int t = 0; t < G; t++) e[q][t] = c[t];
             } else if (owner) {   // DUE: e keeps the stored bits
@@ -1916,15 +1947,11 @@ __global__ void k_vec_check(uint64_t* d, int64_t n, int64_t npad, double* out, D
 #pragma unroll
     for (int t = 0; t < G; t++) o0[t] = v[t] = d[g * G + t];
     int word = 0;
-    int o = vec_check_group<VS>(v, &word);
+    int o = vec_check_group<VS>(v, &word, due);
     if (o == CORRECTED && scrub == 2) o = DUE;   // detection only
     if (o == CORRECTED) {
       bool won = true;
-      if (scrub) {
-        uint64_t ow = o0[word >> 1], nw = v[word >> 1];
-        won = scrub32(reinterpret_cast<uint32_t*>(d + g * G) + word, (word & 1) ? hi32(ow) : lo32(ow),
-                      (word & 1) ? hi32(nw) : lo32(nw));
-      }
+      if (scrub) won = scrub_group32(reinterpret_cast<uint32_t*>(d + g * G), o0, v, G);
       if (won) cnt_add(cnt, T_VEC, VS, CORRECTED);
     } else if (o == DUE) {
 #pragma unroll
@@ -2012,10 +2039,10 @@ __global__ void k_check_rowptr(uint32_t* rowptr, int64_t len, DevCounts* cnt, in
     uint32_t e[G], o0[G];
     for (int t = 0; t < G; t++) o0[t] = e[t] = rowptr[g * G + t];
     int word = 0;
-    int o = rp_check_group<RS>(e, &word);
+    int o = rp_check_group<RS>(e, &word, due);
     if (o == CORRECTED && scrub == 2) o = DUE;   // detection only (interval mode's final check)
     if (o == CORRECTED) {
-      bool won = scrub ? scrub32(rowptr + g * G + word, o0[word], e[word]) : true;
+      bool won = scrub ? scrub_entries32(rowptr + g * G, o0, e, G) : true;
       if (won) cnt_add(cnt, T_ROWPTR, RS, CORRECTED);
     } else if (o == DUE) {
       cnt_add(cnt, T_ROWPTR, RS, DUE);
@@ -2026,7 +2053,7 @@ __global__ void k_check_rowptr(uint32_t* rowptr, int64_t len, DevCounts* cnt, in
 // rowptr entry idx, its group checked and corrected in registers (a DUE group
 // gives its stored bits), masked.
 template <int RS>
-__device__ uint32_t rp_decoded(const uint32_t* rowptr, int64_t idx, bool detect_only) {
+__device__ uint32_t rp_decoded(const uint32_t* rowptr, int64_t idx, bool detect_only, const int* cfg) {
   constexpr int G = rgrp(RS);
   uint32_t e[G];
   const int64_t g0 = idx / G * G;
@@ -2036,7 +2063,7 @@ __device__ uint32_t rp_decoded(const uint32_t* rowptr, int64_t idx, bool detect_
   uint32_t w = raw;
   if (RS != NONE && !detect_only) {   // detection only: a correctable group is a DUE (stored bits)
     int word = 0;
-    if (rp_check_group<RS>(e, &word) == CORRECTED) {
+    if (rp_check_group<RS>(e, &word, cfg) == CORRECTED) {
 #pragma unroll
       for (int t = 0; t < G; t++) if (t == idx - g0) w = e[t];
     }
@@ -2050,7 +2077,7 @@ __global__ void k_check_rows(uint64_t* val, uint32_t* col, const uint32_t* rowpt
   for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < nrows; i += (int64_t)gridDim.x * blockDim.x) {
     // decoded entries (corrected in registers, not counted: the rowptr pass
     // counts), so count-only sweeps see the same ranges as scrubbing ones
-    const uint32_t s = rp_decoded<RS>(rowptr, i, scrub == 2), t = rp_decoded<RS>(rowptr, i + 1, scrub == 2);
+    const uint32_t s = rp_decoded<RS>(rowptr, i, scrub == 2, due), t = rp_decoded<RS>(rowptr, i + 1, scrub == 2, due);
     if (!(s <= t && (int64_t)t <= nnz)) {
       if (RS != NONE) { cnt_range(cnt, T_ROWPTR, RS); *due = 1; }
       continue;
@@ -2067,13 +2094,14 @@ __global__ void k_check_rows(uint64_t* val, uint32_t* col, const uint32_t* rowpt
         bad = (crc ^ 0xFFFFFFFFu) != st;
       }
       // scrub: 0 count only, 1 count + correct in place, 2 detection only
-      uint32_t* fa = nullptr;
-      int fb = 0;
-      if (bad) ecrc_fix(val, col, s, t - s, scrub == 1 ? 1 : scrub == 2 ? 2 : 0, cnt, due, &fa, &fb);
+      uint32_t* fa[2] = {nullptr, nullptr};
+      int fb[2] = {0, 0};
+      if (bad) ecrc_fix(val, col, s, t - s, scrub == 1 ? 1 : scrub == 2 ? 2 : 0, cnt, due, fa, fb);
       // the row is the codeword: range-check its columns as decoded by it
       for (uint32_t j = s; j < t; j++) {
         uint32_t c = *(volatile uint32_t*)(col + j);
-        if (fa == col + j && scrub == 0) c ^= 1u << fb;
+        for (int q = 0; q < 2; q++)
+          if (fa[q] == col + j && scrub == 0) c ^= 1u << fb[q];
         if ((int64_t)(c & 0x00FFFFFFu) >= ncols) { cnt_range(cnt, T_ELEM, CRC32C); *due = 1; }
       }
     }

@@ -121,3 +121,90 @@ def test_crc_check_all_parity(abft, ctx, scrub):
     assert np.array_equal(cg, cnt_o), (cg[:, S].tolist(), cnt_o[:, S].tolist())
     assert np.array_equal(col_words(Ag), Ao.col) and np.array_equal(val_words(Ag), Ao.val)
     assert np.array_equal(rowptr_words(Ag), Ao.rowptr)
+
+
+# ------------------------------------------------ 2EC3ED (reading R9b)
+@pytest.fixture
+def two_ec(abft, ctx):
+    orc.set_crc_correct(2)
+    ctx.set_crc_correction(2)
+    yield
+    orc.set_crc_correct(1)
+    ctx.set_crc_correction(1)
+
+
+@pytest.mark.parametrize("stencil", [True, False])
+@pytest.mark.parametrize("nbits", [2, 3])
+def test_crc_2ec_spmv_parity(abft, ctx, two_ec, stencil, nbits):
+    """Pair correction enabled: double flips in E-CRC rows, R-CRC octets and
+    V-CRC quads of the SpMV input are corrected (both words scrubbed, counted
+    once); triple flips stay DUEs — bit-exact against the oracle's 2EC3ED."""
+    n = 256 if stencil else 48
+    Ao, Ag, N = _both(abft, ctx, n, stencil)
+    rng = np.random.default_rng(300 + 10 * nbits + stencil)
+    for r in range(16):
+        row = (37 * r + 5) % N
+        for b in rng.choice(480, nbits, replace=False):
+            _flip_el(abft, ctx, Ao, Ag, 5 * row + int(b) // 96, int(b) % 96)
+    for g in rng.choice(len(Ao.rowptr) // 8 - 1, 16, replace=False):
+        for b in rng.choice(256, nbits, replace=False):
+            Ao.rowptr[8 * g + b // 32] ^= np.uint32(1 << int(b % 32))
+            abft.inject_bitflip(ctx, Ag.rowptr, 256 * int(g) + int(b))
+    xo = orc.vec_encode(gen.uniform_pm1(N, 4) * 2.0, S)
+    xg = gpu_vec_from_words(abft, xo, N, S)
+    for q in rng.choice(N // 4, 16, replace=False):
+        for b in rng.choice(256, nbits, replace=False):
+            xo[4 * q + b // 64] ^= np.uint64(1 << int(b % 64))
+            abft.inject_bitflip(ctx, xg.data, 256 * int(q) + int(b))
+    yo = np.zeros_like(xo)
+    cnt_o = orc.new_counts()
+    orc.spmv(Ao, xo, N, S, yo, N, cnt_o)
+    yg = abft.Vector.empty(N, S)
+    cnt_g = abft.Counters()
+    abft.spmv(ctx, Ag, xg, yg, cnt_g)
+    torch.cuda.synchronize()
+    cg = cnt_g.read()
+    assert np.array_equal(cg, cnt_o), (cg[:, S].tolist(), cnt_o[:, S].tolist())
+    if nbits == 2:
+        assert cg[orc.ELEM, S, orc.COR] == 16 and cg[orc.ROWPTR, S, orc.COR] == 16 and cg[orc.VEC, S, orc.COR] == 16
+        assert cg[:, S, orc.UNC].sum() == 0
+    else:
+        assert cg[:, S, orc.COR].sum() == 0
+    keep = np.uint64(~np.uint64(0xFF))
+    both_nan = np.isnan((words_of(yg)[:N] & keep).view(np.float64)) & np.isnan((yo[:N] & keep).view(np.float64))
+    assert np.all((words_of(yg)[:N] == yo[:N]) | both_nan)
+    assert np.array_equal(val_words(Ag), Ao.val) and np.array_equal(col_words(Ag), Ao.col)
+    assert np.array_equal(rowptr_words(Ag), Ao.rowptr)
+    assert np.array_equal(words_of(xg)[:N], xo[:N])
+
+
+@pytest.mark.parametrize("scrub", [0, 1, 2])
+def test_crc_2ec_check_all_parity(abft, ctx, two_ec, scrub):
+    Ao, Ag, N = _both(abft, ctx, 40, False)
+    rng = np.random.default_rng(50 + scrub)
+    for row in rng.choice(N, 8, replace=False):
+        for b in rng.choice(480, 2, replace=False):
+            _flip_el(abft, ctx, Ao, Ag, 5 * int(row) + int(b) // 96, int(b) % 96)
+    for g in rng.choice(len(Ao.rowptr) // 8 - 1, 6, replace=False):
+        for b in rng.choice(256, 2, replace=False):
+            Ao.rowptr[8 * g + b // 32] ^= np.uint32(1 << int(b % 32))
+            abft.inject_bitflip(ctx, Ag.rowptr, 256 * int(g) + int(b))
+    xo = orc.vec_encode(gen.uniform_pm1(N, 10), S)
+    xg = gpu_vec_from_words(abft, xo, N, S)
+    for q in rng.choice(N // 4, 6, replace=False):
+        for b in rng.choice(256, 2, replace=False):
+            xo[4 * q + b // 64] ^= np.uint64(1 << int(b % 64))
+            abft.inject_bitflip(ctx, xg.data, 256 * int(q) + int(b))
+    cnt_o = orc.new_counts()
+    Ao.check(cnt_o, scrub=scrub)
+    orc.vec_check(xo, N, S, cnt_o, scrub=(scrub == 1))
+    cnt_g = abft.Counters()
+    abft.check_all(ctx, Ag, [xg] if scrub != 2 else [], cnt_g, scrub=scrub)
+    cg = cnt_g.read()
+    if scrub == 2:
+        cnt_o[orc.VEC] = 0
+    assert np.array_equal(cg, cnt_o), (cg[:, S].tolist(), cnt_o[:, S].tolist())
+    assert np.array_equal(col_words(Ag), Ao.col) and np.array_equal(val_words(Ag), Ao.val)
+    assert np.array_equal(rowptr_words(Ag), Ao.rowptr)
+    if scrub != 2:
+        assert np.array_equal(words_of(xg)[:N], xo[:N])
