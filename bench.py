@@ -134,7 +134,7 @@ def build_problem(n: int, ny: int, rank: int, world: int, device, chunk_rows=Non
 class Solver:
     """One configuration (protected or unprotected twin) of the solve."""
 
-    def __init__(self, abft, ctx, P, es, rs, vs, dist=None, check_interval=1):
+    def __init__(self, abft, ctx, P, es, rs, vs, dist=None, check_interval=1, sr=False):
         import torch
         self.abft, self.ctx, self.P, self.dist = abft, ctx, P, dist
         self.check_interval = check_interval
@@ -150,7 +150,8 @@ class Solver:
             self.A.append(M)
             self.raw.append((ch["col"], rp_raw))
         n_ext = N + 2 * halo
-        self.vecs = [abft.Vector.empty(n_ext, vs, device=dev) for _ in range(5)]  # b x r p w
+        self.sr = sr   # single-reduction CG: a sixth vector s
+        self.vecs = [abft.Vector.empty(n_ext, vs, device=dev) for _ in range(6 if sr else 5)]  # b x r p w [s]
         self.counts = abft.Counters(device=dev)
         self.b_raw = P["b"]
         self.N, self.halo = N, halo
@@ -182,7 +183,14 @@ class Solver:
                 raise RuntimeError(f"encode failed: {self.abft.last_error()}")
         self.vecs[0].encode(self.ctx)
         self.vecs[1].encode(self.ctx)
-        if self.dist is not None:
+        if self.sr:
+            if self.dist is not None:
+                res = self.dist.cg_solve_sr(self.ctx, self.A, self.halo, *self.vecs, tol=tol, max_iters=max_iters,
+                                            due_policy=1, counts=self.counts, poll_every=32)
+            else:
+                res = self.abft.cg_solve_sr(self.ctx, self.A, *self.vecs, tol=tol, max_iters=max_iters, due_policy=1,
+                                            counts=self.counts, poll_every=32)
+        elif self.dist is not None:
             res = self.dist.cg_solve(self.ctx, self.A, self.halo, *self.vecs, tol=tol, max_iters=max_iters,
                                      due_policy=1, counts=self.counts, poll_every=32,
                                      check_interval=self.check_interval)
@@ -366,6 +374,8 @@ def main():
     ap.add_argument("--fuse", action="store_true", help="main line on the fused calc_p path (DESIGN.md §6.1)")
     ap.add_argument("--no-pdl", action="store_true", help="plain launches in the CG loop (DESIGN.md §6.2)")
     ap.add_argument("--no-fused-extra", action="store_true", help="skip the fused-calc_p side measurement")
+    ap.add_argument("--no-sr-extra", action="store_true",
+                    help="skip the single-reduction CG side measurement (DESIGN.md §4.1)")
     args = ap.parse_args()
     if args.impl == "reference":
         return run_reference(args)
@@ -430,6 +440,23 @@ def main():
                "bytes_per_row_per_iter": CG_BYTES_PER_ROW if fused else FUSED_CG_BYTES_PER_ROW,
                "kernel_ms": {"spmv": ms_a[0] / max(n_a[0], 1), "calc_ur": ms_a[1] / max(n_a[1], 1),
                              "calc_p": ms_a[2] / max(n_a[2], 1), "reductions": ms_a[3] / max(n_a[3], 1)}}
+
+    # side measurement: the single-reduction CG (one reduction per iteration), protected and unprotected
+    alt_sr = None
+    if not args.no_sr_extra:
+        s_p = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj, sr=True)
+        r_sp = timed(s_p, args.steps, 1, args.tol, args.max_iters, dist_on)
+        del s_p
+        s_u = Solver(abft, ctx, P, abft.NONE, abft.NONE, abft.NONE, dobj, sr=True)
+        r_su = timed(s_u, args.steps, 1, args.tol, args.max_iters, dist_on)
+        del s_u
+        eq_ = P["N"] / float(4096 * 4096)
+        ip, iu = r_sp["ms"] / max(r_sp["iters"], 1), r_su["ms"] / max(r_su["iters"], 1)
+        alt_sr = {"value": world * r_sp["iters"] / (r_sp["ms"] / 1000.0) * eq_,
+                  "unprotected_value": world * r_su["iters"] / (r_su["ms"] / 1000.0) * eq_,
+                  "iters_per_step": r_sp["iters"] / args.steps,
+                  "overhead_pct_per_iter": 100.0 * (ip / iu - 1.0), "bytes_per_row_per_iter": CG_BYTES_PER_ROW,
+                  "statuses": sorted(r_sp["statuses"])}
 
     e2e = None
     if not args.no_e2e:
@@ -502,6 +529,7 @@ def main():
                         "calc_p_ms": ms_u[2] / max(n_u[2], 1), "reductions_ms": ms_u[3] / max(n_u[3], 1)},
         "overhead_pct_per_iter": 100.0 * (iter_ms_p / iter_ms_u - 1.0),
         "alt_calc_p_arrangement": alt,
+        "alt_single_reduction_cg": alt_sr,
         "clocks": clocks,
         "gpu_launches": r_p["launches"],
         "e2e": e2e,

@@ -91,6 +91,9 @@ def lib():
         L.or_cheby_solve.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, C.c_int, C.c_double, C.c_double,
                                      C.c_double, C.c_int, C.c_int, C.c_void_p, C.c_void_p]
         L.or_set_crc_correct.argtypes = [C.c_int]
+        L.or_ppcg_solve.argtypes = [C.c_void_p, u64p, u64p, u64p, u64p, u64p, u64p, u64p, u64p, C.c_int,
+                                    C.c_double, C.c_double, C.c_int, C.c_double, C.c_int, C.c_int, C.c_void_p,
+                                    C.c_void_p]
         L.or_vec_masked.argtypes = [u64p, C.c_int64, C.c_int, dp]
         L.or_round_k.restype = C.c_uint64
         L.or_round_k.argtypes = [C.c_uint64, C.c_int]
@@ -387,3 +390,15 @@ def cheby_solve(A: Matrix, b, u, r, p, w, scheme, eigmin, eigmax, tol=1e-10, max
 def set_crc_correct(t: int):
     """CRC32C correction capability: 1 = 1EC4ED (default), 2 = 2EC3ED."""
     lib().or_set_crc_correct(int(t))
+
+
+def ppcg_solve(A: Matrix, b, x, r, p, w, z, rin, pin, scheme, eigmin, eigmax, inner=10, tol=1e-10, max_iters=10000,
+               due_policy=1, counts=None):
+    """Protected polynomially preconditioned CG (TeaLeaf PPCG):
+    the preconditioner is `inner` Chebyshev steps on [eigmin, eigmax] from z = 0."""
+    s = A.cstruct()
+    res = CGResult()
+    st = lib().or_ppcg_solve(C.byref(s), *[_p(v, C.c_uint64) for v in (b, x, r, p, w, z, rin, pin)], scheme,
+                             float(eigmin), float(eigmax), int(inner), tol, max_iters, due_policy, C.byref(res),
+                             counts.ctypes.data if counts is not None else None)
+    return st, res

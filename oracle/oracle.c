@@ -20,6 +20,8 @@
  *         Chebyshev  TeaLeaf's Chebyshev iteration (S§8(f) f4), DESIGN.md §4.3
  *                    (reading R32), or_cheby_solve; CG coefficient log
  *                    or_cg_solve_log for the spectrum estimate
+ *         PPCG       CG with an m-step Chebyshev polynomial preconditioner
+ *                    (S§8(f) f4), DESIGN.md §4.4 (reading R34), or_ppcg_solve
  *         faults     O10 scheduled bit flips (S§8(c) O10): XOR before init /
  *                    before iteration k's SpMV, or_cg_solve_sched
  *         CRC fix    1EC4ED single-bit correction (2EC3ED pair correction with
@@ -1167,6 +1169,90 @@ int or_cheby_solve(or_csr* A, uint64_t* b, uint64_t* u, uint64_t* r, uint64_t* p
     dues += cheb_update(b, w, p, u, r, n, vs, 0, theta, alpha, beta, cnt, &rr);
     res->iters = k; res->rrn = rr;
     int conv = sqrt(rr) <= tol * sqrt(rr0);
+    if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+    if (conv) return OK;
+  }
+  res->status = (max_iters > 0) ? E_NOT_CONVERGED : OK;
+  return res->status;
+}
+
+/* ---------------------------------------------------------- PPCG
+ * S§8(f) f4: TeaLeaf's polynomially preconditioned CG (ref [19]; reading R34,
+ * DESIGN.md §4.4): CG whose preconditioner z = M^-1 r is m steps of the
+ * Chebyshev iteration of R32 on A z = r from z = 0, bounds [eigmin, eigmax]
+ * (the step coefficients are the same recurrence, restarted for every
+ * application).  Every vector read checked, every write re-encoded.
+ *  apply(r -> z): rin = r (no SpMV of z = 0); pin = enc(rin'/theta);
+ *                 z = enc(pin');  for j = 1..m-1: w = A z; rin = enc(r - w);
+ *                 pin = enc(fma(alpha_j, pin', beta_j rin')); z = enc(z' + pin').
+ *  Init: w = A x0; r = enc(b - w); rr0 = r.r (0 -> 0 iterations); z = M^-1 r;
+ *        rz = r.z; p = z (word copy).
+ *  Iter k: w = A p, pw = p.w; alpha = rz/pw; x = enc(fma(alpha, p, x));
+ *        r = enc(fma(-alpha, w, r)); rr = r.r; converged if sqrt(rr) <= tol sqrt(rr0);
+ *        z = M^-1 r; rz' = r.z; beta = rz'/rz; p = enc(fma(beta, p, z)); rz = rz'. */
+static int64_t ppcg_apply(or_csr* A, uint64_t* r, uint64_t* z, uint64_t* w, uint64_t* rin, uint64_t* pin, int64_t n,
+                          int vs, double eigmin, double eigmax, int m, counts_t* cnt) {
+  double theta = (eigmax + eigmin) / 2.0, delta = (eigmax - eigmin) / 2.0;
+  double sigma = theta / delta, rho = 1.0 / sigma, rr;
+  double* R = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* P = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  int64_t dues = vdec(r, n, vs, R, cnt);
+  venc(rin, R, n, vs);                       /* rin = r (re-encoded) */
+  vmasked(rin, n, vs, R);
+  for (int64_t i = 0; i < n; i++) P[i] = R[i] / theta;
+  venc(pin, P, n, vs);
+  vmasked(pin, n, vs, P);
+  venc(z, P, n, vs);                         /* z = 0 + pin */
+  free(R); free(P);
+  for (int j = 1; j < m; j++) {
+    double rho_new = 1.0 / (2.0 * sigma - rho);
+    double alpha = rho_new * rho, beta = (2.0 * rho_new) / delta;
+    rho = rho_new;
+    dues += or_spmv_mode(A, z, n, vs, w, n, cnt, NULL, M_CORRECT);
+    dues += cheb_update(r, w, pin, z, rin, n, vs, 0, theta, alpha, beta, cnt, &rr);
+  }
+  return dues;
+}
+
+/* r.z over the masked stored values (RED-1), both operands checked */
+static int64_t dot_checked(uint64_t* a, uint64_t* b, int64_t n, int vs, counts_t* cnt, double* out) {
+  double* A_ = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  double* B_ = (double*)malloc(sizeof(double) * (size_t)(n + 1));
+  int64_t dues = vdec(a, n, vs, A_, cnt) + vdec(b, n, vs, B_, cnt);
+  *out = or_dot_red1(A_, B_, n);
+  free(A_); free(B_);
+  return dues;
+}
+
+int or_ppcg_solve(or_csr* A, uint64_t* b, uint64_t* x, uint64_t* r, uint64_t* p, uint64_t* w, uint64_t* z,
+                  uint64_t* rin, uint64_t* pin, int vs, double eigmin, double eigmax, int inner, double tol,
+                  int max_iters, int due_policy, or_cg_result* res, counts_t* cnt) {
+  init_instances();
+  int64_t n = A->nrows;
+  double rr0, rr, rz, rzn, pw;
+  res->iters = 0; res->status = OK; res->rr0 = 0.0; res->rrn = 0.0;
+  int64_t dues = or_spmv_mode(A, x, n, vs, w, n, cnt, NULL, M_CORRECT);
+  dues += or_cg_init_r(b, w, r, p, n, vs, cnt, &rr0);
+  res->rr0 = rr0; res->rrn = rr0;
+  if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+  if (rr0 == 0.0) return OK;
+  dues = ppcg_apply(A, r, z, w, rin, pin, n, vs, eigmin, eigmax, inner, cnt);
+  dues += dot_checked(r, z, n, vs, cnt, &rz);
+  memcpy(p, z, sizeof(uint64_t) * (size_t)or_vec_padded_len(n, vs));
+  if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
+  for (int k = 1; k <= max_iters; k++) {
+    dues = or_spmv_mode(A, p, n, vs, w, n, cnt, &pw, M_CORRECT);
+    double alpha = rz / pw;
+    dues += or_calc_ur(x, p, r, w, n, vs, alpha, cnt, &rr);
+    res->iters = k; res->rrn = rr;
+    int conv = sqrt(rr) <= tol * sqrt(rr0);
+    if (!conv) {
+      dues += ppcg_apply(A, r, z, w, rin, pin, n, vs, eigmin, eigmax, inner, cnt);
+      dues += dot_checked(r, z, n, vs, cnt, &rzn);
+      double beta = rzn / rz;
+      dues += or_calc_p(p, z, n, vs, beta, cnt);
+      rz = rzn;
+    }
     if (dues && due_policy == 0) { res->status = E_DUE; return E_DUE; }
     if (conv) return OK;
   }
