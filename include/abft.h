@@ -175,6 +175,16 @@ int abft_cg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, ab
 int abft_cheby_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
                      abft_vec* w, double eigmin, double eigmax, const abft_cg_opts* opts, abft_cg_result* res,
                      abft_counts* dcnt, void* stream);
+/* Protected PPCG (S§8(f) f4: TeaLeaf's polynomially preconditioned CG;
+ * DESIGN.md §4.4, reading R34): CG whose preconditioner z = M^-1 r is `inner`
+ * (1..64) Chebyshev steps (as abft_cheby_solve's, bounds [eigmin, eigmax]) on
+ * A z = r from z = 0; beta = (r.z)'/(r.z), p = z + beta p.  z, rin, pin are
+ * three more vectors like the others (the preconditioner's iterate, residual
+ * and direction).  Same conventions, counters and statuses as abft_cg_solve;
+ * single GPU, every access checked. */
+int abft_ppcg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                    abft_vec* w, abft_vec* z, abft_vec* rin, abft_vec* pin, double eigmin, double eigmax, int inner,
+                    const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream);
 /* TeaLeaf's spectrum estimate (reading R33): `steps` (2..128)
  * protected CG iterations from x (opts supply the policy; tol is ignored),
  * then the extreme eigenvalues of the Lanczos tridiagonal built from the CG

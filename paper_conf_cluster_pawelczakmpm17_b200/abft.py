@@ -75,6 +75,8 @@ _sig = {
     "abft_cheby_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                    C.POINTER(Vec), C.POINTER(Vec), C.c_double, C.c_double, C.POINTER(CGOpts),
                                    C.POINTER(CGResult), _P, _P]),
+    "abft_ppcg_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int] + [C.POINTER(Vec)] * 8 +
+                        [C.c_double, C.c_double, C.c_int, C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
     "abft_cg_spectrum": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                    C.POINTER(Vec), C.POINTER(Vec), C.c_int, C.POINTER(CGOpts),
                                    C.POINTER(C.c_double), C.POINTER(C.c_double), C.POINTER(CGResult), _P, _P]),
@@ -361,6 +363,20 @@ def cheby_solve(ctx: Context, A, b: Vector, u: Vector, r: Vector, p: Vector, w: 
     code = _lib.abft_cheby_solve(ctx.h, arr, n, *[C.byref(v) for v in vs], float(eigmin), float(eigmax),
                                  C.byref(opts), C.byref(res), counts.ptr if counts else None, _stream(stream))
     _check(code, "abft_cheby_solve", allow=(E_DUE, E_NOT_CONVERGED))
+    return res
+
+
+def ppcg_solve(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vector, z: Vector, rin: Vector,
+               pin: Vector, eigmin: float, eigmax: float, inner=10, tol=1e-10, max_iters=10000, due_policy=0,
+               counts: Counters | None = None, poll_every=16, stream=None) -> CGResult:
+    """Protected PPCG: CG with an `inner`-step Chebyshev preconditioner (abft_ppcg_solve)."""
+    arr, n = _chunks(A)
+    opts = CGOpts(tol, max_iters, due_policy, poll_every, 1)
+    res = CGResult()
+    vs = [v.cstruct() for v in (b, x, r, p, w, z, rin, pin)]
+    code = _lib.abft_ppcg_solve(ctx.h, arr, n, *[C.byref(v) for v in vs], float(eigmin), float(eigmax), int(inner),
+                                C.byref(opts), C.byref(res), counts.ptr if counts else None, _stream(stream))
+    _check(code, "abft_ppcg_solve", allow=(E_DUE, E_NOT_CONVERGED))
     return res
 
 

@@ -448,6 +448,10 @@ struct RankRun {
   VecArgs va_sr{};
   bool cheb = false;           // Chebyshev iteration with bounds [eigmin, eigmax]; x is u
   double eigmin = 0.0, eigmax = 0.0;
+  int ppcg_inner = 0;          // PPCG: inner Chebyshev steps; z, rin, pin its vectors
+  abft_vec* z = nullptr;
+  abft_vec* rin = nullptr;
+  abft_vec* pin = nullptr;
   DevCounts* cnt = nullptr;
   int64_t n = 0, nrb = 0, n_ext = 0;
   VecArgs va{};
@@ -602,6 +606,43 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   // single-reduction CG (Chronopoulos-Gear, S§8(f) f3): one GPU, every access checked
   const bool sr = R[0].s_vec != nullptr;
   const bool cheb = R[0].cheb;
+  const bool ppcg = R[0].ppcg_inner > 0;
+  std::vector<double> pc_alpha, pc_beta;   // PPCG inner step coefficients (host, rounded as written)
+  double pc_theta = 0.0;
+  VecArgs vpc{}, vdot{}, vcp{};
+  if (ppcg) {
+    if (d || nl != 1) return fail(ABFT_E_SHAPE, "PPCG runs on one GPU");
+    if (opts->check_interval > 1) return fail(ABFT_E_SHAPE, "PPCG checks every access");
+    if (!(R[0].eigmax > R[0].eigmin)) return fail(ABFT_E_INVALID, "PPCG bounds need eigmax > eigmin");
+    abft_vec* extra[3] = {R[0].z, R[0].rin, R[0].pin};
+    for (int i = 0; i < 3; i++) {
+      int e0 = check_vec(extra[i], "z/rin/pin");
+      if (e0) return e0;
+      if (extra[i]->scheme != scheme || extra[i]->n != R[0].n_ext)
+        return fail(ABFT_E_INVALID, "PPCG vectors: scheme/length differ");
+      for (int j = 0; j < 5; j++) if (R[0].v[j]->data == extra[i]->data) return fail(ABFT_E_INVALID, "vectors alias");
+      for (int j = 0; j < i; j++) if (extra[j]->data == extra[i]->data) return fail(ABFT_E_INVALID, "vectors alias");
+    }
+    pc_theta = (R[0].eigmax + R[0].eigmin) / 2.0;
+    const double delta = (R[0].eigmax - R[0].eigmin) / 2.0, sigma = pc_theta / delta;
+    double rho = 1.0 / sigma;
+    for (int j = 1; j < R[0].ppcg_inner; j++) {
+      const double rho_new = 1.0 / (2.0 * sigma - rho);
+      pc_alpha.push_back(rho_new * rho);
+      pc_beta.push_back((2.0 * rho_new) / delta);
+      rho = rho_new;
+    }
+    auto ptr = [](abft_vec* v) { return reinterpret_cast<uint64_t*>(v->data); };
+    vpc = R[0].va;      // preconditioner: rhs r, u = z, direction pin, residual rin, A z -> w
+    vpc.b = ptr(R[0].r());
+    vpc.x = ptr(R[0].z);
+    vpc.p = ptr(R[0].pin);
+    vpc.r = ptr(R[0].rin);
+    vdot = R[0].va;     // r . z
+    vdot.x = ptr(R[0].z);
+    vcp = R[0].va;      // p = z + beta p
+    vcp.r = ptr(R[0].z);
+  }
   if (cheb) {
     if (d || nl != 1) return fail(ABFT_E_SHAPE, "Chebyshev iteration runs on one GPU");
     if (opts->check_interval > 1) return fail(ABFT_E_SHAPE, "Chebyshev iteration checks every access");
@@ -637,7 +678,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   // G = 1 vector scheme; p is double-buffered with ctx->p_alt
   const int64_t npad_ext = vec_padded_len(R[0].n_ext, scheme);
   // (a fault schedule addresses the caller's p: the double-buffered fused CG is off then)
-  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0 && ctx->nfaults == 0 && !sr && !cheb;
+  bool fused = ctx->fuse_p && !multi && G == 1 && n_halo == 0 && ctx->nfaults == 0 && !sr && !cheb && !ppcg;
   abft_vec* const p = R[0].p();
   abft_vec* const r = R[0].r();
   if (fused) {
@@ -667,6 +708,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   h.abort_policy = opts->due_policy == 0 ? 1 : 0;
   h.dist = multi ? 1 : 0;
   h.fused = fused ? 1 : 0;
+  h.pcg = ppcg ? 1 : 0;
   h.alpha_log = ctx->cg_log;
   h.beta_log = ctx->cg_log + CG_LOG;
   if (cheb) {   // host arithmetic, rounded as written
@@ -696,7 +738,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   if (!cheb)
     for (int q = 0; q < nl; q++) count_launch(launch_init_r(R[q].va, scheme, s));
   if (cheb) {   // r = b - A u0; p = r/theta; u += p; rr0
-    count_launch(launch_cheb(R[0].va, scheme, 1, s));
+    count_launch(launch_cheb(R[0].va, scheme, 1, 0.0, 0.0, 0.0, s));
     if ((e = finish_dot(R, nl, d, 8, s))) return e;
   } else if (sr) {
     // p = s = encoded +0.0, then w = A r with both dots (gamma = r.r, delta = w.r)
@@ -713,6 +755,23 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     if ((e = finish_sr(R, nl, d, 7, s))) return e;
   } else if ((e = finish_dot(R, nl, d, 1, s))) {
     return e;
+  }
+  // PPCG's preconditioner z = M^-1 r: inner Chebyshev steps from z = 0
+  auto apply_prec = [&](cudaStream_t ss) -> int {
+    count_launch(launch_cheb(vpc, scheme, 3, 0.0, 0.0, pc_theta, ss));
+    for (size_t j = 0; j < pc_alpha.size(); j++) {
+      int e2 = spmv_chunks(ctx, R[0].A, R[0].nchunks, R[0].z, R[0].w(), 0, R[0].cnt, ctx->state, ss, nullptr);
+      if (e2) return e2;
+      count_launch(launch_cheb(vpc, scheme, 2, pc_alpha[j], pc_beta[j], pc_theta, ss));
+    }
+    return ABFT_OK;
+  };
+  if (ppcg) {   // z = M^-1 r0; rz = r.z; p = z
+    if ((e = apply_prec(s))) return e;
+    count_launch(launch_dot(vdot, scheme, s));
+    if ((e = finish_dot(R, nl, d, 12, s))) return e;
+    count_launch(launch_copy_running(reinterpret_cast<uint64_t*>(R[0].p()->data),
+                                     reinterpret_cast<const uint64_t*>(R[0].z->data), npad_ext, ctx->state, s));
   }
   CUDA_TRY(cudaGetLastError());
 
@@ -774,7 +833,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
         prof.end();
         if (e2) return e2;
         prof.begin(1);
-        count_launch(launch_cheb(R[0].va, scheme, 0, ss));
+        count_launch(launch_cheb(R[0].va, scheme, 0, 0.0, 0.0, 0.0, ss));
         prof.end();
         prof.begin(3);
         if ((e2 = finish_dot(R, nl, d, 9, ss))) return e2;
@@ -811,7 +870,18 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
       prof.begin(3);
       if ((e2 = finish_dot(R, nl, d, 3, ss))) return e2;
       prof.end();
-      if (!fused) {
+      if (ppcg) {   // z = M^-1 r; beta = (r.z)'/(r.z); p = z + beta p
+        prof.begin(2);
+        if ((e2 = apply_prec(ss))) return e2;
+        count_launch(launch_dot(vdot, scheme, ss));
+        prof.end();
+        prof.begin(3);
+        if ((e2 = finish_dot(R, nl, d, 11, ss))) return e2;
+        prof.end();
+        prof.begin(2);
+        count_launch(launch_calc_p(vcp, scheme, ss));
+        prof.end();
+      } else if (!fused) {
         prof.begin(2);
         for (int q = 0; q < nl; q++) count_launch(launch_calc_p(R[q].va, scheme, ss));
         prof.end();
@@ -993,6 +1063,22 @@ int abft_cheby_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b,
   R.cheb = true;
   R.eigmin = eigmin;
   R.eigmax = eigmax;
+  return cg_run(&R, 1, nullptr, 0, opts, res, (cudaStream_t)stream);
+}
+
+int abft_ppcg_solve(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* b, abft_vec* x, abft_vec* r, abft_vec* p,
+                    abft_vec* w, abft_vec* z, abft_vec* rin, abft_vec* pin, double eigmin, double eigmax, int inner,
+                    const abft_cg_opts* opts, abft_cg_result* res, abft_counts* dcnt, void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  if (inner < 1 || inner > 64) return fail(ABFT_E_INVALID, "PPCG inner steps must be in [1, 64]");
+  if (!z || !rin || !pin) return fail(ABFT_E_INVALID, "null PPCG vector");
+  RankRun R = make_rank(ctx, A, nchunks, b, x, r, p, w, dcnt);
+  R.ppcg_inner = inner;
+  R.eigmin = eigmin;
+  R.eigmax = eigmax;
+  R.z = z;
+  R.rin = rin;
+  R.pin = pin;
   return cg_run(&R, 1, nullptr, 0, opts, res, (cudaStream_t)stream);
 }
 

@@ -24,6 +24,7 @@ struct CgState {
   // bounds and the recurrence's rho (alpha / beta above hold its step
   // coefficients)
   double ch_theta, ch_delta, ch_sigma, ch_rho;
+  int32_t pcg;   // PPCG: rro holds r.z, kept by k_post_p
   // CG step coefficients of the first CG_LOG iterations (Lanczos data of the
   // spectrum estimate, abft_cg_spectrum): ctx-owned device arrays [CG_LOG]
   double* alpha_log;
@@ -143,8 +144,15 @@ int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* 
 // (r.r) in RED-1 order and apply op 7 (init) / 6 (iteration)
 int launch_reduce_sr(const double* partials, const double* partials2, int64_t nrb, double* roots, double* roots2,
                      uint32_t* ticket, int op, CgState* st, const int* due, cudaStream_t s);
-// Chebyshev update: init = 1 -> the first step (p = r/theta)
-int launch_cheb(const VecArgs& a, int vs, int init, cudaStream_t s);
+// Chebyshev update (DESIGN.md §4.3 / §4.4).  mode: 0 step, 1 first step (p =
+// r/theta), coefficients from the CG state; 2 step, 3 first step from u = 0
+// (no w, no u read), coefficients alpha / beta / theta as given (the PPCG
+// preconditioner's inner steps).
+int launch_cheb(const VecArgs& a, int vs, int mode, double alpha, double beta, double theta, cudaStream_t s);
+// checked dot a.r . a.x (RED-1 partials; PPCG's r.z)
+int launch_dot(const VecArgs& a, int vs, cudaStream_t s);
+// dst = src (encoded words, npad entries) unless the solve stopped
+int launch_copy_running(uint64_t* dst, const uint64_t* src, int64_t npad, const CgState* st, cudaStream_t s);
 // single-reduction CG update: p, s, x, r (VecArgs.b carries s)
 int launch_calc_sr(const VecArgs& a, int vs, cudaStream_t s);
 // single-reduction CG, multi-rank: op 10 -> out[0..3) = (w.r root, DUE flag, r.r root)

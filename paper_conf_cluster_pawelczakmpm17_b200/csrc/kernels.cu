@@ -134,21 +134,42 @@ int launch_calc_sr(const VecArgs& a, int vs, cudaStream_t s) {
   }
   return 1;
 }
-template <bool INIT>
-static void launch_cheb_t(const VecArgs& a, int vs, cudaStream_t s) {
+template <int MODE>
+static void launch_cheb_t(const VecArgs& a, int vs, double al, double be, double th, cudaStream_t s) {
   int nb = blocks_rb(a.n);
   switch (vs) {
-    case NONE: launch_k(k_cheb<NONE, INIT>, nb, 256, 0, s, a); break;
-    case SED: launch_k(k_cheb<SED, INIT>, nb, 256, 0, s, a); break;
-    case SECDED64: launch_k(k_cheb<SECDED64, INIT>, nb, 256, 0, s, a); break;
-    case SECDED128: launch_k(k_cheb<SECDED128, INIT>, nb, 256, 0, s, a); break;
-    default: launch_k(k_cheb<CRC32C, INIT>, nb, 256, vec_dyn_smem<CRC32C>(), s, a); break;
+    case NONE: launch_k(k_cheb<NONE, MODE>, nb, 256, 0, s, a, al, be, th); break;
+    case SED: launch_k(k_cheb<SED, MODE>, nb, 256, 0, s, a, al, be, th); break;
+    case SECDED64: launch_k(k_cheb<SECDED64, MODE>, nb, 256, 0, s, a, al, be, th); break;
+    case SECDED128: launch_k(k_cheb<SECDED128, MODE>, nb, 256, 0, s, a, al, be, th); break;
+    default: launch_k(k_cheb<CRC32C, MODE>, nb, 256, vec_dyn_smem<CRC32C>(), s, a, al, be, th); break;
   }
 }
-int launch_cheb(const VecArgs& a, int vs, int init, cudaStream_t s) {
+int launch_cheb(const VecArgs& a, int vs, int mode, double alpha, double beta, double theta, cudaStream_t s) {
   if (a.n <= 0) return 0;
-  if (init) launch_cheb_t<true>(a, vs, s);
-  else launch_cheb_t<false>(a, vs, s);
+  switch (mode) {
+    case 0: launch_cheb_t<0>(a, vs, alpha, beta, theta, s); break;
+    case 1: launch_cheb_t<1>(a, vs, alpha, beta, theta, s); break;
+    case 2: launch_cheb_t<2>(a, vs, alpha, beta, theta, s); break;
+    default: launch_cheb_t<3>(a, vs, alpha, beta, theta, s); break;
+  }
+  return 1;
+}
+int launch_dot(const VecArgs& a, int vs, cudaStream_t s) {
+  if (a.n <= 0) return 0;
+  int nb = blocks_rb(a.n);
+  switch (vs) {
+    case NONE: launch_k(k_dot<NONE>, nb, 256, 0, s, a); break;
+    case SED: launch_k(k_dot<SED>, nb, 256, 0, s, a); break;
+    case SECDED64: launch_k(k_dot<SECDED64>, nb, 256, 0, s, a); break;
+    case SECDED128: launch_k(k_dot<SECDED128>, nb, 256, 0, s, a); break;
+    default: launch_k(k_dot<CRC32C>, nb, 256, vec_dyn_smem<CRC32C>(), s, a); break;
+  }
+  return 1;
+}
+int launch_copy_running(uint64_t* dst, const uint64_t* src, int64_t npad, const CgState* st, cudaStream_t s) {
+  if (npad <= 0) return 0;
+  launch_k(k_copy_running, grid_for(npad, 256), 256, 0, s, dst, src, npad, st);
   return 1;
 }
 int launch_init_r(const VecArgs& a, int vs, cudaStream_t s) {

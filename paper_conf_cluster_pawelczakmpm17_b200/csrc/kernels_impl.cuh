@@ -1526,7 +1526,7 @@ static __global__ void k_post_p(CgState* st, const int* due) {
   if (st->stop) return;
   if (!st->dist && st->abort_policy && *((volatile const int*)due)) { st->stop = 1; st->status = ABFT_E_DUE; }
   else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
-  st->rro = st->rrn;
+  if (!st->pcg) st->rro = st->rrn;
 }
 
 // Single-reduction CG update (S§8(f) f3): p = enc(fma(beta,
@@ -1575,8 +1575,11 @@ __global__ void __launch_bounds__(256) k_calc_sr(VecArgs a) {
 // Chebyshev update (TeaLeaf tea_leaf_cheby, reading R32):
 // r = enc(b - w); p = enc(r'/theta) (INIT) or enc(fma(alpha, p', beta r'));
 // u = enc(u' + p'); RED-1 partials of r'.r'.  Checks b, w, (p), u; VecArgs.x is u.
-template <int VS, bool INIT>
-__global__ void __launch_bounds__(256) k_cheb(VecArgs a) {
+// MODE 0 / 1: step / first step with the state's coefficients (abft_cheby_solve);
+// MODE 2 / 3: step / first step from u = 0 with the given coefficients (PPCG).
+template <int VS, int MODE>
+__global__ void __launch_bounds__(256) k_cheb(VecArgs a, double c_alpha, double c_beta, double c_theta) {
+  constexpr bool INIT = (MODE == 1 || MODE == 3), ZERO = (MODE == 3);
   __shared__ __align__(16) uint8_t s_lut[128];
   extern __shared__ __align__(16) uint8_t s_dyn_v[];
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -1584,11 +1587,12 @@ __global__ void __launch_bounds__(256) k_cheb(VecArgs a) {
   pdl_wait();
   pdl_trigger();
   const int stop = a.state->stop;
-  const double alpha = a.state->alpha, beta = a.state->beta, theta = a.state->ch_theta;
+  const double alpha = MODE >= 2 ? c_alpha : a.state->alpha, beta = MODE >= 2 ? c_beta : a.state->beta;
+  const double theta = MODE >= 2 ? c_theta : a.state->ch_theta;
   const uint8_t* cs = vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
   (void)cs;
   __syncthreads();
-  if ((!INIT && stop) || rb * 256 >= a.n) return;
+  if (stop || rb * 256 >= a.n) return;
   const uint64_t keep = vkeep(VS);
   double dot = 0.0;
   for (int k = 0; k < 8; k++) {
@@ -1598,22 +1602,60 @@ __global__ void __launch_bounds__(256) k_cheb(VecArgs a) {
     const bool valid = i < a.n;
     const int64_t lim = a.npad;
     const uint64_t bw = v_load_check<VS>(a.b, i, lim, lane, true, a.counts, a.due);
-    const uint64_t ww = v_load_check<VS>(a.w, i, lim, lane, true, a.counts, a.due);
+    const uint64_t ww = ZERO ? 0ull : v_load_check<VS>(a.w, i, lim, lane, true, a.counts, a.due);
     const uint64_t pw = INIT ? 0ull : v_load_check<VS>(a.p, i, lim, lane, true, a.counts, a.due);
-    const uint64_t uw = v_load_check<VS>(a.x, i, lim, lane, true, a.counts, a.due);
-    const uint64_t rr = valid ? round_k(as_u(__dsub_rn(as_d(bw & keep), as_d(ww & keep))), vk(VS)) : 0ull;
+    const uint64_t uw = ZERO ? 0ull : v_load_check<VS>(a.x, i, lim, lane, true, a.counts, a.due);
+    const uint64_t rr = !valid ? 0ull
+                        : ZERO ? round_k(bw & keep, vk(VS))
+                               : round_k(as_u(__dsub_rn(as_d(bw & keep), as_d(ww & keep))), vk(VS));
     const uint64_t re = v_encode<VS>(rr, lane, s_lut);
     const double rm = as_d(re & keep);
     const double pn = INIT ? rm / theta : fma(alpha, as_d(pw & keep), __dmul_rn(beta, rm));
     const uint64_t pe = v_encode<VS>(valid ? round_k(as_u(pn), vk(VS)) : 0ull, lane, s_lut);
-    const uint64_t ue =
-        v_encode<VS>(valid ? round_k(as_u(__dadd_rn(as_d(uw & keep), as_d(pe & keep))), vk(VS)) : 0ull, lane, s_lut);
+    const double un = ZERO ? as_d(pe & keep) : __dadd_rn(as_d(uw & keep), as_d(pe & keep));
+    const uint64_t ue = v_encode<VS>(valid ? round_k(as_u(un), vk(VS)) : 0ull, lane, s_lut);
     if (i < a.npad) { a.r[i] = re; a.p[i] = pe; a.x[i] = ue; }
     if (valid) dot = fma(rm, rm, dot);
   }
 #pragma unroll
   for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
   if (lane == 0) a.partials[rb] = dot;
+}
+
+// Checked dot a.r . a.x over the masked stored values (PPCG's r.z; RED-1
+// partials); both operands checked as their owner (O9).
+template <int VS>
+__global__ void __launch_bounds__(256) k_dot(VecArgs a) {
+  __shared__ __align__(16) uint8_t s_lut[128];
+  extern __shared__ __align__(16) uint8_t s_dyn_v[];
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int64_t rb = (int64_t)blockIdx.x * 8 + warp;
+  pdl_wait();
+  pdl_trigger();
+  const int stop = a.state->stop;
+  (void)vec_codec_smem<VS>(s_lut, s_dyn_v, a.crc);
+  __syncthreads();
+  if (stop || rb * 256 >= a.n) return;
+  const uint64_t keep = vkeep(VS);
+  double dot = 0.0;
+  for (int k = 0; k < 8; k++) {
+    const int64_t pb = rb * 256 + k * 32;
+    if (pb >= a.n) break;
+    const int64_t i = pb + lane;
+    const uint64_t rw = v_load_check<VS>(a.r, i, a.npad, lane, true, a.counts, a.due);
+    const uint64_t zw = v_load_check<VS>(a.x, i, a.npad, lane, true, a.counts, a.due);
+    if (i < a.n) dot = fma(as_d(rw & keep), as_d(zw & keep), dot);
+  }
+#pragma unroll
+  for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
+  if (lane == 0) a.partials[rb] = dot;
+}
+static __global__ void k_copy_running(uint64_t* dst, const uint64_t* src, int64_t npad, const CgState* st) {
+  pdl_wait();
+  pdl_trigger();
+  if (st->stop) return;
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < npad; i += (int64_t)gridDim.x * blockDim.x)
+    dst[i] = src[i];
 }
 
 // init (a2): r = enc(round(b - w)), p = r, rr0 partials
@@ -1689,6 +1731,12 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
     else if (conv) { st->stop = 1; st->status = ABFT_OK; st->converged = 1; }
     else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
     else cheb_next(st);
+    return;
+  }
+  if (op == 12) { st->rro = res; return; }   // PPCG init: rz = r.z
+  if (op == 11) {                             // PPCG: beta = rz'/rz, rz = rz'
+    st->beta = res / st->rro;
+    st->rro = res;
     return;
   }
   if (op == 1) {  // rr0
