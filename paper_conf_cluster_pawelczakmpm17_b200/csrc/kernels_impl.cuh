@@ -632,10 +632,17 @@ constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
 constexpr int TILE_OFF_BAR = TILE_OFF_RP + TILE_TY * TILE_RP * 4;
 constexpr int TILE_OFF_CRC = TILE_OFF_BAR + 64;                // CRC32C tables (only for CRC schemes)
 constexpr int TILE_SMEM = TILE_OFF_CRC + 128;                   // + alignment slack
+// ABFT_CRC_SLICE_SMEM = 0: the tiled SpMV reads the 4 KB slicing tables of
+// E-CRC / R-CRC through L1 instead of staging them in SMEM (keeps 3 CTAs per
+// SM for CRC32C matrices)
+#ifndef ABFT_CRC_SLICE_SMEM
+#define ABFT_CRC_SLICE_SMEM 1
+#endif
 // dynamic SMEM of one tile kernel: + slicing tables (E-CRC / R-CRC), + V-CRC position tables
 template <int ES, int RS, int VS>
 constexpr int tile_smem() {
-  return TILE_SMEM + ((ES == CRC32C || RS == CRC32C) ? 4 * CRC_SLICE_WORDS : 0) + (VS == CRC32C ? 4 * CRC_VPOS_WORDS : 0);
+  return TILE_SMEM + ((ABFT_CRC_SLICE_SMEM && (ES == CRC32C || RS == CRC32C)) ? 4 * CRC_SLICE_WORDS : 0) +
+         (VS == CRC32C ? 4 * CRC_VPOS_WORDS : 0);
 }
 
 static __device__ __forceinline__ uint32_t smem_u32(const void* p) { return (uint32_t)__cvta_generic_to_shared(p); }
@@ -832,8 +839,8 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   uint64_t* winbar = empty + TILE_NST;   // the TMA-staged `in` window
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   uint32_t* srp = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_RP) + warp * TILE_RP;
-  constexpr bool SLICE = (ES == CRC32C || RS == CRC32C);
-  uint32_t* s_slice = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_CRC);
+  constexpr bool SLICE = ABFT_CRC_SLICE_SMEM && (ES == CRC32C || RS == CRC32C);
+  const uint32_t* s_slice = SLICE ? reinterpret_cast<const uint32_t*>(s_dyn + TILE_OFF_CRC) : &a.crc->slice[0][0];
   uint8_t* s_vpos = s_dyn + TILE_OFF_CRC + (SLICE ? 4 * CRC_SLICE_WORDS : 0);
   const int64_t n = a.stencil_n;
   const int64_t ny = a.nrows / n;
@@ -854,7 +861,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
     for (int k = 0; k < TILE_NST; k++) tile_produce(tm, s_dyn + k * TILE_STAGE, &full[k], tx0, ty0, k);
   }
   if (VS == SECDED64) load_lut(s_lut);
-  if (SLICE) smem_fill(s_slice, &a.crc->slice[0][0], CRC_SLICE_WORDS);
+  if (SLICE) smem_fill(const_cast<uint32_t*>(s_slice), &a.crc->slice[0][0], CRC_SLICE_WORDS);
   if (VS == CRC32C) smem_fill(reinterpret_cast<uint32_t*>(s_vpos), &a.crc->vpos[0][0][0], CRC_VPOS_WORDS);
   const uint8_t* cs = (VS == CRC32C) ? s_vpos : s_lut;   // vector codec tables
   const int64_t gy = ty0 + warp;

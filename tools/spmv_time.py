@@ -28,8 +28,10 @@ def main():
     P = bench.build_problem(a.grid, a.grid, 0, 1, torch.device("cuda", 0))
     ctx = abft.Context(0)
     out = {"so": os.environ.get("ABFT_SO", "default")}
-    for s in [int(t) for t in a.schemes.split(",")]:
-        sol = bench.Solver(abft, ctx, P, s, s, s)
+    for spec in a.schemes.split(","):
+        # "s" = all structures with scheme s; "e/r/v" = element / rowptr / vector schemes
+        es, rs, s = (int(t) for t in spec.split("/")) if "/" in spec else (int(spec),) * 3
+        sol = bench.Solver(abft, ctx, P, es, rs, s)
         sol.step(0.0, 1)
         b, x, r, p, w = sol.vecs
         cnt = sol.counts
@@ -66,7 +68,7 @@ def main():
         torch.cuda.synchronize()
         res["cg_step_ms_200it"] = e0.elapsed_time(e1)
         res["counts"] = int(cnt.read().sum())
-        out[f"scheme{s}"] = res
+        out[f"scheme{spec}" if "/" in spec else f"scheme{s}"] = res
         del sol
     print(json.dumps(out))
 
