@@ -58,7 +58,6 @@ struct abft_ctx {
   double prof_ms[4] = {0, 0, 0, 0};
   int64_t prof_n[4] = {0, 0, 0, 0};
   std::vector<cudaEvent_t> events;
-  RedState* red = nullptr;   // fused-reduction counters/roots (zero between reductions)
   CrcTables* crc = nullptr;  // CRC32C lookup tables (device)
   bool fuse_p = false;       // fused calc_p in the CG's SpMV when eligible (opt-in)
   bool pdl = false;          // programmatic dependent launch between the CG iteration kernels (opt-in, §6.2)
@@ -110,7 +109,7 @@ int check_chunks(const abft_csr* A, int nchunks) {
 // probe = true only builds the arguments and reports whether every chunk can
 // take the fused tiled kernel (nothing is launched).
 int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, int dot,
-                DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total, RedArgs red = RedArgs{},
+                DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total,
                 int check_mode = MODE_CORRECT, int check_interval = 0, uint64_t* p_cur = nullptr,
                 uint64_t* r_f = nullptr, bool probe = false, int part = 0) {
   const int64_t base0 = A[0].row_base;
@@ -157,8 +156,6 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.counts = cnt;
     a.due = ctx->due;
     a.state = st;
-    a.red = red;
-    if (a.red.rs) a.red.nrb = nrb_all;
     a.check_mode = check_mode;
     a.check_interval = check_interval;
     a.crc = ctx->crc;
@@ -222,8 +219,6 @@ int abft_ctx_create(int device, abft_ctx** out) {
   CUDA_TRY(cudaMalloc(&c->due, sizeof(int) * 4));
   CUDA_TRY(cudaMemset(c->due, 0, sizeof(int) * 4));
   CUDA_TRY(cudaMalloc(&c->flags, sizeof(uint32_t) * 4));
-  CUDA_TRY(cudaMalloc(&c->red, sizeof(RedState)));
-  CUDA_TRY(cudaMemset(c->red, 0, sizeof(RedState)));
   CUDA_TRY(cudaMallocHost(&c->h_state, sizeof(CgState)));
   CUDA_TRY(cudaMallocHost(&c->h_flags, sizeof(uint32_t) * 4));
   {
@@ -271,7 +266,6 @@ int abft_ctx_destroy(abft_ctx* c) {
   cudaFree(c->p_alt);
   cudaFree(c->faults);
   cudaFree(c->cg_log);
-  cudaFree(c->red);
   cudaFree(c->crc);
   cudaFreeHost(c->h_state);
   cudaFreeHost(c->h_flags);
@@ -342,7 +336,7 @@ int abft_spmv_ex(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, ab
   cudaStream_t s = (cudaStream_t)stream;
   int64_t nrb = 0;
   e = spmv_chunks(ctx, A, nchunks, in, out, dot_out != nullptr, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb,
-                  RedArgs{}, check_mode);
+                  check_mode);
   if (e) return e;
   if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
   CUDA_TRY(cudaGetLastError());
@@ -683,8 +677,8 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   abft_vec* const r = R[0].r();
   if (fused) {
     abft_vec ptmp = *p;
-    fused = spmv_chunks(ctx, R[0].A, R[0].nchunks, &ptmp, R[0].w(), true, R[0].cnt, nullptr, s, nullptr, RedArgs{},
-                        MODE_CORRECT, 0, reinterpret_cast<uint64_t*>(p->data), reinterpret_cast<uint64_t*>(r->data),
+    fused = spmv_chunks(ctx, R[0].A, R[0].nchunks, &ptmp, R[0].w(), true, R[0].cnt, nullptr, s, nullptr, MODE_CORRECT,
+                        0, reinterpret_cast<uint64_t*>(p->data), reinterpret_cast<uint64_t*>(r->data),
                         true) == ABFT_OK;
   }
   if (fused && ctx->p_alt_len < npad_ext) {
@@ -699,7 +693,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   bool overlap = multi && d->nranks > 1 && n_halo > 0;
   for (int q = 0; q < nl && overlap; q++)
     overlap = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].p(), R[q].w(), true, R[q].cnt, nullptr, s, nullptr,
-                          RedArgs{}, MODE_CORRECT, 0, nullptr, nullptr, true) == ABFT_OK;
+                          MODE_CORRECT, 0, nullptr, nullptr, true) == ABFT_OK;
   (void)cudaGetLastError();
 
   CgState h{};
@@ -731,7 +725,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   prof.begin(0);
   for (int q = 0; q < nl; q++) {
     e = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].x(), R[q].w(), false, R[q].cnt, nullptr, s, nullptr,
-                    RedArgs{}, MODE_CORRECT, interval);
+                    MODE_CORRECT, interval);
     if (e) return e;
   }
   prof.end();
@@ -793,13 +787,13 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
       abft_vec pprev = *p;
       pprev.data = reinterpret_cast<double*>(P[kk & 1]);
       return spmv_chunks(ctx, R[0].A, R[0].nchunks, &pprev, R[0].w(), true, R[0].cnt, ctx->state, ss, nullptr,
-                         RedArgs{}, MODE_CORRECT, interval, P[(kk - 1) & 1], reinterpret_cast<uint64_t*>(r->data));
+                         MODE_CORRECT, interval, P[(kk - 1) & 1], reinterpret_cast<uint64_t*>(r->data));
     }
     if (!overlap) {
       if ((e2 = halo_exchange(d, R, nl, vi, n_halo, ss))) return e2;
       for (int q = 0; q < nl; q++)
         if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].v[vi], R[q].w(), dots, R[q].cnt, R[q].ctx->state,
-                              ss, nullptr, RedArgs{}, MODE_CORRECT, interval)))
+                              ss, nullptr, MODE_CORRECT, interval)))
           return e2;
       return ABFT_OK;
     }
@@ -812,7 +806,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
       if (part == 2) CUDA_TRY(cudaStreamWaitEvent(ss, d->ev_join, 0));
       for (int q = 0; q < nl; q++)
         if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].v[vi], R[q].w(), dots, R[q].cnt, R[q].ctx->state,
-                              ss, nullptr, RedArgs{}, MODE_CORRECT, interval, nullptr, nullptr, false, part)))
+                              ss, nullptr, MODE_CORRECT, interval, nullptr, nullptr, false, part)))
           return e2;
     }
     return ABFT_OK;
@@ -976,7 +970,6 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
       t.max_iters = 0x7FFFFFFF;
       count_launch(launch_set_state(t, ctx->state, s));
       VecArgs vp = R[0].va;
-      vp.red = RedArgs{};
       count_launch(launch_calc_p(vp, scheme, s));
       CUDA_TRY(cudaStreamSynchronize(s));
     }
@@ -1348,11 +1341,11 @@ int abft_calc_p_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* p_
   DevCounts* cnt = reinterpret_cast<DevCounts*>(dcnt);
   uint64_t* pc = reinterpret_cast<uint64_t*>(p_out->data);
   uint64_t* rf = reinterpret_cast<uint64_t*>(r->data);
-  if (spmv_chunks(ctx, A, nchunks, p_prev, out, true, cnt, nullptr, s, nullptr, RedArgs{}, MODE_CORRECT, 0, pc, rf,
+  if (spmv_chunks(ctx, A, nchunks, p_prev, out, true, cnt, nullptr, s, nullptr, MODE_CORRECT, 0, pc, rf,
                   true) != ABFT_OK)
     return fail(ABFT_E_SHAPE, "fused calc_p + SpMV needs the tiled stencil path for every chunk");
   int64_t nrb = 0;
-  e = spmv_chunks(ctx, A, nchunks, p_prev, out, true, cnt, ctx->state, s, &nrb, RedArgs{}, MODE_CORRECT, 0, pc, rf);
+  e = spmv_chunks(ctx, A, nchunks, p_prev, out, true, cnt, ctx->state, s, &nrb, MODE_CORRECT, 0, pc, rf);
   if (e) return e;
   if (dot_out) count_launch(launch_reduce(ctx->partials, nrb, ctx->roots, ctx->ticket, 0, nullptr, dot_out, ctx->due, s));
   CUDA_TRY(cudaGetLastError());

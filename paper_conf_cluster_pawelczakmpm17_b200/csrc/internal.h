@@ -49,25 +49,6 @@ struct CrcTables {
 };
 void build_crc_tables(CrcTables* host_out);
 
-// Fused RED-1 reduction state (ctx scratch, zero between reductions): the warp
-// that writes the last partial of a 1024-leaf group reduces the group, the
-// warp that completes the last group reduces the group roots and applies the
-// CG scalar logic (op) — no separate reduction kernel.
-struct RedState {
-  unsigned int group_ctr[1024];
-  unsigned int top_ctr;
-  unsigned int pad[3];
-  double roots[1024];
-};
-struct RedArgs {
-  RedState* rs;     // null: no fused finish (partials only)
-  int64_t nrb;      // total reduction blocks of the vector (all chunks)
-  int op;           // 0 dot -> out[0], 1 rr0, 2 pw, 3 rrn, 4 root+due -> out[0..2)
-  double* out;
-  CgState* st;
-  const int* due;
-};
-
 // arguments of one SpMV chunk launch
 struct SpmvArgs {
   int64_t nrows, ncols, nnz, row_base, col_base, n_in, npad_in, npad_out, rb_offset;
@@ -85,7 +66,6 @@ struct SpmvArgs {
   DevCounts* counts; // may be null
   int* due;          // DUE / range flag (never null)
   const CgState* state;  // may be null
-  RedArgs red;
   // matrix check mode of this access: MODE_CORRECT / DETECT /
   // RANGE; with check_interval > 1 the kernel derives it from the device
   // iteration counter instead (access k = state->iters + 1, init = 0)
@@ -113,7 +93,6 @@ struct VecArgs {
   int* due;
   CgState* state;
   double* out_masked;
-  RedArgs red;
   const CrcTables* crc;   // device tables (CRC32C schemes only)
 };
 

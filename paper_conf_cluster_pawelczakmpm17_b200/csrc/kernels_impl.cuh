@@ -206,8 +206,6 @@ static __device__ __forceinline__ int spmv_mode(const SpmvArgs& a) {
   return a.check_mode;
 }
 
-struct RedArgs;
-static __device__ void red_push(double* partials, int64_t rb, double val, const RedArgs& r, int lane);
 
 // Cold path of a single-codeword vector check (G = 1 schemes).
 template <int VS>
@@ -570,8 +568,7 @@ __global__ void __launch_bounds__(256) k_spmv(SpmvArgs a) {
   if (DOT) {
 #pragma unroll
     for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-    if (a.red.rs) red_push(a.partials, a.rb_offset + rb, dot, a.red, lane);
-    else if (lane == 0) a.partials[a.rb_offset + rb] = dot;
+    if (lane == 0) a.partials[a.rb_offset + rb] = dot;
   }
   if (DOT == 2) {
 #pragma unroll
@@ -1202,8 +1199,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   if (DOT && has_seg) {
 #pragma unroll
     for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-    if (a.red.rs) red_push(a.partials, a.rb_offset + (rowseg >> 8), dot, a.red, lane);
-    else if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
+    if (lane == 0) a.partials[a.rb_offset + (rowseg >> 8)] = dot;
   }
   if (DOT == 2 && has_seg) {
 #pragma unroll
@@ -1460,8 +1456,7 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 3 : ABFT_UR_MINB) k_calc_u
   }
 #pragma unroll
   for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-  if (a.red.rs) red_push(a.partials, rb, dot, a.red, lane);
-  else if (lane == 0) a.partials[rb] = dot;
+  if (lane == 0) a.partials[rb] = dot;
 }
 
 template <int VS>
@@ -1691,8 +1686,7 @@ __global__ void __launch_bounds__(256) k_init_r(VecArgs a) {
   }
 #pragma unroll
   for (int off = 16; off >= 1; off >>= 1) dot = dot + __shfl_xor_sync(0xffffffffu, dot, off);
-  if (a.red.rs) red_push(a.partials, rb, dot, a.red, lane);
-  else if (lane == 0) a.partials[rb] = dot;
+  if (lane == 0) a.partials[rb] = dot;
 }
 
 // ============================================================ reduction (a6)
@@ -1774,13 +1768,6 @@ static __device__ void apply_op(int op, double res, CgState* st, bool dueflag) {
   }
 }
 
-// ---- fused RED-1 finish: called by a whole warp after it
-// produced the partial of reduction block rb.
-static __device__ __forceinline__ int64_t p2ceil(int64_t v) {
-  int64_t p = 1;
-  while (p < v) p <<= 1;
-  return p;
-}
 // Pairwise tree of m = 2^j values held by lanes 0..m-1 (m <= 32): butterfly
 // over offsets 1..m/2 combines adjacent subtrees first; lane 0 gets the root.
 static __device__ __forceinline__ double warp_tree(double v, int m) {
@@ -1803,42 +1790,6 @@ static __device__ double warp_subtree(const double* src, int64_t L, int64_t vali
     for (int i = 0; i < m / 2; i++) t[i] = t[2 * i] + t[2 * i + 1];
   return warp_tree(t[0], 32);
 }
-static __device__ void red_push(double* partials, int64_t rb, double val, const RedArgs& r, int lane) {
-  const int64_t P2 = p2ceil(r.nrb);
-  const int64_t L = P2 < 1024 ? P2 : 1024;
-  const int64_t g = rb / L;
-  const int64_t ngr = (r.nrb + L - 1) / L;   // groups holding real partials
-  unsigned last = 0;
-  if (lane == 0) {
-    partials[rb] = val;
-    __threadfence();
-    const int64_t expect = (r.nrb - g * L) < L ? (r.nrb - g * L) : L;
-    last = (atomicAdd(&r.rs->group_ctr[g], 1u) == (unsigned)expect - 1u);
-  }
-  last = __shfl_sync(0xffffffffu, last, 0);
-  if (!last) return;
-  __threadfence();
-  const double root = warp_subtree(partials + g * L, L, r.nrb - g * L, lane);
-  unsigned top = 0;
-  if (lane == 0) {
-    r.rs->group_ctr[g] = 0;
-    r.rs->roots[g] = root;
-    __threadfence();
-    top = (atomicAdd(&r.rs->top_ctr, 1u) == (unsigned)ngr - 1u);
-  }
-  top = __shfl_sync(0xffffffffu, top, 0);
-  if (!top) return;
-  __threadfence();
-  const int64_t ng = P2 / L;
-  const double res = warp_subtree(r.rs->roots, ng, ngr, lane);
-  if (lane != 0) return;
-  r.rs->top_ctr = 0;
-  const int dueflag = *((volatile const int*)r.due);
-  if (r.op == 0) r.out[0] = res;
-  else if (r.op == 4) { r.out[0] = res; r.out[1] = (double)dueflag; }
-  else apply_op(r.op, res, r.st, dueflag != 0);
-}
-
 // Single-reduction CG scalar logic: g = r.r, d = w.r of the
 // SpMV w = A r.  op 7: init (rr0); op 6: end of an iteration.
 static __device__ void apply_op_sr(int op, double g, double d, CgState* st, bool dueflag) {
