@@ -888,8 +888,21 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
       }
     }
   }
+  // the fast check of the loaded groups is pure arithmetic on matrix data: done
+  // before the grid dependency resolves (overlapping the previous kernel's
+  // tail under PDL); R-CRC needs the SMEM tables, so it waits for the barrier
+  constexpr bool EARLY_RP = (RS != CRC32C);
+  uint32_t rp_fast = 0;
+  if (EARLY_RP && has_seg) {
+#pragma unroll
+    for (int q = 0; q < PER; q++)
+      if (RS != NONE && lane + 32 * q < NG) rp_fast |= rp_acc<RS>(e[q]);
+  }
   pdl_wait();   // the previous kernel's writes (p / r, CG state, counters) are visible from here
   pdl_trigger();
+  // the CG state's stop flag: loaded first, its latency overlapping the
+  // window TMA issue and the CTA barrier below
+  const int stop_v = a.state ? *(volatile const int*)&a.state->stop : 0;
   // fused calc_p: iteration 1 multiplies by p_cur as init
   // wrote it; later iterations build p_cur from (in = p_{k-1}, r) in the window
   const bool fz = FUSED && a.state->iters > 0;
@@ -914,15 +927,18 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   // every warp waits on winbar / the stage barriers below: thread 0's
   // mbarrier.init (and the SMEM tables) must be visible to the whole CTA first
   __syncthreads();
-  const int stop_v = a.state ? a.state->stop : 0;
   const int mode = spmv_mode(a);
   if (has_seg) {
     if (!stop_v) {
       uint32_t acc = 0;
       if (mode != MODE_RANGE) {
+        if (EARLY_RP) {
+          acc = rp_fast;
+        } else {
 #pragma unroll
-        for (int q = 0; q < PER; q++)
-          if (RS != NONE && lane + 32 * q < NG) acc |= (RS == CRC32C) ? rcrc_acc_tab(e[q], s_slice) : rp_acc<RS>(e[q]);
+          for (int q = 0; q < PER; q++)
+            if (RS != NONE && lane + 32 * q < NG) acc |= rcrc_acc_tab(e[q], s_slice);
+        }
       }
       if (RS != NONE && (acc & 1u)) {  // cold: locate, correct, count (owner), per group
 #pragma unroll
