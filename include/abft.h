@@ -131,6 +131,14 @@ typedef enum {
 int abft_spmv_ex(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, double* dot_out,
                  abft_counts* dcnt, int32_t check_mode, void* stream);
 
+/* a3 alone, for timing the dominant kernel: the CG iteration's SpMV kernel
+ * instantiation (the p.w partial of every reduction block written to the
+ * context's scratch) with NO dot reduction launched after it.
+ * Same arguments, checks and counters as abft_spmv; the partials are not
+ * returned.  bench.py times back-to-back launches of it (roofline). */
+int abft_spmv_partials(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out,
+                       abft_counts* dcnt, void* stream);
+
 typedef struct {
   double tol;          /* stop when sqrt(r.r) <= tol*sqrt(r0.r0) (R15) */
   int32_t max_iters;

@@ -67,6 +67,7 @@ _sig = {
     "abft_vec_decode": (C.c_int, [_P, C.POINTER(Vec), _P, _P, _P]),
     "abft_spmv": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), _P, _P, _P]),
     "abft_spmv_ex": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), _P, _P, C.c_int32, _P]),
+    "abft_spmv_partials": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), _P, _P]),
     "abft_cg_solve": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                 C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
     "abft_cg_solve_sr": (C.c_int, [_P, C.POINTER(CSR), C.c_int, C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
@@ -324,6 +325,14 @@ def spmv(ctx: Context, A, x: Vector, y: Vector, counts: Counters | None = None, 
     vx, vy = x.cstruct(), y.cstruct()
     _check(_lib.abft_spmv_ex(ctx.h, arr, n, C.byref(vx), C.byref(vy), dot.data_ptr() if dot is not None else None,
                              counts.ptr if counts else None, int(mode), _stream(stream)), "abft_spmv_ex")
+
+
+def spmv_partials(ctx: Context, A, x: Vector, y: Vector, counts: Counters | None = None, stream=None):
+    """abft_spmv_partials: the CG SpMV kernel alone (p.w partials in ctx scratch, no reduction) — for timing."""
+    arr, n = _chunks(A)
+    vx, vy = x.cstruct(), y.cstruct()
+    _check(_lib.abft_spmv_partials(ctx.h, arr, n, C.byref(vx), C.byref(vy), counts.ptr if counts else None,
+                                   _stream(stream)), "abft_spmv_partials")
 
 
 def cg_solve(ctx: Context, A, b: Vector, x: Vector, r: Vector, p: Vector, w: Vector, tol=1e-10, max_iters=10000,

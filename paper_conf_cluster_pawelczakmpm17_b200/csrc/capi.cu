@@ -343,6 +343,23 @@ int abft_spmv_ex(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, ab
   return ABFT_OK;
 }
 
+int abft_spmv_partials(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, abft_counts* dcnt,
+                       void* stream) {
+  if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
+  int e = check_chunks(A, nchunks);
+  if (e) return e;
+  if ((e = check_vec(in, "in")) || (e = check_vec(out, "out"))) return e;
+  if (in->data == out->data) return fail(ABFT_E_INVALID, "in and out alias");
+  if (in->scheme != out->scheme) return fail(ABFT_E_INVALID, "in/out schemes differ");
+  cudaStream_t s = (cudaStream_t)stream;
+  int64_t nrb = 0;
+  e = spmv_chunks(ctx, A, nchunks, in, out, true, reinterpret_cast<DevCounts*>(dcnt), nullptr, s, &nrb,
+                  ABFT_CHECK_CORRECT);
+  if (e) return e;
+  CUDA_TRY(cudaGetLastError());
+  return ABFT_OK;
+}
+
 int abft_profile(abft_ctx* ctx, int enable) {
   if (!ctx) return fail(ABFT_E_INVALID, "null ctx");
   ctx->profile = enable;

@@ -208,10 +208,45 @@ int launch_vec_check(uint64_t* d, int64_t n, int64_t npad, int vs, double* out, 
   }
   return 1;
 }
+// Cluster reduction (k_reduce_cl) when the padded leaf count allows it
+// (ABFT_RED_CL = 0 or p2 > RED_CL_MAX: the multi-block ticket form k_reduce).
+#ifndef ABFT_RED_CL
+#define ABFT_RED_CL 1
+#endif
+template <bool TWO>
+static bool launch_reduce_cl(const double* partials, const double* partials2, int64_t nrb, int64_t p2, int op,
+                             CgState* st, double* out, const int* due, cudaStream_t s) {
+  if (!ABFT_RED_CL || p2 > RED_CL_MAX) return false;
+  const int C = p2 >= 4096 ? 8 : (p2 >= 512 ? (int)(p2 / 512) : 1);
+  const int64_t L = p2 / C;
+  const int lpt = L > 512 ? (int)(L / 512) : 1;
+  const int nt = (int)(L / lpt);
+  cudaLaunchConfig_t cfg{};
+  cfg.gridDim = dim3(C);
+  cfg.blockDim = dim3(nt < 32 ? 32 : nt);
+  cfg.dynamicSmemBytes = 0;
+  cfg.stream = s;
+  cudaLaunchAttribute at[2];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = C;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  int na = 1;
+  if (g_pdl) {
+    at[1].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[1].val.programmaticStreamSerializationAllowed = 1;
+    na = 2;
+  }
+  cfg.attrs = at;
+  cfg.numAttrs = na;
+  return cudaLaunchKernelEx(&cfg, k_reduce_cl<TWO>, partials, nrb, nt, lpt, op, st, out, due, partials2) ==
+         cudaSuccess;
+}
 int launch_reduce(const double* partials, int64_t nrb, double* roots, uint32_t* ticket, int op, CgState* st,
                   double* out, const int* due, cudaStream_t s) {
   int64_t p2 = 1;
   while (p2 < nrb) p2 <<= 1;
+  if (launch_reduce_cl<false>(partials, nullptr, nrb, p2, op, st, out, due, s)) return 1;
   int64_t leaves = p2 < 1024 ? p2 : 1024;
   int blocks = (int)(p2 / leaves);
   launch_k(k_reduce<false>, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, op, st, out, due,
@@ -222,6 +257,7 @@ int launch_reduce_sr(const double* partials, const double* partials2, int64_t nr
                      uint32_t* ticket, int op, CgState* st, const int* due, cudaStream_t s) {
   int64_t p2 = 1;
   while (p2 < nrb) p2 <<= 1;
+  if (launch_reduce_cl<true>(partials, partials2, nrb, p2, op, st, nullptr, due, s)) return 1;
   int64_t leaves = p2 < 1024 ? p2 : 1024;
   int blocks = (int)(p2 / leaves);
   launch_k(k_reduce<true>, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, op, st, (double*)nullptr, due,
@@ -235,6 +271,7 @@ int launch_reduce_sr_root(const double* partials, const double* partials2, int64
   while (p2 < nrb) p2 <<= 1;
   int64_t leaves = p2 < 1024 ? p2 : 1024;
   int blocks = (int)(p2 / leaves);
+  if (launch_reduce_cl<true>(partials, partials2, nrb, p2, 10, nullptr, out, due, s)) return 1;
   launch_k(k_reduce<true>, blocks, 256, 0, s, partials, nrb, leaves, roots, ticket, 10, (CgState*)nullptr, out, due,
            partials2, roots2);
   return 1;
