@@ -111,7 +111,7 @@ int check_chunks(const abft_csr* A, int nchunks) {
 int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abft_vec* out, int dot,
                 DevCounts* cnt, const CgState* st, cudaStream_t s, int64_t* nrb_total,
                 int check_mode = MODE_CORRECT, int check_interval = 0, uint64_t* p_cur = nullptr,
-                uint64_t* r_f = nullptr, bool probe = false, int part = 0) {
+                uint64_t* r_f = nullptr, bool probe = false, int part = 0, bool early_in = false) {
   const int64_t base0 = A[0].row_base;
   const int64_t npad_in = vec_padded_len(in->n, in->scheme);
   const int64_t npad_out = vec_padded_len(out->n, out->scheme);
@@ -161,6 +161,7 @@ int spmv_chunks(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* in, abf
     a.crc = ctx->crc;
     a.p_cur = p_cur;
     a.r_f = r_f;
+    a.early_in = early_in ? 1 : 0;
     if (probe) {
       // probe: p_cur set -> can the fused calc_p kernel run; else -> is every chunk tileable
       if (p_cur ? !spmv_fusable(a, in->scheme) : !spmv_tileable(a, in->scheme)) return ABFT_E_SHAPE;
@@ -808,10 +809,17 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     }
     if (!overlap) {
       if ((e2 = halo_exchange(d, R, nl, vi, n_halo, ss))) return e2;
-      for (int q = 0; q < nl; q++)
+      for (int q = 0; q < nl; q++) {
+        // standard CG: p was last written by calc_p (iteration 1: init), and
+        // the kernel between it and this SpMV (k_post_p / the rr0 reduction)
+        // writes no vector, so the window TMA may precede the PDL wait — unless
+        // a fault-injection kernel sits between (PPCG's init copies p right
+        // before iteration 1)
+        const bool early = vi == 3 && !ppcg && (!pdl_on || R[q].ctx->nfaults == 0);
         if ((e2 = spmv_chunks(R[q].ctx, R[q].A, R[q].nchunks, R[q].v[vi], R[q].w(), dots, R[q].cnt, R[q].ctx->state,
-                              ss, nullptr, MODE_CORRECT, interval)))
+                              ss, nullptr, MODE_CORRECT, interval, nullptr, nullptr, false, 0, early)))
           return e2;
+      }
       return ABFT_OK;
     }
     // halo on the comm stream while the interior tile rows run on ss; then the boundary rows

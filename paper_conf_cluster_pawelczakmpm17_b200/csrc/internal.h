@@ -82,6 +82,11 @@ struct SpmvArgs {
   uint64_t* r_f;
   double beta_f;
   int32_t fz;
+  // 1: no kernel between the one that last wrote `in` and this SpMV's direct
+  // predecessor writes `in` (the CG loop's SpMV of p after calc_p + k_post_p,
+  // no fault schedule), so the tiled kernel may issue its `in` window TMA
+  // before the PDL wait
+  int32_t early_in;
 };
 enum { MODE_CORRECT = 0, MODE_DETECT = 1, MODE_RANGE = 2 };
 

@@ -824,6 +824,13 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
 // decoded-window variant knob: 1 = every slot of the thread loaded and checked
 // with one OR-accumulated branch; 0 (default) = the per-slot loop with a branch
 // per codeword (measured faster on the same box: 0.2561 vs 0.2623 ms, r2k)
+#ifndef ABFT_RP_AFTER_WAIT
+#define ABFT_RP_AFTER_WAIT 1
+#endif
+// window TMA before the PDL wait when the host marks `in` final (early_in)
+#ifndef ABFT_EARLY_WIN
+#define ABFT_EARLY_WIN 1
+#endif
 #ifndef ABFT_WIN_ACC
 #define ABFT_WIN_ACC 0
 #endif
@@ -862,6 +869,10 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
 #pragma unroll
     for (int k = 0; k < TILE_NST; k++) tile_produce(tm, s_dyn + k * TILE_STAGE, &full[k], tx0, ty0, k);
+    if (ABFT_EARLY_WIN && !FUSED && a.early_in && vgrp(VS) == 1 && tm.has_vmaps) {   // `in` is final already
+      mbar_expect_tx(winbar, TILE_WIN_BYTES);
+      tma_3d(s_win, &tm.vin, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 - 1), winbar);
+    }
   }
   if (VS == SECDED64) load_lut(s_lut);
   if (SLICE) smem_fill(const_cast<uint32_t*>(s_slice), &a.crc->slice[0][0], CRC_SLICE_WORDS);
@@ -894,12 +905,15 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
       }
     }
   }
-  // the fast check of the loaded groups is pure arithmetic on matrix data: done
-  // before the grid dependency resolves (overlapping the previous kernel's
-  // tail under PDL); R-CRC needs the SMEM tables, so it waits for the barrier
+  // the fast check of the loaded groups is pure arithmetic on matrix data;
+  // R-CRC needs the SMEM tables, so it waits for the barrier.  ABFT_RP_AFTER_WAIT
+  // = 0: computed before the PDL wait (overlapping the previous kernel's tail —
+  // only the first wave of CTAs waits there); 1 (default): after the wait, once
+  // the CG state's stop flag load is in flight, so the two latencies overlap in
+  // every CTA
   constexpr bool EARLY_RP = (RS != CRC32C);
   uint32_t rp_fast = 0;
-  if (EARLY_RP && has_seg) {
+  if (EARLY_RP && !ABFT_RP_AFTER_WAIT && has_seg) {
 #pragma unroll
     for (int q = 0; q < PER; q++)
       if (RS != NONE && lane + 32 * q < NG) rp_fast |= rp_acc<RS>(e[q]);
@@ -907,8 +921,13 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   pdl_wait();   // the previous kernel's writes (p / r, CG state, counters) are visible from here
   pdl_trigger();
   // the CG state's stop flag: loaded first, its latency overlapping the
-  // window TMA issue and the CTA barrier below
+  // rowptr check, the window TMA issue and the CTA barrier below
   const int stop_v = a.state ? *(volatile const int*)&a.state->stop : 0;
+  if (EARLY_RP && ABFT_RP_AFTER_WAIT && has_seg) {
+#pragma unroll
+    for (int q = 0; q < PER; q++)
+      if (RS != NONE && lane + 32 * q < NG) rp_fast |= rp_acc<RS>(e[q]);
+  }
   // fused calc_p: iteration 1 multiplies by p_cur as init
   // wrote it; later iterations build p_cur from (in = p_{k-1}, r) in the window
   const bool fz = FUSED && a.state->iters > 0;
@@ -918,7 +937,8 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   // place.  Unfused, it is issued right here, before the CG-state load below,
   // so the window's latency overlaps it (a stopped solve drains it).
   const bool tma_win = vgrp(VS) == 1 && !(FUSED && fz) && tm.has_vmaps;
-  if (tma_win && threadIdx.x == 0) {
+  const bool win_issued = ABFT_EARLY_WIN && !FUSED && a.early_in;
+  if (tma_win && !win_issued && threadIdx.x == 0) {
     mbar_expect_tx(winbar, TILE_WIN_BYTES);
     tma_3d(s_win, (FUSED && !fz) ? &tm.vcur : &tm.vin, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 - 1), winbar);
   }
@@ -1189,8 +1209,10 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   uint64_t acc_prev = 0;   // SECDED128: rounded result of the even pass awaiting its pair
   double p_prev = 0.0;
   const uint32_t seg_e = (uint32_t)(5 * rowseg);   // assumed element start of the segment
+// pass-loop unroll: 8 (full) measured 0.2525 vs 0.2573 ms (r2l, same box):
+// the stage index / phase / address arithmetic of every pass folds away
 #ifndef ABFT_TILE_UNROLL
-#define ABFT_TILE_UNROLL 1
+#define ABFT_TILE_UNROLL 8
 #endif
   constexpr int kPassUnroll = ABFT_TILE_UNROLL;
 #pragma unroll kPassUnroll
@@ -1232,7 +1254,8 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
                                             : v_encode<VS>(rounded, lane, s_lut);
         a.out[own] = enc;
         if (FUSED && fz) a.p_cur[own] = v_encode<VS>(as_u(p_own), lane, s_lut);   // enc(p_k), own cell
-        if (DOT) dot = fma(p_own, as_d(enc & vkeep(VS)), dot);
+        // enc & vkeep == rounded: the encoders only fill the k bits round_k cleared
+        if (DOT) dot = fma(p_own, as_d(rounded), dot);
         if (DOT == 2) dot2 = fma(p_own, p_own, dot2);
       }
     }
@@ -1417,7 +1440,18 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
                                        uint64_t r0, uint64_t r1, uint64_t p0, uint64_t p1) {
   uint64_t* P = a.p + base + lane;
   uint64_t* R = a.r + base + lane;
-#if ABFT_P_PREFETCH
+#if ABFT_P_PREFETCH == 2
+  // every word of the RB in flight at once (16 loads per lane), then the steps
+  uint64_t rr[8], pp[8];
+  rr[0] = r0; rr[1] = r1; pp[0] = p0; pp[1] = p1;
+#pragma unroll
+  for (int j = 1; j < 4; j++) {
+    rr[2 * j] = ldg64(R + 64 * j); rr[2 * j + 1] = ldg64(R + 64 * j + 32);
+    pp[2 * j] = ldg64(P + 64 * j); pp[2 * j + 1] = ldg64(P + 64 * j + 32);
+  }
+#pragma unroll
+  for (int j = 0; j < 4; j++) p_step<VS>(a, P, R, 64 * j, rr[2 * j], rr[2 * j + 1], pp[2 * j], pp[2 * j + 1], beta, lane, cs);
+#elif ABFT_P_PREFETCH
   // Register double buffer: step k+64's four words are in flight while step k
   // decodes / encodes (the codec ALU otherwise serialises with the next loads).
 #if ABFT_P_UNROLL

@@ -88,7 +88,11 @@ static bool spmv_tile_launch(const SpmvArgs& a, cudaStream_t s) {
   const int64_t lo = a.ty_lo, hi = a.ty_hi > 0 ? a.ty_hi : nty;
   const int64_t blocks = (a.stencil_n / 256) * (hi - lo);
   if (blocks <= 0) return true;
-  launch_k(k_spmv_tile<ES, RS, VS, DOT, FUSED>, (unsigned)blocks, 256, smem, s, a, tm);
+  // a launch without PDL starts after every earlier kernel of the stream has
+  // finished, so its `in` window may always be fetched before the (no-op) wait
+  SpmvArgs b = a;
+  if (!g_pdl) b.early_in = 1;
+  launch_k(k_spmv_tile<ES, RS, VS, DOT, FUSED>, (unsigned)blocks, 256, smem, s, b, tm);
   return true;
 }
 // Returns false only when a fused-calc_p launch (a.p_cur set) was requested

@@ -15,5 +15,5 @@ T = os.environ.get("T", "r2k")
 for l in open(f"gpurun_out/ab_{T}.jsonl"):
     try: d = json.loads(l)
     except Exception: print(l[:200]); continue
-    print(d["so"].split("/")[-1], {k: (round(v["spmv_ms"], 4), round(v["calc_ur_ms"], 4), round(v["calc_p_ms"], 4), round(v["cg_step_ms_200it"] / 200, 4)) for k, v in d.items() if k != "so"})
+    print(d["so"].split("/")[-1], {k: (round(v["spmv_ms"], 4), round(v.get("spmv_partials_ms", 0), 4), round(v["calc_ur_ms"], 4), round(v["calc_p_ms"], 4), round(v["cg_step_ms_200it"] / 200, 4)) for k, v in d.items() if k != "so"})
 PY

@@ -35,6 +35,7 @@ def main():
     ap.add_argument("--out", default=os.path.join(ROOT, "gpurun_out", "sweep.json"))
     ap.add_argument("--intervals", default="", help="comma-separated check intervals (matrix-only configs)")
     ap.add_argument("--no-schemes", action="store_true", help="skip the per-scheme sweep")
+    ap.add_argument("--only", default="SED,SECDED64,CRC32C", help="schemes of the interval sweep")
     a = ap.parse_args()
     import torch
     import bench
@@ -52,7 +53,7 @@ def main():
             configs.append(("rowptr", s, ("NONE", s, "NONE"), 1))
             configs.append(("vectors", s, ("NONE", "NONE", s), 1))
     for N in [int(t) for t in a.intervals.split(",") if t]:
-        for s in ("SED", "SECDED64", "CRC32C"):
+        for s in a.only.split(","):
             configs.append(("matrix", s, (s, s, "NONE"), N))
     rows = []
     base = None
