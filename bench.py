@@ -245,27 +245,6 @@ def timed(solver, steps, warmup, tol, max_iters, dist_on, host=None, out_host=No
     return dict(ms=ms, iters=iters, launches=launches, prof=prof, statuses=statuses)
 
 
-def spmv_burst(solver, reps=100):
-    """Steady-state duration of the dominant kernel on the solve's own final
-    operands: `reps` back-to-back launches of the CG SpMV (+ p.w partials, no
-    reduction) between ONE pair of CUDA events on the launch stream, plain
-    launches (no PDL overlap between them).  Returns ms per launch."""
-    import torch
-    abft = solver.abft
-    b, x, r, p, w = solver.vecs[:5]
-    fn = lambda: abft.spmv_partials(solver.ctx, solver.A, p, w, solver.counts)  # noqa: E731
-    for _ in range(3):
-        fn()
-    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    torch.cuda.synchronize()
-    e0.record()
-    for _ in range(reps):
-        fn()
-    e1.record()
-    torch.cuda.synchronize()
-    return e0.elapsed_time(e1) / reps
-
-
 def read_traffic():
     """dram bytes per SpMV launch from the committed ncu --set full summary (or None)."""
     p = os.path.join(ROOT, "profiles", "spmv_traffic.json")
@@ -430,10 +409,6 @@ def main():
         # roofline pass: same workload, every SpMV launch bracketed by CUDA events on
         # the launch stream (event-timed solves launch kernels directly, no graph)
         r_ps = timed(prot, args.steps, 0, args.tol, args.max_iters, dist_on, profile=1)
-        # and back to back on the final operands (one event pair, no per-launch events)
-        ctx.set_pdl(False)
-        burst_ms = spmv_burst(prot) if not fused else None
-        ctx.set_pdl(not args.no_pdl)
     clocks = clk.summary()
     # per-kernel breakdown: one extra, untimed, fully profiled step
     r_pk = timed(prot, 1, 0, args.tol, args.max_iters, dist_on, profile=15)
@@ -541,9 +516,7 @@ def main():
                      "frac": (spmv_gbs / peak) if spmv_gbs else None,
                      "traffic": traffic.get("bytes_per_launch") if traffic_matches(traffic, args.grid, world, fused) else None,
                      "bytes_per_launch_algorithmic": spmv_bpr * N, "peak_source": peak_src,
-                     "avg_launch_ms": spmv_ms,
-                     "avg_launch_ms_burst": burst_ms,
-                     "achieved_burst": (spmv_bpr * N / (burst_ms / 1000.0) / 1e9) if burst_ms else None},
+                     "avg_launch_ms": spmv_ms},
         "cg_bandwidth": {"achieved_gbs": cg_bpr * N / (iter_ms_p / 1000.0) / 1e9,
                          "frac_of_measured": cg_bpr * N / (iter_ms_p / 1000.0) / 1e9 / peak,
                          "frac_of_8tbs": cg_bpr * N / (iter_ms_p / 1000.0) / 1e9 / 8000.0,

@@ -20,6 +20,8 @@ def main():
     ap.add_argument("--grid", type=int, default=4096)
     ap.add_argument("--reps", type=int, default=50)
     ap.add_argument("--schemes", default="2,0")
+    ap.add_argument("--mode", type=int, default=0, help="matrix check mode of the timed SpMVs (0 correct, 2 range)")
+    ap.add_argument("--spmv-only", action="store_true", help="time the SpMV kernels only")
     a = ap.parse_args()
     import torch
     import bench
@@ -49,8 +51,14 @@ def main():
             torch.cuda.synchronize()
             return e0.elapsed_time(e1) / a.reps
         res = {
-            "spmv_ms": t(lambda: abft.spmv(ctx, sol.A, p, w, cnt, dot=dot)),
+            "spmv_ms": t(lambda: abft.spmv(ctx, sol.A, p, w, cnt, dot=dot, mode=a.mode)),
             "spmv_partials_ms": t(lambda: abft.spmv_partials(ctx, sol.A, p, w, cnt)),
+        }
+        if a.spmv_only:
+            out[f"scheme{spec}" if "/" in spec else f"scheme{s}"] = res
+            del sol
+            continue
+        res |= {
             "calc_ur_ms": t(lambda: abft.calc_ur(ctx, x, p, r, w, 1e-30, rrn=dot, counts=cnt)),
             "calc_p_ms": t(lambda: abft.calc_p(ctx, p, r, 1e-30, counts=cnt)),
         }
