@@ -292,6 +292,36 @@ int abft_cg_solve_dist(abft_dist* d, abft_ctx* ctx, const abft_csr* A, int nchun
  * CUDA graph) is the code the NCCL transport runs.  Errors: ABFT_E_INVALID
  * (nranks < 1 or > 1024), ABFT_E_CUDA. */
 int abft_dist_init_loopback(abft_dist** out, int nranks, int device);
+
+/* Peer-memory halos (SURVEY S§8(f) f3 "NVLink P2P / symmetric-memory halos";
+ * the halo exchange of PAPER.md P:300-301 §V-A's decomposed grid done by the
+ * producer of p): with enable = 1 the standard CG's calc_p also stores the
+ * encoded p of its first / last local grid row straight into the neighbours'
+ * ghost rows, k_post_p then raises the neighbours' arrival flags
+ * (system-scope fence + atomic store of the iteration count), and each SpMV's
+ * halo step becomes a one-thread wait on this rank's two flags (on the comm
+ * stream, overlapped with the interior tile rows).  Iteration 1 still copies
+ * the init p once.  Same words, counters and results as the copy exchange.
+ * Used only for the standard CG with equal strips and no fault schedule;
+ * otherwise the copy exchange runs.
+ *   loopback transport: peer_p / peer_flag ignored (the ranks' own buffers).
+ *   NCCL transport: peer_p[0] / peer_p[1] = rank-1's / rank+1's halo-extended
+ *   p data mapped into this process (abft_ipc_open_handle; NULL where there is
+ *   no neighbour), peer_flag[0] = rank-1's flags + 1, peer_flag[1] = rank+1's
+ *   flags + 0 (abft_dist_flags of the neighbour, mapped).  The buffers must
+ *   stay valid for the solves that use them.
+ * enable = 0 restores the copy exchange.  ABFT_E_INVALID on missing pointers. */
+int abft_dist_set_peer_halo(abft_dist* d, int enable, void* const* peer_p, int* const* peer_flag);
+/* This rank's two arrival-flag words (device memory of the transport; [0] is
+ * raised by rank-1, [1] by rank+1) — to be shared with the neighbours. */
+int abft_dist_flags(abft_dist* d, int** flags);
+/* CUDA IPC for the NCCL transport's peer halos: the 64-byte handle of the
+ * allocation holding dev_ptr and dev_ptr's offset in it; open maps a peer's
+ * handle (+ offset) into this process (peer access enabled lazily); close
+ * unmaps (pass the same offset). */
+int abft_ipc_get_handle(const void* dev_ptr, void* handle64, int64_t* offset);
+int abft_ipc_open_handle(const void* handle64, int64_t offset, void** dev_ptr);
+int abft_ipc_close_handle(void* dev_ptr, int64_t offset);
 /* Distributed protected CG over a loopback transport: per rank q, ctxs[q] (one
  * context per rank, all on the transport's device), its chunk array A[q] of
  * nchunks[q] chunks, its halo-extended vectors vecs[5q .. 5q+4] = b, x, r, p, w,
@@ -316,7 +346,10 @@ int abft_cg_solve_loopback_sr(abft_dist* d, abft_ctx* const* ctxs, const abft_cs
 
 /* Host-side codec hooks (no GPU needed): run the exact __host__ __device__
  * codec functions on the CPU for the unit tests.  inst: 0 E-SECDED, 1 V-SECDED64,
- * 2 R-SECDED64, 3 R-SECDED128, 4 V-SECDED128.  Returns 0 clean, 1 corrected, 2 DUE. */
+ * 2 R-SECDED64, 3 R-SECDED128, 4 V-SECDED128.  Returns 0 clean, 1 corrected, 2 DUE.
+ * inst 5 / 6 (check only): the tiled SpMV's pair-packed fast checks of two
+ * E-SECDED codewords words[0..2], words[3..5] / two V-SECDED64 codewords
+ * words[0..1], words[2..3]: 0 iff both are clean, else 2. */
 int abft_codec_host_check(int inst, uint32_t* words);
 void abft_codec_host_encode(int inst, uint32_t* words);
 

@@ -102,6 +102,11 @@ _sig = {
                                      C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(CGOpts),
                                      C.POINTER(CGResult), _P, _P]),
     "abft_dist_init_loopback": (C.c_int, [C.POINTER(C.c_void_p), C.c_int, C.c_int]),
+    "abft_dist_set_peer_halo": (C.c_int, [_P, C.c_int, _P, _P]),
+    "abft_dist_flags": (C.c_int, [_P, C.POINTER(C.c_void_p)]),
+    "abft_ipc_get_handle": (C.c_int, [_P, _P, C.POINTER(C.c_int64)]),
+    "abft_ipc_open_handle": (C.c_int, [_P, C.c_int64, C.POINTER(C.c_void_p)]),
+    "abft_ipc_close_handle": (C.c_int, [_P, C.c_int64]),
     "abft_cg_solve_sr_dist": (C.c_int, [_P, _P, C.POINTER(CSR), C.c_int, C.c_int64, C.POINTER(Vec), C.POINTER(Vec),
                                         C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec), C.POINTER(Vec),
                                         C.POINTER(CGOpts), C.POINTER(CGResult), _P, _P]),
@@ -481,8 +486,53 @@ class Dist:
 
     def close(self):
         if self.h:
+            self.disable_peer_halo()
             _lib.abft_dist_destroy(self.h)
             self.h = None
+
+    def enable_peer_halo(self, p: "Vector", group=None):
+        """Peer-memory halos (abft_dist_set_peer_halo) for solves whose p is the
+        halo-extended vector `p`: every rank shares the CUDA IPC handles of its p
+        and of its arrival flags (abft_ipc_get_handle, all-gathered over
+        torch.distributed), maps its neighbours' (abft_ipc_open_handle) and hands
+        the pointers to the transport.  Collective over the ranks."""
+        import torch.distributed as dist
+        flags = C.c_void_p()
+        _check(_lib.abft_dist_flags(self.h, C.byref(flags)), "abft_dist_flags")
+        mine = []
+        for ptr in (p.data.data_ptr(), flags.value):
+            hb = (C.c_uint8 * 64)()
+            off = C.c_int64()
+            _check(_lib.abft_ipc_get_handle(C.c_void_p(ptr), C.cast(hb, C.c_void_p), C.byref(off)),
+                   "abft_ipc_get_handle")
+            mine.append((bytes(hb), off.value))
+        allh = [None] * self.nranks
+        dist.all_gather_object(allh, mine, group=group)
+        self._mapped = []
+        peer_p = (C.c_void_p * 2)()
+        peer_f = (C.c_void_p * 2)()
+        for k, nb in enumerate((self.rank - 1, self.rank + 1)):
+            if not 0 <= nb < self.nranks:
+                continue
+            ptrs = []
+            for (hbytes, off) in allh[nb]:
+                raw = (C.c_uint8 * 64)(*hbytes)
+                out = C.c_void_p()
+                _check(_lib.abft_ipc_open_handle(C.cast(raw, C.c_void_p), off, C.byref(out)), "abft_ipc_open_handle")
+                self._mapped.append((out.value, off))
+                ptrs.append(out.value)
+            peer_p[k] = ptrs[0]
+            # rank-1 is signalled through its flags[1], rank+1 through its flags[0]
+            peer_f[k] = ptrs[1] + (4 if k == 0 else 0)
+        _check(_lib.abft_dist_set_peer_halo(self.h, 1, C.cast(peer_p, C.c_void_p), C.cast(peer_f, C.c_void_p)),
+               "abft_dist_set_peer_halo")
+
+    def disable_peer_halo(self):
+        if self.h:
+            _lib.abft_dist_set_peer_halo(self.h, 0, None, None)
+        for (ptr, off) in getattr(self, "_mapped", []):
+            _lib.abft_ipc_close_handle(C.c_void_p(ptr), off)
+        self._mapped = []
 
     def cg_solve(self, ctx: Context, A, n_halo: int, b, x, r, p, w, tol=1e-10, max_iters=10000, due_policy=0,
                  counts: Counters | None = None, poll_every=16, stream=None, check_interval=1) -> CGResult:
@@ -522,6 +572,10 @@ class Loopback:
         if self.h:
             _lib.abft_dist_destroy(self.h)
             self.h = None
+
+    def set_peer_halo(self, enable: bool):
+        """Peer-memory halos between the loopback ranks (abft_dist_set_peer_halo)."""
+        _check(_lib.abft_dist_set_peer_halo(self.h, 1 if enable else 0, None, None), "abft_dist_set_peer_halo")
 
     def __del__(self):
         try:

@@ -1,6 +1,8 @@
 // capi.cu — the C ABI of libabft.so (include/abft.h): argument validation,
 // scratch ownership, and the device-resident CG driver.
 // Host code only; every arithmetic step runs in kernels.cu.
+#include <cuda.h>
+#include <cudaTypedefs.h>
 #include <cuda_runtime.h>
 
 #include <atomic>
@@ -440,6 +442,12 @@ struct abft_dist {
   double* gathered = nullptr;  // all ranks' payloads [GATHER_W * nranks] (loopback: rank r writes its own slot)
   cudaStream_t comm_stream = nullptr;   // halo exchange, overlapped with the interior SpMV
   cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
+  // peer-memory halos (S§8(f) f3): p's ghost rows are stored by
+  // the neighbours' calc_p straight into this rank's vector; arrival flags
+  int peer_halo = 0;
+  int* flags = nullptr;         // [2] this rank's (NCCL) / [2 * nranks] every loopback rank's: [0] from rank-1, [1] from rank+1
+  uint64_t* peer_p[2] = {};     // NCCL: the neighbours' halo-extended p, mapped here ([0] rank-1, [1] rank+1)
+  int* peer_flag[2] = {};       // NCCL: where this rank signals: rank-1's flags[1], rank+1's flags[0] (mapped)
 };
 
 namespace {
@@ -707,6 +715,33 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     ctx->p_alt_len = npad_ext;
   }
   uint64_t* const P[2] = {reinterpret_cast<uint64_t*>(p->data), ctx->p_alt};
+  // peer-memory halos: calc_p stores p's boundary rows into the
+  // neighbours' ghost rows and k_post_p raises their arrival flags; the SpMV's
+  // halo step becomes a wait on this rank's flags.  Standard CG only, equal
+  // strips, no fault schedule (an injected p fault must reach the ghost copy)
+  bool peer = multi && d->peer_halo && d->nranks > 1 && n_halo > 0 && !sr && !cheb && !ppcg;
+  for (int q = 0; q < nl && peer; q++) peer = R[q].ctx->nfaults == 0 && R[q].n == R[0].n;
+  if (peer) {
+    auto ext = [](abft_vec* v) { return reinterpret_cast<uint64_t*>(v->data); };
+    for (int q = 0; q < nl; q++) {
+      VecArgs& va = R[q].va;
+      va.halo_n = n_halo;
+      if (d->loopback) {
+        va.halo_up = q > 0 ? ext(R[q - 1].p()) + n_halo + R[q - 1].n : nullptr;
+        va.halo_dn = q < nl - 1 ? ext(R[q + 1].p()) : nullptr;
+        va.sig_up = q > 0 ? d->flags + 2 * (q - 1) + 1 : nullptr;
+        va.sig_dn = q < nl - 1 ? d->flags + 2 * (q + 1) : nullptr;
+      } else {
+        va.halo_up = d->rank > 0 ? d->peer_p[0] + n_halo + R[0].n : nullptr;
+        va.halo_dn = d->rank < d->nranks - 1 ? d->peer_p[1] : nullptr;
+        va.sig_up = d->rank > 0 ? d->peer_flag[0] : nullptr;
+        va.sig_dn = d->rank < d->nranks - 1 ? d->peer_flag[1] : nullptr;
+      }
+    }
+    // (ordered before any neighbour's first signal: that comes after the init
+    // all-gather, which needs this rank)
+    CUDA_TRY(cudaMemsetAsync(d->flags, 0, sizeof(int) * 2 * (d->loopback ? nl : 1), s));
+  }
   // halo overlap: P > 1 and every chunk of every rank on the tiled kernel
   bool overlap = multi && d->nranks > 1 && n_halo > 0;
   for (int q = 0; q < nl && overlap; q++)
@@ -749,6 +784,10 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   prof.end();
   if (!cheb)
     for (int q = 0; q < nl; q++) count_launch(launch_init_r(R[q].va, scheme, s));
+  // peer-memory halos: iteration 1's p (= r, written by init) reaches the
+  // ghost rows by one copy exchange; from then on the neighbours' calc_p
+  // stores them (the loop's wait then passes on flags >= 0 at iteration 1)
+  if (peer && (e = halo_exchange(d, R, nl, 3, n_halo, s))) return e;
   if (cheb) {   // r = b - A u0; p = r/theta; u += p; rr0
     count_launch(launch_cheb(R[0].va, scheme, 1, 0.0, 0.0, 0.0, s));
     if ((e = finish_dot(R, nl, d, 8, s))) return e;
@@ -799,6 +838,20 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
   const bool pdl_on = ctx->pdl && !multi;
   // the protected SpMV of one iteration, all ranks (halo first, or overlapped)
   // vi: the SpMV's input vector (3 = p; 2 = r for the single-reduction CG), dots 1 or 2
+  // the p halo of an iteration's SpMV: copied (NCCL send/recv, loopback
+  // copies) or, with peer-memory halos, already stored by the neighbours'
+  // calc_p — then wait for their arrival flags (identical in every graph replay)
+  auto halo_step = [&](int vi, cudaStream_t hs) -> int {
+    if (peer && vi == 3) {
+      for (int q = 0; q < nl; q++) {
+        const bool up = d->loopback ? q > 0 : d->rank > 0;
+        const bool dn = d->loopback ? q < nl - 1 : d->rank < d->nranks - 1;
+        count_launch(launch_wait_halo(d->flags + (d->loopback ? 2 * q : 0), R[q].ctx->state, up, dn, hs));
+      }
+      return ABFT_OK;
+    }
+    return halo_exchange(d, R, nl, vi, n_halo, hs);
+  };
   auto spmv_iter = [&](int64_t kk, cudaStream_t ss, int vi, int dots) -> int {
     int e2;
     if (fused) {
@@ -808,7 +861,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
                          MODE_CORRECT, interval, P[(kk - 1) & 1], reinterpret_cast<uint64_t*>(r->data));
     }
     if (!overlap) {
-      if ((e2 = halo_exchange(d, R, nl, vi, n_halo, ss))) return e2;
+      if ((e2 = halo_step(vi, ss))) return e2;
       for (int q = 0; q < nl; q++) {
         // standard CG: p was last written by calc_p (iteration 1: init), and
         // the kernel between it and this SpMV (k_post_p / the rr0 reduction)
@@ -825,7 +878,7 @@ int cg_run(RankRun* R, int nl, abft_dist* d, int64_t n_halo, const abft_cg_opts*
     // halo on the comm stream while the interior tile rows run on ss; then the boundary rows
     CUDA_TRY(cudaEventRecord(d->ev_fork, ss));
     CUDA_TRY(cudaStreamWaitEvent(d->comm_stream, d->ev_fork, 0));
-    if ((e2 = halo_exchange(d, R, nl, vi, n_halo, d->comm_stream))) return e2;
+    if ((e2 = halo_step(vi, d->comm_stream))) return e2;
     CUDA_TRY(cudaEventRecord(d->ev_join, d->comm_stream));
     for (int part = 1; part <= 2; part++) {
       if (part == 2) CUDA_TRY(cudaStreamWaitEvent(ss, d->ev_join, 0));
@@ -1183,6 +1236,7 @@ int abft_dist_init(abft_dist** out, const void* uid, int rank, int nranks, int d
   if (!e && cudaMalloc(&d->sendbuf, sizeof(double) * GATHER_W) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc sendbuf");
   if (!e && cudaMalloc(&d->gathered, sizeof(double) * GATHER_W * nranks) != cudaSuccess)
     e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
+  if (!e && cudaMalloc(&d->flags, sizeof(int) * 2) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc flags");
   if (e) {
     abft_dist_destroy(d);
     return e;
@@ -1201,6 +1255,7 @@ int abft_dist_init_loopback(abft_dist** out, int nranks, int device) {
   int e = dist_streams(d);
   if (!e && cudaMalloc(&d->gathered, sizeof(double) * GATHER_W * nranks) != cudaSuccess)
     e = fail(ABFT_E_CUDA, "cudaMalloc gathered");
+  if (!e && cudaMalloc(&d->flags, sizeof(int) * 2 * nranks) != cudaSuccess) e = fail(ABFT_E_CUDA, "cudaMalloc flags");
   if (e) {
     abft_dist_destroy(d);
     return e;
@@ -1209,11 +1264,78 @@ int abft_dist_init_loopback(abft_dist** out, int nranks, int device) {
   return ABFT_OK;
 }
 
+int abft_dist_set_peer_halo(abft_dist* d, int enable, void* const* peer_p, int* const* peer_flag) {
+  if (!d) return fail(ABFT_E_INVALID, "null dist");
+  if (!enable) {
+    d->peer_halo = 0;
+    return ABFT_OK;
+  }
+  if (!d->loopback) {
+    if (!peer_p || !peer_flag) return fail(ABFT_E_INVALID, "NCCL transport: the neighbours' p and flags are needed");
+    const bool up = d->rank > 0, dn = d->rank < d->nranks - 1;
+    if ((up && (!peer_p[0] || !peer_flag[0])) || (dn && (!peer_p[1] || !peer_flag[1])))
+      return fail(ABFT_E_INVALID, "missing neighbour pointer");
+    for (int k = 0; k < 2; k++) {
+      d->peer_p[k] = reinterpret_cast<uint64_t*>(peer_p[k]);
+      d->peer_flag[k] = peer_flag[k];
+    }
+  }
+  d->peer_halo = 1;
+  return ABFT_OK;
+}
+
+int abft_dist_flags(abft_dist* d, int** flags) {
+  if (!d || !flags) return fail(ABFT_E_INVALID, "null dist/flags");
+  *flags = d->flags;
+  return ABFT_OK;
+}
+
+int abft_ipc_get_handle(const void* dev_ptr, void* handle, int64_t* offset) {
+  if (!dev_ptr || !handle || !offset) return fail(ABFT_E_INVALID, "null argument");
+  CUdeviceptr base = 0;
+  size_t size = 0;
+  cudaPointerAttributes at{};
+  CUDA_TRY(cudaPointerGetAttributes(&at, dev_ptr));
+  // the allocation's base address: IPC handles name whole allocations
+  static PFN_cuMemGetAddressRange_v3020 range = [] {
+    void* p = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    return (cudaGetDriverEntryPoint("cuMemGetAddressRange", &p, cudaEnableDefault, &q) == cudaSuccess &&
+            q == cudaDriverEntryPointSuccess)
+               ? reinterpret_cast<PFN_cuMemGetAddressRange_v3020>(p)
+               : static_cast<PFN_cuMemGetAddressRange_v3020>(nullptr);
+  }();
+  if (!range || range(&base, &size, reinterpret_cast<CUdeviceptr>(dev_ptr)) != CUDA_SUCCESS)
+    return fail(ABFT_E_CUDA, "cuMemGetAddressRange failed");
+  cudaIpcMemHandle_t h;
+  CUDA_TRY(cudaIpcGetMemHandle(&h, reinterpret_cast<void*>(base)));
+  memcpy(handle, &h, sizeof(h));
+  *offset = (int64_t)(reinterpret_cast<CUdeviceptr>(dev_ptr) - base);
+  return ABFT_OK;
+}
+
+int abft_ipc_open_handle(const void* handle, int64_t offset, void** dev_ptr) {
+  if (!handle || !dev_ptr) return fail(ABFT_E_INVALID, "null argument");
+  cudaIpcMemHandle_t h;
+  memcpy(&h, handle, sizeof(h));
+  void* base = nullptr;
+  CUDA_TRY(cudaIpcOpenMemHandle(&base, h, cudaIpcMemLazyEnablePeerAccess));
+  *dev_ptr = static_cast<char*>(base) + offset;
+  return ABFT_OK;
+}
+
+int abft_ipc_close_handle(void* dev_ptr, int64_t offset) {
+  if (!dev_ptr) return ABFT_OK;
+  CUDA_TRY(cudaIpcCloseMemHandle(static_cast<char*>(dev_ptr) - offset));
+  return ABFT_OK;
+}
+
 int abft_dist_destroy(abft_dist* d) {
   if (!d) return ABFT_OK;
   if (d->comm) ncclCommDestroy(d->comm);
   cudaFree(d->sendbuf);
   cudaFree(d->gathered);
+  cudaFree(d->flags);
   if (d->ev_fork) cudaEventDestroy(d->ev_fork);
   if (d->ev_join) cudaEventDestroy(d->ev_join);
   if (d->comm_stream) cudaStreamDestroy(d->comm_stream);

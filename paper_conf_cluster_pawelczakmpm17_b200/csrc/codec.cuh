@@ -296,6 +296,11 @@ ABFT_HD void v64_acc(uint32_t a, uint32_t b, uint32_t& acc_r, uint32_t& acc_p) {
   acc_r |= moebius32(v64_fold(a, b));
   acc_p |= (uint32_t)(popc32(b ^ (a & 0x80u)) | popc32(a & 0x8Eu));
 }
+// Two V-SECDED64 codewords at once (the decoded SpMV window's slot pairs):
+// the fold registers' 4-step Moebius shared as in e96_acc2, par(lo) of each
+// fold and the two code rows by POPC.  Nonzero (acc_u & MOEB2_SYN_MASK, or
+// acc_p bit 0) iff either codeword fails v64_bad.
+ABFT_HD void v64_acc2(uint32_t a1, uint32_t b1, uint32_t a2, uint32_t b2, uint32_t& acc_u, uint32_t& acc_p);
 ABFT_HD uint32_t v64_bad(uint32_t a, uint32_t b) {
   uint32_t r = moebius32(v64_fold(a, b));
   uint32_t s56 = (uint32_t)(popc32(b ^ (a & 0x80u)) | popc32(a & 0x8Eu)) & 1u;
@@ -560,6 +565,43 @@ ABFT_HD uint32_t e96_fold(uint32_t a, uint32_t b, uint32_t c) {
 ABFT_HD void e96_acc(uint32_t a, uint32_t b, uint32_t c, uint32_t& acc_r, uint32_t& acc_p) {
   acc_r |= moebius32(e96_fold(a, b, c));
   acc_p |= (uint32_t)(popc32(lop3<0x78>(b, c, 0x9F000000u)) | popc32(lop3<0xE4>(b, c, 0x80000000u)));
+}
+
+// Two E-SECDED codewords at once (the hot path's element pairs): the five
+// index-syndrome bits and the overall parity of a fold F are parities of its
+// 16-bit halves' XOR u = lo ^ hi (R31, R30, R29, R27, R23 = the 4-step
+// Moebius transform of u at bits 15, 14, 13, 11, 7) plus par(lo) (R15).  The
+// two codewords' u share one register, so the 4 Moebius steps run once for
+// both; par(lo) of each is a POPC next to the code-row POPCs.  OR-accumulates
+// into acc_u (test with MOEB2_SYN_MASK) and acc_p (bit 0): nonzero iff either
+// codeword's syndrome or parity is nonzero — exactly e96_bad of each.
+constexpr uint32_t MOEB2_SYN_MASK = 0xE880E880u;
+ABFT_HD void e96_acc2(uint32_t a1, uint32_t b1, uint32_t c1, uint32_t a2, uint32_t b2, uint32_t c2, uint32_t& acc_u,
+                      uint32_t& acc_p) {
+  const uint32_t f1 = e96_fold(a1, b1, c1), f2 = e96_fold(a2, b2, c2);
+  const uint32_t x = byte_perm(f1, f2, 0x5410u), y = byte_perm(f1, f2, 0x7632u);   // lo halves, hi halves
+  uint32_t u = x ^ y;
+  u ^= (u << 1) & 0xAAAAAAAAu;
+  u ^= (u << 2) & 0xCCCCCCCCu;
+  u ^= (u << 4) & 0xF0F0F0F0u;
+  u ^= (u << 8) & 0xFF00FF00u;
+  acc_u |= u;
+  acc_p |= (uint32_t)(popc32(x & 0xFFFFu) | popc32(x >> 16) | popc32(lop3<0x78>(b1, c1, 0x9F000000u)) |
+                      popc32(lop3<0xE4>(b1, c1, 0x80000000u)) | popc32(lop3<0x78>(b2, c2, 0x9F000000u)) |
+                      popc32(lop3<0xE4>(b2, c2, 0x80000000u)));
+}
+
+ABFT_HD void v64_acc2(uint32_t a1, uint32_t b1, uint32_t a2, uint32_t b2, uint32_t& acc_u, uint32_t& acc_p) {
+  const uint32_t f1 = v64_fold(a1, b1), f2 = v64_fold(a2, b2);
+  const uint32_t x = byte_perm(f1, f2, 0x5410u), y = byte_perm(f1, f2, 0x7632u);
+  uint32_t u = x ^ y;
+  u ^= (u << 1) & 0xAAAAAAAAu;
+  u ^= (u << 2) & 0xCCCCCCCCu;
+  u ^= (u << 4) & 0xF0F0F0F0u;
+  u ^= (u << 8) & 0xFF00FF00u;
+  acc_u |= u;
+  acc_p |= (uint32_t)(popc32(x & 0xFFFFu) | popc32(x >> 16) | popc32(b1 ^ (a1 & 0x80u)) | popc32(a1 & 0x8Eu) |
+                      popc32(b2 ^ (a2 & 0x80u)) | popc32(a2 & 0x8Eu));
 }
 
 ABFT_HD uint32_t e96_bad(uint32_t a, uint32_t b, uint32_t c) {

@@ -99,6 +99,16 @@ struct VecArgs {
   CgState* state;
   double* out_masked;
   const CrcTables* crc;   // device tables (CRC32C schemes only)
+  // peer-memory halos (multi-rank): calc_p also stores the
+  // encoded p of its first / last halo_n local rows straight into the
+  // neighbours' ghost rows (halo_up: rank-1's bottom ghost row, halo_dn:
+  // rank+1's top ghost row; null = no such neighbour), and k_post_p then raises
+  // the neighbours' arrival flags (sig_up / sig_dn) to the iteration count
+  uint64_t* halo_up;
+  uint64_t* halo_dn;
+  int64_t halo_n;
+  int* sig_up;
+  int* sig_dn;
 };
 
 // PDL for the CG driver's iteration launches
@@ -149,6 +159,7 @@ int launch_pack_due(double* out, const int* due, cudaStream_t s);
 int launch_csr_encode(abft_csr* A, uint32_t* flags, cudaStream_t s);
 int launch_check_csr(const abft_csr* A, DevCounts* c, int* due, int scrub, cudaStream_t s);
 int launch_inject(void* base, uint64_t bit, cudaStream_t s);
+int launch_wait_halo(const int* flags, const CgState* st, int need_up, int need_dn, cudaStream_t s);
 // phase 0: the faults of iteration 0 (before init); phase 1: those of
 // iteration state->iters + 1 (skipped once the solve stopped)
 int launch_inject_sched(const DevFault* f, int n, const CgState* st, int phase, cudaStream_t s);

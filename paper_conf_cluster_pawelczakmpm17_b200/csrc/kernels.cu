@@ -118,7 +118,7 @@ int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s) {
 #if ABFT_P_TICKET
   return 1;
 #else
-  launch_k(k_post_p, 1, 1, 0, s, a.state, (const int*)a.due);
+  launch_k(k_post_p, 1, 1, 0, s, a.state, (const int*)a.due, a.sig_up, a.sig_dn);
   return 2;
 #endif
 }
@@ -376,6 +376,10 @@ int launch_inject_sched(const DevFault* f, int n, const CgState* st, int phase, 
   return 1;
 }
 
+int launch_wait_halo(const int* flags, const CgState* st, int need_up, int need_dn, cudaStream_t s) {
+  k_wait_halo<<<1, 1, 0, s>>>(flags, st, need_up, need_dn);
+  return 1;
+}
 int launch_inject(void* base, uint64_t bit, cudaStream_t s) {
   k_inject<<<1, 1, 0, s>>>(reinterpret_cast<uint32_t*>(base), bit);
   return 1;
@@ -417,6 +421,16 @@ extern "C" int abft_codec_host_check(int inst, uint32_t* w) {
       int o = v128_check(d, &word);
       if (o == CORRECTED) { w[0] = lo32(d[0]); w[1] = hi32(d[0]); w[2] = lo32(d[1]); w[3] = hi32(d[1]); }
       return o;
+    }
+    case 5: {   // the tiled SpMV's pair-packed E-SECDED fast check of two codewords w[0..2], w[3..5]
+      uint32_t u = 0, p = 0;
+      e96_acc2(w[0], w[1], w[2], w[3], w[4], w[5], u, p);
+      return ((u & MOEB2_SYN_MASK) | (p & 1u)) ? DUE : CLEAN;
+    }
+    case 6: {   // the decoded window's pair-packed V-SECDED64 fast check of w[0..1], w[2..3]
+      uint32_t u = 0, p = 0;
+      v64_acc2(w[0], w[1], w[2], w[3], u, p);
+      return ((u & MOEB2_SYN_MASK) | (p & 1u)) ? DUE : CLEAN;
     }
   }
   return -1;

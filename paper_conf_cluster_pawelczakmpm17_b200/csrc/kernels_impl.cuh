@@ -624,11 +624,7 @@ constexpr int TILE_STAGE_VAL = TILE_TY * TILE_PE * 8;          // 10240
 constexpr int TILE_STAGE = TILE_STAGE_VAL + TILE_TY * TILE_PE * 4;   // + 5120
 constexpr int TILE_WIN_BYTES = (TILE_TY + 2) * TILE_WW * 8;    // 21120
 constexpr int TILE_RP = 264;                                   // rowptr entries staged per warp
-constexpr int TILE_OFF_WIN = TILE_NST * TILE_STAGE;            // stages first (128-B aligned)
-constexpr int TILE_OFF_RP = TILE_OFF_WIN + TILE_WIN_BYTES;
-constexpr int TILE_OFF_BAR = TILE_OFF_RP + TILE_TY * TILE_RP * 4;
-constexpr int TILE_OFF_CRC = TILE_OFF_BAR + 64;                // CRC32C tables (only for CRC schemes)
-constexpr int TILE_SMEM = TILE_OFF_CRC + 128;                   // + alignment slack
+// SMEM layout (tile_off_*): stages, window, row pointers, mbarriers, CRC tables
 // ABFT_CRC_SLICE_SMEM = 0: the tiled SpMV reads the 4 KB slicing tables of
 // E-CRC / R-CRC through L1 instead of staging them in SMEM (keeps 3 CTAs per
 // SM for CRC32C matrices)
@@ -636,9 +632,22 @@ constexpr int TILE_SMEM = TILE_OFF_CRC + 128;                   // + alignment s
 #define ABFT_CRC_SLICE_SMEM 1
 #endif
 // dynamic SMEM of one tile kernel: + slicing tables (E-CRC / R-CRC), + V-CRC position tables
+// E-CRC / R-CRC instantiations run 2 stages: their 4 KB of slicing tables
+// would otherwise push the CTA past 76 KB (2 CTAs per SM instead of 3, the
+// range-only accesses of interval mode then +13 %, r2n / r2o)
+#ifndef ABFT_CRC_NST
+#define ABFT_CRC_NST 2
+#endif
+template <int ES, int RS>
+constexpr int tile_nst() { return (ES == CRC32C || RS == CRC32C) ? ABFT_CRC_NST : TILE_NST; }
+constexpr int tile_off_win(int nst) { return nst * TILE_STAGE; }
+constexpr int tile_off_rp(int nst) { return tile_off_win(nst) + TILE_WIN_BYTES; }
+constexpr int tile_off_bar(int nst) { return tile_off_rp(nst) + TILE_TY * TILE_RP * 4; }
+constexpr int tile_off_crc(int nst) { return tile_off_bar(nst) + 64; }
 template <int ES, int RS, int VS>
 constexpr int tile_smem() {
-  return TILE_SMEM + ((ABFT_CRC_SLICE_SMEM && (ES == CRC32C || RS == CRC32C)) ? 4 * CRC_SLICE_WORDS : 0) +
+  return tile_off_crc(tile_nst<ES, RS>()) + 128 +
+         ((ABFT_CRC_SLICE_SMEM && (ES == CRC32C || RS == CRC32C)) ? 4 * CRC_SLICE_WORDS : 0) +
          (VS == CRC32C ? 4 * CRC_VPOS_WORDS : 0);
 }
 
@@ -752,6 +761,14 @@ static __device__ __noinline__ double tile_row(const SpmvArgs& a, uint32_t start
   return acc;
 }
 
+// E-SECDED fast check of the stencil rows' elements in pairs (codec e96_acc2)
+#ifndef ABFT_PAIR_E
+#define ABFT_PAIR_E 1
+#endif
+// V-SECDED64 fast check of the decoded window in slot pairs (codec v64_acc2)
+#ifndef ABFT_PAIR_W
+#define ABFT_PAIR_W 1
+#endif
 // 5-entry stencil rows (the TeaLeaf layout, reading R16) at the assumed
 // position start = s0 + 5 lane: straight-line code, one uniform branch for
 // "any element needs correction / any index is not the canonical stencil
@@ -775,7 +792,7 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
     v[t] = sval[5 * lane + t];
     c[t] = scol[5 * lane + t];
   }
-  uint32_t acc_r = 0, acc_p = 0;
+  uint32_t acc_r = 0, acc_p = 0, acc_u = 0;
   if (mode != MODE_RANGE) {   // uniform: interval mode's unchecked accesses skip the codec
     if (ES == CRC32C) {       // E-CRC over the row, slicing-by-4 tables
       uint32_t crc = 0xFFFFFFFFu, st = 0;
@@ -788,10 +805,16 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
       }
       acc_p = ((crc ^ 0xFFFFFFFFu) != st) ? 1u : 0u;
     }
+    if ((ES == SECDED64 || ES == SECDED128) && ABFT_PAIR_E) {   // elements (0,1), (2,3) pair-packed, 4 alone
+      e96_acc2(lo32(v[0]), hi32(v[0]), c[0], lo32(v[1]), hi32(v[1]), c[1], acc_u, acc_p);
+      e96_acc2(lo32(v[2]), hi32(v[2]), c[2], lo32(v[3]), hi32(v[3]), c[3], acc_u, acc_p);
+      e96_acc(lo32(v[4]), hi32(v[4]), c[4], acc_r, acc_p);
+    } else {
 #pragma unroll
-    for (int t = 0; t < 5; t++) {
-      if (ES == SED) acc_p |= (uint32_t)(popc64(v[t]) + popc32(c[t]));
-      else if (ES == SECDED64 || ES == SECDED128) e96_acc(lo32(v[t]), hi32(v[t]), c[t], acc_r, acc_p);
+      for (int t = 0; t < 5; t++) {
+        if (ES == SED) acc_p |= (uint32_t)(popc64(v[t]) + popc32(c[t]));
+        else if (ES == SECDED64 || ES == SECDED128) e96_acc(lo32(v[t]), hi32(v[t]), c[t], acc_r, acc_p);
+      }
     }
   }
   // canonical stencil neighbours [i-n, i-1, i, i+1, i+n] or the row itself (R16)
@@ -806,7 +829,7 @@ static __device__ __forceinline__ double tile_row5(const SpmvArgs& a, const Spmv
   const bool canon = (d[0] == 0 || d[0] == -n32) && ((unsigned)(d[1] + 1) <= 1u) && d[2] == 0 &&
                      ((unsigned)d[3] <= 1u) && (d[4] == 0 || d[4] == n32);
   const bool in_range = (ES == NONE) || cmax < (uint32_t)a.ncols;
-  if ((ES != NONE && syn_bad(acc_r, acc_p)) || !canon || !in_range)
+  if ((ES != NONE && (syn_bad(acc_r, acc_p) || (acc_u & MOEB2_SYN_MASK) != 0u)) || !canon || !in_range)
     return tile_row<ES, RS, VS>(sa, start, end, sval, scol, true, win, oslot, p_own, own, s0, s1, mode);
   // slot offsets: d itself for +-1 / 0, +-window width for +-n
   const int o0 = d[0] ? -TILE_WW : 0, o4 = d[4] ? TILE_WW : 0;
@@ -843,39 +866,44 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   // the kernel parameters are never spilled to local memory
   __shared__ SpmvArgs s_args;
   uint8_t* s_dyn = s_raw + ((128u - (smem_u32(s_raw) & 127u)) & 127u);
-  double* s_win = reinterpret_cast<double*>(s_dyn + TILE_OFF_WIN);
-  uint64_t* full = reinterpret_cast<uint64_t*>(s_dyn + TILE_OFF_BAR);
-  uint64_t* empty = full + TILE_NST;
-  uint64_t* winbar = empty + TILE_NST;   // the TMA-staged `in` window
+  constexpr int NST = tile_nst<ES, RS>();   // pipeline stages of this instantiation
+  double* s_win = reinterpret_cast<double*>(s_dyn + tile_off_win(NST));
+  uint64_t* full = reinterpret_cast<uint64_t*>(s_dyn + tile_off_bar(NST));
+  uint64_t* empty = full + NST;
+  uint64_t* winbar = empty + NST;   // the TMA-staged `in` window
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  uint32_t* srp = reinterpret_cast<uint32_t*>(s_dyn + TILE_OFF_RP) + warp * TILE_RP;
+  uint32_t* srp = reinterpret_cast<uint32_t*>(s_dyn + tile_off_rp(NST)) + warp * TILE_RP;
   constexpr bool SLICE = ABFT_CRC_SLICE_SMEM && (ES == CRC32C || RS == CRC32C);
-  const uint32_t* s_slice = SLICE ? reinterpret_cast<const uint32_t*>(s_dyn + TILE_OFF_CRC) : &a.crc->slice[0][0];
-  uint8_t* s_vpos = s_dyn + TILE_OFF_CRC + (SLICE ? 4 * CRC_SLICE_WORDS : 0);
+  const uint32_t* s_slice = SLICE ? reinterpret_cast<const uint32_t*>(s_dyn + tile_off_crc(NST)) : &a.crc->slice[0][0];
+  uint8_t* s_vpos = s_dyn + tile_off_crc(NST) + (SLICE ? 4 * CRC_SLICE_WORDS : 0);
   const int64_t n = a.stencil_n;
   const int64_t ny = a.nrows / n;
   const int64_t tiles_x = n >> 8;
   const int64_t tx0 = (blockIdx.x % tiles_x) << 8;
   const int64_t ty0 = ((int64_t)(blockIdx.x / tiles_x) + a.ty_lo) * TILE_TY;
-  // ---- 0. producer: barriers, then the first TILE_NST passes in flight (the
+  // ---- 0. producer: barriers, then the first NST passes in flight (the
   // matrix: loaded before the PDL grid dependency resolves)
   if (threadIdx.x == 0) {
 #pragma unroll
-    for (int s = 0; s < TILE_NST; s++) {
+    for (int s = 0; s < NST; s++) {
       mbar_init(&full[s], 1);
       mbar_init(&empty[s], TILE_TY);
     }
     mbar_init(winbar, 1);
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
 #pragma unroll
-    for (int k = 0; k < TILE_NST; k++) tile_produce(tm, s_dyn + k * TILE_STAGE, &full[k], tx0, ty0, k);
+    for (int k = 0; k < NST; k++) tile_produce(tm, s_dyn + k * TILE_STAGE, &full[k], tx0, ty0, k);
     if (ABFT_EARLY_WIN && !FUSED && a.early_in && vgrp(VS) == 1 && tm.has_vmaps) {   // `in` is final already
       mbar_expect_tx(winbar, TILE_WIN_BYTES);
       tma_3d(s_win, &tm.vin, 0, (int)(tx0 / 2 - 1), (int)(a.row_base / n + ty0 - 1), winbar);
     }
   }
   if (VS == SECDED64) load_lut(s_lut);
-  if (SLICE) smem_fill(const_cast<uint32_t*>(s_slice), &a.crc->slice[0][0], CRC_SLICE_WORDS);
+  // E-CRC / R-CRC slicing tables: only range-checked accesses (interval mode)
+  // never read them, so a known-range launch skips the 4 KB fill; interval
+  // launches learn their mode after the PDL wait and fill below if checked
+  if (SLICE && a.check_interval <= 1 && a.check_mode != MODE_RANGE)
+    smem_fill(const_cast<uint32_t*>(s_slice), &a.crc->slice[0][0], CRC_SLICE_WORDS);
   if (VS == CRC32C) smem_fill(reinterpret_cast<uint32_t*>(s_vpos), &a.crc->vpos[0][0][0], CRC_VPOS_WORDS);
   const uint8_t* cs = (VS == CRC32C) ? s_vpos : s_lut;   // vector codec tables
   const int64_t gy = ty0 + warp;
@@ -950,10 +978,12 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
       s_args.beta_f = fz ? a.state->beta : 0.0;
     }
   }
+  const int mode = spmv_mode(a);
+  if (SLICE && a.check_interval > 1 && mode != MODE_RANGE)
+    smem_fill(const_cast<uint32_t*>(s_slice), &a.crc->slice[0][0], CRC_SLICE_WORDS);
   // every warp waits on winbar / the stage barriers below: thread 0's
   // mbarrier.init (and the SMEM tables) must be visible to the whole CTA first
   __syncthreads();
-  const int mode = spmv_mode(a);
   if (has_seg) {
     if (!stop_v) {
       uint32_t acc = 0;
@@ -1009,7 +1039,7 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   }
   if (stop_v) {  // uniform per grid: drain the producer's copies before the CTA exits
     if (threadIdx.x == 0) {
-      for (int s = 0; s < TILE_NST; s++) mbar_wait(&full[s], 0u);
+      for (int s = 0; s < NST; s++) mbar_wait(&full[s], 0u);
       if (tma_win) mbar_wait(winbar, 0u);
     }
     return;
@@ -1045,6 +1075,33 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
       for (int q = 0; q < WQ; q++) {
         const int sl = threadIdx.x + 256 * q;
         if (q < WQ - 1 || sl < WS) s_win[sl] = as_d(wv[q] & vkeep(VS));
+      }
+    } else
+#endif
+#if ABFT_PAIR_W
+    if (VS == SECDED64) {   // slot pairs (sl, sl + 256): one shared fast check, the per-slot path when it fails
+      auto slot = [&](int sl, uint64_t w) {
+        if (v64_bad(lo32(w), hi32(w))) {
+          const int wy = sl / TILE_WW, j = sl - wy * TILE_WW;
+          const int64_t idx = win0 + (int64_t)wy * n + j;
+          const bool owner = wy >= 1 && wy <= TILE_TY && ty0 + wy - 1 < ny && j >= TILE_WX0 && j < TILE_WX0 + 256;
+          w = v1_check<VS>(w, pin + idx, owner, a.counts, a.due);
+        }
+        s_win[sl] = as_d(w & vkeep(VS));
+      };
+#pragma unroll 1
+      for (int sl = threadIdx.x; sl < WS; sl += 512) {
+        const bool two = sl + 256 < WS;
+        uint64_t w0 = raw[sl], w1 = two ? raw[sl + 256] : 0ull;   // zero is a clean codeword
+        uint32_t au = 0, ap = 0;
+        v64_acc2(lo32(w0), hi32(w0), lo32(w1), hi32(w1), au, ap);
+        if (((au & MOEB2_SYN_MASK) | (ap & 1u)) == 0u) {
+          s_win[sl] = as_d(w0 & vkeep(VS));
+          if (two) s_win[sl + 256] = as_d(w1 & vkeep(VS));
+        } else {   // cold
+          slot(sl, w0);
+          if (two) slot(sl + 256, w1);
+        }
       }
     } else
 #endif
@@ -1217,8 +1274,8 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
   constexpr int kPassUnroll = ABFT_TILE_UNROLL;
 #pragma unroll kPassUnroll
   for (int k = 0; k < 8; k++) {
-    const int st = k % TILE_NST;
-    const uint32_t ph = (uint32_t)((k / TILE_NST) & 1);
+    const int st = k % NST;
+    const uint32_t ph = (uint32_t)((k / NST) & 1);
     uint8_t* stage = s_dyn + st * TILE_STAGE;
     mbar_wait(&full[st], ph);
     if (has_seg) {
@@ -1261,9 +1318,9 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
     }
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[st]);
-    if (k + TILE_NST < 8 && threadIdx.x == 0) {  // refill the stage once every warp released it
+    if (k + NST < 8 && threadIdx.x == 0) {  // refill the stage once every warp released it
       mbar_wait(&empty[st], ph);
-      tile_produce(tm, stage, &full[st], tx0, ty0, k + TILE_NST);
+      tile_produce(tm, stage, &full[st], tx0, ty0, k + NST);
     }
   }
   if (DOT && has_seg) {
@@ -1285,6 +1342,11 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
 // (RED-1).  G = 1 schemes check each word in its lane; G = 2 / 4 schemes use
 // the lane-split group codecs (pair gather / V-CRC partials), the pass pair
 // (k, k+32) being exactly what the SECDED128 pair gather needs.
+// BLAS-1 V-SECDED64 fast checks in pairs (codec v64_acc2): off — calc_ur
+// measured 0.1537 vs 0.1347 ms with it (r2o)
+#ifndef ABFT_PAIR_V
+#define ABFT_PAIR_V 0
+#endif
 // OR-accumulated fast check of up to 8 G=1 codewords (zero words are clean in
 // every scheme): true iff any of them needs the per-word cold path.
 template <int VS>
@@ -1292,6 +1354,14 @@ __device__ __forceinline__ bool vacc_bad(uint64_t w0, uint64_t w1, uint64_t w2, 
                                          uint64_t w6, uint64_t w7) {
   if (VS == SED) return ((popc64(w0) | popc64(w1) | popc64(w2) | popc64(w3) | popc64(w4) | popc64(w5) |
                           popc64(w6) | popc64(w7)) & 1) != 0;
+  if (VS == SECDED64 && ABFT_PAIR_V) {   // pair-packed fast checks (codec v64_acc2); zero words fold away
+    uint32_t u = 0, p = 0;
+    v64_acc2(lo32(w0), hi32(w0), lo32(w1), hi32(w1), u, p);
+    v64_acc2(lo32(w2), hi32(w2), lo32(w3), hi32(w3), u, p);
+    v64_acc2(lo32(w4), hi32(w4), lo32(w5), hi32(w5), u, p);
+    v64_acc2(lo32(w6), hi32(w6), lo32(w7), hi32(w7), u, p);
+    return ((u & MOEB2_SYN_MASK) | (p & 1u)) != 0u;
+  }
   if (VS == SECDED64) {
     uint32_t r = 0, p = 0;
     v64_acc(lo32(w0), hi32(w0), r, p);
@@ -1398,9 +1468,16 @@ __device__ __forceinline__ void ur_step(const VecArgs& a, uint64_t* X, uint64_t*
   dot = fma(m0, m0, dot);
   dot = fma(m1, m1, dot);
 }
+// peer-memory halo: the encoded word of local row i also goes to the
+// neighbour ghost row that mirrors it (VecArgs.halo_up / halo_dn)
+__device__ __forceinline__ void halo_store(const VecArgs& a, int64_t i, uint64_t e) {
+  if (a.halo_up && i < a.halo_n) a.halo_up[i] = e;
+  if (a.halo_dn && i >= a.n - a.halo_n && i < a.n) a.halo_dn[i - (a.n - a.halo_n)] = e;
+}
 template <int VS>
 __device__ __forceinline__ void p_step(const VecArgs& a, uint64_t* P, uint64_t* R, int k, uint64_t r0, uint64_t r1,
-                                       uint64_t p0, uint64_t p1, double beta, int lane, const uint8_t* cs) {
+                                       uint64_t p0, uint64_t p1, double beta, int lane, const uint8_t* cs,
+                                       int64_t row0 = 0, bool edge = false) {
   const uint64_t keep = vkeep(VS);
   if (vgrp(VS) == 1) {
     if (vacc_bad<VS>(r0, r1, p0, p1, 0ull, 0ull, 0ull, 0ull)) {  // cold: locate per word
@@ -1420,6 +1497,10 @@ __device__ __forceinline__ void p_step(const VecArgs& a, uint64_t* P, uint64_t* 
   venc2<VS>(round_k(as_u(n0), vk(VS)), round_k(as_u(n1), vk(VS)), lane, cs, e0, e1);
   P[k] = e0;
   P[k + 32] = e1;
+  if (edge) {   // warp-uniform: this RB holds rows of the first / last grid row of the strip
+    halo_store(a, row0 + k, e0);
+    halo_store(a, row0 + k + 32, e1);
+  }
 }
 // 0 (default): calc_p's end-of-iteration logic runs in a one-thread kernel
 // after it (measured r2c: protected calc_p 0.0758 -> 0.0723 ms at 4096^2);
@@ -1440,6 +1521,8 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
                                        uint64_t r0, uint64_t r1, uint64_t p0, uint64_t p1) {
   uint64_t* P = a.p + base + lane;
   uint64_t* R = a.r + base + lane;
+  const bool edge = a.halo_n > 0 && (base < a.halo_n || base + 256 > a.n - a.halo_n);
+  const int64_t row0 = base + lane;
 #if ABFT_P_PREFETCH == 2
   // every word of the RB in flight at once (16 loads per lane), then the steps
   uint64_t rr[8], pp[8];
@@ -1450,7 +1533,8 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
     pp[2 * j] = ldg64(P + 64 * j); pp[2 * j + 1] = ldg64(P + 64 * j + 32);
   }
 #pragma unroll
-  for (int j = 0; j < 4; j++) p_step<VS>(a, P, R, 64 * j, rr[2 * j], rr[2 * j + 1], pp[2 * j], pp[2 * j + 1], beta, lane, cs);
+  for (int j = 0; j < 4; j++)
+    p_step<VS>(a, P, R, 64 * j, rr[2 * j], rr[2 * j + 1], pp[2 * j], pp[2 * j + 1], beta, lane, cs, row0, edge);
 #elif ABFT_P_PREFETCH
   // Register double buffer: step k+64's four words are in flight while step k
   // decodes / encodes (the codec ALU otherwise serialises with the next loads).
@@ -1465,14 +1549,15 @@ __device__ __forceinline__ void p_full(const VecArgs& a, int64_t base, int lane,
       nr0 = ldg64(R + k + 64); nr1 = ldg64(R + k + 96);
       np0 = ldg64(P + k + 64); np1 = ldg64(P + k + 96);
     }
-    p_step<VS>(a, P, R, k, r0, r1, p0, p1, beta, lane, cs);
+    p_step<VS>(a, P, R, k, r0, r1, p0, p1, beta, lane, cs, row0, edge);
     r0 = nr0; r1 = nr1; p0 = np0; p1 = np1;
   }
 #else
-  p_step<VS>(a, P, R, 0, r0, r1, p0, p1, beta, lane, cs);
+  p_step<VS>(a, P, R, 0, r0, r1, p0, p1, beta, lane, cs, row0, edge);
 #pragma unroll 1
   for (int k = 64; k < 256; k += 64)
-    p_step<VS>(a, P, R, k, ldg64(R + k), ldg64(R + k + 32), ldg64(P + k), ldg64(P + k + 32), beta, lane, cs);
+    p_step<VS>(a, P, R, k, ldg64(R + k), ldg64(R + k + 32), ldg64(P + k), ldg64(P + k + 32), beta, lane, cs, row0,
+               edge);
 #endif
 }
 
@@ -1578,6 +1663,7 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : ABFT_P_MINB) k_calc_p(
       double P = fma(beta, as_d(pw & keep), as_d(rw & keep));
       uint64_t pe = v_encode<VS>(valid ? round_k(as_u(P), vk(VS)) : 0ull, lane, s_lut);
       if (i < a.npad) a.p[i] = pe;
+      if (a.halo_n > 0) halo_store(a, i, pe);
     }
   }
 #if ABFT_P_TICKET
@@ -1603,13 +1689,36 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : ABFT_P_MINB) k_calc_p(
 }
 // ABFT_P_TICKET = 0: the end-of-iteration logic runs in this one-thread kernel
 // after calc_p instead of in calc_p's last block (no per-CTA fence + ticket).
-static __global__ void k_post_p(CgState* st, const int* due) {
+static __global__ void k_post_p(CgState* st, const int* due, int* sig_up, int* sig_dn) {
   pdl_wait();
   pdl_trigger();
   if (st->stop) return;
   if (!st->dist && st->abort_policy && *((volatile const int*)due)) { st->stop = 1; st->status = ABFT_E_DUE; }
   else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
   if (!st->pcg) st->rro = st->rrn;
+  if (sig_up || sig_dn) {
+    // peer-memory halo: calc_p (the previous kernel, complete) stored this
+    // iteration's boundary rows into the neighbours' ghost rows; publish them
+    // system-wide, then raise the neighbours' arrival flags to the iteration
+    __threadfence_system();
+    if (sig_up) atomicExch_system(sig_up, st->iters);
+    if (sig_dn) atomicExch_system(sig_dn, st->iters);
+  }
+}
+// Peer-memory halo, consumer side: before the SpMV of iteration iters + 1
+// (boundary tile rows), wait until both neighbours' calc_p of iteration
+// `iters` has published p's ghost rows (flags[0]: from rank - 1, flags[1]: from
+// rank + 1).  A stopped solve does not wait.
+static __global__ void k_wait_halo(const int* flags, const CgState* st, int need_up, int need_dn) {
+  const volatile CgState* vs = st;
+  if (vs->stop) return;
+  const int it = vs->iters;
+  const volatile int* f = flags;
+  while ((need_up && f[0] < it) || (need_dn && f[1] < it)) {
+    if (vs->stop) return;
+    __nanosleep(64);
+  }
+  __threadfence_system();   // acquire: the ghost rows are read after the flags
 }
 
 // Single-reduction CG update (S§8(f) f3): p = enc(fma(beta,

@@ -50,7 +50,7 @@ def _oracle(n, S, vflips, eflips, policy, max_iters, interval=1):
     return st, res, xo[:N], cnt
 
 
-def _loopback(abft, n, P, S, stencil, vflips, eflips, policy, max_iters, interval=1, poll=8, sr=False):
+def _loopback(abft, n, P, S, stencil, vflips, eflips, policy, max_iters, interval=1, poll=8, sr=False, peer=False):
     rows = n // P
     h = n
     ctxs, As, vecs, cnts = [], [], [], []
@@ -83,6 +83,8 @@ def _loopback(abft, n, P, S, stencil, vflips, eflips, policy, max_iters, interva
         vecs.append(vs)
         cnts.append(abft.Counters())
     d = abft.Loopback(P, 0)
+    if peer:
+        d.set_peer_halo(True)
     if sr:
         res = d.cg_solve_sr(ctxs, As, h, vecs, tol=1e-10, max_iters=max_iters, due_policy=policy, counts=cnts,
                             poll_every=poll)
@@ -188,4 +190,51 @@ def test_loopback_single_reduction_cg(abft, n, stencil, P, policy):
     for q in range(P):
         assert res[q].iters == res_o.iters and res[q].status == st and res[q].rrn == res_o.rrn
     assert np.array_equal(x, xo[:N])
+    assert np.array_equal(cnt, cnt_o)
+
+
+@pytest.mark.parametrize("n,stencil,P", [(64, 0, 2), (64, 0, 8), (256, 256, 2), (256, 256, 4), (256, 256, 8)])
+@pytest.mark.parametrize("policy", [0, 1])
+def test_loopback_peer_halo_matches_oracle(abft, n, stencil, P, policy):
+    """Peer-memory halos (abft_dist_set_peer_halo): calc_p stores p's boundary
+    rows straight into the neighbours' ghost rows and the SpMV waits on arrival
+    flags — iterations, residuals, x and counters bit-exact against the
+    single-domain oracle, flips in halo cells included (tiled strips: the wait
+    overlaps the interior tile rows on the comm stream)."""
+    S = orc.SECDED64
+    rows = n // P
+    vflips = [((rows - 1) * n + 5, [9]), (rows * n + 7, [40]), (rows * n // 2 + 3, [0]), (n * n - 1, [63])]
+    eflips = [(5 * (rows * n - 2) + 4, 17), (5 * (n * n // 2 + 11) + 2, 60)]
+    st, res_o, xo, cnt_o = _oracle(n, S, vflips, eflips, policy, 400)
+    l0 = abft.launch_count()
+    res, x, cnt = _loopback(abft, n, P, S, stencil, vflips, eflips, policy, 400, peer=True)
+    l_peer = abft.launch_count() - l0
+    assert st == 0
+    for q in range(P):
+        assert res[q].iters == res_o.iters and res[q].status == st, (q, res[q].iters, res_o.iters)
+        assert res[q].rrn == res_o.rrn and res[q].rr0 == res_o.rr0
+    assert np.array_equal(x, xo)
+    assert np.array_equal(cnt, cnt_o), (cnt, cnt_o)
+    # the halo step ran as flag waits (one kernel per rank and iteration), not copies
+    l0 = abft.launch_count()
+    _loopback(abft, n, P, S, stencil, vflips, eflips, policy, 400)
+    l_copy = abft.launch_count() - l0
+    assert l_peer - l_copy >= P * res_o.iters, (l_peer, l_copy)
+
+
+@pytest.mark.parametrize("P", [2, 4])
+@pytest.mark.parametrize("policy", [0, 1])
+def test_loopback_peer_halo_due(abft, P, policy):
+    """A same-word double flip (DUE) in a halo row of x0 with peer halos:
+    the DUE consensus and the statuses / counters match the oracle."""
+    n, S = 256, orc.SECDED64
+    rows = n // P
+    vflips = [(rows * n + 3, [5, 6])]
+    st, res_o, xo, cnt_o = _oracle(n, S, vflips, [], policy, 60)
+    res, x, cnt = _loopback(abft, n, P, S, n, vflips, [], policy, 60, peer=True)
+    for q in range(P):
+        assert res[q].iters == res_o.iters and res[q].status == st
+    if policy == 0:
+        assert st == orc.E_DUE
+    assert np.array_equal(x, xo)
     assert np.array_equal(cnt, cnt_o)

@@ -75,3 +75,49 @@ def test_host_codec_matches_oracle(lib, orc, inst_name):
             w[a // 32] ^= np.uint32(1 << (a % 32))
             w[b // 32] ^= np.uint32(1 << (b % 32))
             assert lib.codec_host_check(inst, list(w)) == orc.DUE
+
+
+def test_host_pair_fast_check_matches_oracle(lib, orc):
+    """The tiled SpMV's pair-packed E-SECDED fast check (codec e96_acc2, host
+    hook inst 5) says 'clean' exactly when the oracle finds both codewords
+    clean: every single flip of either codeword, random doubles within one and
+    across both, and random 3-flip patterns."""
+    rng = np.random.default_rng(77)
+    inst = orc.I_E_SECDED
+    for _ in range(20):
+        cws = []
+        for _ in range(2):
+            data = _rand_words(orc, inst, rng)
+            cws.append(orc.secded_encode(inst, data))
+        both = np.concatenate(cws)
+        assert lib.codec_host_check(5, list(both)) == orc.CLEAN
+        patterns = [[b] for b in range(192)]
+        patterns += [list(rng.choice(192, 2, replace=False)) for _ in range(200)]
+        patterns += [list(rng.choice(192, 3, replace=False)) for _ in range(100)]
+        for pat in patterns:
+            w = both.copy()
+            for b in pat:
+                w[b // 32] ^= np.uint32(1 << (b % 32))
+            ref = [orc.secded_check(inst, w[3 * k:3 * k + 3].copy()) for k in range(2)]
+            clean = all(o[0] == orc.CLEAN for o in ref)
+            assert (lib.codec_host_check(5, list(w)) == orc.CLEAN) == clean, pat
+
+
+def test_host_pair_window_check_matches_oracle(lib, orc):
+    """The decoded window's pair-packed V-SECDED64 fast check (codec v64_acc2,
+    host hook inst 6) says 'clean' exactly when the oracle finds both codewords
+    clean (singles of either word, random doubles and triples)."""
+    rng = np.random.default_rng(78)
+    inst = orc.I_V_SECDED64
+    for _ in range(20):
+        both = np.concatenate([orc.secded_encode(inst, _rand_words(orc, inst, rng)) for _ in range(2)])
+        assert lib.codec_host_check(6, list(both)) == orc.CLEAN
+        patterns = [[b] for b in range(128)]
+        patterns += [list(rng.choice(128, 2, replace=False)) for _ in range(200)]
+        patterns += [list(rng.choice(128, 3, replace=False)) for _ in range(100)]
+        for pat in patterns:
+            w = both.copy()
+            for b in pat:
+                w[b // 32] ^= np.uint32(1 << (b % 32))
+            clean = all(orc.secded_check(inst, w[2 * k:2 * k + 2].copy())[0] == orc.CLEAN for k in range(2))
+            assert (lib.codec_host_check(6, list(w)) == orc.CLEAN) == clean, pat

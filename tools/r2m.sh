@@ -6,7 +6,7 @@ python -c "import __graft_entry__ as g; g.build()" > gpurun_out/build_$T.log 2>&
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw,power.limit --format=csv > gpurun_out/gpu_$T.txt
 T=$T VARIANTS="$VARIANTS" TESTS="$TESTS" bash tools/r2k.sh
 if [ -n "$CRC" ]; then
-  for so in default $CRC; do
+  for so in default $(echo $CRC | sed "s/^-$//"); do
     if [ $so = default ]; then unset ABFT_SO; else export ABFT_SO=variants/libabft_$so.so; fi
     timeout 900 python tools/sweep.py --grid 8192 --iters 200 --no-schemes --intervals 1,128 --only CRC32C,SECDED64 \
       --out gpurun_out/sweep_crc_${so}_$T.json > gpurun_out/sweep_crc_${so}_$T.log 2>&1
