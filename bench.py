@@ -134,9 +134,10 @@ def build_problem(n: int, ny: int, rank: int, world: int, device, chunk_rows=Non
 class Solver:
     """One configuration (protected or unprotected twin) of the solve."""
 
-    def __init__(self, abft, ctx, P, es, rs, vs, dist=None, check_interval=1, sr=False):
+    def __init__(self, abft, ctx, P, es, rs, vs, dist=None, check_interval=1, sr=False, peer=False):
         import torch
         self.abft, self.ctx, self.P, self.dist = abft, ctx, P, dist
+        self.peer = peer and dist is not None and not sr   # peer-memory halos (DESIGN.md §8)
         self.check_interval = check_interval
         self.es, self.rs, self.vs = es, rs, vs
         N, halo = P["N"], P["halo"]
@@ -191,6 +192,15 @@ class Solver:
                 res = self.abft.cg_solve_sr(self.ctx, self.A, *self.vecs, tol=tol, max_iters=max_iters, due_policy=1,
                                             counts=self.counts, poll_every=32)
         elif self.dist is not None:
+            # peer-memory halos name this solver's p: map the neighbours' p once
+            # (collective), and never leave another solver's mapping enabled
+            owner = getattr(self.dist, "_peer_owner", None)
+            if owner is not (self if self.peer else None):
+                self.dist.disable_peer_halo()
+                self.dist._peer_owner = None
+                if self.peer:
+                    self.dist.enable_peer_halo(self.vecs[3])
+                    self.dist._peer_owner = self
             res = self.dist.cg_solve(self.ctx, self.A, self.halo, *self.vecs, tol=tol, max_iters=max_iters,
                                      due_policy=1, counts=self.counts, poll_every=32,
                                      check_interval=self.check_interval)
@@ -374,6 +384,8 @@ def main():
     ap.add_argument("--fuse", action="store_true", help="main line on the fused calc_p path (DESIGN.md §6.1)")
     ap.add_argument("--no-pdl", action="store_true", help="plain launches in the CG loop (DESIGN.md §6.2)")
     ap.add_argument("--no-fused-extra", action="store_true", help="skip the fused-calc_p side measurement")
+    ap.add_argument("--peer-halo", action="store_true",
+                    help="N > 1: p's halo stored by the neighbours' calc_p over NVLink peer memory (DESIGN.md §8)")
     ap.add_argument("--no-sr-extra", action="store_true",
                     help="skip the single-reduction CG side measurement (DESIGN.md §4.1)")
     args = ap.parse_args()
@@ -403,7 +415,7 @@ def main():
     spmv_bpr = FUSED_SPMV_BYTES_PER_ROW if fused else SPMV_BYTES_PER_ROW
     cg_bpr = FUSED_CG_BYTES_PER_ROW if fused else CG_BYTES_PER_ROW
     dobj = abft.Dist(rank, world, local) if dist_on else None
-    prot = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj)
+    prot = Solver(abft, ctx, P, abft.SECDED64, abft.SECDED64, abft.SECDED64, dobj, peer=args.peer_halo)
     with ClockSampler(local) as clk:
         r_p = timed(prot, args.steps, args.warmup, args.tol, args.max_iters, dist_on)
         # roofline pass: same workload, every SpMV launch bracketed by CUDA events on
@@ -413,7 +425,7 @@ def main():
     # per-kernel breakdown: one extra, untimed, fully profiled step
     r_pk = timed(prot, 1, 0, args.tol, args.max_iters, dist_on, profile=15)
     del prot
-    twin = Solver(abft, ctx, P, abft.NONE, abft.NONE, abft.NONE, dobj)
+    twin = Solver(abft, ctx, P, abft.NONE, abft.NONE, abft.NONE, dobj, peer=args.peer_halo)
     r_u = timed(twin, args.steps, max(1, args.warmup // 2), args.tol, args.max_iters, dist_on)
     r_uk = timed(twin, 1, 0, args.tol, args.max_iters, dist_on, profile=15)
     del twin
@@ -508,7 +520,8 @@ def main():
                    "tol": args.tol, "iters_per_step": r_p["iters"] / args.steps,
                    "l2": f"inputs larger than L2 ({cg_bpr * N / 1e9:.2f} GB moved per CG iteration vs 126 MB L2)",
                    "parallelism": f"row-block strips x{world}" if world > 1 else "single GPU",
-                   "fused_calc_p": fused, "pdl": not args.no_pdl and not dist_on, "bytes_per_row_per_iter": cg_bpr},
+                   "fused_calc_p": fused, "pdl": not args.no_pdl and not dist_on, "bytes_per_row_per_iter": cg_bpr,
+                   "halo": ("peer-memory" if args.peer_halo else "nccl send/recv") if world > 1 else None},
         "roofline": {"bound": "hbm",
                      "kernel": "k_spmv_tile (fused calc_p + protected SpMV + p.w)" if fused
                      else "k_spmv_tile (protected SpMV + p.w)",

@@ -2007,6 +2007,12 @@ static __device__ void apply_op_sr(int op, double g, double d, CgState* st, bool
   else if (st->iters >= st->max_iters) { st->stop = 1; st->status = ABFT_E_NOT_CONVERGED; }
 }
 
+// ABFT_RED_PREFETCH (default 1): stop flag, CG state and DUE flag loaded at
+// the start of k_reduce (their latency overlapping the subtree loads); the
+// scalar logic runs on a register copy of the state
+#ifndef ABFT_RED_PREFETCH
+#define ABFT_RED_PREFETCH 1
+#endif
 // TWO: also reduce partials2 (second tree, same order) and apply the
 // single-reduction CG logic (op 6 / 7) to both results.
 template <bool TWO>
@@ -2021,18 +2027,35 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
   __shared__ bool s_last;
   pdl_wait();   // partials of the producing kernel
   pdl_trigger();
-  if (st && op != 1 && op != 7 && op != 8 && op != 10 && st->stop) return;
+  const bool check_stop = st && op != 1 && op != 7 && op != 8 && op != 10;
+#if ABFT_RED_PREFETCH
+  // the stop flag, the CG state and the DUE flag are loaded now, in flight
+  // while the subtree is reduced (thread 0: used by the last block)
+  const int stopv = check_stop ? *(volatile const int*)&st->stop : 0;
+  CgState loc;
+  bool due_pre = false;
+  if (threadIdx.x == 0) {
+    if (st) loc = *st;
+    due_pre = *((volatile const int*)due) != 0;
+  }
+#else
+  if (check_stop && st->stop) return;
+#endif
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int64_t base = (int64_t)blockIdx.x * leaves;
   const int nw = leaves >= 8 ? 8 : 1;
   const int64_t per = leaves / nw;
+  double r = 0.0, r2 = 0.0;
   if (warp < nw) {
-    const double r = warp_subtree(partials + base + warp * per, per, nrb - base - warp * per, lane);
-    if (lane == 0) s_w[warp] = r;
-    if (TWO) {
-      const double r2 = warp_subtree(partials2 + base + warp * per, per, nrb - base - warp * per, lane);
-      if (lane == 0) s_w2[warp] = r2;
-    }
+    r = warp_subtree(partials + base + warp * per, per, nrb - base - warp * per, lane);
+    if (TWO) r2 = warp_subtree(partials2 + base + warp * per, per, nrb - base - warp * per, lane);
+  }
+#if ABFT_RED_PREFETCH
+  if (stopv) return;   // uniform over the grid
+#endif
+  if (warp < nw && lane == 0) {
+    s_w[warp] = r;
+    if (TWO) s_w2[warp] = r2;
   }
   __syncthreads();
   double root = 0.0, root2 = 0.0;
@@ -2055,12 +2078,21 @@ static __global__ void __launch_bounds__(256) k_reduce(const double* partials, i
   }
   if (threadIdx.x != 0) return;
   if (gridDim.x > 1) *ticket = 0;
+#if ABFT_RED_PREFETCH
+  const bool dueflag = due_pre;
+  CgState* const sp = &loc;   // the scalar logic on the register copy, written back once
+#else
   const bool dueflag = *((volatile const int*)due) != 0;
+  CgState* const sp = st;
+#endif
   if (TWO && op == 10) { out[0] = root; out[1] = (double)(dueflag ? 1 : 0); out[2] = root2; return; }
-  if (TWO) { apply_op_sr(op, root2, root, st, dueflag); return; }
   if (op == 0) { *out = root; return; }
   if (op == 4) { out[0] = root; out[1] = (double)(dueflag ? 1 : 0); out[2] = 0.0; return; }
-  apply_op(op, root, st, dueflag);
+  if (TWO) apply_op_sr(op, root2, root, sp, dueflag);
+  else apply_op(op, root, sp, dueflag);
+#if ABFT_RED_PREFETCH
+  *st = loc;
+#endif
 }
 
 // Cluster form of k_reduce (a6) for p2 <= RED_CL_MAX padded leaves: one thread

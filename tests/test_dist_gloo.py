@@ -203,3 +203,91 @@ def test_bench_traffic_only_for_the_captured_workload():
     assert not bench.traffic_matches(t, 4096, 2, False)
     assert not bench.traffic_matches(t, 4096, 1, True)
     assert not bench.traffic_matches(None, 4096, 1, False)
+
+
+# ---------------------------------------------------------------- peer-memory halo handshake
+def _peer_worker(rank, world, port, q):
+    """Dist.enable_peer_halo's host logic over gloo with the CUDA IPC calls
+    faked: every rank publishes (handle, offset) of its p and of its flag
+    words, maps its neighbours' and hands abft_dist_set_peer_halo rank-1's p
+    and flags[1], rank+1's p and flags[0]."""
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import ctypes as C
+        from paper_conf_cluster_pawelczakmpm17_b200 import abft
+        P_BASE, F_BASE = 0x10000000, 0x20000000   # fake device addresses of rank r: base + r * 0x1000
+
+        class FakeLib:
+            def abft_dist_flags(self, h, out):
+                out._obj.value = F_BASE + rank * 0x1000
+                return 0
+
+            def abft_ipc_get_handle(self, ptr, hb, off):   # handle = allocation base, 8 bytes LE
+                o = 8 if ptr.value >= F_BASE else 16
+                base = ptr.value - o
+                buf = (C.c_uint8 * 64).from_address(hb.value)
+                for i in range(8):
+                    buf[i] = base >> (8 * i) & 0xFF
+                off._obj.value = o
+                return 0
+
+            def abft_ipc_open_handle(self, hb, off, out):
+                buf = (C.c_uint8 * 64).from_address(hb.value)
+                out._obj.value = sum(buf[i] << (8 * i) for i in range(8)) + off
+                return 0
+
+            def abft_ipc_close_handle(self, ptr, off):
+                return 0
+
+            def abft_dist_set_peer_halo(self, h, enable, pp, pf):
+                if enable:
+                    pa = (C.c_void_p * 2).from_address(pp.value)
+                    fa = (C.c_void_p * 2).from_address(pf.value)
+                    self.got = ([pa[0], pa[1]], [fa[0], fa[1]])
+                return 0
+
+        fake = FakeLib()
+        real = abft._lib
+        abft._lib = fake
+        try:
+            d = abft.Dist.__new__(abft.Dist)
+            d.h, d.rank, d.nranks = C.c_void_p(1), rank, world
+
+            class FakeVec:
+                class data:
+                    @staticmethod
+                    def data_ptr():
+                        return P_BASE + rank * 0x1000
+
+            d.enable_peer_halo(FakeVec())
+            q.put((rank, fake.got))
+        finally:
+            abft._lib = real
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_peer_halo_handshake_gloo(world):
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = 29650 + world
+    procs = [ctx.Process(target=_peer_worker, args=(r, world, port, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    got = dict(q.get(timeout=240) for _ in range(world))
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    P_BASE, F_BASE = 0x10000000, 0x20000000
+    for r in range(world):
+        pp, pf = got[r]
+        up, dn = r > 0, r < world - 1
+        # rank-1's and rank+1's p, mapped at their own addresses (handle + offset)
+        assert pp[0] == (P_BASE + (r - 1) * 0x1000 if up else None)
+        assert pp[1] == (P_BASE + (r + 1) * 0x1000 if dn else None)
+        # rank-1 is signalled in its flags[1] (+4 bytes), rank+1 in its flags[0]
+        assert pf[0] == (F_BASE + (r - 1) * 0x1000 + 4 if up else None)
+        assert pf[1] == (F_BASE + (r + 1) * 0x1000 if dn else None)
