@@ -51,6 +51,39 @@ def main():
         res = abft.cg_solve(ctx, A, b, xs, rr, pp, ww, tol=1e-10, max_iters=6, due_policy=1, counts=cnt, poll_every=3)
         torch.cuda.synchronize()
         print(f"scheme {S}: cg iters {res.iters} counts {int(cnt.read().sum())}", flush=True)
+        if S == abft.SECDED64:   # the bench's arrangement: PDL between the CG kernels (early window TMA)
+            ctx.set_pdl(True)
+            res = abft.cg_solve(ctx, A, b, xs, rr, pp, ww, tol=1e-10, max_iters=6, due_policy=1, counts=cnt,
+                                poll_every=3)
+            ctx.set_pdl(False)
+            torch.cuda.synchronize()
+            print(f"scheme {S} + PDL: cg iters {res.iters}", flush=True)
+    # peer-memory halos between two loopback ranks (calc_p's stores into the
+    # neighbour's ghost rows, arrival flags, the SpMV's wait)
+    m, P = 256, 2
+    S = abft.SECDED64
+    rows = m // P
+    ctxs, As, vecs = [], [], []
+    for q in range(P):
+        vq, cq, rq = gen.strip_csr(m, q * rows, (q + 1) * rows, ny=m, col_offset=m, device="cuda")
+        cx = abft.Context(0)
+        Aq = abft.Matrix(vq, cq.to(torch.int32), rq.to(torch.int32), rows * m, rows * m + 2 * m, S, S, row_base=m,
+                         col_base=0, stencil_n=m)
+        assert Aq.encode(cx) == 0
+        bq = torch.zeros(rows * m + 2 * m, dtype=torch.float64, device="cuda")
+        bq[m:m + rows * m] = gen.tealeaf_rhs(m, q * rows, (q + 1) * rows, ny=m).cuda()
+        bv = abft.Vector.from_values(cx, bq, S)
+        xv = abft.Vector.from_values(cx, bq.clone(), S)
+        ctxs.append(cx)
+        As.append(Aq)
+        vecs.append([bv, xv] + [abft.Vector.empty(rows * m + 2 * m, S) for _ in range(3)])
+    d = abft.Loopback(P, 0)
+    d.set_peer_halo(True)
+    res = d.cg_solve(ctxs, As, m, vecs, tol=1e-10, max_iters=8, due_policy=1, counts=[abft.Counters() for _ in range(P)],
+                     poll_every=4)
+    torch.cuda.synchronize()
+    d.close()
+    print(f"loopback peer halo: iters {[r.iters for r in res]}", flush=True)
 
 
 if __name__ == "__main__":
