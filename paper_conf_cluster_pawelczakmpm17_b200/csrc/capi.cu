@@ -230,6 +230,7 @@ int abft_ctx_create(int device, abft_ctx** out) {
     CUDA_TRY(cudaMalloc(&c->crc, sizeof(CrcTables)));
     CUDA_TRY(cudaMemcpy(c->crc, h.data(), sizeof(CrcTables), cudaMemcpyHostToDevice));
   }
+  prepare_kernels(device);
   int e = ensure_partials(c, 1024);
   if (e) return e;
   *out = c;

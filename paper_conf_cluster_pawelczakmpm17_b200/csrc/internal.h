@@ -160,6 +160,7 @@ int launch_csr_encode(abft_csr* A, uint32_t* flags, cudaStream_t s);
 int launch_check_csr(const abft_csr* A, DevCounts* c, int* due, int scrub, cudaStream_t s);
 int launch_inject(void* base, uint64_t bit, cudaStream_t s);
 int launch_wait_halo(const int* flags, const CgState* st, int need_up, int need_dn, cudaStream_t s);
+void prepare_kernels(int device);
 // phase 0: the faults of iteration 0 (before init); phase 1: those of
 // iteration state->iters + 1 (skipped once the solve stopped)
 int launch_inject_sched(const DevFault* f, int n, const CgState* st, int phase, cudaStream_t s);

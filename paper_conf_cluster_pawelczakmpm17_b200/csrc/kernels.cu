@@ -17,6 +17,8 @@
 // issues fully coalesced 8-byte loads of the vectors (one 256-byte line per
 // warp-instruction).  The codec fast path ("is this codeword clean?") is
 // inline; locating/correcting a flip is a __noinline__ cold path.
+#include <atomic>
+
 #include "kernels_impl.cuh"
 
 namespace abft {
@@ -105,9 +107,43 @@ int launch_calc_ur(const VecArgs& a, int vs, cudaStream_t s) {
   }
   return 1;
 }
+// ABFT_P_BULK (default 1): G = 1 schemes on whole CP_STAGE-row stages take the
+// bulk-copy staged persistent kernel k_calc_p_bulk
+#ifndef ABFT_P_BULK
+#define ABFT_P_BULK 1
+#endif
+// per-device function attributes of the kernels with > 48 KB of dynamic SMEM
+// that may first launch inside a CG-graph capture (abft_ctx_create calls this)
+void prepare_kernels(int device) {
+  (void)device;
+  cudaFuncSetAttribute(k_calc_p_bulk<NONE>, cudaFuncAttributeMaxDynamicSharedMemorySize, CP_SMEM);
+  cudaFuncSetAttribute(k_calc_p_bulk<SED>, cudaFuncAttributeMaxDynamicSharedMemorySize, CP_SMEM);
+  cudaFuncSetAttribute(k_calc_p_bulk<SECDED64>, cudaFuncAttributeMaxDynamicSharedMemorySize, CP_SMEM);
+}
+template <int VS>
+static void calc_p_bulk(const VecArgs& a, cudaStream_t s) {
+  static std::atomic<int> grid{0};   // CTAs resident at once (persistent grid)
+  if (!grid.load(std::memory_order_relaxed)) {
+    int dev = 0, sms = 0;
+    cudaGetDevice(&dev);
+    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+    grid.store(sms * CP_CTAS_PER_SM, std::memory_order_relaxed);
+  }
+  const int64_t nstage = a.n / CP_STAGE;
+  const int gmax = grid.load(std::memory_order_relaxed);
+  const int g = (int)(nstage < gmax ? nstage : gmax);
+  launch_k(k_calc_p_bulk<VS>, g, 256, CP_SMEM, s, a);
+}
 int launch_calc_p(const VecArgs& a, int vs, cudaStream_t s) {
   if (a.n <= 0) return 0;
   int nb = blocks_rb(a.n);
+  if (ABFT_P_BULK && (a.n % CP_STAGE) == 0 && (vs == NONE || vs == SED || vs == SECDED64)) {
+    if (vs == NONE) calc_p_bulk<NONE>(a, s);
+    else if (vs == SED) calc_p_bulk<SED>(a, s);
+    else calc_p_bulk<SECDED64>(a, s);
+    launch_k(k_post_p, 1, 1, 0, s, a.state, (const int*)a.due, a.sig_up, a.sig_dn);
+    return 2;
+  }
   switch (vs) {
     case NONE: launch_k(k_calc_p<NONE>, nb, 256, 0, s, a); break;
     case SED: launch_k(k_calc_p<SED>, nb, 256, 0, s, a); break;

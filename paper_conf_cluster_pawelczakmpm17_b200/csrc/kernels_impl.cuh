@@ -1271,7 +1271,9 @@ __global__ void __launch_bounds__(256, ABFT_TILE_MINB) k_spmv_tile(const SpmvArg
 #ifndef ABFT_TILE_UNROLL
 #define ABFT_TILE_UNROLL 8
 #endif
-  constexpr int kPassUnroll = ABFT_TILE_UNROLL;
+  // (G > 1 vector codecs and the CRC element / rowptr codecs spill at 80
+  // registers when the 8 passes are unrolled: they keep the rolled loop)
+  constexpr int kPassUnroll = (vgrp(VS) == 1 && ES != CRC32C && RS != CRC32C) ? ABFT_TILE_UNROLL : 1;
 #pragma unroll kPassUnroll
   for (int k = 0; k < 8; k++) {
     const int st = k % NST;
@@ -1687,6 +1689,93 @@ __global__ void __launch_bounds__(256, vgrp(VS) > 1 ? 4 : ABFT_P_MINB) k_calc_p(
   }
 #endif
 }
+// calc_p staged by bulk copies (a5, G = 1 vector schemes): a persistent grid
+// (CP_CTAS_PER_SM CTAs per SM) walks the vector in stages of CP_STAGE rows;
+// thread 0 keeps CP_NST stages of r and p in flight (two 1-D
+// cp.async.bulk copies into SMEM per stage, an mbarrier each), so the codec
+// work of one stage never stalls the loads of the next.  Each row is checked
+// (owner: counts + scrub), p = enc(round(fma(beta, p, r))) stored back, and
+// the peer-memory halo rows mirrored — word for word what k_calc_p does.
+constexpr int CP_STAGE = 1024;   // rows per stage: 8 KB of r + 8 KB of p
+constexpr int CP_NST = 3;
+constexpr int CP_CTAS_PER_SM = 4;
+constexpr int CP_SMEM = CP_NST * 2 * CP_STAGE * 8 + 128;
+static __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                   smem_u32(dst)),
+               "l"(reinterpret_cast<uint64_t>(src)), "r"(bytes), "r"(smem_u32(bar))
+               : "memory");
+}
+template <int VS>
+__global__ void __launch_bounds__(256, CP_CTAS_PER_SM) k_calc_p_bulk(VecArgs a) {
+  static_assert(vgrp(VS) == 1, "G = 1 vector schemes");
+  extern __shared__ __align__(128) uint8_t s_cp[];
+  __shared__ __align__(16) uint8_t s_lut[128];
+  __shared__ __align__(8) uint64_t s_bar[CP_NST];
+  uint64_t* sbuf = reinterpret_cast<uint64_t*>(s_cp + ((128u - (smem_u32(s_cp) & 127u)) & 127u));
+  const int64_t nstage = a.n / CP_STAGE;   // host: n % CP_STAGE == 0
+  const int64_t G = gridDim.x;
+  const int64_t mine = nstage > blockIdx.x ? (nstage - blockIdx.x + G - 1) / G : 0;   // stages of this CTA
+  auto issue = [&](int64_t j) {   // j-th stage of this CTA into ring slot j % CP_NST
+    const int slot = (int)(j % CP_NST);
+    const int64_t row = (blockIdx.x + j * G) * CP_STAGE;
+    uint64_t* dst = sbuf + (int64_t)slot * 2 * CP_STAGE;
+    mbar_expect_tx(&s_bar[slot], 2 * CP_STAGE * 8);
+    bulk_g2s(dst, a.r + row, CP_STAGE * 8, &s_bar[slot]);
+    bulk_g2s(dst + CP_STAGE, a.p + row, CP_STAGE * 8, &s_bar[slot]);
+  };
+  if (threadIdx.x == 0) {   // r and p were last written >= 2 kernels back: loaded before the PDL wait
+    for (int k = 0; k < CP_NST; k++) mbar_init(&s_bar[k], 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    for (int64_t j = 0; j < CP_NST && j < mine; j++) issue(j);
+  }
+  if (VS == SECDED64) load_lut(s_lut);
+  pdl_wait();   // beta / stop from the rrn reduction
+  pdl_trigger();
+  const int stop = a.state->stop;
+  const double beta = a.state->beta;
+  __syncthreads();   // barriers initialised, LUT in place
+  if (stop) {   // drain the copies in flight before the CTA exits
+    if (threadIdx.x == 0)
+      for (int64_t j = 0; j < CP_NST && j < mine; j++) mbar_wait(&s_bar[j], 0u);
+    return;
+  }
+  const uint64_t keep = vkeep(VS);
+  const int lane = threadIdx.x & 31;
+  for (int64_t j = 0; j < mine; j++) {
+    const int slot = (int)(j % CP_NST);
+    mbar_wait(&s_bar[slot], (uint32_t)((j / CP_NST) & 1));
+    const uint64_t* sr = sbuf + (int64_t)slot * 2 * CP_STAGE;
+    const uint64_t* sp = sr + CP_STAGE;
+    const int64_t row = (blockIdx.x + j * G) * CP_STAGE;
+    uint64_t rv[4], pv[4];
+#pragma unroll
+    for (int t = 0; t < 4; t++) {
+      rv[t] = sr[threadIdx.x + 256 * t];
+      pv[t] = sp[threadIdx.x + 256 * t];
+    }
+    if (vacc_bad<VS>(rv[0], rv[1], rv[2], rv[3], pv[0], pv[1], pv[2], pv[3])) {   // cold: per word, owner
+#pragma unroll 1
+      for (int t = 0; t < 4; t++) {
+        const int64_t i = row + threadIdx.x + 256 * t;
+        rv[t] = v1_check<VS>(rv[t], a.r + i, true, a.counts, a.due);
+        pv[t] = v1_check<VS>(pv[t], a.p + i, true, a.counts, a.due);
+      }
+    }
+    const bool edge = a.halo_n > 0 && (row < a.halo_n || row + CP_STAGE > a.n - a.halo_n);
+#pragma unroll
+    for (int t = 0; t < 4; t++) {
+      const int64_t i = row + threadIdx.x + 256 * t;
+      const double P = fma(beta, as_d(pv[t] & keep), as_d(rv[t] & keep));
+      const uint64_t e = v_encode<VS>(round_k(as_u(P), vk(VS)), lane, s_lut);
+      a.p[i] = e;
+      if (edge) halo_store(a, i, e);
+    }
+    __syncthreads();   // every thread is done with this slot
+    if (threadIdx.x == 0 && j + CP_NST < mine) issue(j + CP_NST);
+  }
+}
+
 // ABFT_P_TICKET = 0: the end-of-iteration logic runs in this one-thread kernel
 // after calc_p instead of in calc_p's last block (no per-CTA fence + ticket).
 static __global__ void k_post_p(CgState* st, const int* due, int* sig_up, int* sig_dn) {
