@@ -111,7 +111,9 @@ int abft_vec_encode(abft_ctx* ctx, abft_vec* v, void* stream);
 
 /* Check every codeword of v, write the masked values to out_masked (device
  * f64[n], may be NULL), count into dcnt (device, may be NULL), scrub single
- * flips in place. */
+ * flips in place.  The vector read of PAPER.md P:441-451 (§VI: the reserved
+ * low mantissa bits are masked to 0 when the value is used) as a standalone
+ * call; checks and counts follow DESIGN.md §3.6 / §3.8. */
 int abft_vec_decode(abft_ctx* ctx, abft_vec* v, double* out_masked, abft_counts* dcnt, void* stream);
 
 /* a3: protected SpMV out = A*in over nchunks chunks.
@@ -230,7 +232,11 @@ int abft_calc_p_spmv(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* p_
 
 /* Check every codeword of the matrix chunks and of the nvec vectors, counting
  * into dcnt.  scrub: 0 count only, 1 count and correct single flips in place,
- * 2 detection only (every failing codeword is a DUE, nothing is written). */
+ * 2 detection only (every failing codeword is a DUE, nothing is written).
+ * The whole-structure check of PAPER.md P:398-425 (§VI "less frequent
+ * correctness checking": the full check at the end of a solve whose
+ * interval does not divide the iteration count) and the config-5 campaign's
+ * per-trial check (SURVEY S§8(d)); semantics DESIGN.md §3.8 / §3.9. */
 int abft_check_all(abft_ctx* ctx, const abft_csr* A, int nchunks, abft_vec* vecs, int nvec, int scrub,
                    abft_counts* dcnt, void* stream);
 
@@ -253,7 +259,10 @@ typedef struct { int32_t iter; int32_t target; int64_t word; int32_t bit; int32_
 int abft_ctx_set_faults(abft_ctx* ctx, const abft_fault* faults, int nfaults, const abft_csr* A, int nchunks,
                         abft_vec* const* vecs /* [5]: b, x, r, p, w */);
 
-/* Copy the device counters to host_out[ABFT_T_COUNT*ABFT_SCHEME_COUNT].  Syncs. */
+/* Copy the device counters to host_out[ABFT_T_COUNT*ABFT_SCHEME_COUNT].  Syncs.
+ * The per-scheme detected / corrected / uncorrectable counts the paper's
+ * evaluation reports (§VII) and north_star asks for;
+ * counting rule DESIGN.md §3.8 (first logical read, owner counts). */
 int abft_counts_read(const abft_counts* dcnt, abft_counts* host_out, void* stream);
 int abft_counts_reset(abft_counts* dcnt, void* stream);
 
